@@ -1,0 +1,320 @@
+"""Pins for the CPU oracle (no GPU).  Each test checks the oracle against
+something other than itself: dense Gaussian elimination, LAPACK dgtsv, closed
+forms of the 1-D Poisson matrix, exact dyadic PCR values, brute-force
+orderings, or values printed in the paper (tests/golden/)."""
+import math
+import os
+
+import numpy as np
+import pytest
+import scipy.linalg.lapack as lapack
+
+import oracle
+from oracle import plan as rplan
+from paper_conf_ipps_davidsonzo11_b200 import inputs
+
+GOLDEN = os.path.join(os.path.dirname(__file__), "golden")
+EPS64 = np.finfo(np.float64).eps
+
+
+def dense(a, b, c):
+    n = b.shape[-1]
+    A = np.diag(b.astype(np.float64))
+    if n > 1:
+        A += np.diag(a[1:].astype(np.float64), -1) + np.diag(c[:-1].astype(np.float64), 1)
+    return A
+
+
+# ---------------------------------------------------------------- Thomas ----
+
+@pytest.mark.parametrize("n", [1, 2, 3, 5, 8, 17, 31, 32, 33, 64])
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+def test_thomas_vs_dense_ge(n, dtype):
+    """North_star pin 1: brute-force dense Gaussian elimination (partial
+    pivoting, LAPACK gesv through numpy) for N <= 64."""
+    a, b, c, d = inputs.generate(n, 6, dtype, seed=7)
+    x = oracle.thomas(a, b, c, d)
+    for s in range(6):
+        xr = np.linalg.solve(dense(a[s], b[s], c[s]), d[s].astype(np.float64))
+        err = np.abs(x[s] - xr).max() / max(np.abs(xr).max(), 1e-300)
+        assert err <= 1e-13, (n, s, err)
+
+
+@pytest.mark.parametrize("n", [2, 9, 64])
+def test_thomas_nonsymmetric_and_ignored_corners(n):
+    """a[0] and c[n-1] are outside the matrix: garbage there must not change x
+    (reading R3).  Also a non-symmetric, non-generator matrix vs dense GE."""
+    rng = np.random.default_rng(3)
+    a = rng.uniform(-1, 1, n); c = rng.uniform(-3, 3, n)
+    b = np.abs(a) + np.abs(c) + rng.uniform(0.5, 2, n) * np.sign(rng.uniform(-1, 1, n))
+    d = rng.uniform(-5, 5, n)
+    x0 = oracle.thomas(a, b, c, d)
+    a2, c2 = a.copy(), c.copy()
+    a2[0] = 1e30; c2[-1] = -1e30
+    x1 = oracle.thomas(a2, b, c2, d)
+    assert np.array_equal(x0, x1)
+    A = dense(a, b, c)
+    xr = np.linalg.solve(A, d)
+    assert np.abs(x0 - xr).max() <= 1e-12 * np.abs(xr).max()
+
+
+def test_thomas_special_cases():
+    """N=1: x = d/b; N=2: Cramer's rule; diagonal A: x = d/b (exact)."""
+    x = oracle.thomas([0.0], [4.0], [0.0], [2.0])
+    assert x[0] == 0.5
+    a0, b0, c0, d0 = 0.0, 3.0, 1.0, 5.0
+    a1, b1, c1, d1 = 2.0, 7.0, 0.0, -1.0
+    x = oracle.thomas([a0, a1], [b0, b1], [c0, c1], [d0, d1])
+    det = b0 * b1 - c0 * a1
+    assert np.allclose(x, [(d0 * b1 - c0 * d1) / det, (b0 * d1 - a1 * d0) / det], rtol=1e-15)
+    n = 100
+    rng = np.random.default_rng(1)
+    b = rng.uniform(1, 2, n); d = rng.uniform(-1, 1, n)
+    x = oracle.thomas(np.zeros(n), b, np.zeros(n), d)
+    assert np.array_equal(x, d / b)
+
+
+def poisson_kappa(n):
+    """2-norm condition number of tridiag(-1,2,-1): sin^2(n pi/2(n+1)) / sin^2(pi/2(n+1))."""
+    h = math.pi / (2 * (n + 1))
+    return math.sin(n * h) ** 2 / math.sin(h) ** 2
+
+
+@pytest.mark.parametrize("n", [1, 2, 10, 1024, 65536, 1 << 20])
+def test_thomas_poisson_closed_form_ones(n):
+    """North_star pin 2: tridiag(-1,2,-1) x = 1 has x_i = i(n+1-i)/2 (1-based i)."""
+    a, b, c, d = inputs.generate(n, 1, np.float64, family="poisson_ones")
+    x = oracle.thomas(a, b, c, d)[0]
+    i = np.arange(1, n + 1, dtype=np.float64)
+    xe = i * (n + 1 - i) / 2
+    err = np.abs(x - xe).max() / np.abs(xe).max()
+    assert err <= 10 * poisson_kappa(n) * EPS64, (n, err)
+    assert oracle.backward_error(a, b, c, d, x) <= 1e-14
+
+
+@pytest.mark.parametrize("n", [3, 100, 4096, 1 << 18])
+def test_thomas_poisson_closed_form_eigvec(n):
+    """d_i = sin(i pi/(n+1)) is the smallest eigenvector: x = d / (4 sin^2(pi/(2(n+1))))."""
+    i = np.arange(1, n + 1, dtype=np.float64)
+    d = np.sin(i * math.pi / (n + 1))
+    a = -np.ones(n); c = -np.ones(n); b = 2 * np.ones(n)
+    x = oracle.thomas(a, b, c, d)
+    xe = d / (4 * math.sin(math.pi / (2 * (n + 1))) ** 2)
+    err = np.abs(x - xe).max() / np.abs(xe).max()
+    assert err <= 10 * poisson_kappa(n) * EPS64, (n, err)
+
+
+@pytest.mark.parametrize("n,m", [(64, 8), (1024, 16), (65536, 4), (1 << 20, 2)])
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+def test_thomas_residual_invariant(n, m, dtype):
+    """North_star pin 3: ||Ax-d||_inf/||d||_inf <= 1e-12 on the generated
+    diagonally dominant family (reading R17: the plain residual is applied to
+    this family; the Poisson family uses the backward error above)."""
+    a, b, c, d = inputs.generate(n, m, dtype, seed=11)
+    x = oracle.thomas(a, b, c, d)
+    assert oracle.residual(a, b, c, d, x) <= 1e-12
+
+
+@pytest.mark.parametrize("n", [2, 50, 4097])
+def test_thomas_vs_lapack_dgtsv(n):
+    """Library pin: LAPACK dgtsv (partial pivoting) through scipy."""
+    a, b, c, d = inputs.generate(n, 3, np.float64, seed=5, mu=0.3)
+    x = oracle.thomas(a, b, c, d)
+    for s in range(3):
+        _, _, _, xl, info = lapack.dgtsv(a[s, 1:].copy(), b[s].copy(), c[s, :-1].copy(), d[s].copy())
+        assert info == 0
+        assert np.abs(x[s] - xl).max() <= 1e-12 * np.abs(xl).max()
+
+
+def test_thomas_batch_independence_and_threads():
+    a, b, c, d = inputs.generate(300, 40, np.float64, seed=2)
+    x1 = oracle.thomas(a, b, c, d, threads=1)
+    x4 = oracle.thomas(a, b, c, d, threads=4)
+    assert np.array_equal(x1, x4)
+    xs = oracle.thomas(a[17], b[17], c[17], d[17])
+    assert np.array_equal(xs, x1[17])
+
+
+# ------------------------------------------------------------- generator ----
+
+def test_generator_recipe():
+    """Counter-hash generator: deterministic, exact dyadic values in [-1,1),
+    corners zero, b = |a|+|c|+mu in the target precision, shard-invariant."""
+    for dt, bits in ((np.float32, 23), (np.float64, 52)):
+        a, b, c, d = inputs.generate(1000, 5, dt, seed=3)
+        a2, b2, c2, d2 = inputs.generate(1000, 5, dt, seed=3)
+        assert all(np.array_equal(u, v) for u, v in zip((a, b, c, d), (a2, b2, c2, d2)))
+        assert a.dtype == dt
+        assert np.all(a[:, 0] == 0) and np.all(c[:, -1] == 0)
+        for v in (a, c, d):
+            assert v.min() >= -1 and v.max() < 1
+            scaled = v.astype(np.float64) * 2.0 ** bits
+            assert np.array_equal(scaled, np.round(scaled))
+        assert np.array_equal(b, (np.abs(a) + np.abs(c)) + dt(1))
+        # the first system of a shard equals the corresponding system of the whole batch
+        sa, sb, sc, sd = inputs.generate(1000, 2, dt, seed=3, first_system=3)
+        assert np.array_equal(sd, d[3:5]) and np.array_equal(sb, b[3:5])
+    # different array ids / seeds decorrelate
+    a, _, c, _ = inputs.generate(4096, 1, np.float32, seed=1)
+    assert abs(np.corrcoef(a[0, 1:-1], c[0, 1:-1])[0, 1]) < 0.05
+
+
+def test_splitmix64_known_values():
+    """splitmix64 reference outputs for state 0 (Vigna's generator: the first
+    outputs of the sequence seeded with 0 are these published constants)."""
+    z = inputs.splitmix64(np.array([0, 0x9E3779B97F4A7C15], dtype=np.uint64))
+    assert int(z[0]) == 0xE220A8397B1DCDAF
+    assert int(z[1]) == 0x6E789E6AA1B965F4
+
+
+# ---------------------------------------------------------------- PCR split ----
+
+@pytest.mark.parametrize("n", [8, 37, 64, 100, 1000])
+def test_pcr_split_decouples(n):
+    """After k PCR levels, each residue class mod 2^k is an independent
+    tridiagonal system whose solution is x restricted to that class (Fig. 3a,
+    P:L386-394).  A dropped term, wrong sign or wrong neighbour index in any
+    of the four update formulas breaks this."""
+    a, b, c, d = inputs.generate(n, 3, np.float64, seed=9, mu=0.5)
+    x = oracle.thomas(a, b, c, d)
+    for k in range(0, math.ceil(math.log2(n)) + 1):
+        sa, sb, sc, sd = oracle.pcr_split(a, b, c, d, k)
+        step = 1 << k
+        for r in range(min(step, n)):
+            xs = oracle.thomas(*oracle.subsystem(sa, sb, sc, sd, k, r))
+            assert np.abs(xs - x[:, r::step]).max() <= 1e-12 * np.abs(x).max(), (n, k, r)
+
+
+def test_pcr_split_full_is_diagonal():
+    """k = ceil(log2 n): pure PCR, every row decoupled: x = d'/b'."""
+    n = 100
+    a, b, c, d = inputs.generate(n, 2, np.float64, seed=4)
+    sa, sb, sc, sd = oracle.pcr_split(a, b, c, d, 7)
+    assert np.all(sa == 0) and np.all(sc == 0)
+    x = oracle.thomas(a, b, c, d)
+    assert np.abs(sd / sb - x).max() <= 1e-13 * np.abs(x).max()
+
+
+@pytest.mark.parametrize("n,k", [(300, 1), (300, 4), (300, 7), (1000, 5), (77, 3)])
+def test_pcr_split_exact_zeros(n, k):
+    """Structural pin: after k levels a' = 0 at the first row and c' = 0 at the
+    last row of every residue class (their neighbours are identity rows)."""
+    a, b, c, d = inputs.generate(n, 2, np.float64, seed=1)
+    sa, sb, sc, sd = oracle.pcr_split(a, b, c, d, k)
+    step = 1 << k
+    for r in range(min(step, n)):
+        rows = np.arange(r, n, step)
+        assert np.all(sa[:, rows[0]] == 0)
+        assert np.all(sc[:, rows[-1]] == 0)
+
+
+@pytest.mark.parametrize("k", [1, 2, 5, 7])
+def test_pcr_split_poisson_interior_exact(k):
+    """Structural pin: on tridiag(-1,2,-1), rows 2^k <= i <= n-1-2^k after k
+    unnormalised levels are exactly a' = c' = -2^-k, b' = 2^(1-k) (k1 = k2 =
+    -1/2 at every level: all arithmetic is dyadic and exact)."""
+    n = 600
+    a, b, c, d = inputs.generate(n, 1, np.float64, family="poisson")
+    d = np.round(d * 3)  # integer d in [-3, 3]
+    sa, sb, sc, sd = oracle.pcr_split(a, b, c, d, k)
+    lo, hi = 1 << k, n - 1 - (1 << k)
+    assert np.all(sa[0, lo:hi + 1] == -2.0 ** -k)
+    assert np.all(sc[0, lo:hi + 1] == -2.0 ** -k)
+    assert np.all(sb[0, lo:hi + 1] == 2.0 ** (1 - k))
+    # d' is the exact rational combination: d'_i = 2^-k sum_t w_t d_{i+t s} with the
+    # binomial-like weights of PCR; check against exact integer arithmetic for k=1.
+    if k == 1:
+        i = np.arange(lo, hi + 1)
+        assert np.array_equal(sd[0, i], d[0, i] + 0.5 * (d[0, i - 1] + d[0, i + 1]))
+
+
+def test_pcr_split_composes():
+    """k1 levels, take a residue-class subsystem, k2 more levels on it ==
+    k1+k2 levels on the full system, bit-exactly (same formula, same operands)."""
+    n, k1, k2 = 333, 2, 3
+    a, b, c, d = inputs.generate(n, 2, np.float64, seed=8)
+    full = oracle.pcr_split(a, b, c, d, k1 + k2)
+    first = oracle.pcr_split(a, b, c, d, k1)
+    for r1 in range(1 << k1):
+        sub = oracle.subsystem(*first, k1, r1)
+        second = oracle.pcr_split(*sub, k2)
+        rows = np.arange(r1, n, 1 << k1)
+        for u, v in zip(second, full):
+            assert np.array_equal(u, v[:, rows])
+
+
+# ------------------------------------------------------------ permutation ----
+
+def test_permutation_golden_fig3():
+    with open(os.path.join(GOLDEN, "fig3_permutation.txt")) as f:
+        rows = [l.split() for l in f if l.strip() and not l.startswith("#")]
+    assert rows
+    for r in rows:
+        n, k, perm = int(r[0]), int(r[1]), [int(v) for v in r[2:]]
+        assert oracle.permutation(n, k).tolist() == perm
+
+
+@pytest.mark.parametrize("n", [1, 2, 7, 8, 100, 1023, 4096])
+def test_permutation_bruteforce(n):
+    """Closed form == stable sort of rows by residue (brute force)."""
+    for k in range(0, 12):
+        p = oracle.permutation(n, k)
+        bf = np.argsort(np.arange(n) % (1 << k), kind="stable")
+        assert np.array_equal(p, bf)
+
+
+# --------------------------------------------------------------- planner ----
+
+def _golden_params():
+    out = {}
+    with open(os.path.join(GOLDEN, "paper_parameters.txt")) as f:
+        for l in f:
+            l = l.split("#")[0].split()
+            if l:
+                out[l[0]] = [int(v) for v in l[1:]]
+    return out
+
+
+def test_planner_paper_values():
+    g = _golden_params()
+    p = rplan.make_plan(rplan.B200, rplan.F32, 1 << 20, 16, mode=rplan.DEFAULT)
+    assert p.n_sub_target == g["default_nsub_target"][0]
+    assert p.theta == g["default_theta"][0]
+    assert p.n_sub <= 256 and p.k == 12
+    ps = rplan.make_plan(rplan.B200, rplan.F32, 1 << 20, 16, mode=rplan.STATIC)
+    assert ps.thomas_chains == g["static_thomas_chains"][0]
+    assert ps.theta == rplan.B200.sm_count
+
+
+def test_planner_static_onchip_sizes():
+    """Static on-chip size = largest power of two whose 4 arrays fit in shared
+    memory: 512 (16 KB) / 2048 (48 KB) on Table I, 8192 fp32 / 4096 fp64 on B200."""
+    t = rplan.TABLE_I
+    assert rplan.n_onchip_max(t["GeForce 8800 GTX"], rplan.F32) == 512
+    assert rplan.n_onchip_max(t["GeForce GTX 280"], rplan.F32) == 512
+    assert rplan.n_onchip_max(t["GeForce GTX 470"], rplan.F32) == 2048
+    assert rplan.n_onchip_max(rplan.B200, rplan.F32) == 8192
+    assert rplan.n_onchip_max(rplan.B200, rplan.F64) == 4096
+
+
+@pytest.mark.parametrize("dtype,n,m,k,passes,nsub", [
+    (rplan.F32, 1024, 1, 0, 0, 1024),
+    (rplan.F32, 65536, 256, 3, 1, 8192),
+    (rplan.F32, 1 << 20, 16, 7, 1, 8192),
+    (rplan.F64, 1 << 20, 16, 8, 1, 4096),
+    (rplan.F32, 16384, 4096, 1, 1, 8192),
+    (rplan.F32, 1 << 28, 1, 15, 2, 8192),
+])
+def test_planner_static_configs(dtype, n, m, k, passes, nsub):
+    """The STATIC plans of SURVEY.md §8(a) A1 at the BASELINE.json configs."""
+    p = rplan.make_plan(rplan.B200, dtype, n, m, mode=rplan.STATIC)
+    assert (p.k, p.passes, p.n_sub) == (k, passes, nsub)
+    assert sum(p.k_pass) == k
+    assert p.k_pass[:passes] == sorted(p.k_pass[:passes], reverse=True)
+    assert max(p.k_pass) - min(p.k_pass[:max(passes, 1)]) <= 1 or passes <= 1
+
+
+def test_decoupled_trial_count_arithmetic():
+    """§IV-D: decoupling makes trials additive, not multiplicative."""
+    g = _golden_params()["decoupled_trials"]
+    assert g[0] + g[1] == g[2] and g[0] * g[1] == g[3]
