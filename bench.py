@@ -1,0 +1,423 @@
+#!/usr/bin/env python
+"""Benchmark: batched tridiagonal solves on B200 (BASELINE.json metric:
+equations solved/sec, fp32, and % of HBM roofline).
+
+    python bench.py [--gpus N --steps K --warmup W] [--config 3] [--dtype f32]
+                    [--mode tuned|static|default] [--impl tds|reference]
+
+One step = one pass of the whole hot path (every split pass + the on-chip
+kernel) over one batch of synthetic systems already resident in HBM.  Under
+torchrun (N > 1) every rank solves its own batch of the same shape (weak
+scaling: the systems are independent, no data-path collective); value = all
+ranks' equations / max-over-ranks device time.  ``--impl reference`` times
+the CPU oracle (fp64 Thomas, OpenMP over systems) on the same workload.
+Prints ONE JSON line on rank 0.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import shutil
+import statistics
+import subprocess
+import sys
+import tempfile
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+METRIC = "equations solved/sec (fp32, 1/2/4/8 B200) and % of HBM roofline"
+CONFIGS = {  # BASELINE.json configs: (n, m)
+    1: (1024, 1),
+    2: (65536, 256),
+    3: (1 << 20, 16),
+    4: (16384, 4096),
+    5: (1 << 28, 1),
+}
+L2_BYTES = 126 * 2 ** 20
+
+
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=50)
+    ap.add_argument("--warmup", type=int, default=5)
+    ap.add_argument("--config", type=int, default=3, choices=sorted(CONFIGS))
+    ap.add_argument("--dtype", default="f32", choices=["f32", "f64"])
+    ap.add_argument("--mode", default="tuned", choices=["tuned", "static", "default"])
+    ap.add_argument("--impl", default="tds", choices=["tds", "reference"])
+    ap.add_argument("--tune-cache", default=None, help="tds_tune cache file (default: a fresh temp file)")
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--soak-s", type=float, default=1.5, help="untimed load before timing (clock sampling)")
+    return ap.parse_args()
+
+
+def dist_env():
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    return world, rank, local
+
+
+# ------------------------------------------------------------------ clocks
+
+class ClockSampler:
+    """nvidia-smi sampling of SM clocks / throttle reasons during the timed region."""
+    FIELDS = ["clocks.sm", "clocks.max.sm", "utilization.gpu", "power.draw", "clocks_event_reasons.active",
+              "clocks_event_reasons.hw_slowdown", "clocks_event_reasons.hw_thermal_slowdown",
+              "clocks_event_reasons.sw_thermal_slowdown", "clocks_event_reasons.sw_power_cap"]
+
+    def __init__(self, index: int):
+        self.index = index
+        self.proc = None
+        self.path = None
+
+    def start(self):
+        if not shutil.which("nvidia-smi"):
+            return self
+        fd, self.path = tempfile.mkstemp(suffix=".csv")
+        os.close(fd)
+        self.proc = subprocess.Popen(["nvidia-smi", f"--id={self.index}", "--query-gpu=" + ",".join(self.FIELDS),
+                                      "--format=csv,noheader,nounits", "-lms", "100"],
+                                     stdout=open(self.path, "w"), stderr=subprocess.DEVNULL)
+        time.sleep(0.3)
+        return self
+
+    def stop(self) -> dict:
+        if self.proc is None:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvidia-smi unavailable"]}
+        self.proc.terminate()
+        try:
+            self.proc.wait(timeout=5)
+        except subprocess.TimeoutExpired:
+            self.proc.kill()
+        rows = []
+        with open(self.path) as f:
+            for line in f:
+                parts = [p.strip() for p in line.split(",")]
+                if len(parts) == len(self.FIELDS):
+                    rows.append(parts)
+        os.unlink(self.path)
+        if not rows:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": [], "samples": 0}
+
+        def num(v):
+            try:
+                return float(v)
+            except ValueError:
+                return None
+        busy = [r for r in rows if (num(r[2]) or 0) >= 50] or rows
+        sm = [num(r[0]) for r in busy if num(r[0]) is not None]
+        mx = [num(r[1]) for r in rows if num(r[1]) is not None]
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = sorted({names[i] for r in busy for i in range(4) if r[5 + i].lower().startswith("active")})
+        pw = [num(r[3]) for r in busy if num(r[3]) is not None]
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": max(mx) if mx else None,
+                "reasons": reasons, "samples": len(rows), "samples_under_load": len(busy),
+                "power_w_max": max(pw) if pw else None}
+
+
+# ------------------------------------------------------------------ helpers
+
+def algorithmic_bytes(info: dict, s: int):
+    """Bytes per launch the method must move: split
+    pass 1 reads a,b,c,d and writes normalised a',c',d' (7 s/eq); a later pass
+    reads and writes 3 arrays (6 s/eq); the on-chip kernel reads 3 (or the 4
+    raw arrays when k = 0) and writes x (4 s or 5 s per equation)."""
+    eqs = info["n"] * info["m"]
+    out = []
+    for p in range(info["passes"]):
+        out.append((7 if p == 0 else 6) * s * eqs)
+    out.append((5 if info["passes"] == 0 else 4) * s * eqs)
+    return out
+
+
+def stage_names(info):
+    return [f"split_pass_{p}(k_p={info['k_pass'][p]})" for p in range(info["passes"])] + ["onchip_cr_pcr_thomas"]
+
+
+def measured_peaks():
+    try:
+        with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
+            return json.load(f), "measured"
+    except (OSError, ValueError):
+        return {"hbm_gbs": 6650.0}, "fallback (B200_PROFILING.md)"
+
+
+def ncu_traffic(config_key: str, stage: str):
+    """dram__bytes_read.sum + dram__bytes_write.sum per launch from the committed
+    ncu --set full summary (profiles/ncu_traffic.json), or None."""
+    try:
+        with open(os.path.join(ROOT, "profiles", "ncu_traffic.json")) as f:
+            t = json.load(f)
+        v = t.get(config_key, {}).get(stage.split("(")[0])
+        return v
+    except (OSError, ValueError):
+        return None
+
+
+def host_cores():
+    try:
+        return len(os.sched_getaffinity(0))
+    except AttributeError:
+        return os.cpu_count() or 1
+
+
+def cpu_oracle_time(a, b, c, d, repeats=3, budget_s=25.0):
+    """Time the oracle (as it stands) on a bounded sample of the workload.
+    Returns (eq/s, threads, sample description, x of the sample)."""
+    import oracle
+    m, n = d.shape
+    # bounded sample: as many whole systems as fit ~2^25 rows (all of them for configs 1-3)
+    ms = max(1, min(m, (1 << 25) // n))
+    a64, b64, c64, d64 = (np.ascontiguousarray(v[:ms], dtype=np.float64) for v in (a, b, c, d))  # upcast: untimed
+    threads = min(oracle.num_threads(), ms)
+    times, x = [], None
+    t_start = time.perf_counter()
+    for _ in range(repeats):
+        t0 = time.perf_counter()
+        x = oracle.thomas(a64, b64, c64, d64, threads=threads)
+        times.append(time.perf_counter() - t0)
+        if time.perf_counter() - t_start > budget_s:
+            break
+    t = statistics.median(times)
+    sample = f"{ms} of {m} systems x {n} rows (fp64 Thomas, fp32->fp64 upcast untimed), median of {len(times)}"
+    return ms * n / t, threads, sample, x, ms
+
+
+# ------------------------------------------------------------------ reference arm
+
+def run_reference(args):
+    world, rank, _ = dist_env()
+    if rank != 0:
+        return 0
+    from paper_conf_ipps_davidsonzo11_b200 import inputs
+    import oracle
+    n, m = CONFIGS[args.config]
+    dt = np.float32 if args.dtype == "f32" else np.float64
+    # each step: a bounded sample of the workload (whole systems, <= 2^25 rows)
+    ms = max(1, min(m, (1 << 25) // n))
+    a, b, c, d = inputs.generate(n, ms, dt, seed=inputs.config_seed(args.config, dt))
+    a64, b64, c64, d64 = (np.ascontiguousarray(v, dtype=np.float64) for v in (a, b, c, d))
+    threads = min(oracle.num_threads(), ms)
+    for _ in range(args.warmup):
+        oracle.thomas(a64, b64, c64, d64, threads=threads)
+    t0 = time.perf_counter()
+    for _ in range(args.steps):
+        oracle.thomas(a64, b64, c64, d64, threads=threads)
+    el = time.perf_counter() - t0
+    value = ms * n * args.steps / el
+    sample = f"{ms} of {m} systems x {n} rows per step (fp64 Thomas, upcast untimed)"
+    line = {
+        "impl": "reference", "metric": METRIC, "value": value, "unit": "eq/s", "n_gpus": args.gpus,
+        "steps": args.steps, "warmup": args.warmup, "ms_per_step": el * 1e3 / args.steps,
+        "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f64",
+        "data": "synthetic (splitmix64 counter hash, diagonally dominant, margin 1)",
+        "config": {"workload": f"config{args.config}: {m} x {n} {args.dtype}", "n": n, "m": m,
+                   "oracle": "oracle/thomas.c fp64 Thomas, OpenMP one system per thread"},
+        "cpu_baseline": {"value": value, "unit": "eq/s", "cores": threads, "kind": "oracle", "sample": sample},
+        "e2e": {"value": value, "unit": "eq/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+    }
+    print(json.dumps(line), flush=True)
+    return 0
+
+
+# ------------------------------------------------------------------ tds arm
+
+def run_tds(args):
+    import torch
+    import torch.distributed as dist
+    import paper_conf_ipps_davidsonzo11_b200 as tds
+    from paper_conf_ipps_davidsonzo11_b200 import inputs
+
+    world, rank, local = dist_env()
+    if world != args.gpus and world > 1:
+        print(f"warning: WORLD_SIZE={world} != --gpus {args.gpus}", file=sys.stderr)
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=dev)
+
+    def barrier():
+        if world > 1:
+            dist.barrier()
+
+    n, m = CONFIGS[args.config]
+    dt = np.float32 if args.dtype == "f32" else np.float64
+    tdt = torch.float32 if dt == np.float32 else torch.float64
+    s = np.dtype(dt).itemsize
+    seed = inputs.config_seed(args.config, dt)
+    a, b, c, d = inputs.generate(n, m, dt, seed=seed, first_system=rank * m)
+    ta, tb, tc, td = (torch.from_numpy(v).to(dev) for v in (a, b, c, d))
+    x = torch.empty_like(td)
+
+    plan = tds.Plan(n, m, "float32" if dt == np.float32 else "float64", device=local,
+                    mode="static" if args.mode == "tuned" else args.mode)
+    trials = 0
+    tune_s = 0.0
+    if args.mode == "tuned":
+        # rank 0 tunes; the integer plan is broadcast so every rank runs identical kernels
+        if rank == 0:
+            cache = args.tune_cache or tempfile.mktemp(suffix=".tds_tune")
+            t0 = time.perf_counter()
+            trials = plan.tune(cache_path=cache)
+            tune_s = time.perf_counter() - t0
+            if not args.tune_cache and os.path.exists(cache):
+                os.unlink(cache)
+        if world > 1:
+            p = plan.params
+            vec = torch.tensor([p.k, p.passes] + list(p.k_pass) + [p.cr_levels, p.thomas_chains,
+                                                                    p.split_tile_rows, p.split_threads, p.theta],
+                               dtype=torch.int64, device=dev)
+            dist.broadcast(vec, 0)
+            v = vec.tolist()
+            if rank != 0:
+                plan.set_params(k_pass=[k for k in v[2:10] if k], cr_levels=v[10], thomas_chains=v[11],
+                                split_tile_rows=v[12], split_threads=v[13], theta=v[14])
+    info = plan.info
+    ws = plan.workspace()
+    P = info["passes"]
+    stream = torch.cuda.current_stream()
+
+    def step():
+        tds.solve_batched(plan, ta, tb, tc, td, out=x, workspace=ws)
+
+    # warm-up (W steps) + soak for clock sampling, sampler covers the timed region
+    sampler = ClockSampler(local).start()
+    for _ in range(max(args.warmup, 3)):
+        step()
+    torch.cuda.synchronize()
+    t_end = time.perf_counter() + args.soak_s
+    while time.perf_counter() < t_end:
+        for _ in range(20):
+            step()
+        torch.cuda.synchronize()
+
+    # ---- timed region: K steps, events between the kernels of each step
+    K = args.steps
+    ev = [[torch.cuda.Event(enable_timing=True) for _ in range(P + 2)] for _ in range(K)]
+    barrier()
+    torch.cuda.synchronize()
+    for i in range(K):
+        for st in range(P + 1):
+            ev[i][st].record(stream)
+            tds.api.solve_stages(plan, ta, tb, tc, td, x, ws, st, st)
+        ev[i][P + 1].record(stream)
+    torch.cuda.synchronize()
+    barrier()
+    clocks = sampler.stop()
+    total_ms = ev[0][0].elapsed_time(ev[K - 1][P + 1])
+    stage_ms = [sum(ev[i][st].elapsed_time(ev[i][st + 1]) for i in range(K)) / K for st in range(P + 1)]
+    if world > 1:
+        t = torch.tensor([total_ms], dtype=torch.float64, device=dev)
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        total_ms = float(t.item())
+    eqs_per_step = n * m
+    value = world * eqs_per_step * K / (total_ms / 1e3)
+
+    # ---- roofline for the dominant kernel
+    peaks, peak_kind = measured_peaks()
+    hbm_peak = float(peaks.get("hbm_gbs", 6650.0))
+    abytes = algorithmic_bytes(info, s)
+    names = stage_names(info)
+    dom = int(np.argmax(stage_ms))
+    achieved = abytes[dom] / (stage_ms[dom] / 1e3) / 1e9
+    ws_fp = "x".join(str(v) for v in (m, n))
+    roofline = {
+        "bound": "hbm", "kernel": names[dom], "achieved": achieved, "peak": hbm_peak, "unit": "GB/s",
+        "frac": achieved / hbm_peak, "traffic": ncu_traffic(f"config{args.config}_{args.dtype}", names[dom]),
+        "peak_kind": peak_kind, "frac_of_8TBs": achieved / 8000.0,
+        "algorithmic_bytes_per_launch": abytes[dom], "share_of_step": stage_ms[dom] / sum(stage_ms),
+        "per_kernel": [{"kernel": nm, "ms": ms_, "algorithmic_bytes": ab, "gbs": ab / (ms_ / 1e3) / 1e9}
+                       for nm, ms_, ab in zip(names, stage_ms, abytes)],
+        "step": {"algorithmic_bytes": sum(abytes), "bytes_per_eq": sum(abytes) / eqs_per_step,
+                 "gbs": sum(abytes) / (total_ms / K / 1e3) / 1e9,
+                 "frac": sum(abytes) / (total_ms / K / 1e3) / 1e9 / hbm_peak,
+                 "frac_of_8TBs": sum(abytes) / (total_ms / K / 1e3) / 1e9 / 8000.0},
+    }
+
+    # ---- end to end through the public API with host buffers
+    e2e = None
+    if not args.no_e2e:
+        ha, hb, hc, hd = (torch.from_numpy(v).pin_memory() for v in (a, b, c, d))
+        hx = torch.empty(hd.shape, dtype=tdt).pin_memory()
+        Ke = max(1, min(K, 10))
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+
+        def e2e_step():
+            for src, dst in ((ha, ta), (hb, tb), (hc, tc), (hd, td)):
+                dst.copy_(src, non_blocking=True)
+            tds.solve_batched(plan, ta, tb, tc, td, out=x, workspace=ws)
+            hx.copy_(x, non_blocking=True)
+        e2e_step()
+        torch.cuda.synchronize()
+        barrier()
+        e0.record(stream)
+        for _ in range(Ke):
+            e2e_step()
+        e1.record(stream)
+        torch.cuda.synchronize()
+        e_ms = e0.elapsed_time(e1)
+        if world > 1:
+            t = torch.tensor([e_ms], dtype=torch.float64, device=dev)
+            dist.all_reduce(t, op=dist.ReduceOp.MAX)
+            e_ms = float(t.item())
+        e2e = {"value": world * eqs_per_step * Ke / (e_ms / 1e3), "unit": "eq/s",
+               "h2d_bytes_per_step": 4 * eqs_per_step * s, "d2h_bytes_per_step": eqs_per_step * s,
+               "steps": Ke, "ms_per_step": e_ms / Ke}
+        assert torch.equal(hx, x.cpu())
+
+    # ---- CPU baseline: the oracle on the host cores (rank 0, N = 1 only)
+    cpu = None
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+        v, thr, sample, xo, ms_ = cpu_oracle_time(a, b, c, d)
+        import oracle
+        xg = x[:ms_].cpu().numpy()
+        cpu = {"value": v, "unit": "eq/s", "cores": thr, "host_cores": host_cores(), "kind": "oracle",
+               "sample": sample, "gpu_vs_oracle_rel_err": oracle.rel_err(xg, xo),
+               "gpu_residual": oracle.residual(a[:ms_], b[:ms_], c[:ms_], d[:ms_], xg)}
+
+    if world > 1:
+        dist.destroy_process_group()
+    if rank != 0:
+        return 0
+    line = {
+        "metric": METRIC, "value": value, "unit": "eq/s", "n_gpus": world, "steps": K, "warmup": args.warmup,
+        "ms_per_step": total_ms / K, "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
+        "dtype": args.dtype, "data": "synthetic (splitmix64 counter hash, diagonally dominant, margin 1)",
+        "config": {"workload": f"config{args.config}: {m} x {n} {args.dtype} per GPU", "n": n, "m": m,
+                   "mode": args.mode, "plan": {k: info[k] for k in ("k", "passes", "k_pass", "n_sub",
+                                                                     "cr_levels", "thomas_chains",
+                                                                     "split_tile_rows", "split_threads",
+                                                                     "theta", "split_segments",
+                                                                     "onchip_threads", "workspace_bytes")},
+                   "tune_trials": trials, "tune_s": round(tune_s, 2),
+                   "l2": f"no flush: per-step working set {(5 * eqs_per_step * s + info['workspace_bytes']) / 2**20:.0f} MiB > L2 126 MiB"
+                   if 5 * eqs_per_step * s + info["workspace_bytes"] > L2_BYTES else
+                   "working set fits L2: warm-L2 latency number",
+                   "parallelism": f"batch-sharded x{world} (independent systems, no data-path collective)"},
+        "roofline": roofline,
+        "cpu_baseline": cpu,
+        "e2e": e2e,
+        "gpu_launches": K * (P + 1),
+        "clocks": clocks,
+    }
+    print(json.dumps(line), flush=True)
+    return 0
+
+
+def main():
+    args = parse()
+    if args.impl == "reference":
+        return run_reference(args)
+    return run_tds(args)
+
+
+if __name__ == "__main__":
+    sys.exit(main())

@@ -1,0 +1,214 @@
+/*
+ * tds.h -- C ABI of libtds, the B200-native multi-stage batched tridiagonal
+ * solver (Davidson, Zhang & Owens, "An Auto-tuned Method for Solving Large
+ * Tridiagonal Systems on the GPU", IPDPS 2011).  "P:Lx" = line x of the
+ * paper's text; "§8" = SURVEY.md §8, the hot-path contract.
+ *
+ * WHAT IS SOLVED.  m independent tridiagonal systems of n equations
+ *        a_i x_{i-1} + b_i x_i + c_i x_{i+1} = d_i,   i = 0..n-1
+ * ("tridiagonal systems of any size and number, as long as they fit into
+ * global memory"; the workload [m, n] of Fig. 1).
+ * a_0 and c_{n-1} of every system are ignored (treated as 0).
+ *
+ * HOW (the paper's four stages in sm_100a kernels, §III):
+ *   stages 1+2  k global PCR splitting levels in
+ *               one or more fused HBM passes -> 2^k interleaved subsystems;
+ *   stages 3+4  each subsystem solved on-chip by the hybrid kernel: c CR
+ *               levels in registers, PCR on the reduced system until T
+ *               independent chains, Thomas per chain, CR back substitution
+ *               (base kernel §III-A; switch points §III-D).
+ * The switch points come from one of the paper's three parameter-selection
+ * methods (§IV): DEFAULT (machine-oblivious), STATIC (device
+ * query) or TUNED (self-tuned from the static seed, tds_tune).
+ *
+ * NUMERICS.  No pivoting (the paper's solvers do not pivot): the precondition
+ * is a nonsingular, diagonally dominant (or SPD) system.  Breakdown is NOT
+ * detected: a zero pivot yields inf/NaN in x.  fp32 uses the hardware
+ * approximate reciprocal; fp64 uses IEEE division.
+ *
+ * CONVENTIONS (every entry point):
+ *  - Layout: element i of system s is at ptr[s * batch_stride + i]
+ *    (system-major; batch_stride >= n; batch_stride == 0 means n).
+ *  - Device pointers are caller-owned device memory of the plan's dtype,
+ *    aligned to sizeof(T).  Host pointers are documented as such.
+ *  - Plans are host objects and own NO device memory.  A plan is immutable
+ *    except through tds_tune / tds_plan_set_params; concurrent solves with one
+ *    plan on different streams need separate workspaces.
+ *  - Streams: a cudaStream_t passed as void* (NULL = legacy default stream).
+ *    Solve entry points only enqueue work and return (asynchronous).
+ *  - Errors: every call returns tds_status; no exception crosses the ABI.
+ *    Argument errors are detected before anything is enqueued.  Launch
+ *    failures return TDS_ERR_CUDA.  tds_last_error() gives a thread-local
+ *    human-readable detail for the most recent failing call.
+ */
+#ifndef TDS_H_
+#define TDS_H_
+
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+#define TDS_VERSION 100 /* 1.0.0 */
+#define TDS_MAX_PASSES 8
+
+typedef enum {
+    TDS_OK = 0,
+    TDS_ERR_INVALID_ARG = 1,     /* bad pointer, size, stride, mode, overlap      */
+    TDS_ERR_UNSUPPORTED = 2,     /* valid request the kernels cannot run          */
+    TDS_ERR_NO_MEMORY = 3,       /* host or device allocation failed              */
+    TDS_ERR_WORKSPACE = 4,       /* workspace NULL / too small / misaligned       */
+    TDS_ERR_CUDA = 5,            /* CUDA runtime or launch error                  */
+    TDS_ERR_TUNE = 6,            /* tuner failed (trial error, cache I/O)         */
+    TDS_ERR_DEVICE_MISMATCH = 7  /* current device differs from the plan's device */
+} tds_status;
+
+typedef enum { TDS_F32 = 0, TDS_F64 = 1 } tds_dtype;
+
+/* Parameter-selection methods of §IV. */
+typedef enum {
+    TDS_PARAMS_DEFAULT = 0, /* §IV-B: 256-element on-chip entry, 16 systems, T = 32 */
+    TDS_PARAMS_STATIC = 1,  /* §IV-C: device-query seeds (smem size, SM count, 2x warp) */
+    TDS_PARAMS_TUNED = 2    /* §IV-D: set by tds_tune only (not accepted by tds_plan) */
+} tds_param_mode;
+
+typedef struct tds_plan_st *tds_plan_t;
+
+/* Queryable device properties used by the planner (Table II). */
+typedef struct {
+    int32_t sm_count;              /* "Processors"                               */
+    int32_t smem_optin_bytes;      /* max dynamic shared memory per block        */
+    int32_t smem_per_sm_bytes;     /* "Shared Memory" per processor              */
+    int32_t regs_per_sm;           /* "Register Memory"                          */
+    int32_t max_threads_per_block;
+    int32_t warp_size;
+    int32_t cc_major, cc_minor;
+    int64_t l2_bytes;
+    int64_t global_mem_bytes;      /* "Global Mem"                               */
+} tds_device_props;
+
+/* The tunable integers of a plan (the switch points of §III-D). */
+typedef struct {
+    int32_t k;                       /* total split levels: 2^k subsystems per system   */
+    int32_t passes;                  /* HBM split passes (0 iff k == 0)                 */
+    int32_t k_pass[TDS_MAX_PASSES];  /* levels fused in each pass, sum == k             */
+    int32_t cr_levels;               /* c: CR levels in registers (R = 2^c rows/thread)  */
+    int32_t thomas_chains;           /* T: Thomas chains of the reduced system (pow2)   */
+    int32_t split_tile_rows;         /* split-pass tile (pow2, >= 2^k_pass[i])          */
+    int32_t split_threads;           /* split-pass CTA size (multiple of 32)            */
+    int32_t theta;                   /* stage 1->2 switch: independent systems needed   */
+} tds_params;
+
+/* Everything a plan decided (read-only view). */
+typedef struct {
+    int32_t dtype, mode, tuned;
+    int32_t device;
+    int64_t n, m, batch_stride;
+    tds_params params;
+    int64_t n_sub;            /* longest subsystem: ceil(n / 2^k)                      */
+    int64_t num_subsystems;   /* m * min(2^k, n)                                       */
+    int32_t n_sub_target;     /* stage 2->3 switch (subsystem size) the plan aimed at  */
+    int32_t n_onchip_max;     /* largest on-chip subsystem for this device and dtype   */
+    int32_t split_kp_max;     /* max levels per split pass                             */
+    int32_t onchip_threads;   /* on-chip kernel CTA size                               */
+    int32_t subsys_per_cta;   /* on-chip subsystems per CTA (1)                        */
+    int32_t cluster;          /* CTAs per cluster (1)                                  */
+    int32_t split_segments;   /* CTAs cooperating on one system in pass 1 (stage 1)    */
+    int32_t pad_;
+    int64_t slot_rows;        /* workspace rows reserved per subsystem (final pass)    */
+    size_t workspace_bytes;   /* bytes tds_solve_batched needs (0 when k == 0)         */
+} tds_plan_info;
+
+/* ---- planning (host only, no device work) -------------------------------- */
+
+/* Plan a solve of m systems of n equations on CUDA device `device` with the
+ * DEFAULT or STATIC method.  *out receives a new plan (free with
+ * tds_plan_destroy).  Errors: INVALID_ARG (n < 1, m < 1, 0 < batch_stride < n,
+ * bad dtype/mode, out == NULL), CUDA (device query failed). */
+tds_status tds_plan(tds_plan_t *out, int device, tds_dtype dtype, int64_t n, int64_t m,
+                    int64_t batch_stride, tds_param_mode mode);
+
+/* Same as tds_plan, from explicit (possibly fake) device properties (host
+ * pointer, read only during the call).  The plan's device is -1: it can be
+ * inspected but tds_solve_batched rejects it (DEVICE_MISMATCH). */
+tds_status tds_plan_from_props(tds_plan_t *out, const tds_device_props *props, tds_dtype dtype,
+                               int64_t n, int64_t m, int64_t batch_stride, tds_param_mode mode);
+
+/* Fill *out (host) with the properties of CUDA device `device`. */
+tds_status tds_device_props_query(int device, tds_device_props *out);
+
+tds_status tds_plan_info_get(const tds_plan_t plan, tds_plan_info *out);
+
+/* Replace the plan's tunable parameters (host struct) after validating them
+ * against the kernels' limits; derived fields (n_sub, threads, workspace) are
+ * recomputed and the plan's mode becomes TUNED.  INVALID_ARG / UNSUPPORTED on
+ * a rejected set (the plan is then unchanged). */
+tds_status tds_plan_set_params(tds_plan_t plan, const tds_params *params);
+
+/* Canonical subsystem order after k levels (Fig. 3a): residue r
+ * ascending, then row ascending: perm[off(r) + j] = r + 2^k j, off(r) =
+ * sum_{r'<r} ceil((n - r')/2^k).  perm_host: host array of len == n entries. */
+tds_status tds_plan_permutation(const tds_plan_t plan, int64_t *perm_host, int64_t len);
+
+tds_status tds_plan_destroy(tds_plan_t plan);
+
+/* ---- self-tuning (§IV-D) -------------------------------------- */
+
+/* Tune the plan's switch points on its device: decoupled, seeded hill climb
+ * over timed trials on generated diagonally dominant systems of the plan's
+ * shape (the on-chip switch (c, T) and the split schedule (k, passes, tile,
+ * theta) are searched independently, starting from the STATIC seed).
+ * Allocates and frees its own device buffers; synchronises `cuda_stream`.
+ * cache_path (host string, may be NULL => $TDS_TUNE_CACHE or no cache): a
+ * text file of saved results keyed by device, dtype, n and m ("save those
+ * results for future runs"); a hit skips the search.
+ * Errors: INVALID_ARG, DEVICE_MISMATCH, NO_MEMORY, CUDA, TUNE. */
+tds_status tds_tune(tds_plan_t plan, void *cuda_stream, const char *cache_path);
+
+/* Trials run by the most recent tds_tune on this plan (0 on a cache hit). */
+tds_status tds_plan_tune_trials(const tds_plan_t plan, int32_t *trials);
+
+/* ---- solving ---------------------------------------------------------------- */
+
+/* x = A^{-1} d for every system.  a, b, c, d: device, dtype, m x batch_stride.
+ * x: device, same layout; may alias d exactly (in-place), must not otherwise
+ * overlap a, b, c or d.  workspace: device, >= info.workspace_bytes bytes,
+ * 256-byte aligned (may be NULL when info.workspace_bytes == 0).  Enqueued on
+ * cuda_stream; returns immediately.  Errors (nothing enqueued): INVALID_ARG,
+ * WORKSPACE, DEVICE_MISMATCH, UNSUPPORTED; CUDA on a launch failure. */
+tds_status tds_solve_batched(const tds_plan_t plan, const void *a, const void *b, const void *c,
+                             const void *d, void *x, void *workspace, size_t workspace_bytes,
+                             void *cuda_stream);
+
+/* Run only kernels first_stage..last_stage (inclusive) of the solve sequence
+ * tds_solve_batched enqueues: stage p < passes is split pass p (PAPER.md
+ * stages 1-2), stage == passes is the on-chip kernel (stages 3-4).  Calling
+ * stages 0..passes in order on one stream is identical to tds_solve_batched
+ * (used to time each kernel with events between them).  Same arguments and
+ * errors as tds_solve_batched; INVALID_ARG if the range is empty or outside
+ * [0, passes]. */
+tds_status tds_solve_stages(const tds_plan_t plan, const void *a, const void *b, const void *c,
+                            const void *d, void *x, void *workspace, size_t workspace_bytes,
+                            void *cuda_stream, int32_t first_stage, int32_t last_stage);
+
+/* Diagnostic: run only the split stage (stages 1-2) and write the split
+ * system in CANONICAL order, normalised so that b' = 1: for system s,
+ * out[s*n + off(r) + j] holds the coefficient of original row r + 2^k j
+ * (the tds_plan_permutation order).  a_out, c_out, d_out: device, dtype,
+ * m x n (dense).  Requires k >= 1.  Same workspace rules as the solve. */
+tds_status tds_split_batched(const tds_plan_t plan, const void *a, const void *b, const void *c,
+                             const void *d, void *a_out, void *c_out, void *d_out,
+                             void *workspace, size_t workspace_bytes, void *cuda_stream);
+
+/* ---- misc ---------------------------------------------------------------------- */
+
+const char *tds_status_string(tds_status status);
+const char *tds_last_error(void);
+int tds_version(void);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* TDS_H_ */

@@ -135,6 +135,13 @@ def slot_rows(n: int, kk: int, dtype: int) -> int:
     return round_up(cdiv(n, 1 << kk), 16 // dsize(dtype))
 
 
+def split_smem_bytes(dtype: int, tile: int, kp: int) -> int:
+    """Split-pass shared memory: 3 normalised arrays of the tile plus a
+    (2^kp - 1)-row halo per side, padded by index >> max(kp, 5) against bank conflicts."""
+    e = tile + 2 * ((1 << kp) - 1)
+    return 3 * (e + (e >> max(kp, 5)) + 1) * dsize(dtype)
+
+
 def segments(m_in: int, tiles: int, theta: int) -> int:
     """Stage 1 (cooperative, several CTAs per system) until theta independent
     systems exist, else Stage 2 (one CTA per system) -- Fig. 1 P:L169-187."""
@@ -167,7 +174,7 @@ def make_plan(props: Props, dtype: int, n: int, m: int, batch_stride: int = 0,
         g1t = STATIC_SPLIT_THREADS
         kpmax = 9 if dtype == F32 else 8
         budget = props.smem_optin_bytes - SMEM_RESERVE
-        while kpmax > 1 and ((tile + 2 * ((1 << kpmax) - 1)) * 3 * s > budget
+        while kpmax > 1 and (split_smem_bytes(dtype, tile, kpmax) > budget
                              or (1 << kpmax) > tile):
             kpmax -= 1
         g2cap = props.max_threads_per_block // 2
@@ -198,6 +205,14 @@ def make_plan(props: Props, dtype: int, n: int, m: int, batch_stride: int = 0,
     p.cr_levels = R.bit_length() - 1
     p.onchip_threads = max(32, round_up(nred, 32))
     p.thomas_chains = min(T, pow2ceil(nred))
+
+    # Kernel limits (the C++ planner rejects these plans as UNSUPPORTED).
+    budget = props.smem_optin_bytes - SMEM_RESERVE
+    for i in range(P):
+        if split_smem_bytes(dtype, tile, p.k_pass[i]) > budget:
+            raise ValueError("unsupported: split tile + halo exceeds shared memory")
+    if (9 * p.onchip_threads + 8) * s > budget:
+        raise ValueError("unsupported: on-chip shared memory")
 
     # Workspace: split output (normalised a, c, d) in fixed slots; ping-pong if P >= 2.
     if P:

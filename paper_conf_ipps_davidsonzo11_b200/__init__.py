@@ -1,10 +1,12 @@
 """B200-native multi-stage batched tridiagonal solver (Davidson, Zhang & Owens, IPDPS 2011).
 
-The compute path lives in ``libtds.so`` (csrc/, sm_100a CUDA + a C ABI declared
-in include/tds.h).  This package is a thin ctypes binding over that library;
-the native library is loaded lazily on first use and its absence is an error
-(there is no CPU fallback).
+The compute path lives in ``libtds.so`` (csrc/: sm_100a CUDA kernels and the C
+ABI declared in include/tds.h).  This package is a thin ctypes binding with the
+same names; the native library is loaded on first use and its absence is an
+error (there is no CPU fallback).
 """
 from . import inputs  # noqa: F401  (seeded generator; no solver arithmetic)
+from ._lib import TdsError  # noqa: F401
+from .api import Plan, device_props, solve_batched, split_batched, version  # noqa: F401
 
-__all__ = ["inputs"]
+__all__ = ["Plan", "solve_batched", "split_batched", "device_props", "version", "TdsError", "inputs"]

@@ -1,0 +1,196 @@
+"""Python face of libtds: the same names as the C ABI (include/tds.h).
+
+Argument marshalling only -- every step of the solve runs in libtds's sm_100a
+kernels.  PyTorch supplies device memory (tensors) and streams.
+"""
+from __future__ import annotations
+
+import ctypes
+from typing import Optional
+
+import numpy as np
+
+from . import _lib as L
+
+_DTYPES = {"float32": L.TDS_F32, "float64": L.TDS_F64}
+MODES = {"default": L.TDS_PARAMS_DEFAULT, "static": L.TDS_PARAMS_STATIC, "tuned": L.TDS_PARAMS_TUNED}
+
+
+def _dtype_code(dtype) -> int:
+    name = str(dtype).replace("torch.", "")
+    if name not in _DTYPES:
+        raise TypeError(f"unsupported dtype {dtype}: float32 or float64")
+    return _DTYPES[name]
+
+
+def _stream_ptr(stream) -> Optional[int]:
+    import torch
+    if stream is None:
+        stream = torch.cuda.current_stream()
+    return stream.cuda_stream
+
+
+def device_props(device: int = 0) -> dict:
+    lib = L.load()
+    p = L.DeviceProps()
+    L.check(lib.tds_device_props_query(int(device), ctypes.byref(p)))
+    return {f: getattr(p, f) for f, _ in L.DeviceProps._fields_}
+
+
+def params_to_dict(p: L.Params) -> dict:
+    return {"k": p.k, "passes": p.passes, "k_pass": list(p.k_pass)[: max(p.passes, 0)],
+            "cr_levels": p.cr_levels, "thomas_chains": p.thomas_chains,
+            "split_tile_rows": p.split_tile_rows, "split_threads": p.split_threads, "theta": p.theta}
+
+
+class Plan:
+    """tds_plan / tds_plan_from_props wrapper (host object; owns no device memory)."""
+
+    def __init__(self, n: int, m: int, dtype="float32", device: int = 0, mode: str = "static",
+                 batch_stride: int = 0, props: Optional[dict] = None):
+        self._lib = L.load()
+        self._h = ctypes.c_void_p()
+        code = _dtype_code(dtype)
+        if props is not None:
+            dp = L.DeviceProps(**props)
+            L.check(self._lib.tds_plan_from_props(ctypes.byref(self._h), ctypes.byref(dp), code, int(n),
+                                                  int(m), int(batch_stride), MODES[mode]))
+        else:
+            L.check(self._lib.tds_plan(ctypes.byref(self._h), int(device), code, int(n), int(m),
+                                       int(batch_stride), MODES[mode]))
+        self.dtype = "float32" if code == L.TDS_F32 else "float64"
+
+    def __del__(self):
+        h = getattr(self, "_h", None)
+        if h is not None and h.value:
+            self._lib.tds_plan_destroy(h)
+            self._h = None
+
+    @property
+    def handle(self):
+        return self._h
+
+    def info_struct(self) -> L.PlanInfo:
+        info = L.PlanInfo()
+        L.check(self._lib.tds_plan_info_get(self._h, ctypes.byref(info)))
+        return info
+
+    @property
+    def info(self) -> dict:
+        s = self.info_struct()
+        out = {f: getattr(s, f) for f, _ in L.PlanInfo._fields_ if f not in ("params", "pad_")}
+        out.update(params_to_dict(s.params))
+        return out
+
+    @property
+    def params(self) -> L.Params:
+        return self.info_struct().params
+
+    @property
+    def workspace_bytes(self) -> int:
+        return int(self.info_struct().workspace_bytes)
+
+    def set_params(self, **kw) -> None:
+        """tds_plan_set_params: replace tunables (k, k_pass, cr_levels, thomas_chains, ...)."""
+        p = self.params
+        for key, val in kw.items():
+            if key == "k_pass":
+                vals = list(val) + [0] * (L.TDS_MAX_PASSES - len(val))
+                for i in range(L.TDS_MAX_PASSES):
+                    p.k_pass[i] = vals[i]
+                p.passes = len(val)
+                p.k = sum(val)
+            else:
+                setattr(p, key, int(val))
+        L.check(self._lib.tds_plan_set_params(self._h, ctypes.byref(p)))
+
+    def permutation(self) -> np.ndarray:
+        n = self.info_struct().n
+        out = np.empty(n, dtype=np.int64)
+        L.check(self._lib.tds_plan_permutation(self._h, out.ctypes.data, int(n)))
+        return out
+
+    def tune(self, stream=None, cache_path: Optional[str] = None) -> int:
+        """tds_tune; returns the number of timed trials (0 on a cache hit)."""
+        cp = cache_path.encode() if cache_path else None
+        L.check(self._lib.tds_tune(self._h, _stream_ptr(stream), cp))
+        t = ctypes.c_int32()
+        L.check(self._lib.tds_plan_tune_trials(self._h, ctypes.byref(t)))
+        return int(t.value)
+
+    def workspace(self):
+        import torch
+        nbytes = self.workspace_bytes
+        if nbytes == 0:
+            return None
+        return torch.empty(nbytes, dtype=torch.uint8, device=f"cuda:{self.info_struct().device}")
+
+
+def _ptr(t) -> int:
+    return t.data_ptr()
+
+
+def _check_tensor(t, plan_info, name):
+    import torch
+    if not isinstance(t, torch.Tensor) or not t.is_cuda:
+        raise TypeError(f"{name} must be a CUDA tensor")
+    want = torch.float32 if plan_info.dtype == L.TDS_F32 else torch.float64
+    if t.dtype != want:
+        raise TypeError(f"{name} has dtype {t.dtype}, plan expects {want}")
+    need = (plan_info.m - 1) * plan_info.batch_stride + plan_info.n
+    if t.numel() < need or not t.is_contiguous():
+        raise ValueError(f"{name} must be contiguous with >= {need} elements")
+
+
+def solve_batched(plan: Plan, a, b, c, d, out=None, workspace=None, stream=None):
+    """x = A^{-1} d for every system (tds_solve_batched).  a, b, c, d: CUDA
+    tensors laid out as the plan says (m x batch_stride).  Returns x."""
+    import torch
+    info = plan.info_struct()
+    for name, t in (("a", a), ("b", b), ("c", c), ("d", d)):
+        _check_tensor(t, info, name)
+    if out is None:
+        out = torch.empty_like(d)
+    _check_tensor(out, info, "out")
+    if workspace is None:
+        workspace = plan.workspace()
+    wptr = _ptr(workspace) if workspace is not None else None
+    wbytes = workspace.numel() * workspace.element_size() if workspace is not None else 0
+    L.check(plan._lib.tds_solve_batched(plan.handle, _ptr(a), _ptr(b), _ptr(c), _ptr(d), _ptr(out), wptr,
+                                        wbytes, _stream_ptr(stream)))
+    return out
+
+
+def solve_stages(plan: Plan, a, b, c, d, out, workspace, first: int, last: int, stream=None):
+    """tds_solve_stages: run kernels first..last of the solve sequence (split
+    passes 0..P-1, on-chip kernel P) -- for per-kernel timing."""
+    info = plan.info_struct()
+    for name, t in (("a", a), ("b", b), ("c", c), ("d", d), ("out", out)):
+        _check_tensor(t, info, name)
+    wptr = _ptr(workspace) if workspace is not None else None
+    wbytes = workspace.numel() * workspace.element_size() if workspace is not None else 0
+    L.check(plan._lib.tds_solve_stages(plan.handle, _ptr(a), _ptr(b), _ptr(c), _ptr(d), _ptr(out), wptr,
+                                       wbytes, _stream_ptr(stream), int(first), int(last)))
+    return out
+
+
+def split_batched(plan: Plan, a, b, c, d, workspace=None, stream=None):
+    """Diagnostic split stage (tds_split_batched): returns (a', c', d') (m, n)
+    in canonical order, normalised so that b' = 1."""
+    import torch
+    info = plan.info_struct()
+    for name, t in (("a", a), ("b", b), ("c", c), ("d", d)):
+        _check_tensor(t, info, name)
+    shape = (info.m, info.n)
+    oa, oc, od = (torch.empty(shape, dtype=d.dtype, device=d.device) for _ in range(3))
+    if workspace is None:
+        workspace = plan.workspace()
+    wptr = _ptr(workspace) if workspace is not None else None
+    wbytes = workspace.numel() * workspace.element_size() if workspace is not None else 0
+    L.check(plan._lib.tds_split_batched(plan.handle, _ptr(a), _ptr(b), _ptr(c), _ptr(d), _ptr(oa), _ptr(oc),
+                                        _ptr(od), wptr, wbytes, _stream_ptr(stream)))
+    return oa, oc, od
+
+
+def version() -> int:
+    return int(L.load().tds_version())

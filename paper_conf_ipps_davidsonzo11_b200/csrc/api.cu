@@ -1,0 +1,294 @@
+// api.cu -- the solve half of the C ABI: device query, argument validation,
+// the stream-ordered launch sequence (split passes, then the on-chip kernel)
+// and the diagnostic split-only entry point.  See include/tds.h.
+#include <algorithm>
+#include <cstring>
+#include <string>
+
+#include "common.cuh"
+
+namespace tds {
+
+static bool overlaps(const void *p, size_t pb, const void *q, size_t qb) {
+    const char *a = static_cast<const char *>(p), *b = static_cast<const char *>(q);
+    return a < b + qb && b < a + pb;
+}
+
+static tds_status cuda_fail(cudaError_t e, const char *what) {
+    return fail(TDS_ERR_CUDA, std::string(what) + ": " + cudaGetErrorString(e));
+}
+
+static tds_status check_device(const tds_plan_st *plan) {
+    int dev = -1;
+    cudaError_t e = cudaGetDevice(&dev);
+    if (e != cudaSuccess) return cuda_fail(e, "cudaGetDevice");
+    if (plan->info.device < 0 || dev != plan->info.device)
+        return fail(TDS_ERR_DEVICE_MISMATCH, "current device " + std::to_string(dev) + " != plan device " +
+                                                 std::to_string(plan->info.device));
+    return TDS_OK;
+}
+
+static tds_status check_workspace(const tds_plan_info &I, const void *ws, size_t ws_bytes) {
+    if (I.workspace_bytes == 0) return TDS_OK;
+    if (!ws) return fail(TDS_ERR_WORKSPACE, "workspace is NULL");
+    if (ws_bytes < I.workspace_bytes)
+        return fail(TDS_ERR_WORKSPACE, "workspace " + std::to_string(ws_bytes) + " < required " +
+                                           std::to_string(I.workspace_bytes));
+    if (reinterpret_cast<uintptr_t>(ws) % 256) return fail(TDS_ERR_WORKSPACE, "workspace not 256-byte aligned");
+    return TDS_OK;
+}
+
+// Workspace buffer i holds normalised (a, c, d) arrays of E elements each.
+template <typename T>
+struct WsBufs {
+    T *a[2], *c[2], *d[2];
+};
+
+template <typename T>
+static WsBufs<T> ws_bufs(const tds_plan_info &I, void *ws) {
+    WsBufs<T> w{};
+    const int nbuf = I.params.passes >= 2 ? 2 : 1;
+    const int64_t E = int64_t(I.workspace_bytes / (size_t(nbuf) * 3 * sizeof(T)));
+    T *base = static_cast<T *>(ws);
+    for (int i = 0; i < nbuf; ++i) {
+        w.a[i] = base + (3 * i + 0) * E;
+        w.c[i] = base + (3 * i + 1) * E;
+        w.d[i] = base + (3 * i + 2) * E;
+    }
+    if (nbuf == 1) {
+        w.a[1] = w.a[0];
+        w.c[1] = w.c[0];
+        w.d[1] = w.d[0];
+    }
+    return w;
+}
+
+// Launch the P split passes; returns the index of the buffer holding the result.
+template <typename T>
+static tds_status run_split(const tds_plan_info &I, const T *a, const T *b, const T *c, const T *d,
+                            const WsBufs<T> &w, cudaStream_t st, int *out_buf, int first = 0,
+                            int last = 1 << 30) {
+    const tds_params &P = I.params;
+    int kprev = 0;
+    for (int p = 0; p < P.passes; ++p) {
+        const int kp = P.k_pass[p];
+        if (p < first || p > last) {
+            kprev += kp;
+            continue;
+        }
+        SplitArgs<T> A{};
+        const bool raw = (p == 0);
+        if (raw) {
+            A.a = a;
+            A.b = b;
+            A.c = c;
+            A.d = d;
+            A.in_stride = I.batch_stride;
+        } else {
+            const int ib = (p - 1) & 1;
+            A.a = w.a[ib];
+            A.b = nullptr;
+            A.c = w.c[ib];
+            A.d = w.d[ib];
+            A.in_stride = slot_rows(I.n, kprev, I.dtype);
+        }
+        const int ob = p & 1;
+        A.oa = w.a[ob];
+        A.oc = w.c[ob];
+        A.od = w.d[ob];
+        A.n = I.n;
+        A.out_slot = slot_rows(I.n, kprev + kp, I.dtype);
+        A.kp = kp;
+        A.tile = P.split_tile_rows;
+        A.geom.npass = p;
+        for (int q = 0; q < kMaxPasses; ++q) A.geom.kpass[q] = q < p ? P.k_pass[q] : 0;
+        const int64_t m_in = I.m << kprev;
+        const int64_t len_in = cdiv(I.n, int64_t(1) << kprev);
+        A.segs = split_segments(m_in, cdiv(len_in, P.split_tile_rows), P.theta);
+        const int64_t e = P.split_tile_rows + 2 * ((int64_t(1) << kp) - 1);
+        A.ep = int32_t(e + (e >> std::max(kp, 5)) + 1);
+        const int64_t grid = m_in * A.segs;
+        if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "split grid exceeds 2^31-1 CTAs");
+        const size_t smem = split_smem_bytes(I.dtype, P.split_tile_rows, kp);
+        cudaError_t err = launch_split_pass<T>(A, raw, grid, P.split_threads, smem, st);
+        if (err != cudaSuccess) return cuda_fail(err, "split_pass launch");
+        kprev += kp;
+    }
+    *out_buf = (P.passes - 1) & 1;
+    return TDS_OK;
+}
+
+template <typename T>
+static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, const T *c, const T *d, T *x,
+                             void *ws, cudaStream_t st, int first = 0, int last = 1 << 30) {
+    const tds_params &P = I.params;
+    OnchipArgs<T> A{};
+    A.x = x;
+    A.n = I.n;
+    A.batch_stride = I.batch_stride;
+    A.K = P.k;
+    int t = P.thomas_chains, l2 = 0;
+    while ((1 << l2) < t) ++l2;
+    A.log2T = l2;
+    int64_t grid;
+    if (P.k == 0) {
+        A.a = a;
+        A.b = b;
+        A.c = c;
+        A.d = d;
+        grid = I.m;
+    } else {
+        WsBufs<T> w = ws_bufs<T>(I, ws);
+        int ob = 0;
+        tds_status s = run_split<T>(I, a, b, c, d, w, st, &ob, first, last);
+        if (s != TDS_OK) return s;
+        A.a = w.a[ob];
+        A.b = nullptr;
+        A.c = w.c[ob];
+        A.d = w.d[ob];
+        A.slot = I.slot_rows;
+        A.geom.npass = P.passes;
+        for (int q = 0; q < kMaxPasses; ++q) A.geom.kpass[q] = P.k_pass[q];
+        grid = I.m << P.k;
+    }
+    if (P.passes < first || P.passes > last) return TDS_OK;  // on-chip stage not requested
+    if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "on-chip grid exceeds 2^31-1 CTAs");
+    const size_t smem = onchip_smem_bytes(I.dtype, I.onchip_threads);
+    cudaError_t err = launch_onchip<T>(A, P.cr_levels, P.k == 0, grid, I.onchip_threads, smem, st);
+    if (err != cudaSuccess) return cuda_fail(err, "onchip launch");
+    return TDS_OK;
+}
+
+// Gather workspace slots into the canonical order (diagnostic path only).
+template <typename T>
+__global__ void gather_canonical_kernel(const T *sa, const T *sc, const T *sd, T *oa, T *oc, T *od, int64_t n,
+                                        int32_t K, int64_t slot, PassGeom geom) {
+    const int64_t sigma = blockIdx.x;
+    const int64_t sys = sigma >> K;
+    const int64_t r = slot_residue(sigma & ((int64_t(1) << K) - 1), geom.npass, geom.kpass);
+    if (r >= n) return;
+    const int64_t L = (n - r + (int64_t(1) << K) - 1) >> K;
+    const int64_t q = n >> K, rem = n & ((int64_t(1) << K) - 1);
+    const int64_t off = r * q + (r < rem ? r : rem);
+    for (int64_t j = threadIdx.x; j < L; j += blockDim.x) {
+        const int64_t i = sigma * slot + j, o = sys * n + off + j;
+        oa[o] = sa[i];
+        oc[o] = sc[i];
+        od[o] = sd[i];
+    }
+}
+
+template <typename T>
+static tds_status split_impl(const tds_plan_info &I, const T *a, const T *b, const T *c, const T *d, T *oa,
+                             T *oc, T *od, void *ws, cudaStream_t st) {
+    WsBufs<T> w = ws_bufs<T>(I, ws);
+    int ob = 0;
+    tds_status s = run_split<T>(I, a, b, c, d, w, st, &ob);
+    if (s != TDS_OK) return s;
+    PassGeom g{};
+    g.npass = I.params.passes;
+    for (int q = 0; q < kMaxPasses; ++q) g.kpass[q] = I.params.k_pass[q];
+    const int64_t grid = I.m << I.params.k;
+    if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "grid too large");
+    gather_canonical_kernel<T><<<(unsigned)grid, 256, 0, st>>>(w.a[ob], w.c[ob], w.d[ob], oa, oc, od, I.n,
+                                                                 I.params.k, I.slot_rows, g);
+    cudaError_t err = cudaGetLastError();
+    if (err != cudaSuccess) return cuda_fail(err, "gather launch");
+    return TDS_OK;
+}
+
+static tds_status check_arrays(const tds_plan_info &I, std::initializer_list<const void *> ptrs) {
+    const size_t es = size_t(dsize(I.dtype));
+    for (const void *p : ptrs) {
+        if (!p) return fail(TDS_ERR_INVALID_ARG, "NULL array pointer");
+        if (reinterpret_cast<uintptr_t>(p) % es) return fail(TDS_ERR_INVALID_ARG, "array not aligned to sizeof(T)");
+    }
+    return TDS_OK;
+}
+
+}  // namespace tds
+
+using namespace tds;
+
+extern "C" {
+
+tds_status tds_device_props_query(int device, tds_device_props *out) {
+    if (!out) return fail(TDS_ERR_INVALID_ARG, "out is NULL");
+    cudaDeviceProp p;
+    cudaError_t e = cudaGetDeviceProperties(&p, device);
+    if (e != cudaSuccess) return cuda_fail(e, "cudaGetDeviceProperties");
+    int optin = 0;
+    e = cudaDeviceGetAttribute(&optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, device);
+    if (e != cudaSuccess) return cuda_fail(e, "cudaDeviceGetAttribute");
+    std::memset(out, 0, sizeof(*out));
+    out->sm_count = p.multiProcessorCount;
+    out->smem_optin_bytes = optin;
+    out->smem_per_sm_bytes = (int32_t)p.sharedMemPerMultiprocessor;
+    out->regs_per_sm = p.regsPerMultiprocessor;
+    out->max_threads_per_block = p.maxThreadsPerBlock;
+    out->warp_size = p.warpSize;
+    out->cc_major = p.major;
+    out->cc_minor = p.minor;
+    out->l2_bytes = p.l2CacheSize;
+    out->global_mem_bytes = (int64_t)p.totalGlobalMem;
+    return TDS_OK;
+}
+
+tds_status tds_solve_batched(const tds_plan_t plan, const void *a, const void *b, const void *c, const void *d,
+                             void *x, void *workspace, size_t workspace_bytes, void *cuda_stream) {
+    if (!plan) return fail(TDS_ERR_INVALID_ARG, "plan is NULL");
+    return tds_solve_stages(plan, a, b, c, d, x, workspace, workspace_bytes, cuda_stream, 0,
+                            plan->info.params.passes);
+}
+
+tds_status tds_solve_stages(const tds_plan_t plan, const void *a, const void *b, const void *c, const void *d,
+                            void *x, void *workspace, size_t workspace_bytes, void *cuda_stream,
+                            int32_t first_stage, int32_t last_stage) {
+    if (!plan) return fail(TDS_ERR_INVALID_ARG, "plan is NULL");
+    const tds_plan_info &I = plan->info;
+    if (first_stage < 0 || last_stage > I.params.passes || first_stage > last_stage)
+        return fail(TDS_ERR_INVALID_ARG, "stage range outside [0, passes]");
+    tds_status s = check_arrays(I, {a, b, c, d, x});
+    if (s != TDS_OK) return s;
+    const size_t bytes = size_t(((I.m - 1) * I.batch_stride + I.n) * dsize(I.dtype));
+    for (const void *p : {a, b, c})
+        if (overlaps(x, bytes, p, bytes)) return fail(TDS_ERR_INVALID_ARG, "x overlaps a, b or c");
+    if (x != d && overlaps(x, bytes, d, bytes))
+        return fail(TDS_ERR_INVALID_ARG, "x partially overlaps d (only x == d is allowed)");
+    if ((s = check_workspace(I, workspace, workspace_bytes)) != TDS_OK) return s;
+    if (workspace && I.workspace_bytes)
+        for (const void *p : {a, b, c, d, (const void *)x})
+            if (overlaps(workspace, I.workspace_bytes, p, bytes))
+                return fail(TDS_ERR_INVALID_ARG, "workspace overlaps an array");
+    if ((s = check_device(plan)) != TDS_OK) return s;
+    cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
+    s = I.dtype == TDS_F32
+            ? solve_impl<float>(I, (const float *)a, (const float *)b, (const float *)c, (const float *)d,
+                                (float *)x, workspace, st, first_stage, last_stage)
+            : solve_impl<double>(I, (const double *)a, (const double *)b, (const double *)c, (const double *)d,
+                                 (double *)x, workspace, st, first_stage, last_stage);
+    if (s == TDS_OK) clear_error();
+    return s;
+}
+
+tds_status tds_split_batched(const tds_plan_t plan, const void *a, const void *b, const void *c, const void *d,
+                             void *a_out, void *c_out, void *d_out, void *workspace, size_t workspace_bytes,
+                             void *cuda_stream) {
+    if (!plan) return fail(TDS_ERR_INVALID_ARG, "plan is NULL");
+    const tds_plan_info &I = plan->info;
+    if (I.params.k < 1) return fail(TDS_ERR_INVALID_ARG, "tds_split_batched needs k >= 1");
+    tds_status s = check_arrays(I, {a, b, c, d, a_out, c_out, d_out});
+    if (s != TDS_OK) return s;
+    if ((s = check_workspace(I, workspace, workspace_bytes)) != TDS_OK) return s;
+    if ((s = check_device(plan)) != TDS_OK) return s;
+    cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
+    s = I.dtype == TDS_F32
+            ? split_impl<float>(I, (const float *)a, (const float *)b, (const float *)c, (const float *)d,
+                                (float *)a_out, (float *)c_out, (float *)d_out, workspace, st)
+            : split_impl<double>(I, (const double *)a, (const double *)b, (const double *)c, (const double *)d,
+                                 (double *)a_out, (double *)c_out, (double *)d_out, workspace, st);
+    if (s == TDS_OK) clear_error();
+    return s;
+}
+
+}  // extern "C"

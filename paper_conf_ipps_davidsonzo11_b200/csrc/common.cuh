@@ -1,0 +1,98 @@
+// common.cuh -- device helpers shared by the libtds kernels (not by the oracle).
+#pragma once
+#include <cuda_runtime.h>
+#include <stdint.h>
+
+#include "tds_internal.h"
+
+namespace tds {
+
+constexpr int kMaxPasses = TDS_MAX_PASSES;
+
+// Reciprocal.  fp32: the SFU approximation (MUFU.RCP, <= 1 ulp) -- the
+// north_star's fp32 tolerance (1e-4 error, 1e-5 residual) leaves room for it
+// (reading R16).  fp64: IEEE division.
+__device__ __forceinline__ float rcp(float x) {
+    float r;
+    asm("rcp.approx.ftz.f32 %0, %1;" : "=f"(r) : "f"(x));
+    return r;
+}
+__device__ __forceinline__ double rcp(double x) { return 1.0 / x; }
+
+// One PCR/CR row update in NORMALISED form (every row scaled so b = 1).
+// With the textbook update (Hockney & Jesshope [11], cited
+// PAPER.md P:L199-200) applied to normalised rows and the result rescaled
+// by 1/b':
+//   r  = 1 / (1 - a_i c_{i-s} - c_i a_{i+s})
+//   a' = -a_i a_{i-s} r,  c' = -c_i c_{i+s} r,  d' = (d_i - a_i d_{i-s} - c_i d_{i+s}) r
+// Identity neighbours (outside the system) are (a, c, d) = (0, 0, 0).
+template <typename T>
+__device__ __forceinline__ void row_update(T &a, T &c, T &d, T al, T cl, T dl, T ar, T cr, T dr) {
+    const T den = fma(-c, ar, fma(-a, cl, T(1)));
+    const T r = rcp(den);
+    const T ma = -a * r;
+    const T mc = -c * r;
+    const T nd = fma(ma, dl, fma(mc, dr, d * r));
+    a = ma * al;
+    c = mc * cr;
+    d = nd;
+}
+
+// Original residue (mod 2^K) of workspace slot index rho after `npass`
+// passes: each pass appends its residue digit as the LOW digit of the slot
+// index, while in the original row numbering that digit has weight
+// 2^(levels of the earlier passes).
+__device__ __forceinline__ int64_t slot_residue(int64_t rho, int npass, const int32_t *kpass) {
+    int kcum = 0;
+    for (int p = 0; p < npass; ++p) kcum += kpass[p];
+    int64_t r = 0;
+    for (int p = npass - 1; p >= 0; --p) {
+        kcum -= kpass[p];
+        r += (rho & ((int64_t(1) << kpass[p]) - 1)) << kcum;
+        rho >>= kpass[p];
+    }
+    return r;
+}
+
+struct PassGeom {
+    int32_t npass;                 // passes already applied to the input
+    int32_t kpass[kMaxPasses];     // their level counts
+};
+
+
+template <typename T>
+struct SplitArgs {
+    const T *a, *b, *c, *d;  // input (RAW: original a,b,c,d; else normalised a,c,d slots)
+    int64_t in_stride;       // RAW: batch_stride; else input slot capacity
+    int64_t n;               // original system size
+    T *oa, *oc, *od;         // output slots (normalised)
+    int64_t out_slot;        // output slot capacity
+    int32_t kp;              // levels fused in this pass
+    int32_t tile;            // TILE rows (power of two, >= 2^kp)
+    int32_t segs;            // CTAs per input slot
+    int32_t ep;              // padded shared-memory length per array
+    PassGeom geom;           // passes applied to the input
+};
+
+template <typename T>
+struct OnchipArgs {
+    const T *a, *b, *c, *d;  // RAW (K == 0): original arrays; else normalised a,c,d slots
+    T *x;
+    int64_t n;
+    int64_t batch_stride;    // original layout (input when RAW, always for x)
+    int64_t slot;            // workspace slot capacity (K > 0)
+    int32_t K;               // total split levels
+    int32_t log2T;           // PCR levels on the reduced system (T = 2^log2T chains)
+    PassGeom geom;           // passes applied (for the slot -> residue map)
+};
+
+__host__ __device__ constexpr int ilog2c(int v) { return v <= 1 ? 0 : 1 + ilog2c(v / 2); }
+
+template <typename T>
+cudaError_t launch_split_pass(const SplitArgs<T> &A, bool raw, int64_t grid, int threads, size_t smem,
+                              cudaStream_t st);
+template <typename T>
+cudaError_t launch_onchip(const OnchipArgs<T> &A, int cr_levels, bool raw, int64_t grid, int threads,
+                          size_t smem, cudaStream_t st);
+
+}  // namespace tds

@@ -1,0 +1,317 @@
+// plan.cpp -- the planner: the paper's DEFAULT and machine-query ("static")
+// parameter selection (§IV-B/C) turned into an integer
+// plan for the B200 kernels, plus the plan-handling half of the C ABI.
+//
+// The rules:
+//   DEFAULT  n_sub_target = 256, theta = 16 systems,
+//            T = 32 (reading R10), split tile 1024 x 256 threads, <= 8
+//            levels per pass, on-chip CTA <= 256 threads.
+//   STATIC   n_sub_target = n_onchip_max: largest power of two whose four
+//            arrays fit in shared memory ("switch as soon as it fits",
+//            P:L704-705), T = 2 x warp size, theta = #SMs
+//            (P:L650-655), split tile = n_onchip_max x 512 threads, <= 9
+//            (fp32) / 8 (fp64) levels per pass, on-chip CTA <= half the
+//            maximum block size.
+//   both     k = min{k : ceil(n/2^k) <= n_sub_target}; passes = ceil(k/kp_max)
+//            with levels as equal as possible, larger first; R = 2^c the
+//            smallest power of two with ceil(n_sub/R) <= on-chip cap.
+#include <algorithm>
+#include <cstring>
+#include <new>
+#include <string>
+
+#include "tds_internal.h"
+
+namespace tds {
+
+static thread_local std::string g_last_error;
+
+tds_status fail(tds_status st, const std::string &msg) {
+    g_last_error = msg;
+    return st;
+}
+void clear_error() { g_last_error.clear(); }
+
+static int ilog2(int64_t v) {
+    int l = 0;
+    while ((int64_t(1) << (l + 1)) <= v) ++l;
+    return l;
+}
+static bool is_pow2(int64_t v) { return v > 0 && (v & (v - 1)) == 0; }
+static int64_t pow2ceil(int64_t v) {
+    int64_t p = 1;
+    while (p < v) p <<= 1;
+    return p;
+}
+
+int64_t slot_rows(int64_t n, int kk, int32_t dtype) {
+    // ceil(n / 2^kk) rounded up to 16 bytes so every slot is 16-byte aligned
+    return round_up(cdiv(n, int64_t(1) << kk), 16 / dsize(dtype));
+}
+
+int32_t split_segments(int64_t m_in, int64_t tiles, int32_t theta) {
+    // Fig. 1: cooperative splitting (stage 1, several CTAs per
+    // system) only while there are fewer than theta independent systems.
+    if (m_in >= theta) return 1;
+    return (int32_t)std::max<int64_t>(1, std::min<int64_t>(tiles, cdiv(theta, m_in)));
+}
+
+size_t split_smem_bytes(int32_t dtype, int32_t tile, int kp) {
+    int64_t halo = (int64_t(1) << kp) - 1;
+    int64_t e = tile + 2 * halo;
+    int64_t ep = e + (e >> std::max(kp, 5)) + 1;  // bank-conflict padding: index + (index >> max(kp,5))
+    return size_t(3 * ep * dsize(dtype));
+}
+
+size_t onchip_smem_bytes(int32_t dtype, int32_t threads) {
+    return size_t((9 * int64_t(threads) + 8) * dsize(dtype));
+}
+
+static int n_onchip_max(const tds_device_props &p, int32_t dtype) {
+    const int cap = dtype == TDS_F64 ? 4096 : 8192;  // on-chip kernel: R_max x 512 threads
+    const int64_t budget = int64_t(p.smem_optin_bytes) - kSmemReserve;
+    int n = 1;
+    while (n * 2 <= cap && 4 * int64_t(n * 2) * dsize(dtype) <= budget) n *= 2;
+    return n;
+}
+
+static int kp_limit(const tds_device_props &props, int32_t dtype, int32_t tile) {
+    int kp = 12;
+    while (kp > 1 && ((int64_t(1) << kp) > tile ||
+                      (int64_t)split_smem_bytes(dtype, tile, kp) >
+                          int64_t(props.smem_optin_bytes) - kSmemReserve))
+        --kp;
+    return kp;
+}
+
+tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_params &p) {
+    const int64_t n = info.n, m = info.m;
+    const int32_t dtype = info.dtype;
+    // --- validate the tunables against the kernels' limits
+    if (p.k < 0 || p.k > 40) return fail(TDS_ERR_INVALID_ARG, "k out of range");
+    if ((p.k == 0) != (p.passes == 0) || p.passes < 0 || p.passes > TDS_MAX_PASSES)
+        return fail(TDS_ERR_INVALID_ARG, "passes must be 0 iff k == 0, <= 8");
+    int ksum = 0;
+    for (int i = 0; i < TDS_MAX_PASSES; ++i) {
+        if (i < p.passes) {
+            if (p.k_pass[i] < 1) return fail(TDS_ERR_INVALID_ARG, "k_pass[i] >= 1");
+            ksum += p.k_pass[i];
+        } else if (p.k_pass[i] != 0) {
+            return fail(TDS_ERR_INVALID_ARG, "unused k_pass entries must be 0");
+        }
+    }
+    if (ksum != p.k) return fail(TDS_ERR_INVALID_ARG, "sum(k_pass) != k");
+    if (p.cr_levels < 0 || (1 << p.cr_levels) > r_max(dtype))
+        return fail(TDS_ERR_UNSUPPORTED, "cr_levels exceeds the on-chip kernel's R_max");
+    if (!is_pow2(p.thomas_chains)) return fail(TDS_ERR_INVALID_ARG, "thomas_chains must be a power of two");
+    if (p.theta < 1) return fail(TDS_ERR_INVALID_ARG, "theta >= 1");
+    const int64_t n_sub = cdiv(n, int64_t(1) << std::min(p.k, 62));
+    const int R = 1 << p.cr_levels;
+    const int64_t nred = cdiv(n_sub, R);
+    const int64_t threads = std::max<int64_t>(32, round_up(nred, 32));
+    if (threads > (R >= 8 ? kMaxOnchipThreadsWide : kMaxOnchipThreads))
+        return fail(TDS_ERR_UNSUPPORTED, "subsystem too large for the on-chip kernel (n_sub / 2^c > 1024, or > 512 when 2^c >= 8)");
+    if (p.thomas_chains > threads) return fail(TDS_ERR_INVALID_ARG, "thomas_chains > on-chip threads");
+    if ((int64_t)onchip_smem_bytes(dtype, (int32_t)threads) > int64_t(props.smem_optin_bytes) - kSmemReserve)
+        return fail(TDS_ERR_UNSUPPORTED, "on-chip shared memory exceeds the device limit");
+    if (p.passes > 0) {
+        if (!is_pow2(p.split_tile_rows) || p.split_tile_rows < 32 || p.split_tile_rows > (1 << 15))
+            return fail(TDS_ERR_INVALID_ARG, "split_tile_rows must be a power of two in [32, 32768]");
+        if (p.split_threads < 32 || p.split_threads > kMaxSplitThreads || p.split_threads % 32)
+            return fail(TDS_ERR_INVALID_ARG, "split_threads must be a multiple of 32 in [32, 512]");
+        for (int i = 0; i < p.passes; ++i) {
+            const int kp = p.k_pass[i];
+            if ((int64_t(1) << kp) > p.split_tile_rows)
+                return fail(TDS_ERR_INVALID_ARG, "2^k_pass exceeds split_tile_rows");
+            const int64_t e = p.split_tile_rows + 2 * ((int64_t(1) << kp) - 1);
+            if (e > int64_t(p.split_threads) * kSplitQMax)
+                return fail(TDS_ERR_UNSUPPORTED, "split tile + halo exceeds threads x 24 rows");
+            if ((int64_t)split_smem_bytes(dtype, p.split_tile_rows, kp) >
+                int64_t(props.smem_optin_bytes) - kSmemReserve)
+                return fail(TDS_ERR_UNSUPPORTED, "split tile + halo exceeds shared memory");
+        }
+    }
+    // --- derived fields
+    info.params = p;
+    info.n_sub = n_sub;
+    info.num_subsystems = m * std::min<int64_t>(int64_t(1) << std::min(p.k, 62), n);
+    info.onchip_threads = (int32_t)threads;
+    info.subsys_per_cta = 1;
+    info.cluster = 1;
+    if (p.passes > 0) {
+        int kk = 0;
+        int64_t elems = 0;
+        for (int i = 0; i < p.passes; ++i) {
+            kk += p.k_pass[i];
+            elems = std::max<int64_t>(elems, m * (int64_t(1) << kk) * slot_rows(n, kk, dtype));
+        }
+        const int64_t E = round_up(elems, 64);
+        info.slot_rows = slot_rows(n, p.k, dtype);
+        info.workspace_bytes = size_t((p.passes == 1 ? 1 : 2) * 3 * E * dsize(dtype));
+        info.split_segments = split_segments(m, cdiv(n, p.split_tile_rows), p.theta);
+    } else {
+        info.slot_rows = 0;
+        info.workspace_bytes = 0;
+        info.split_segments = 0;
+    }
+    return TDS_OK;
+}
+
+static tds_status seed(tds_plan_info &info, const tds_device_props &props, tds_params &p) {
+    const int32_t dtype = info.dtype;
+    const int64_t n = info.n;
+    int64_t target;
+    int32_t T, theta, tile, g1threads, kpmax, g2cap;
+    info.n_onchip_max = n_onchip_max(props, dtype);
+    if (info.mode == TDS_PARAMS_DEFAULT) {
+        target = 256;
+        theta = 16;
+        T = 32;               // reading R10
+        tile = 1024;
+        g1threads = 256;
+        kpmax = 8;
+        g2cap = 256;
+    } else {
+        target = info.n_onchip_max;
+        T = 2 * props.warp_size;
+        theta = props.sm_count;
+        tile = info.n_onchip_max;
+        g1threads = 512;
+        kpmax = std::min(dtype == TDS_F32 ? 9 : 8, kp_limit(props, dtype, tile));
+        g2cap = props.max_threads_per_block / 2;
+    }
+    info.n_sub_target = (int32_t)target;
+    info.split_kp_max = kpmax;
+    std::memset(&p, 0, sizeof(p));
+    int k = 0;
+    while (cdiv(n, int64_t(1) << k) > target) ++k;
+    p.k = k;
+    const int P = k > 0 ? (int)cdiv(k, kpmax) : 0;
+    if (P > TDS_MAX_PASSES) return fail(TDS_ERR_UNSUPPORTED, "system needs more than 8 split passes");
+    p.passes = P;
+    for (int i = 0; i < P; ++i) p.k_pass[i] = k / P + (i < k % P ? 1 : 0);
+    const int64_t n_sub = cdiv(n, int64_t(1) << k);
+    int R = 1;
+    while (cdiv(n_sub, R) > g2cap && R < r_max(dtype)) R *= 2;
+    p.cr_levels = ilog2(R);
+    p.thomas_chains = (int32_t)std::min<int64_t>(T, pow2ceil(cdiv(n_sub, R)));
+    p.split_tile_rows = tile;
+    p.split_threads = g1threads;
+    p.theta = theta;
+    return TDS_OK;
+}
+
+static tds_status make_plan(tds_plan_t *out, const tds_device_props &props, int device, tds_dtype dtype,
+                            int64_t n, int64_t m, int64_t batch_stride, tds_param_mode mode) {
+    if (!out) return fail(TDS_ERR_INVALID_ARG, "out is NULL");
+    *out = nullptr;
+    if (dtype != TDS_F32 && dtype != TDS_F64) return fail(TDS_ERR_INVALID_ARG, "dtype");
+    if (mode != TDS_PARAMS_DEFAULT && mode != TDS_PARAMS_STATIC)
+        return fail(TDS_ERR_INVALID_ARG, "mode must be DEFAULT or STATIC (TUNED comes from tds_tune)");
+    if (n < 1 || m < 1) return fail(TDS_ERR_INVALID_ARG, "n and m must be >= 1");
+    if (batch_stride == 0) batch_stride = n;
+    if (batch_stride < n) return fail(TDS_ERR_INVALID_ARG, "batch_stride < n");
+    if (props.sm_count < 1 || props.warp_size < 1 || props.max_threads_per_block < 32 ||
+        props.smem_optin_bytes < 4096)
+        return fail(TDS_ERR_INVALID_ARG, "implausible device properties");
+    tds_plan_st *pl = new (std::nothrow) tds_plan_st();
+    if (!pl) return fail(TDS_ERR_NO_MEMORY, "host allocation");
+    std::memset(&pl->info, 0, sizeof(pl->info));
+    pl->props = props;
+    pl->info.dtype = dtype;
+    pl->info.mode = mode;
+    pl->info.device = device;
+    pl->info.n = n;
+    pl->info.m = m;
+    pl->info.batch_stride = batch_stride;
+    tds_params p;
+    tds_status st = seed(pl->info, props, p);
+    if (st == TDS_OK) st = derive(pl->info, props, p);
+    if (st != TDS_OK) {
+        delete pl;
+        return st;
+    }
+    *out = pl;
+    clear_error();
+    return TDS_OK;
+}
+
+}  // namespace tds
+
+using namespace tds;
+
+extern "C" {
+
+tds_status tds_plan_from_props(tds_plan_t *out, const tds_device_props *props, tds_dtype dtype, int64_t n,
+                               int64_t m, int64_t batch_stride, tds_param_mode mode) {
+    if (!props) return fail(TDS_ERR_INVALID_ARG, "props is NULL");
+    return make_plan(out, *props, -1, dtype, n, m, batch_stride, mode);
+}
+
+tds_status tds_plan(tds_plan_t *out, int device, tds_dtype dtype, int64_t n, int64_t m, int64_t batch_stride,
+                    tds_param_mode mode) {
+    tds_device_props props;
+    tds_status st = tds_device_props_query(device, &props);
+    if (st != TDS_OK) return st;
+    return make_plan(out, props, device, dtype, n, m, batch_stride, mode);
+}
+
+tds_status tds_plan_info_get(const tds_plan_t plan, tds_plan_info *out) {
+    if (!plan || !out) return fail(TDS_ERR_INVALID_ARG, "NULL argument");
+    *out = plan->info;
+    return TDS_OK;
+}
+
+tds_status tds_plan_set_params(tds_plan_t plan, const tds_params *params) {
+    if (!plan || !params) return fail(TDS_ERR_INVALID_ARG, "NULL argument");
+    tds_plan_info info = plan->info;
+    tds_status st = derive(info, plan->props, *params);
+    if (st != TDS_OK) return st;
+    info.mode = TDS_PARAMS_TUNED;
+    plan->info = info;
+    clear_error();
+    return TDS_OK;
+}
+
+tds_status tds_plan_permutation(const tds_plan_t plan, int64_t *perm, int64_t len) {
+    if (!plan || !perm) return fail(TDS_ERR_INVALID_ARG, "NULL argument");
+    const int64_t n = plan->info.n;
+    if (len != n) return fail(TDS_ERR_INVALID_ARG, "len must equal n");
+    const int k = plan->info.params.k;
+    const int64_t step = int64_t(1) << std::min(k, 62);
+    int64_t o = 0;
+    for (int64_t r = 0; r < std::min(step, n); ++r)
+        for (int64_t i = r; i < n; i += step) perm[o++] = i;
+    return TDS_OK;
+}
+
+tds_status tds_plan_destroy(tds_plan_t plan) {
+    delete plan;
+    return TDS_OK;
+}
+
+tds_status tds_plan_tune_trials(const tds_plan_t plan, int32_t *trials) {
+    if (!plan || !trials) return fail(TDS_ERR_INVALID_ARG, "NULL argument");
+    *trials = plan->tune_trials;
+    return TDS_OK;
+}
+
+const char *tds_status_string(tds_status s) {
+    switch (s) {
+        case TDS_OK: return "TDS_OK";
+        case TDS_ERR_INVALID_ARG: return "TDS_ERR_INVALID_ARG: invalid argument";
+        case TDS_ERR_UNSUPPORTED: return "TDS_ERR_UNSUPPORTED: unsupported configuration";
+        case TDS_ERR_NO_MEMORY: return "TDS_ERR_NO_MEMORY: allocation failed";
+        case TDS_ERR_WORKSPACE: return "TDS_ERR_WORKSPACE: workspace missing, too small or misaligned";
+        case TDS_ERR_CUDA: return "TDS_ERR_CUDA: CUDA error";
+        case TDS_ERR_TUNE: return "TDS_ERR_TUNE: tuning failed";
+        case TDS_ERR_DEVICE_MISMATCH: return "TDS_ERR_DEVICE_MISMATCH: current device differs from the plan's";
+    }
+    return "unknown tds_status";
+}
+
+const char *tds_last_error(void) { return g_last_error.c_str(); }
+
+int tds_version(void) { return TDS_VERSION; }
+
+}  // extern "C"

@@ -1,0 +1,38 @@
+// Internal (non-ABI) declarations shared by the libtds translation units.
+#pragma once
+#include <string>
+
+#include "../../include/tds.h"
+
+struct tds_plan_st {
+    tds_plan_info info;
+    tds_device_props props;
+    int32_t tune_trials = 0;
+};
+
+namespace tds {
+
+// Kernel limits the planner validates against.
+constexpr int kSplitQMax = 24;        // rows per thread held in registers by the split pass
+constexpr int kSmemReserve = 1024;    // per-CTA shared memory reserved by the runtime
+constexpr int kMaxOnchipThreads = 1024;     // on-chip CTA size for R <= 4
+constexpr int kMaxOnchipThreadsWide = 512;  // ... and for R >= 8 (register budget)
+constexpr int kMaxSplitThreads = 512;
+
+inline int dsize(int32_t dtype) { return dtype == TDS_F64 ? 8 : 4; }
+inline int r_max(int32_t dtype) { return dtype == TDS_F64 ? 8 : 16; }
+inline int64_t cdiv(int64_t a, int64_t b) { return (a + b - 1) / b; }
+inline int64_t round_up(int64_t a, int64_t b) { return cdiv(a, b) * b; }
+
+// Thread-local error detail (tds_last_error).
+tds_status fail(tds_status st, const std::string &msg);
+void clear_error();
+
+// Planner helpers (plan.cpp).
+int64_t slot_rows(int64_t n, int kk, int32_t dtype);
+int32_t split_segments(int64_t m_in, int64_t tiles, int32_t theta);
+size_t split_smem_bytes(int32_t dtype, int32_t tile, int kp);
+size_t onchip_smem_bytes(int32_t dtype, int32_t threads);
+tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_params &p);
+
+}  // namespace tds

@@ -1,0 +1,335 @@
+// tune.cu -- the self-tuner (§IV-D).
+//
+// The paper's two pruning ideas, applied to the B200 plan parameters:
+//  (1) decouple parameters that do not interact: the stage 3->4
+//      switch (on-chip: CR levels c, Thomas chains T) depends only on the
+//      subsystem size; the stage 2->3 switch (split levels k) is compared
+//      "vs. two times the number of systems at half the size" re-tuning the
+//      3->4 switch for each; the stage 1->2 threshold theta and
+//      the split geometry (tile, CTA size) are tuned last with the others
+//      fixed.  Trials therefore add up instead of multiplying.
+//  (2) start every search at the machine-query seed (the STATIC plan) and hill
+//      climb to a local minimum ("a local minimum in a hyperbolic search
+//      space").
+// Results are saved to a cache file for future runs.
+// Ties: candidates within 2% of the incumbent do not replace it; neighbours
+// are visited in a fixed order (decrease before increase).
+#include <algorithm>
+#include <chrono>
+#include <cstdio>
+#include <cstdlib>
+#include <cstring>
+#include <fstream>
+#include <sstream>
+#include <string>
+#include <vector>
+
+#include "common.cuh"
+
+namespace tds {
+
+__device__ __forceinline__ uint64_t mix64(uint64_t z) {
+    z += 0x9E3779B97F4A7C15ull;
+    z = (z ^ (z >> 30)) * 0xBF58476D1CE4E5B9ull;
+    z = (z ^ (z >> 27)) * 0x94D049BB133111EBull;
+    return z ^ (z >> 31);
+}
+
+// Trial data: diagonally dominant random systems (margin 1), tuner-private.
+template <typename T>
+__global__ void fill_dd_kernel(T *a, T *b, T *c, T *d, int64_t n, int64_t m, int64_t stride) {
+    const int64_t total = n * m;
+    for (int64_t idx = blockIdx.x * int64_t(blockDim.x) + threadIdx.x; idx < total;
+         idx += int64_t(gridDim.x) * blockDim.x) {
+        const int64_t s = idx / n, i = idx - s * n;
+        const uint64_t h1 = mix64(uint64_t(idx) * 3 + 1), h2 = mix64(uint64_t(idx) * 3 + 2),
+                       h3 = mix64(uint64_t(idx) * 3 + 3);
+        const T va = i > 0 ? T(2) * T(double(h1 >> 11) * 0x1p-53) - T(1) : T(0);
+        const T vc = i < n - 1 ? T(2) * T(double(h2 >> 11) * 0x1p-53) - T(1) : T(0);
+        const T vd = T(2) * T(double(h3 >> 11) * 0x1p-53) - T(1);
+        const int64_t o = s * stride + i;
+        a[o] = va;
+        c[o] = vc;
+        d[o] = vd;
+        b[o] = fabs(va) + fabs(vc) + T(1);
+    }
+}
+
+struct TuneCtx {
+    tds_plan_st *plan;
+    cudaStream_t st;
+    void *a = nullptr, *b = nullptr, *c = nullptr, *d = nullptr, *x = nullptr, *ws = nullptr;
+    size_t ws_bytes = 0;
+    int trials = 0;
+    int reps = 7;
+    std::chrono::steady_clock::time_point t_start;
+    double budget_s = 50.0;
+};
+
+static bool out_of_time(const TuneCtx &C) {
+    return std::chrono::duration<double>(std::chrono::steady_clock::now() - C.t_start).count() > C.budget_s;
+}
+
+// Median time (ms) of the full solve with parameters p; +inf if rejected.
+static double trial(TuneCtx &C, const tds_params &p) {
+    tds_plan_st tmp = *C.plan;
+    if (derive(tmp.info, tmp.props, p) != TDS_OK) return 1e30;
+    if (tmp.info.workspace_bytes > C.ws_bytes) {
+        if (C.ws) cudaFree(C.ws);
+        C.ws = nullptr;
+        C.ws_bytes = 0;
+        if (cudaMalloc(&C.ws, tmp.info.workspace_bytes) != cudaSuccess) {
+            cudaGetLastError();
+            return 1e30;
+        }
+        C.ws_bytes = tmp.info.workspace_bytes;
+    }
+    ++C.trials;
+    cudaEvent_t e0, e1;
+    cudaEventCreate(&e0);
+    cudaEventCreate(&e1);
+    std::vector<float> ms;
+    bool ok = true;
+    for (int r = 0; r < C.reps + 2 && ok; ++r) {
+        cudaEventRecord(e0, C.st);
+        ok = tds_solve_batched(&tmp, C.a, C.b, C.c, C.d, C.x, C.ws, C.ws_bytes, C.st) == TDS_OK;
+        cudaEventRecord(e1, C.st);
+        if (cudaEventSynchronize(e1) != cudaSuccess) ok = false;
+        float t = 0;
+        cudaEventElapsedTime(&t, e0, e1);
+        if (r >= 2) ms.push_back(t);
+    }
+    cudaEventDestroy(e0);
+    cudaEventDestroy(e1);
+    if (!ok) {
+        cudaGetLastError();
+        return 1e30;
+    }
+    std::sort(ms.begin(), ms.end());
+    return ms[ms.size() / 2];
+}
+
+static bool better(double t_new, double t_best) { return t_new < 0.98 * t_best; }
+
+static int ilog2i(int64_t v) {
+    int l = 0;
+    while ((int64_t(1) << (l + 1)) <= v) ++l;
+    return l;
+}
+
+// Stage 3->4: hill climb over (c, T) for the current k.
+static void tune_onchip(TuneCtx &C, tds_params &best, double &t_best) {
+    const tds_plan_info &I = C.plan->info;
+    bool improved = true;
+    while (improved && !out_of_time(C)) {
+        improved = false;
+        tds_params cand[4];
+        int nc = 0;
+        if (best.thomas_chains > 1) { cand[nc] = best; cand[nc++].thomas_chains /= 2; }
+        cand[nc] = best; cand[nc++].thomas_chains *= 2;
+        if (best.cr_levels > 0) { cand[nc] = best; cand[nc++].cr_levels -= 1; }
+        if ((1 << (best.cr_levels + 1)) <= r_max(I.dtype)) { cand[nc] = best; cand[nc++].cr_levels += 1; }
+        for (int i = 0; i < nc; ++i) {
+            // keep T within the reduced system after a change of c
+            const int64_t n_sub = cdiv(I.n, int64_t(1) << cand[i].k);
+            const int64_t thr = std::max<int64_t>(32, round_up(cdiv(n_sub, int64_t(1) << cand[i].cr_levels), 32));
+            if (cand[i].thomas_chains > thr) continue;
+            const double t = trial(C, cand[i]);
+            if (better(t, t_best)) {
+                best = cand[i];
+                t_best = t;
+                improved = true;
+                break;
+            }
+        }
+    }
+}
+
+static void schedule_passes(tds_params &p, int kpmax) {
+    std::memset(p.k_pass, 0, sizeof(p.k_pass));
+    p.passes = p.k > 0 ? int((p.k + kpmax - 1) / kpmax) : 0;
+    for (int i = 0; i < p.passes; ++i) p.k_pass[i] = p.k / p.passes + (i < p.k % p.passes ? 1 : 0);
+}
+
+// Make (c, T) valid for a new k: smallest c whose CTA fits the kernel's cap, T capped.
+static void fit_onchip(const tds_plan_info &I, tds_params &p) {
+    const int64_t n_sub = cdiv(I.n, int64_t(1) << p.k);
+    auto cap = [](int c) { return (1 << c) >= 8 ? kMaxOnchipThreadsWide : kMaxOnchipThreads; };
+    while (round_up(cdiv(n_sub, int64_t(1) << p.cr_levels), 32) > cap(p.cr_levels) &&
+           (1 << (p.cr_levels + 1)) <= r_max(I.dtype))
+        ++p.cr_levels;
+    const int64_t thr = std::max<int64_t>(32, round_up(cdiv(n_sub, int64_t(1) << p.cr_levels), 32));
+    while (p.thomas_chains > thr) p.thomas_chains /= 2;
+}
+
+static std::string cache_key(const tds_plan_st *plan) {
+    cudaDeviceProp prop;
+    std::string name = "unknown";
+    if (plan->info.device >= 0 && cudaGetDeviceProperties(&prop, plan->info.device) == cudaSuccess) name = prop.name;
+    for (auto &ch : name)
+        if (ch == ' ' || ch == '\t') ch = '_';
+    std::ostringstream o;
+    o << name << "|sm" << plan->props.sm_count << "|smem" << plan->props.smem_optin_bytes << "|"
+      << (plan->info.dtype == TDS_F64 ? "f64" : "f32") << "|n" << plan->info.n << "|m" << plan->info.m << "|s"
+      << plan->info.batch_stride;
+    return o.str();
+}
+
+static std::string params_str(const tds_params &p) {
+    std::ostringstream o;
+    o << p.k << " " << p.passes;
+    for (int i = 0; i < TDS_MAX_PASSES; ++i) o << " " << p.k_pass[i];
+    o << " " << p.cr_levels << " " << p.thomas_chains << " " << p.split_tile_rows << " " << p.split_threads << " "
+      << p.theta;
+    return o.str();
+}
+
+static bool cache_lookup(const std::string &path, const std::string &key, tds_params &p) {
+    std::ifstream f(path);
+    if (!f) return false;
+    std::string line;
+    bool found = false;
+    while (std::getline(f, line)) {  // last matching line wins
+        std::istringstream is(line);
+        std::string k;
+        if (!(is >> k) || k != key) continue;
+        tds_params q{};
+        is >> q.k >> q.passes;
+        for (int i = 0; i < TDS_MAX_PASSES; ++i) is >> q.k_pass[i];
+        is >> q.cr_levels >> q.thomas_chains >> q.split_tile_rows >> q.split_threads >> q.theta;
+        if (is) {
+            p = q;
+            found = true;
+        }
+    }
+    return found;
+}
+
+}  // namespace tds
+
+using namespace tds;
+
+extern "C" tds_status tds_tune(tds_plan_t plan, void *cuda_stream, const char *cache_path) {
+    if (!plan) return fail(TDS_ERR_INVALID_ARG, "plan is NULL");
+    int dev = -1;
+    if (cudaGetDevice(&dev) != cudaSuccess || plan->info.device < 0 || dev != plan->info.device)
+        return fail(TDS_ERR_DEVICE_MISMATCH, "tds_tune must run on the plan's device");
+    std::string path = cache_path ? cache_path : (std::getenv("TDS_TUNE_CACHE") ? std::getenv("TDS_TUNE_CACHE") : "");
+    const std::string key = cache_key(plan);
+    if (!path.empty()) {
+        tds_params p{};
+        if (cache_lookup(path, key, p)) {
+            tds_plan_info info = plan->info;
+            if (derive(info, plan->props, p) == TDS_OK) {
+                info.mode = TDS_PARAMS_TUNED;
+                info.tuned = 1;
+                plan->info = info;
+                plan->tune_trials = 0;
+                clear_error();
+                return TDS_OK;
+            }
+        }
+    }
+    TuneCtx C;
+    C.plan = plan;
+    C.st = static_cast<cudaStream_t>(cuda_stream);
+    C.t_start = std::chrono::steady_clock::now();
+    const tds_plan_info &I = plan->info;
+    const size_t es = size_t(dsize(I.dtype));
+    const size_t bytes = size_t((I.m - 1) * I.batch_stride + I.n) * es;
+    void **bufs[5] = {&C.a, &C.b, &C.c, &C.d, &C.x};
+    for (auto p : bufs) {
+        if (cudaMalloc(p, bytes) != cudaSuccess) {
+            cudaGetLastError();
+            for (auto q : bufs)
+                if (*q) cudaFree(*q);
+            return fail(TDS_ERR_NO_MEMORY, "tuner trial buffers");
+        }
+    }
+    const int64_t total = I.n * I.m;
+    const int blocks = (int)std::min<int64_t>(4096, cdiv(total, 256));
+    if (I.dtype == TDS_F32)
+        fill_dd_kernel<float><<<blocks, 256, 0, C.st>>>((float *)C.a, (float *)C.b, (float *)C.c, (float *)C.d, I.n,
+                                                        I.m, I.batch_stride);
+    else
+        fill_dd_kernel<double><<<blocks, 256, 0, C.st>>>((double *)C.a, (double *)C.b, (double *)C.c,
+                                                         (double *)C.d, I.n, I.m, I.batch_stride);
+    if (total < (1 << 20)) C.reps = 15;
+
+    tds_params best = I.params;
+    double t_best = trial(C, best);
+    tds_status result = TDS_OK;
+    if (t_best >= 1e29) {
+        result = fail(TDS_ERR_TUNE, "the seed plan failed to run");
+    } else {
+        // (1) stage 3->4 switch at the seed's subsystem size
+        tune_onchip(C, best, t_best);
+        // (2) stage 2->3 switch: 2x the systems at half the size (k+1), or the reverse
+        for (int dir : {+1, -1}) {
+            bool moved = true;
+            while (moved && !out_of_time(C)) {
+                moved = false;
+                tds_params cand = best;
+                cand.k += dir;
+                if (cand.k < 0 || cand.k > 30 || (int64_t(1) << cand.k) > 2 * I.n) break;
+                const int kpmax = std::max(I.split_kp_max, 1);
+                schedule_passes(cand, kpmax);
+                fit_onchip(I, cand);
+                double t = trial(C, cand);
+                if (t >= 1e29) break;
+                tune_onchip(C, cand, t);
+                if (better(t, t_best)) {
+                    best = cand;
+                    t_best = t;
+                    moved = true;
+                }
+            }
+        }
+        // (3) stage 1->2 threshold theta and split geometry, one dimension at a time
+        if (best.passes > 0) {
+            bool improved = true;
+            while (improved && !out_of_time(C)) {
+                improved = false;
+                std::vector<tds_params> cands;
+                tds_params q = best;
+                if (best.theta > 1) { q = best; q.theta = std::max(1, best.theta / 2); cands.push_back(q); }
+                q = best; q.theta = best.theta * 2; cands.push_back(q);
+                q = best; q.split_tile_rows = best.split_tile_rows / 2; cands.push_back(q);
+                q = best; q.split_tile_rows = best.split_tile_rows * 2; cands.push_back(q);
+                q = best; q.split_threads = best.split_threads / 2; cands.push_back(q);
+                q = best; q.split_threads = best.split_threads * 2; cands.push_back(q);
+                if (best.passes < TDS_MAX_PASSES && best.k > best.passes) {
+                    // one more (shallower) pass: less halo per pass, one more HBM round trip
+                    q = best;
+                    schedule_passes(q, std::max(1, (best.k + best.passes) / (best.passes + 1)));
+                    cands.push_back(q);
+                }
+                for (auto &cnd : cands) {
+                    const double t = trial(C, cnd);
+                    if (better(t, t_best)) {
+                        best = cnd;
+                        t_best = t;
+                        improved = true;
+                        break;
+                    }
+                }
+            }
+        }
+        tds_plan_info info = plan->info;
+        if (derive(info, plan->props, best) == TDS_OK) {
+            info.mode = TDS_PARAMS_TUNED;
+            info.tuned = 1;
+            plan->info = info;
+        }
+        plan->tune_trials = C.trials;
+        if (!path.empty()) {
+            std::ofstream f(path, std::ios::app);
+            if (f) f << key << " " << params_str(best) << "\n";
+        }
+    }
+    cudaStreamSynchronize(C.st);
+    for (auto p : bufs) cudaFree(*p);
+    if (C.ws) cudaFree(C.ws);
+    if (result == TDS_OK) clear_error();
+    return result;
+}

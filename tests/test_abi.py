@@ -1,0 +1,155 @@
+"""C-ABI boundary tests that need no GPU: the library loads, exports every
+symbol include/tds.h declares, the C++ planner matches the reference planner
+bit-exactly, and argument errors are reported before anything is launched."""
+import ctypes
+import dataclasses
+import os
+import re
+
+import numpy as np
+import pytest
+
+import oracle
+from oracle import plan as rp
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+@pytest.fixture(scope="module")
+def tds():
+    lib_path = os.path.join(ROOT, "paper_conf_ipps_davidsonzo11_b200", "libtds.so")
+    if not os.path.exists(lib_path):
+        import __graft_entry__
+        __graft_entry__.build()
+    import paper_conf_ipps_davidsonzo11_b200 as m
+    m._lib.load()
+    return m
+
+
+def header_functions():
+    src = open(os.path.join(ROOT, "include", "tds.h")).read()
+    src = re.sub(r"/\*.*?\*/", "", src, flags=re.S)
+    return sorted(set(re.findall(r"\b(tds_[a-z_]+)\s*\(", src)))
+
+
+def test_exports_every_header_symbol(tds):
+    names = header_functions()
+    assert len(names) >= 12
+    lib = tds._lib.load()
+    for name in names:
+        assert hasattr(lib, name), name
+    assert sorted(tds._lib.EXPORTED) == names
+    assert tds.version() == 100
+
+
+def test_status_strings(tds):
+    lib = tds._lib.load()
+    for code, name in tds._lib.STATUS_NAMES.items():
+        assert lib.tds_status_string(code).decode().startswith(name)
+
+
+def _props(p):
+    return dataclasses.asdict(p)
+
+
+CASES = []
+for pname, props in [("B200", rp.B200)] + list(rp.TABLE_I.items()):
+    for dtype in (rp.F32, rp.F64):
+        for mode in (rp.DEFAULT, rp.STATIC):
+            for n, m in [(1, 1), (2, 3), (255, 2), (256, 1), (257, 1), (1000, 7), (1024, 1), (4097, 3),
+                         (65536, 256), (1 << 20, 16), (16384, 4096), (1 << 28, 1), (3 * 10 ** 6 + 7, 2),
+                         (8192, 1), (8193, 5)]:
+                CASES.append((pname, props, dtype, mode, n, m))
+
+
+@pytest.mark.parametrize("pname,props,dtype,mode,n,m", CASES)
+def test_planner_matches_reference(tds, pname, props, dtype, mode, n, m):
+    """Integer plan bit-exact vs the plain-Python reference planner (oracle/plan.py)."""
+    try:
+        ref = rp.make_plan(props, dtype, n, m, 0, mode)
+    except ValueError as e:
+        assert "unsupported" in str(e)
+        with pytest.raises(tds.TdsError) as ce:
+            tds.Plan(n, m, "float32" if dtype == rp.F32 else "float64", props=_props(props),
+                     mode="default" if mode == rp.DEFAULT else "static")
+        assert ce.value.name == "TDS_ERR_UNSUPPORTED"
+        return
+    p = tds.Plan(n, m, "float32" if dtype == rp.F32 else "float64", props=_props(props),
+                 mode="default" if mode == rp.DEFAULT else "static")
+    got = p.info
+    for f in ("k", "passes", "n_sub", "num_subsystems", "cr_levels", "thomas_chains", "onchip_threads",
+              "split_tile_rows", "split_threads", "split_segments", "theta", "n_sub_target", "n_onchip_max",
+              "split_kp_max", "slot_rows", "workspace_bytes"):
+        assert got[f] == getattr(ref, f), (f, got[f], getattr(ref, f))
+    assert got["k_pass"] == ref.k_pass[:ref.passes]
+
+
+@pytest.mark.parametrize("n", [1, 5, 8, 100, 1023, 70000])
+def test_permutation_matches_oracle(tds, n):
+    for k in range(0, 9):
+        p = tds.Plan(n, 1, props=_props(rp.B200), mode="static")
+        if k:
+            try:
+                p.set_params(k_pass=[k], cr_levels=4 if n > 4096 else 0, thomas_chains=1)
+            except tds.TdsError:
+                continue
+        assert np.array_equal(p.permutation(), oracle.permutation(n, p.info["k"]))
+
+
+def test_plan_argument_errors(tds):
+    lib = tds._lib.load()
+    h = ctypes.c_void_p()
+    props = tds._lib.DeviceProps(**_props(rp.B200))
+    st = lambda *a: lib.tds_plan_from_props(ctypes.byref(h), ctypes.byref(props), *a)
+    assert st(0, 0, 1, 0, 1) == 1          # n < 1
+    assert st(0, 10, 0, 0, 1) == 1         # m < 1
+    assert st(0, 10, 1, 5, 1) == 1         # stride < n
+    assert st(2, 10, 1, 0, 1) == 1         # bad dtype
+    assert st(0, 10, 1, 0, 2) == 1         # TUNED is set by tds_tune only
+    assert st(0, 10, 1, 0, 9) == 1
+    assert lib.tds_plan_from_props(None, ctypes.byref(props), 0, 10, 1, 0, 1) == 1
+    assert st(0, 10, 1, 0, 1) == 0
+    lib.tds_plan_destroy(h)
+
+
+def test_set_params_validation(tds):
+    p = tds.Plan(1 << 20, 4, props=_props(rp.B200))
+    before = p.info
+    with pytest.raises(tds.TdsError) as e:
+        p.set_params(k_pass=[7], cr_levels=5)  # R = 32 > R_max
+    assert e.value.name == "TDS_ERR_UNSUPPORTED"
+    with pytest.raises(tds.TdsError):
+        p.set_params(thomas_chains=48)  # not a power of two
+    with pytest.raises(tds.TdsError):
+        p.set_params(k_pass=[3], cr_levels=0)  # 131072-row subsystems do not fit on chip
+    assert p.info == before  # unchanged after rejections
+    p.set_params(k_pass=[5, 5], cr_levels=3, thomas_chains=16)
+    i = p.info
+    assert (i["k"], i["passes"], i["k_pass"], i["n_sub"], i["mode"]) == (10, 2, [5, 5], 1024, 2)
+    assert i["workspace_bytes"] == 2 * 3 * 4 * max(4 * 32 * rp.slot_rows(1 << 20, 5, 0),
+                                                   4 * 1024 * rp.slot_rows(1 << 20, 10, 0))
+
+
+def test_solve_argument_errors_before_launch(tds):
+    """Argument checks run on the host before any CUDA call; a plan built from
+    fake properties has no device, so a valid call ends in DEVICE_MISMATCH or
+    a CUDA error (no GPU here) -- never in a launch."""
+    lib = tds._lib.load()
+    p = tds.Plan(1000, 4, props=_props(rp.B200))
+    p.set_params(k_pass=[2], cr_levels=0, thomas_chains=32)
+    ws_need = p.workspace_bytes
+    base = 1 << 40
+    nbytes = 4 * 4000
+    A, B, C, D, X = (base + i * (1 << 30) for i in range(5))
+    W = base + 10 * (1 << 30)
+    f = lambda *a: lib.tds_solve_batched(p.handle, *a, None)
+    assert f(None, B, C, D, X, W, ws_need) == 1                 # NULL
+    assert f(A + 2, B, C, D, X, W, ws_need) == 1                # misaligned
+    assert f(A, B, C, D, A + 4, W, ws_need) == 1                # x overlaps a
+    assert f(A, B, C, D, D + 8, W, ws_need) == 1                # x partially overlaps d
+    assert f(A, B, C, D, X, None, ws_need) == 4                 # workspace NULL
+    assert f(A, B, C, D, X, W, ws_need - 1) == 4                # too small
+    assert f(A, B, C, D, X, W + 16, ws_need) == 4               # misaligned workspace
+    assert f(A, B, C, D, X, A, ws_need) == 1                    # workspace overlaps an array
+    assert f(A, B, C, D, D, W, ws_need) in (5, 7)               # valid (x == d): no device here
+    assert nbytes < (1 << 30)

@@ -1,0 +1,329 @@
+"""GPU parity: the CUDA path (through the C ABI) against the CPU oracle on the
+same seeded inputs.  Tolerances (BASELINE.json north_star; R17):
+fp32 normwise relative error <= 1e-4 and residual <= 1e-5; fp64 relative
+error <= 1e-10.  Integer/index outputs (permutation, split structure) bit-exact."""
+import math
+
+import numpy as np
+import pytest
+
+import oracle
+from paper_conf_ipps_davidsonzo11_b200 import inputs
+
+pytestmark = pytest.mark.gpu
+
+TOL = {np.float32: (1e-4, 1e-5), np.float64: (1e-10, 1e-12)}
+
+
+@pytest.fixture(scope="module")
+def tds():
+    import torch
+    assert torch.cuda.is_available()
+    import paper_conf_ipps_davidsonzo11_b200 as m
+    m._lib.load()
+    return m
+
+
+def to_dev(*arrs):
+    import torch
+    return [torch.from_numpy(np.ascontiguousarray(v)).cuda() for v in arrs]
+
+
+def run(tds, a, b, c, d, mode="static", params=None, stride=0, inplace=False):
+    import torch
+    m, n = d.shape
+    dt = "float32" if d.dtype == np.float32 else "float64"
+    plan = tds.Plan(n, m, dt, device=0, mode=mode)
+    if params:
+        plan.set_params(**params)
+    ta, tb, tc, td = to_dev(a, b, c, d)
+    x = tds.solve_batched(plan, ta, tb, tc, td, out=td if inplace else None)
+    torch.cuda.synchronize()
+    return x.cpu().numpy(), plan
+
+
+def check(a, b, c, d, x, dtype, xr=None):
+    if xr is None:
+        xr = oracle.thomas(a, b, c, d)
+    err = oracle.rel_err(x, xr)
+    etol, rtol = TOL[dtype]
+    assert np.all(np.isfinite(x))
+    assert err <= etol, f"rel_err {err:.3e} > {etol}"
+    if dtype == np.float32:
+        res = oracle.residual(a, b, c, d, x)
+        assert res <= rtol, f"residual {res:.3e} > {rtol}"
+    return err
+
+
+# ------------------------------------------------ on-chip kernel alone (k = 0)
+
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("n", [1, 2, 3, 31, 32, 33, 100, 1000, 1024, 4097, 8192])
+def test_onchip_k0_static(tds, dtype, n):
+    if dtype == np.float64 and n > 4096:
+        n = 4096
+    a, b, c, d = inputs.generate(n, 5, dtype, seed=21)
+    x, plan = run(tds, a, b, c, d, params=None)
+    assert plan.info["k"] == 0
+    check(a, b, c, d, x, dtype)
+
+
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("c_lv", [0, 1, 2, 3, 4])
+@pytest.mark.parametrize("T", [1, 4, 32, 64, 1024])
+def test_onchip_switch_points(tds, dtype, c_lv, T):
+    """Every (c, T) switch point of the hybrid CR/PCR-Thomas kernel: c = 0 is the
+    paper's PCR-Thomas; T = threads is pure PCR on the reduced system; T = 1 is
+    a single Thomas chain."""
+    if dtype == np.float64 and c_lv > 3:
+        pytest.skip("R_max = 8 for fp64")
+    n = 1000
+    nred = -(-n // (1 << c_lv))
+    threads = max(32, -(-nred // 32) * 32)
+    if T > threads:
+        pytest.skip("T > threads")
+    a, b, c, d = inputs.generate(n, 3, dtype, seed=5)
+    x, _ = run(tds, a, b, c, d, params=dict(cr_levels=c_lv, thomas_chains=T))
+    check(a, b, c, d, x, dtype)
+
+
+# ------------------------------------------------ split passes + on-chip
+
+SPLIT_CASES = [
+    # n, m, k_pass, c, T, tile
+    (4096, 3, [1], 1, 32, 1024),
+    (4096, 3, [2], 2, 16, 256),
+    (5000, 2, [3], 0, 32, 1024),
+    (65536, 2, [3], 4, 64, 8192),
+    (70001, 2, [4], 4, 64, 4096),
+    (1 << 20, 2, [7], 4, 64, 8192),
+    (1 << 18, 1, [9], 2, 32, 8192),
+    (123457, 1, [5, 4], 2, 32, 2048),
+    (1 << 16, 3, [3, 3, 3], 0, 64, 512),
+    (1000, 2, [6, 4], 0, 1, 1024),   # 2^k > n: empty slots
+    (37, 4, [2, 2, 1], 0, 1, 32),
+]
+
+
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("n,m,kp,c_lv,T,tile", SPLIT_CASES)
+def test_split_then_onchip(tds, dtype, n, m, kp, c_lv, T, tile):
+    if dtype == np.float64 and c_lv > 3:
+        c_lv = 3
+    a, b, c, d = inputs.generate(n, m, dtype, seed=33)
+    params = dict(k_pass=kp, cr_levels=c_lv, thomas_chains=T, split_tile_rows=tile,
+                  split_threads=512 if tile >= 8192 else 256)
+    try:
+        x, plan = run(tds, a, b, c, d, params=params)
+    except tds.TdsError as e:
+        pytest.skip(f"plan rejected: {e}")
+    check(a, b, c, d, x, dtype)
+
+
+@pytest.mark.parametrize("theta", [1, 4, 148, 10 ** 6])
+def test_cooperative_segments(tds, theta):
+    """Stage 1 (several CTAs per system, theta large) and stage 2 (one CTA per
+    system, theta small) produce the same x bit-exactly."""
+    n, m = 200000, 3
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=3)
+    base = dict(k_pass=[5], cr_levels=4, thomas_chains=32, split_tile_rows=4096)
+    x0, _ = run(tds, a, b, c, d, params=dict(base, theta=1))
+    x1, plan = run(tds, a, b, c, d, params=dict(base, theta=theta))
+    assert np.array_equal(x0, x1)
+    check(a, b, c, d, x1, np.float32)
+
+
+# ------------------------------------------------ the split stage itself
+
+def split_gpu(tds, a, b, c, d, params):
+    import torch
+    m, n = d.shape
+    dt = "float32" if d.dtype == np.float32 else "float64"
+    plan = tds.Plan(n, m, dt, device=0)
+    plan.set_params(**params)
+    oa, oc, od = tds.split_batched(plan, *to_dev(a, b, c, d))
+    torch.cuda.synchronize()
+    return oa.cpu().numpy(), oc.cpu().numpy(), od.cpu().numpy(), plan
+
+
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("n,kp", [(1000, [3]), (4096, [5]), (777, [2, 2]), (20000, [4, 3]), (300, [9])])
+def test_split_vs_oracle_pcr(tds, dtype, n, kp):
+    """Split coefficients vs the oracle's textbook PCR (fp64), normalised by b'
+    and put in canonical order (tds_plan_permutation == oracle.permutation)."""
+    a, b, c, d = inputs.generate(n, 2, dtype, seed=12)
+    ga, gc, gd, plan = split_gpu(tds, a, b, c, d, dict(k_pass=kp, cr_levels=0, thomas_chains=1,
+                                                      split_tile_rows=1024, split_threads=256))
+    k = sum(kp)
+    perm = plan.permutation()
+    assert np.array_equal(perm, oracle.permutation(n, k))
+    sa, sb, sc, sd = oracle.pcr_split(a, b, c, d, k)
+    ref = [v[:, perm] / sb[:, perm] for v in (sa, sc, sd)]
+    tol = 1e-5 if dtype == np.float32 else 1e-13
+    for g, r in zip((ga, gc, gd), ref):
+        assert np.abs(g - r).max() <= tol * max(1.0, np.abs(r).max())
+
+
+@pytest.mark.parametrize("n,kp", [(300, [1]), (300, [4]), (1000, [5]), (4099, [3, 3])])
+def test_split_exact_zeros(tds, n, kp):
+    """a' = 0 at the first row and c' = 0 at the last row of every subsystem (bit-exact)."""
+    a, b, c, d = inputs.generate(n, 2, np.float32, seed=1)
+    ga, gc, gd, plan = split_gpu(tds, a, b, c, d, dict(k_pass=kp, cr_levels=0, thomas_chains=1,
+                                                      split_tile_rows=1024, split_threads=256))
+    k = sum(kp)
+    step = 1 << k
+    off = 0
+    for r in range(min(step, n)):
+        nr = -(-(n - r) // step)
+        assert np.all(ga[:, off] == 0) and np.all(gc[:, off + nr - 1] == 0)
+        off += nr
+
+
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("kp", [[1], [3], [7], [4, 3]])
+def test_split_poisson_interior_exact(tds, dtype, kp):
+    """On tridiag(-1,2,-1) every normalised level gives interior a' = c' = -1/2
+    exactly (1 - 1/4 - 1/4 = 1/2, rcp(1/2) = 2): pins long strides bit-exactly."""
+    n = 5000
+    a, b, c, d = inputs.generate(n, 1, dtype, family="poisson")
+    ga, gc, gd, plan = split_gpu(tds, a, b, c, d, dict(k_pass=kp, cr_levels=0, thomas_chains=1,
+                                                      split_tile_rows=1024, split_threads=256))
+    k = sum(kp)
+    perm = plan.permutation()
+    rows = perm  # original row of each canonical position
+    interior = (rows >= (1 << k)) & (rows <= n - 1 - (1 << k))
+    assert interior.sum() > n // 2
+    assert np.all(ga[0, interior] == -0.5) and np.all(gc[0, interior] == -0.5)
+
+
+def test_split_fused_equals_multipass_and_tiles(tds):
+    """Halo exactness: k = 6 fused in one pass == 3 + 3 in two passes == other
+    tile sizes, bit-exactly (same row update on the same operands)."""
+    n = 50000
+    a, b, c, d = inputs.generate(n, 2, np.float32, seed=4)
+    base = dict(cr_levels=0, thomas_chains=1, split_threads=256)
+    r1 = split_gpu(tds, a, b, c, d, dict(base, k_pass=[6], split_tile_rows=1024))
+    r2 = split_gpu(tds, a, b, c, d, dict(base, k_pass=[3, 3], split_tile_rows=1024))
+    r3 = split_gpu(tds, a, b, c, d, dict(base, k_pass=[6], split_tile_rows=4096, theta=1))
+    r4 = split_gpu(tds, a, b, c, d, dict(base, k_pass=[2, 2, 2], split_tile_rows=64))
+    for other in (r2, r3, r4):
+        for u, v in zip(r1[:3], other[:3]):
+            assert np.array_equal(u, v)
+
+
+# ------------------------------------------------ layout, aliasing, isolation
+
+def test_batch_isolation(tds):
+    n, m = 30000, 4
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=8)
+    x0, _ = run(tds, a, b, c, d, params=dict(k_pass=[3], cr_levels=4, thomas_chains=64))
+    d2 = d.copy(); b2 = b.copy()
+    d2[2] *= 1e6; b2[2] += 5
+    x1, _ = run(tds, a, b2, c, d2, params=dict(k_pass=[3], cr_levels=4, thomas_chains=64))
+    for s in (0, 1, 3):
+        assert np.array_equal(x0[s], x1[s])
+
+
+def test_inplace_and_stride(tds):
+    import torch
+    n, m, stride = 10000, 3, 10007
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=9)
+    pad = lambda v: np.pad(v, ((0, 0), (0, stride - n)), constant_values=7.0)
+    A, B, C, D = (pad(v).reshape(-1) for v in (a, b, c, d))
+    plan = tds.Plan(n, m, "float32", device=0, batch_stride=stride)
+    plan.set_params(k_pass=[2], cr_levels=4, thomas_chains=64)
+    ta, tb, tc, td = to_dev(A, B, C, D)
+    x = tds.solve_batched(plan, ta, tb, tc, td, out=td)  # in place
+    torch.cuda.synchronize()
+    xs = x.cpu().numpy().reshape(m, stride)
+    assert np.all(xs[:, n:] == 7.0)  # padding untouched
+    check(a, b, c, d, xs[:, :n], np.float32)
+
+
+def test_workspace_errors(tds):
+    import torch
+    n, m = 4096, 2
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=1)
+    plan = tds.Plan(n, m, "float32", device=0)
+    plan.set_params(k_pass=[2], cr_levels=2, thomas_chains=32)
+    ta, tb, tc, td = to_dev(a, b, c, d)
+    small = torch.empty(plan.workspace_bytes - 256, dtype=torch.uint8, device="cuda")
+    with pytest.raises(tds.TdsError) as e:
+        tds.solve_batched(plan, ta, tb, tc, td, workspace=small)
+    assert e.value.name == "TDS_ERR_WORKSPACE"
+
+
+# ------------------------------------------------ other value families (fp64, kappa-scaled)
+
+@pytest.mark.parametrize("family,kw", [("poisson", {}), ("const", {"param": 0.01}), ("adi", {"param": 10.0}),
+                                       ("weak", {"param": 0.1}), ("weak", {"param": 0.01})])
+def test_families_fp64(tds, family, kw):
+    n, m = 100000, 2
+    a, b, c, d = inputs.generate(n, m, np.float64, seed=2, family=family, **kw)
+    x, _ = run(tds, a, b, c, d, params=dict(k_pass=[5], cr_levels=3, thomas_chains=32))
+    xr = oracle.thomas(a, b, c, d)
+    assert oracle.backward_error(a, b, c, d, x) <= 1e-13
+    if family == "poisson":
+        kappa = 4 * (n + 1) ** 2 / math.pi ** 2
+        assert oracle.rel_err(x, xr) <= 100 * kappa * 2.2e-16
+    else:
+        assert oracle.rel_err(x, xr) <= 1e-10
+
+
+# ------------------------------------------------ BASELINE.json configs (bench launch configuration)
+
+@pytest.mark.parametrize("dtype", [np.float32])
+def test_config1_full(tds, dtype):
+    a, b, c, d = inputs.generate(1024, 1, dtype, seed=inputs.config_seed(1, dtype))
+    for mode in ("default", "static"):
+        x, _ = run(tds, a, b, c, d, mode=mode)
+        check(a, b, c, d, x, dtype)
+
+
+@pytest.mark.parametrize("cfg,n,m,dtype", [(2, 65536, 256, np.float32), (3, 1 << 20, 16, np.float32),
+                                            (3, 1 << 20, 16, np.float64)])
+def test_config_full_static_and_default(tds, cfg, n, m, dtype):
+    a, b, c, d = inputs.generate(n, m, dtype, seed=inputs.config_seed(cfg, dtype))
+    xr = oracle.thomas(a, b, c, d)
+    for mode in ("static", "default"):
+        x, plan = run(tds, a, b, c, d, mode=mode)
+        check(a, b, c, d, x, dtype, xr=xr)
+
+
+def test_config4_sampled(tds):
+    """4096 x 16384 fp32: the full batch on the GPU, 48 sampled systems through the oracle."""
+    n, m = 16384, 4096
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=inputs.config_seed(4, np.float32))
+    x, _ = run(tds, a, b, c, d, mode="static")
+    rng = np.random.default_rng(0)
+    idx = np.sort(np.concatenate([[0, m - 1], rng.choice(m, 46, replace=False)]))
+    check(a[idx], b[idx], c[idx], d[idx], x[idx], np.float32)
+
+
+@pytest.mark.slow
+def test_config5_single_gpu_part(tds):
+    """1 x 2^26 fp32 (the single-GPU half of config 5's schedule: 2 passes)."""
+    n = 1 << 26
+    a, b, c, d = inputs.generate(n, 1, np.float32, seed=5)
+    x, plan = run(tds, a, b, c, d, mode="static")
+    assert plan.info["passes"] == 2
+    check(a, b, c, d, x, np.float32)
+
+
+def test_tuner_runs_and_caches(tds, tmp_path):
+    import torch
+    n, m = 1 << 18, 8
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=1)
+    plan = tds.Plan(n, m, "float32", device=0)
+    cache = str(tmp_path / "tune.txt")
+    trials = plan.tune(cache_path=cache)
+    assert trials >= 3
+    info = plan.info
+    assert info["mode"] == 2 and info["tuned"] == 1
+    ta, tb, tc, td = to_dev(a, b, c, d)
+    x = tds.solve_batched(plan, ta, tb, tc, td)
+    torch.cuda.synchronize()
+    check(a, b, c, d, x.cpu().numpy(), np.float32)
+    plan2 = tds.Plan(n, m, "float32", device=0)
+    assert plan2.tune(cache_path=cache) == 0  # saved result reused
+    assert plan2.info["k"] == info["k"] and plan2.info["thomas_chains"] == info["thomas_chains"]
