@@ -186,7 +186,7 @@ def test_split_poisson_interior_exact(tds, dtype, kp):
     exactly (1 - 1/4 - 1/4 = 1/2, rcp(1/2) = 2): pins long strides bit-exactly."""
     n = 5000
     a, b, c, d = inputs.generate(n, 1, dtype, family="poisson")
-    ga, gc, gd, plan = split_gpu(tds, a, b, c, d, dict(k_pass=kp, cr_levels=0, thomas_chains=1,
+    ga, gc, gd, plan = split_gpu(tds, a, b, c, d, dict(k_pass=kp, cr_levels=3, thomas_chains=1,
                                                       split_tile_rows=1024, split_threads=256))
     k = sum(kp)
     perm = plan.permutation()
