@@ -394,7 +394,7 @@ def run_tds(args):
         "config": {"workload": f"config{args.config}: {m} x {n} {args.dtype} per GPU", "n": n, "m": m,
                    "mode": args.mode, "plan": {k: info[k] for k in ("k", "passes", "k_pass", "n_sub",
                                                                      "cr_levels", "thomas_chains",
-                                                                     "split_tile_rows", "split_threads",
+                                                                     "cluster", "tl_levels", "split_tile_rows", "split_threads",
                                                                      "theta", "split_segments",
                                                                      "onchip_threads", "workspace_bytes")},
                    "tune_trials": trials, "tune_s": round(tune_s, 2),

@@ -96,8 +96,10 @@ typedef struct {
     int32_t k_pass[TDS_MAX_PASSES];  /* levels fused in each pass, sum == k             */
     int32_t cr_levels;               /* c: CR levels in registers (R = 2^c rows/thread)  */
     int32_t thomas_chains;           /* T: Thomas chains of the reduced system (pow2)   */
-    int32_t split_tile_rows;         /* split-pass tile (pow2, >= 2^k_pass[i])          */
-    int32_t split_threads;           /* split-pass CTA size (multiple of 32)            */
+    int32_t cluster;                 /* CTAs (SMs) sharing one subsystem: 1,2,4,8,16    */
+    int32_t tl_levels;               /* c2: CR levels across threads (shared memory)    */
+    int32_t split_tile_rows;         /* shared-memory split pass tile (k_pass > 4 only) */
+    int32_t split_threads;           /* shared-memory split pass CTA size (k_pass > 4)  */
     int32_t theta;                   /* stage 1->2 switch: independent systems needed   */
 } tds_params;
 
@@ -114,9 +116,8 @@ typedef struct {
     int32_t split_kp_max;     /* max levels per split pass                             */
     int32_t onchip_threads;   /* on-chip kernel CTA size                               */
     int32_t subsys_per_cta;   /* on-chip subsystems per CTA (1)                        */
-    int32_t cluster;          /* CTAs per cluster (1)                                  */
     int32_t split_segments;   /* CTAs cooperating on one system in pass 1 (stage 1)    */
-    int32_t pad_;
+    int32_t split_tile_eff;   /* rows one split CTA produces per tile in pass 1        */
     int64_t slot_rows;        /* workspace rows reserved per subsystem (final pass)    */
     size_t workspace_bytes;   /* bytes tds_solve_batched needs (0 when k == 0)         */
 } tds_plan_info;

@@ -84,12 +84,20 @@ def pow2ceil(x: int) -> int:
     return p
 
 
+def static_cluster(props: Props) -> int:
+    """Thread-block clusters exist from compute capability 9.0; 8 CTAs is the
+    portable maximum.  Older devices (Table I) have none: 1."""
+    return 8 if props.cc_major >= 9 else 1
+
+
 def n_onchip_max(props: Props, dtype: int) -> int:
-    """Largest power of two n with 4 n sizeof(T) <= smem_optin - reserve,
-    capped at the on-chip kernel's register capacity (8192 fp32 / 4096 fp64)."""
+    """Largest power of two n whose four arrays fit in the shared memory of one
+    cluster (4 n sizeof(T) <= (smem_optin - reserve) x C), capped at the
+    on-chip kernel's register capacity (R_max x 512 threads x C)."""
     s = dsize(dtype)
-    cap = 8192 if dtype == F32 else 4096
-    budget = props.smem_optin_bytes - SMEM_RESERVE
+    C = static_cluster(props)
+    cap = r_max(dtype) * 512 * C
+    budget = (props.smem_optin_bytes - SMEM_RESERVE) * C
     n = 1
     while n * 2 <= cap and 4 * (n * 2) * s <= budget:
         n *= 2
@@ -98,6 +106,10 @@ def n_onchip_max(props: Props, dtype: int) -> int:
 
 def r_max(dtype: int) -> int:
     return 16 if dtype == F32 else 8
+
+
+REG_SPLIT_MAX_KP = 4          # split passes with k_p <= 4 use the register kernel
+REG_SPLIT_TILE = 16 * 256 - 32  # rows it produces per CTA tile
 
 
 @dataclass
@@ -117,6 +129,7 @@ class Plan:
     onchip_threads: int = 0
     subsys_per_cta: int = 1
     cluster: int = 1
+    tl_levels: int = 0
     split_tile_rows: int = 0
     split_threads: int = 0
     split_segments: int = 0
@@ -166,12 +179,14 @@ def make_plan(props: Props, dtype: int, n: int, m: int, batch_stride: int = 0,
     if mode == DEFAULT:
         target, T, theta = DEFAULT_NSUB_TARGET, DEFAULT_THOMAS, DEFAULT_THETA
         tile, g1t, kpmax, g2cap = DEFAULT_TILE, DEFAULT_SPLIT_THREADS, DEFAULT_KP_MAX, DEFAULT_G2_THREAD_CAP
+        cmax = 1
     else:
         target = p.n_onchip_max
         T = STATIC_THOMAS_PER_WARP * props.warp_size
         theta = props.sm_count
-        tile = p.n_onchip_max
+        tile = min(p.n_onchip_max, r_max(dtype) * 512)
         g1t = STATIC_SPLIT_THREADS
+        cmax = static_cluster(props)
         kpmax = 9 if dtype == F32 else 8
         budget = props.smem_optin_bytes - SMEM_RESERVE
         while kpmax > 1 and (split_smem_bytes(dtype, tile, kpmax) > budget
@@ -196,22 +211,32 @@ def make_plan(props: Props, dtype: int, n: int, m: int, batch_stride: int = 0,
         for i in range(P):
             p.k_pass[i] = base + (1 if i < extra else 0)
 
-    # Stage 3->4 switch inside the on-chip kernel: R = 2^c rows per thread
-    # (c CR levels), then PCR on the reduced system until T Thomas chains.
+    # Stage 3->4 switch inside the on-chip kernel: the smallest cluster of C
+    # CTAs that holds the subsystem, R = 2^c rows per thread (c CR levels),
+    # then PCR on the reduced system until T Thomas chains.
+    C = 1
+    while C < cmax and p.n_sub > C * r_max(dtype) * g2cap:
+        C *= 2
     R = 1
-    while cdiv(p.n_sub, R) > g2cap and R < r_max(dtype):
+    while cdiv(p.n_sub, R * C) > g2cap and R < r_max(dtype):
         R *= 2
-    nred = cdiv(p.n_sub, R)
+    if C > 1 and R < 8:
+        R = 8
+    nred = cdiv(p.n_sub, R * C)
+    p.cluster = C
     p.cr_levels = R.bit_length() - 1
     p.onchip_threads = max(32, round_up(nred, 32))
-    p.thomas_chains = min(T, pow2ceil(nred))
+    # CR across threads until the leader's system has one row per thread
+    p.tl_levels = C.bit_length() - 1
+    p.thomas_chains = min(T, pow2ceil(cdiv(p.n_sub, R) >> p.tl_levels))
 
     # Kernel limits (the C++ planner rejects these plans as UNSUPPORTED).
     budget = props.smem_optin_bytes - SMEM_RESERVE
     for i in range(P):
-        if split_smem_bytes(dtype, tile, p.k_pass[i]) > budget:
+        if p.k_pass[i] > REG_SPLIT_MAX_KP and split_smem_bytes(dtype, tile, p.k_pass[i]) > budget:
             raise ValueError("unsupported: split tile + halo exceeds shared memory")
-    if (9 * p.onchip_threads + 8) * s > budget:
+    nt = p.onchip_threads
+    if (3 * C * (nt >> p.tl_levels) + 4 * nt + 6 * (nt // 32) + 48) * s > budget:
         raise ValueError("unsupported: on-chip shared memory")
 
     # Workspace: split output (normalised a, c, d) in fixed slots; ping-pong if P >= 2.
@@ -223,5 +248,6 @@ def make_plan(props: Props, dtype: int, n: int, m: int, batch_stride: int = 0,
         E = round_up(elems, 64)
         p.slot_rows = slot_rows(n, k, dtype)
         p.workspace_bytes = (1 if P == 1 else 2) * 3 * E * s
-        p.split_segments = segments(m, cdiv(n, tile), theta)
+        tile_eff = REG_SPLIT_TILE if p.k_pass[0] <= REG_SPLIT_MAX_KP else tile
+        p.split_segments = segments(m, cdiv(n, tile_eff), theta)
     return p

@@ -40,7 +40,9 @@ class DeviceProps(ctypes.Structure):
 class Params(ctypes.Structure):
     _fields_ = [("k", ctypes.c_int32), ("passes", ctypes.c_int32),
                 ("k_pass", ctypes.c_int32 * TDS_MAX_PASSES), ("cr_levels", ctypes.c_int32),
-                ("thomas_chains", ctypes.c_int32), ("split_tile_rows", ctypes.c_int32),
+                ("thomas_chains", ctypes.c_int32), ("cluster", ctypes.c_int32),
+                ("tl_levels", ctypes.c_int32),
+                ("split_tile_rows", ctypes.c_int32),
                 ("split_threads", ctypes.c_int32), ("theta", ctypes.c_int32)]
 
 
@@ -51,7 +53,7 @@ class PlanInfo(ctypes.Structure):
                 ("num_subsystems", ctypes.c_int64), ("n_sub_target", ctypes.c_int32),
                 ("n_onchip_max", ctypes.c_int32), ("split_kp_max", ctypes.c_int32),
                 ("onchip_threads", ctypes.c_int32), ("subsys_per_cta", ctypes.c_int32),
-                ("cluster", ctypes.c_int32), ("split_segments", ctypes.c_int32), ("pad_", ctypes.c_int32),
+                ("split_segments", ctypes.c_int32), ("split_tile_eff", ctypes.c_int32),
                 ("slot_rows", ctypes.c_int64), ("workspace_bytes", ctypes.c_size_t)]
 
 

@@ -38,6 +38,15 @@ static tds_status check_workspace(const tds_plan_info &I, const void *ws, size_t
     return TDS_OK;
 }
 
+// 16-byte vector access to the caller's arrays: every system start must be aligned.
+static int vec_ok(const tds_plan_info &I, std::initializer_list<const void *> ptrs) {
+    const int64_t es = dsize(I.dtype);
+    if ((I.batch_stride * es) % 16) return 0;
+    for (const void *p : ptrs)
+        if (reinterpret_cast<uintptr_t>(p) % 16) return 0;
+    return 1;
+}
+
 // Workspace buffer i holds normalised (a, c, d) arrays of E elements each.
 template <typename T>
 struct WsBufs {
@@ -104,13 +113,19 @@ static tds_status run_split(const tds_plan_info &I, const T *a, const T *b, cons
         for (int q = 0; q < kMaxPasses; ++q) A.geom.kpass[q] = q < p ? P.k_pass[q] : 0;
         const int64_t m_in = I.m << kprev;
         const int64_t len_in = cdiv(I.n, int64_t(1) << kprev);
-        A.segs = split_segments(m_in, cdiv(len_in, P.split_tile_rows), P.theta);
+        A.segs = split_segments(m_in, cdiv(len_in, split_tile_eff(P, p)), P.theta);
         const int64_t e = P.split_tile_rows + 2 * ((int64_t(1) << kp) - 1);
         A.ep = int32_t(e + (e >> std::max(kp, 5)) + 1);
+        A.vec = raw ? vec_ok(I, {a, b, c, d}) : 1;
         const int64_t grid = m_in * A.segs;
         if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "split grid exceeds 2^31-1 CTAs");
-        const size_t smem = split_smem_bytes(I.dtype, P.split_tile_rows, kp);
-        cudaError_t err = launch_split_pass<T>(A, raw, grid, P.split_threads, smem, st);
+        cudaError_t err;
+        if (kp <= kRegSplitMaxKp) {
+            err = launch_split_reg<T>(A, raw, grid, st);
+        } else {
+            const size_t smem = split_smem_bytes(I.dtype, P.split_tile_rows, kp);
+            err = launch_split_pass<T>(A, raw, grid, P.split_threads, smem, st);
+        }
         if (err != cudaSuccess) return cuda_fail(err, "split_pass launch");
         kprev += kp;
     }
@@ -130,14 +145,18 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
     int t = P.thomas_chains, l2 = 0;
     while ((1 << l2) < t) ++l2;
     A.log2T = l2;
+    A.cluster = P.cluster;
+    A.tl_levels = P.tl_levels;
     int64_t grid;
     if (P.k == 0) {
         A.a = a;
         A.b = b;
         A.c = c;
         A.d = d;
-        grid = I.m;
+        A.vec = vec_ok(I, {a, b, c, d, x});
+        grid = I.m * P.cluster;
     } else {
+        A.vec = 1;
         WsBufs<T> w = ws_bufs<T>(I, ws);
         int ob = 0;
         tds_status s = run_split<T>(I, a, b, c, d, w, st, &ob, first, last);
@@ -149,11 +168,11 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
         A.slot = I.slot_rows;
         A.geom.npass = P.passes;
         for (int q = 0; q < kMaxPasses; ++q) A.geom.kpass[q] = P.k_pass[q];
-        grid = I.m << P.k;
+        grid = (I.m << P.k) * P.cluster;
     }
     if (P.passes < first || P.passes > last) return TDS_OK;  // on-chip stage not requested
     if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "on-chip grid exceeds 2^31-1 CTAs");
-    const size_t smem = onchip_smem_bytes(I.dtype, I.onchip_threads);
+    const size_t smem = onchip_smem_bytes(I.dtype, I.onchip_threads, P.cluster, P.tl_levels);
     cudaError_t err = launch_onchip<T>(A, P.cr_levels, P.k == 0, grid, I.onchip_threads, smem, st);
     if (err != cudaSuccess) return cuda_fail(err, "onchip launch");
     return TDS_OK;

@@ -42,16 +42,31 @@ __device__ __forceinline__ void row_update(T &a, T &c, T &d, T al, T cl, T dl, T
 // passes: each pass appends its residue digit as the LOW digit of the slot
 // index, while in the original row numbering that digit has weight
 // 2^(levels of the earlier passes).
+// (Fixed-trip unrolled loops keep the kernel-parameter array in the constant
+// bank instead of copying it to local memory for dynamic indexing.)
 __device__ __forceinline__ int64_t slot_residue(int64_t rho, int npass, const int32_t *kpass) {
     int kcum = 0;
-    for (int p = 0; p < npass; ++p) kcum += kpass[p];
+#pragma unroll
+    for (int p = 0; p < TDS_MAX_PASSES; ++p)
+        if (p < npass) kcum += kpass[p];
     int64_t r = 0;
-    for (int p = npass - 1; p >= 0; --p) {
-        kcum -= kpass[p];
-        r += (rho & ((int64_t(1) << kpass[p]) - 1)) << kcum;
-        rho >>= kpass[p];
+#pragma unroll
+    for (int p = TDS_MAX_PASSES - 1; p >= 0; --p) {
+        if (p < npass) {
+            kcum -= kpass[p];
+            r += (rho & ((int64_t(1) << kpass[p]) - 1)) << kcum;
+            rho >>= kpass[p];
+        }
     }
     return r;
+}
+
+__device__ __forceinline__ int pass_levels(int npass, const int32_t *kpass) {
+    int k = 0;
+#pragma unroll
+    for (int p = 0; p < TDS_MAX_PASSES; ++p)
+        if (p < npass) k += kpass[p];
+    return k;
 }
 
 struct PassGeom {
@@ -71,6 +86,7 @@ struct SplitArgs {
     int32_t tile;            // TILE rows (power of two, >= 2^kp)
     int32_t segs;            // CTAs per input slot
     int32_t ep;              // padded shared-memory length per array
+    int32_t vec;             // input rows may be read with 16-byte vector loads
     PassGeom geom;           // passes applied to the input
 };
 
@@ -83,6 +99,9 @@ struct OnchipArgs {
     int64_t slot;            // workspace slot capacity (K > 0)
     int32_t K;               // total split levels
     int32_t log2T;           // PCR levels on the reduced system (T = 2^log2T chains)
+    int32_t cluster;         // CTAs per subsystem (thread-block cluster size)
+    int32_t tl_levels;       // CR levels across threads before the leader's solve
+    int32_t vec;             // 16-byte vector loads/stores allowed
     PassGeom geom;           // passes applied (for the slot -> residue map)
 };
 
@@ -91,6 +110,8 @@ __host__ __device__ constexpr int ilog2c(int v) { return v <= 1 ? 0 : 1 + ilog2c
 template <typename T>
 cudaError_t launch_split_pass(const SplitArgs<T> &A, bool raw, int64_t grid, int threads, size_t smem,
                               cudaStream_t st);
+template <typename T>
+cudaError_t launch_split_reg(const SplitArgs<T> &A, bool raw, int64_t grid, cudaStream_t st);
 template <typename T>
 cudaError_t launch_onchip(const OnchipArgs<T> &A, int cr_levels, bool raw, int64_t grid, int threads,
                           size_t smem, cudaStream_t st);

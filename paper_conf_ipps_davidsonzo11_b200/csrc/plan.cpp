@@ -49,6 +49,14 @@ int64_t slot_rows(int64_t n, int kk, int32_t dtype) {
     return round_up(cdiv(n, int64_t(1) << kk), 16 / dsize(dtype));
 }
 
+int32_t split_tile_eff(const tds_params &p, int pass) {
+    // rows one split CTA produces per tile: the register kernel (k_p <= 4) keeps
+    // 16 rows x 256 threads minus one halo thread per side; the shared-memory
+    // kernel produces split_tile_rows.
+    return p.k_pass[pass] <= kRegSplitMaxKp ? kRegSplitRows * kRegSplitThreads - 2 * kRegSplitRows
+                                            : p.split_tile_rows;
+}
+
 int32_t split_segments(int64_t m_in, int64_t tiles, int32_t theta) {
     // Fig. 1: cooperative splitting (stage 1, several CTAs per
     // system) only while there are fewer than theta independent systems.
@@ -63,15 +71,27 @@ size_t split_smem_bytes(int32_t dtype, int32_t tile, int kp) {
     return size_t(3 * ep * dsize(dtype));
 }
 
-size_t onchip_smem_bytes(int32_t dtype, int32_t threads) {
-    return size_t((9 * int64_t(threads) + 8) * dsize(dtype));
+size_t onchip_smem_bytes(int32_t dtype, int32_t threads, int32_t cluster, int32_t tl_levels) {
+    // leader's reduced system [3][cluster * (threads >> c2)] + thread-level rows [4][threads]
+    // + warp-edge exchange [2][3][threads/32] + ghosts (12 + 30) + 1, rounded up
+    return size_t((3 * int64_t(cluster) * (threads >> tl_levels) + 4 * int64_t(threads) + 6 * (threads / 32) +
+                   48) * dsize(dtype));
 }
 
-static int n_onchip_max(const tds_device_props &p, int32_t dtype) {
-    const int cap = dtype == TDS_F64 ? 4096 : 8192;  // on-chip kernel: R_max x 512 threads
-    const int64_t budget = int64_t(p.smem_optin_bytes) - kSmemReserve;
-    int n = 1;
-    while (n * 2 <= cap && 4 * int64_t(n * 2) * dsize(dtype) <= budget) n *= 2;
+int32_t static_cluster(const tds_device_props &p) {
+    // thread-block clusters (DSMEM) exist from compute capability 9.0; 8 is the portable maximum
+    return p.cc_major >= 9 ? 8 : 1;
+}
+
+static int64_t n_onchip_max(const tds_device_props &p, int32_t dtype) {
+    // "switch as soon as it fits": the largest power of two whose four
+    // arrays fit in the shared memory of one cluster, capped by the on-chip kernel's
+    // register capacity (R_max x 512 threads per CTA).
+    const int64_t C = static_cluster(p);
+    const int64_t cap = int64_t(r_max(dtype)) * kMaxOnchipThreadsWide * C;
+    const int64_t budget = (int64_t(p.smem_optin_bytes) - kSmemReserve) * C;
+    int64_t n = 1;
+    while (n * 2 <= cap && 4 * (n * 2) * dsize(dtype) <= budget) n *= 2;
     return n;
 }
 
@@ -105,14 +125,22 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
         return fail(TDS_ERR_UNSUPPORTED, "cr_levels exceeds the on-chip kernel's R_max");
     if (!is_pow2(p.thomas_chains)) return fail(TDS_ERR_INVALID_ARG, "thomas_chains must be a power of two");
     if (p.theta < 1) return fail(TDS_ERR_INVALID_ARG, "theta >= 1");
-    const int64_t n_sub = cdiv(n, int64_t(1) << std::min(p.k, 62));
+    if (!is_pow2(p.cluster) || p.cluster > 16) return fail(TDS_ERR_INVALID_ARG, "cluster must be 1, 2, 4, 8 or 16");
     const int R = 1 << p.cr_levels;
-    const int64_t nred = cdiv(n_sub, R);
+    if (p.cluster > 1 && (props.cc_major < 9 || R < 8))
+        return fail(TDS_ERR_UNSUPPORTED, "clusters need compute capability >= 9.0 and 2^cr_levels >= 8");
+    const int64_t n_sub = cdiv(n, int64_t(1) << std::min(p.k, 62));
+    const int64_t nred = cdiv(n_sub, int64_t(R) * p.cluster);
     const int64_t threads = std::max<int64_t>(32, round_up(nred, 32));
     if (threads > (R >= 8 ? kMaxOnchipThreadsWide : kMaxOnchipThreads))
-        return fail(TDS_ERR_UNSUPPORTED, "subsystem too large for the on-chip kernel (n_sub / 2^c > 1024, or > 512 when 2^c >= 8)");
-    if (p.thomas_chains > threads) return fail(TDS_ERR_INVALID_ARG, "thomas_chains > on-chip threads");
-    if ((int64_t)onchip_smem_bytes(dtype, (int32_t)threads) > int64_t(props.smem_optin_bytes) - kSmemReserve)
+        return fail(TDS_ERR_UNSUPPORTED, "subsystem too large for the on-chip kernel (n_sub / (2^c cluster) > 1024, "
+                                         "or > 512 when 2^c >= 8)");
+    if (p.tl_levels < 0 || p.tl_levels > 10 || threads % (int64_t(1) << p.tl_levels))
+        return fail(TDS_ERR_INVALID_ARG, "tl_levels must be in [0, 10] and 2^tl_levels must divide the CTA size");
+    if (p.thomas_chains > (threads >> p.tl_levels) * p.cluster)
+        return fail(TDS_ERR_INVALID_ARG, "thomas_chains > leader's reduced system (cluster x threads / 2^tl_levels)");
+    if ((int64_t)onchip_smem_bytes(dtype, (int32_t)threads, p.cluster, p.tl_levels) >
+        int64_t(props.smem_optin_bytes) - kSmemReserve)
         return fail(TDS_ERR_UNSUPPORTED, "on-chip shared memory exceeds the device limit");
     if (p.passes > 0) {
         if (!is_pow2(p.split_tile_rows) || p.split_tile_rows < 32 || p.split_tile_rows > (1 << 15))
@@ -121,6 +149,7 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
             return fail(TDS_ERR_INVALID_ARG, "split_threads must be a multiple of 32 in [32, 512]");
         for (int i = 0; i < p.passes; ++i) {
             const int kp = p.k_pass[i];
+            if (kp <= kRegSplitMaxKp) continue;  // register split kernel: no tile / smem limits
             if ((int64_t(1) << kp) > p.split_tile_rows)
                 return fail(TDS_ERR_INVALID_ARG, "2^k_pass exceeds split_tile_rows");
             const int64_t e = p.split_tile_rows + 2 * ((int64_t(1) << kp) - 1);
@@ -137,7 +166,6 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
     info.num_subsystems = m * std::min<int64_t>(int64_t(1) << std::min(p.k, 62), n);
     info.onchip_threads = (int32_t)threads;
     info.subsys_per_cta = 1;
-    info.cluster = 1;
     if (p.passes > 0) {
         int kk = 0;
         int64_t elems = 0;
@@ -148,11 +176,13 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
         const int64_t E = round_up(elems, 64);
         info.slot_rows = slot_rows(n, p.k, dtype);
         info.workspace_bytes = size_t((p.passes == 1 ? 1 : 2) * 3 * E * dsize(dtype));
-        info.split_segments = split_segments(m, cdiv(n, p.split_tile_rows), p.theta);
+        info.split_tile_eff = split_tile_eff(p, 0);
+        info.split_segments = split_segments(m, cdiv(n, info.split_tile_eff), p.theta);
     } else {
         info.slot_rows = 0;
         info.workspace_bytes = 0;
         info.split_segments = 0;
+        info.split_tile_eff = 0;
     }
     return TDS_OK;
 }
@@ -161,8 +191,8 @@ static tds_status seed(tds_plan_info &info, const tds_device_props &props, tds_p
     const int32_t dtype = info.dtype;
     const int64_t n = info.n;
     int64_t target;
-    int32_t T, theta, tile, g1threads, kpmax, g2cap;
-    info.n_onchip_max = n_onchip_max(props, dtype);
+    int32_t T, theta, tile, g1threads, kpmax, g2cap, cmax;
+    info.n_onchip_max = (int32_t)n_onchip_max(props, dtype);
     if (info.mode == TDS_PARAMS_DEFAULT) {
         target = 256;
         theta = 16;
@@ -171,14 +201,16 @@ static tds_status seed(tds_plan_info &info, const tds_device_props &props, tds_p
         g1threads = 256;
         kpmax = 8;
         g2cap = 256;
+        cmax = 1;
     } else {
         target = info.n_onchip_max;
         T = 2 * props.warp_size;
         theta = props.sm_count;
-        tile = info.n_onchip_max;
+        tile = (int32_t)std::min<int64_t>(info.n_onchip_max, int64_t(r_max(dtype)) * kMaxOnchipThreadsWide);
         g1threads = 512;
         kpmax = std::min(dtype == TDS_F32 ? 9 : 8, kp_limit(props, dtype, tile));
         g2cap = props.max_threads_per_block / 2;
+        cmax = static_cluster(props);
     }
     info.n_sub_target = (int32_t)target;
     info.split_kp_max = kpmax;
@@ -191,10 +223,17 @@ static tds_status seed(tds_plan_info &info, const tds_device_props &props, tds_p
     p.passes = P;
     for (int i = 0; i < P; ++i) p.k_pass[i] = k / P + (i < k % P ? 1 : 0);
     const int64_t n_sub = cdiv(n, int64_t(1) << k);
+    // smallest cluster whose CTAs hold the subsystem, then the fewest rows per thread
+    int C = 1;
+    while (C < cmax && n_sub > int64_t(C) * r_max(dtype) * g2cap) C *= 2;
     int R = 1;
-    while (cdiv(n_sub, R) > g2cap && R < r_max(dtype)) R *= 2;
+    while (cdiv(n_sub, int64_t(R) * C) > g2cap && R < r_max(dtype)) R *= 2;
+    if (C > 1 && R < 8) R = 8;  // the cluster kernel keeps >= 8 rows per thread
+    p.cluster = C;
     p.cr_levels = ilog2(R);
-    p.thomas_chains = (int32_t)std::min<int64_t>(T, pow2ceil(cdiv(n_sub, R)));
+    // CR across threads until the leader's system has one row per thread: c2 = log2(C)
+    p.tl_levels = ilog2(C);
+    p.thomas_chains = (int32_t)std::min<int64_t>(T, pow2ceil(cdiv(n_sub, R) >> p.tl_levels));
     p.split_tile_rows = tile;
     p.split_threads = g1threads;
     p.theta = theta;

@@ -40,8 +40,7 @@ __global__ void __launch_bounds__(512) split_pass_kernel(const SplitArgs<T> A) {
     if (RAW) {
         L = A.n;
     } else {
-        int kprev = 0;
-        for (int p = 0; p < A.geom.npass; ++p) kprev += A.geom.kpass[p];
+        const int kprev = pass_levels(A.geom.npass, A.geom.kpass);
         const int64_t rho = sigma & ((int64_t(1) << kprev) - 1);
         const int64_t r = slot_residue(rho, A.geom.npass, A.geom.kpass);
         L = r < A.n ? (A.n - r + (int64_t(1) << kprev) - 1) >> kprev : 0;

@@ -1,0 +1,262 @@
+// split_reg.cu -- G1, register-resident form for k_p <= 4 fused PCR levels.
+//
+// Same contract as split_pass.cu (one HBM pass of k_p global PCR splitting
+// levels, §III-B/C P:L296-303; output de-interleaved so
+// each subsystem is contiguous), but with no shared-memory tile:
+//   * thread t owns 16 CONSECUTIVE rows in registers (16-byte vector loads);
+//   * level l (stride s = 2^l <= 8) needs the last / first s rows of threads
+//     t-1 / t+1: warp shuffles, plus shared memory only for the two warp-edge
+//     lanes;  the first and last thread of the CTA are the tile's halo
+//     (16 >= 2^k_p - 1 rows per side), so a tile yields 16*(NT-2) rows;
+//   * after k_p levels row v of the thread belongs to residue v mod 2^k_p and
+//     the 16 >> k_p rows of one residue have consecutive positions j, so the
+//     de-interleaved store is a vector store per residue, coalesced across
+//     the warp (consecutive threads -> consecutive j).
+// Per row and level: one normalised row update (9 FMA-pipe ops + 1 MUFU.RCP).
+#include "common.cuh"
+
+namespace tds {
+
+template <typename T, int G>
+__device__ __forceinline__ void store_run(T *p, const T *v) {
+    if constexpr (G * sizeof(T) >= 16) {
+        constexpr int W = 16 / sizeof(T);
+#pragma unroll
+        for (int q = 0; q < G / W; ++q) {
+            if constexpr (sizeof(T) == 4)
+                reinterpret_cast<float4 *>(p)[q] = make_float4(v[4 * q], v[4 * q + 1], v[4 * q + 2], v[4 * q + 3]);
+            else
+                reinterpret_cast<double2 *>(p)[q] = make_double2(v[2 * q], v[2 * q + 1]);
+        }
+    } else if constexpr (G * sizeof(T) == 8 && sizeof(T) == 4) {
+        reinterpret_cast<float2 *>(p)[0] = make_float2(v[0], v[1]);
+    } else {
+#pragma unroll
+        for (int u = 0; u < G; ++u) p[u] = v[u];
+    }
+}
+
+// One PCR level with compile-time stride S on 16 register rows per thread.
+// A level couples only rows of one class rho (mod S): each class is updated in
+// place, ascending, carrying the previous OLD row, so only a few registers
+// beyond the 48 row values stay live.  eL/eR: [2][3][NW][SM] edge buffers.
+template <typename T, int R, int S, int NW, int SM>
+__device__ __forceinline__ void reg_level(T (&ra)[R], T (&rc)[R], T (&rd)[R], T *eL, T *eR, int bsel, int lane,
+                                          int warp) {
+    auto E = [&](T *e, int arr, int w, int u) -> T & { return e[((bsel * 3 + arr) * NW + w) * SM + u]; };
+    if (lane == 0) {
+#pragma unroll
+        for (int u = 0; u < S; ++u) {
+            E(eL, 0, warp, u) = ra[u];
+            E(eL, 1, warp, u) = rc[u];
+            E(eL, 2, warp, u) = rd[u];
+        }
+    }
+    if (lane == 31) {
+#pragma unroll
+        for (int u = 0; u < S; ++u) {
+            E(eR, 0, warp, u) = ra[R - S + u];
+            E(eR, 1, warp, u) = rc[R - S + u];
+            E(eR, 2, warp, u) = rd[R - S + u];
+        }
+    }
+    __syncthreads();
+#pragma unroll
+    for (int rho = 0; rho < S; ++rho) {
+        // left neighbour of row rho: row R-S+rho of thread t-1 (old; same class)
+        T pa = __shfl_up_sync(0xffffffffu, ra[R - S + rho], 1);
+        T pc = __shfl_up_sync(0xffffffffu, rc[R - S + rho], 1);
+        T pd = __shfl_up_sync(0xffffffffu, rd[R - S + rho], 1);
+        // right neighbour of row R-S+rho: row rho of thread t+1 (old)
+        T xa = __shfl_down_sync(0xffffffffu, ra[rho], 1);
+        T xc = __shfl_down_sync(0xffffffffu, rc[rho], 1);
+        T xd = __shfl_down_sync(0xffffffffu, rd[rho], 1);
+        if (lane == 0) {
+            const bool h = warp > 0;
+            const int w = h ? warp - 1 : 0;
+            pa = h ? E(eR, 0, w, rho) : T(0);
+            pc = h ? E(eR, 1, w, rho) : T(0);
+            pd = h ? E(eR, 2, w, rho) : T(0);
+        }
+        if (lane == 31) {
+            const bool h = warp < NW - 1;
+            const int w = h ? warp + 1 : 0;
+            xa = h ? E(eL, 0, w, rho) : T(0);
+            xc = h ? E(eL, 1, w, rho) : T(0);
+            xd = h ? E(eL, 2, w, rho) : T(0);
+        }
+#pragma unroll
+        for (int v = rho; v < R; v += S) {
+            const T oa = ra[v], oc = rc[v], od = rd[v];
+            if constexpr (true) {
+                const bool last = v + S >= R;
+                row_update(ra[v], rc[v], rd[v], pa, pc, pd, last ? xa : ra[(v + S) % R], last ? xc : rc[(v + S) % R],
+                           last ? xd : rd[(v + S) % R]);
+            }
+            pa = oa;
+            pc = oc;
+            pd = od;
+        }
+    }
+}
+
+template <typename T, int KP, bool RAW>
+__global__ void __launch_bounds__(kRegSplitThreads, 2) split_reg_kernel(const SplitArgs<T> A) {
+    constexpr int R = kRegSplitRows;
+    constexpr int NT = kRegSplitThreads;
+    constexpr int NW = NT / 32;
+    constexpr int SM = 1 << (KP - 1);  // largest stride
+    constexpr int NR = 1 << KP;        // residues produced
+    constexpr int G = R >> KP;         // rows per residue per thread
+    constexpr int W = 16 / int(sizeof(T));
+    __shared__ T eL[2][3][NW][SM];  // lane 0's first s rows  -> previous warp's lane 31
+    __shared__ T eR[2][3][NW][SM];  // lane 31's last s rows  -> next warp's lane 0
+    const int t = threadIdx.x, lane = t & 31, warp = t >> 5;
+    constexpr int TV = NT * R - 2 * R;  // valid rows per tile
+
+    const int64_t sigma = int64_t(blockIdx.x) / A.segs;
+    const int g = int(int64_t(blockIdx.x) % A.segs);
+    int64_t L;
+    if (RAW) {
+        L = A.n;
+    } else {
+        const int kprev = pass_levels(A.geom.npass, A.geom.kpass);
+        const int64_t rho = sigma & ((int64_t(1) << kprev) - 1);
+        const int64_t r = slot_residue(rho, A.geom.npass, A.geom.kpass);
+        L = r < A.n ? (A.n - r + (int64_t(1) << kprev) - 1) >> kprev : 0;
+    }
+    const int64_t in_base = sigma * A.in_stride;
+    const int64_t ntiles = (L + TV - 1) / TV;
+    const int64_t t_begin = g * ntiles / A.segs;
+    const int64_t t_end = (g + 1) * ntiles / A.segs;
+
+    for (int64_t ti = t_begin; ti < t_end; ++ti) {
+        const int64_t i0 = ti * TV - R + int64_t(t) * R;  // first row of this thread
+        T ra[R], rc[R], rd[R];
+        if (A.vec && i0 >= 0 && i0 + R <= L) {
+            const int64_t o = in_base + i0;
+#pragma unroll
+            for (int q = 0; q < R / W; ++q) {
+                if constexpr (sizeof(T) == 4) {
+                    const float4 fa = __ldcs(reinterpret_cast<const float4 *>(A.a + o) + q);
+                    const float4 fc = __ldcs(reinterpret_cast<const float4 *>(A.c + o) + q);
+                    const float4 fd = __ldcs(reinterpret_cast<const float4 *>(A.d + o) + q);
+                    ra[4 * q] = fa.x; ra[4 * q + 1] = fa.y; ra[4 * q + 2] = fa.z; ra[4 * q + 3] = fa.w;
+                    rc[4 * q] = fc.x; rc[4 * q + 1] = fc.y; rc[4 * q + 2] = fc.z; rc[4 * q + 3] = fc.w;
+                    rd[4 * q] = fd.x; rd[4 * q + 1] = fd.y; rd[4 * q + 2] = fd.z; rd[4 * q + 3] = fd.w;
+                } else {
+                    const double2 fa = __ldcs(reinterpret_cast<const double2 *>(A.a + o) + q);
+                    const double2 fc = __ldcs(reinterpret_cast<const double2 *>(A.c + o) + q);
+                    const double2 fd = __ldcs(reinterpret_cast<const double2 *>(A.d + o) + q);
+                    ra[2 * q] = fa.x; ra[2 * q + 1] = fa.y;
+                    rc[2 * q] = fc.x; rc[2 * q + 1] = fc.y;
+                    rd[2 * q] = fd.x; rd[2 * q + 1] = fd.y;
+                }
+            }
+            if (RAW) {
+                T rb[R];
+#pragma unroll
+                for (int q = 0; q < R / W; ++q) {
+                    if constexpr (sizeof(T) == 4) {
+                        const float4 fb = __ldcs(reinterpret_cast<const float4 *>(A.b + o) + q);
+                        rb[4 * q] = fb.x; rb[4 * q + 1] = fb.y; rb[4 * q + 2] = fb.z; rb[4 * q + 3] = fb.w;
+                    } else {
+                        const double2 fb = __ldcs(reinterpret_cast<const double2 *>(A.b + o) + q);
+                        rb[2 * q] = fb.x; rb[2 * q + 1] = fb.y;
+                    }
+                }
+#pragma unroll
+                for (int v = 0; v < R; ++v) {
+                    const T inv = rcp(rb[v]);
+                    ra[v] = (i0 + v > 0 ? ra[v] : T(0)) * inv;
+                    rc[v] = (i0 + v < L - 1 ? rc[v] : T(0)) * inv;
+                    rd[v] = rd[v] * inv;
+                }
+            }
+        } else {
+#pragma unroll
+            for (int v = 0; v < R; ++v) {
+                const int64_t row = i0 + v;
+                ra[v] = T(0);
+                rc[v] = T(0);
+                rd[v] = T(0);
+                if (row >= 0 && row < L) {
+                    const int64_t o = in_base + row;
+                    if (RAW) {
+                        const T inv = rcp(A.b[o]);
+                        ra[v] = (row > 0 ? A.a[o] : T(0)) * inv;
+                        rc[v] = (row < L - 1 ? A.c[o] : T(0)) * inv;
+                        rd[v] = A.d[o] * inv;
+                    } else {
+                        ra[v] = A.a[o];
+                        rc[v] = A.c[o];
+                        rd[v] = A.d[o];
+                    }
+                }
+            }
+        }
+
+        T *el = &eL[0][0][0][0], *er = &eR[0][0][0][0];
+        if constexpr (KP >= 1) reg_level<T, R, 1, NW, SM>(ra, rc, rd, el, er, 0, lane, warp);
+        if constexpr (KP >= 2) reg_level<T, R, 2, NW, SM>(ra, rc, rd, el, er, 1, lane, warp);
+        if constexpr (KP >= 3) reg_level<T, R, 4, NW, SM>(ra, rc, rd, el, er, 0, lane, warp);
+        if constexpr (KP >= 4) reg_level<T, R, 8, NW, SM>(ra, rc, rd, el, er, 1, lane, warp);
+
+        // ---- de-interleaved store: residue rho gets rows rho + NR*u, u < G, positions (i0 >> KP) + u
+        if (t >= 1 && t <= NT - 2 && i0 < L) {
+            const int64_t jb = i0 >> KP;
+            const bool full = i0 + R <= L;
+#pragma unroll
+            for (int rho = 0; rho < NR; ++rho) {
+                const int64_t o = ((sigma << KP) + rho) * A.out_slot + jb;
+                T va[G], vc[G], vd[G];
+#pragma unroll
+                for (int u = 0; u < G; ++u) {
+                    va[u] = ra[rho + NR * u];
+                    vc[u] = rc[rho + NR * u];
+                    vd[u] = rd[rho + NR * u];
+                }
+                if (full) {
+                    store_run<T, G>(A.oa + o, va);
+                    store_run<T, G>(A.oc + o, vc);
+                    store_run<T, G>(A.od + o, vd);
+                } else {
+#pragma unroll
+                    for (int u = 0; u < G; ++u) {
+                        if (i0 + rho + NR * u < L) {
+                            A.oa[o + u] = va[u];
+                            A.oc[o + u] = vc[u];
+                            A.od[o + u] = vd[u];
+                        }
+                    }
+                }
+            }
+        }
+        __syncthreads();  // edge buffers are reused by the next tile
+    }
+}
+
+template <typename T, int KP>
+static cudaError_t launch_kp(const SplitArgs<T> &A, bool raw, int64_t grid, cudaStream_t st) {
+    if (raw)
+        split_reg_kernel<T, KP, true><<<(unsigned)grid, kRegSplitThreads, 0, st>>>(A);
+    else
+        split_reg_kernel<T, KP, false><<<(unsigned)grid, kRegSplitThreads, 0, st>>>(A);
+    return cudaGetLastError();
+}
+
+template <typename T>
+cudaError_t launch_split_reg(const SplitArgs<T> &A, bool raw, int64_t grid, cudaStream_t st) {
+    switch (A.kp) {
+        case 1: return launch_kp<T, 1>(A, raw, grid, st);
+        case 2: return launch_kp<T, 2>(A, raw, grid, st);
+        case 3: return launch_kp<T, 3>(A, raw, grid, st);
+        case 4: return launch_kp<T, 4>(A, raw, grid, st);
+        default: return cudaErrorInvalidConfiguration;
+    }
+}
+
+template cudaError_t launch_split_reg<float>(const SplitArgs<float> &, bool, int64_t, cudaStream_t);
+template cudaError_t launch_split_reg<double>(const SplitArgs<double> &, bool, int64_t, cudaStream_t);
+
+}  // namespace tds

@@ -18,6 +18,9 @@ constexpr int kSmemReserve = 1024;    // per-CTA shared memory reserved by the r
 constexpr int kMaxOnchipThreads = 1024;     // on-chip CTA size for R <= 4
 constexpr int kMaxOnchipThreadsWide = 512;  // ... and for R >= 8 (register budget)
 constexpr int kMaxSplitThreads = 512;
+constexpr int kRegSplitMaxKp = 4;       // split passes with k_p <= 4 use the register kernel
+constexpr int kRegSplitRows = 16;       // ... 16 rows per thread
+constexpr int kRegSplitThreads = 256;   // ... 256 threads per CTA
 
 inline int dsize(int32_t dtype) { return dtype == TDS_F64 ? 8 : 4; }
 inline int r_max(int32_t dtype) { return dtype == TDS_F64 ? 8 : 16; }
@@ -32,7 +35,9 @@ void clear_error();
 int64_t slot_rows(int64_t n, int kk, int32_t dtype);
 int32_t split_segments(int64_t m_in, int64_t tiles, int32_t theta);
 size_t split_smem_bytes(int32_t dtype, int32_t tile, int kp);
-size_t onchip_smem_bytes(int32_t dtype, int32_t threads);
+size_t onchip_smem_bytes(int32_t dtype, int32_t threads, int32_t cluster, int32_t tl_levels);
+int32_t split_tile_eff(const tds_params &p, int pass);
+int32_t static_cluster(const tds_device_props &p);
 tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_params &p);
 
 }  // namespace tds

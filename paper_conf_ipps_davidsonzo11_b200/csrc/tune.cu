@@ -117,23 +117,42 @@ static int ilog2i(int64_t v) {
     return l;
 }
 
-// Stage 3->4: hill climb over (c, T) for the current k.
+static int64_t cta_threads(const tds_plan_info &I, const tds_params &p) {
+    const int64_t n_sub = cdiv(I.n, int64_t(1) << p.k);
+    return std::max<int64_t>(32, round_up(cdiv(n_sub, (int64_t(1) << p.cr_levels) * p.cluster), 32));
+}
+
+// Keep (c, C, c2, T) consistent: clusters need >= 8 rows per thread, 2^c2
+// divides the CTA size, T <= the leader's system Z = C * threads / 2^c2.
+static void clamp_onchip(const tds_plan_info &I, tds_params &p) {
+    if (p.cluster > 1 && p.cr_levels < 3) p.cr_levels = 3;
+    const int64_t thr = cta_threads(I, p);
+    while (p.tl_levels > 0 && (thr % (int64_t(1) << p.tl_levels))) --p.tl_levels;
+    const int64_t Z = (thr >> p.tl_levels) * p.cluster;
+    while (p.thomas_chains > Z && p.thomas_chains > 1) p.thomas_chains /= 2;
+}
+
+// Stage 3->4: hill climb over (c, T, cluster) for the current k.
 static void tune_onchip(TuneCtx &C, tds_params &best, double &t_best) {
     const tds_plan_info &I = C.plan->info;
     bool improved = true;
     while (improved && !out_of_time(C)) {
         improved = false;
-        tds_params cand[4];
+        tds_params cand[8];
         int nc = 0;
         if (best.thomas_chains > 1) { cand[nc] = best; cand[nc++].thomas_chains /= 2; }
         cand[nc] = best; cand[nc++].thomas_chains *= 2;
+        if (best.tl_levels > 0) { cand[nc] = best; cand[nc++].tl_levels -= 1; }
+        if (best.tl_levels < 10) { cand[nc] = best; cand[nc++].tl_levels += 1; }
         if (best.cr_levels > 0) { cand[nc] = best; cand[nc++].cr_levels -= 1; }
         if ((1 << (best.cr_levels + 1)) <= r_max(I.dtype)) { cand[nc] = best; cand[nc++].cr_levels += 1; }
+        if (best.cluster > 1) { cand[nc] = best; cand[nc].cluster /= 2; cand[nc++].tl_levels -= best.tl_levels > 0; }
+        if (best.cluster < 16 && C.plan->props.cc_major >= 9) {
+            cand[nc] = best; cand[nc].cluster *= 2; cand[nc++].tl_levels += 1;
+        }
         for (int i = 0; i < nc; ++i) {
-            // keep T within the reduced system after a change of c
-            const int64_t n_sub = cdiv(I.n, int64_t(1) << cand[i].k);
-            const int64_t thr = std::max<int64_t>(32, round_up(cdiv(n_sub, int64_t(1) << cand[i].cr_levels), 32));
-            if (cand[i].thomas_chains > thr) continue;
+            clamp_onchip(I, cand[i]);
+            if (std::memcmp(&cand[i], &best, sizeof(best)) == 0) continue;
             const double t = trial(C, cand[i]);
             if (better(t, t_best)) {
                 best = cand[i];
@@ -151,15 +170,19 @@ static void schedule_passes(tds_params &p, int kpmax) {
     for (int i = 0; i < p.passes; ++i) p.k_pass[i] = p.k / p.passes + (i < p.k % p.passes ? 1 : 0);
 }
 
-// Make (c, T) valid for a new k: smallest c whose CTA fits the kernel's cap, T capped.
-static void fit_onchip(const tds_plan_info &I, tds_params &p) {
+// Make (c, C, T) valid for a new k: grow c, then the cluster, until a CTA fits.
+static void fit_onchip(const tds_plan_info &I, const tds_device_props &props, tds_params &p) {
     const int64_t n_sub = cdiv(I.n, int64_t(1) << p.k);
     auto cap = [](int c) { return (1 << c) >= 8 ? kMaxOnchipThreadsWide : kMaxOnchipThreads; };
-    while (round_up(cdiv(n_sub, int64_t(1) << p.cr_levels), 32) > cap(p.cr_levels) &&
-           (1 << (p.cr_levels + 1)) <= r_max(I.dtype))
-        ++p.cr_levels;
-    const int64_t thr = std::max<int64_t>(32, round_up(cdiv(n_sub, int64_t(1) << p.cr_levels), 32));
-    while (p.thomas_chains > thr) p.thomas_chains /= 2;
+    auto thr = [&](const tds_params &q) {
+        return round_up(cdiv(n_sub, (int64_t(1) << q.cr_levels) * q.cluster), 32);
+    };
+    while (thr(p) > cap(p.cr_levels)) {
+        if ((1 << (p.cr_levels + 1)) <= r_max(I.dtype)) ++p.cr_levels;
+        else if (p.cluster < 16 && props.cc_major >= 9) p.cluster *= 2;
+        else break;
+    }
+    clamp_onchip(I, p);
 }
 
 static std::string cache_key(const tds_plan_st *plan) {
@@ -179,8 +202,8 @@ static std::string params_str(const tds_params &p) {
     std::ostringstream o;
     o << p.k << " " << p.passes;
     for (int i = 0; i < TDS_MAX_PASSES; ++i) o << " " << p.k_pass[i];
-    o << " " << p.cr_levels << " " << p.thomas_chains << " " << p.split_tile_rows << " " << p.split_threads << " "
-      << p.theta;
+    o << " " << p.cr_levels << " " << p.thomas_chains << " " << p.cluster << " " << p.tl_levels << " "
+      << p.split_tile_rows << " " << p.split_threads << " " << p.theta;
     return o.str();
 }
 
@@ -196,7 +219,8 @@ static bool cache_lookup(const std::string &path, const std::string &key, tds_pa
         tds_params q{};
         is >> q.k >> q.passes;
         for (int i = 0; i < TDS_MAX_PASSES; ++i) is >> q.k_pass[i];
-        is >> q.cr_levels >> q.thomas_chains >> q.split_tile_rows >> q.split_threads >> q.theta;
+        is >> q.cr_levels >> q.thomas_chains >> q.cluster >> q.tl_levels >> q.split_tile_rows >> q.split_threads >>
+            q.theta;
         if (is) {
             p = q;
             found = true;
@@ -274,7 +298,7 @@ extern "C" tds_status tds_tune(tds_plan_t plan, void *cuda_stream, const char *c
                 if (cand.k < 0 || cand.k > 30 || (int64_t(1) << cand.k) > 2 * I.n) break;
                 const int kpmax = std::max(I.split_kp_max, 1);
                 schedule_passes(cand, kpmax);
-                fit_onchip(I, cand);
+                fit_onchip(I, plan->props, cand);
                 double t = trial(C, cand);
                 if (t >= 1e29) break;
                 tune_onchip(C, cand, t);

@@ -35,7 +35,7 @@ def run(tds, a, b, c, d, mode="static", params=None, stride=0, inplace=False):
     dt = "float32" if d.dtype == np.float32 else "float64"
     plan = tds.Plan(n, m, dt, device=0, mode=mode)
     if params:
-        plan.set_params(**params)
+        plan.set_params(**dict({"cluster": 1, "tl_levels": 0}, **params))
     ta, tb, tc, td = to_dev(a, b, c, d)
     x = tds.solve_batched(plan, ta, tb, tc, td, out=td if inplace else None)
     torch.cuda.synchronize()
@@ -85,6 +85,49 @@ def test_onchip_switch_points(tds, dtype, c_lv, T):
     a, b, c, d = inputs.generate(n, 3, dtype, seed=5)
     x, _ = run(tds, a, b, c, d, params=dict(cr_levels=c_lv, thomas_chains=T))
     check(a, b, c, d, x, dtype)
+
+
+# ------------------------------------------------ cluster (DSMEM) on-chip kernel
+
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("n", [16384, 65536, 100003, 131072])
+@pytest.mark.parametrize("cl", [2, 4, 8, 16])
+@pytest.mark.parametrize("T", [1, 32, 512])
+@pytest.mark.parametrize("tl", [0, 1, 3, 5])
+def test_onchip_cluster(tds, dtype, n, cl, T, tl):
+    """One subsystem spread over a cluster of C CTAs (k = 0): CR in registers,
+    reduced system gathered on the leader through DSMEM."""
+    c_lv = 4 if dtype == np.float32 else 3
+    R = 1 << c_lv
+    nred = -(-n // (R * cl))
+    threads = max(32, -(-nred // 32) * 32)
+    if threads > 512:
+        pytest.skip("subsystem too large for this cluster")
+    if T > (threads >> tl) * cl:
+        pytest.skip("T > reduced rows")
+    a, b, c, d = inputs.generate(n, 3, dtype, seed=17)
+    x, plan = run(tds, a, b, c, d, params=dict(k_pass=[], cr_levels=c_lv, thomas_chains=T, cluster=cl,
+                                               tl_levels=tl))
+    assert plan.info["cluster"] == cl and plan.info["k"] == 0
+    check(a, b, c, d, x, dtype)
+
+
+@pytest.mark.parametrize("n,tl,T", [(8192, 9, 1), (8192, 4, 32), (5000, 3, 8), (1000, 5, 1), (100, 5, 1)])
+def test_onchip_thread_level_cr(tds, n, tl, T):
+    """CR across threads inside one CTA (C = 1, c2 > 0) down to a tiny leader system."""
+    a, b, c, d = inputs.generate(n, 4, np.float32, seed=23)
+    R = 16 if n > 4096 else 4
+    x, plan = run(tds, a, b, c, d, params=dict(k_pass=[], cr_levels=R.bit_length() - 1, thomas_chains=T,
+                                               tl_levels=tl))
+    check(a, b, c, d, x, np.float32)
+
+
+@pytest.mark.parametrize("n,m,kp,cl", [(1 << 20, 2, [4], 8), (1 << 20, 1, [3], 16), (300001, 2, [2], 16),
+                                       (1 << 19, 3, [1, 1], 16)])
+def test_split_then_cluster(tds, n, m, kp, cl):
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=19)
+    x, plan = run(tds, a, b, c, d, params=dict(k_pass=kp, cr_levels=4, thomas_chains=64, cluster=cl))
+    check(a, b, c, d, x, np.float32)
 
 
 # ------------------------------------------------ split passes + on-chip
@@ -140,7 +183,7 @@ def split_gpu(tds, a, b, c, d, params):
     m, n = d.shape
     dt = "float32" if d.dtype == np.float32 else "float64"
     plan = tds.Plan(n, m, dt, device=0)
-    plan.set_params(**params)
+    plan.set_params(**dict({"cluster": 1, "tl_levels": 0}, **params))
     oa, oc, od = tds.split_batched(plan, *to_dev(a, b, c, d))
     torch.cuda.synchronize()
     return oa.cpu().numpy(), oc.cpu().numpy(), od.cpu().numpy(), plan

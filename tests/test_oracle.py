@@ -287,28 +287,31 @@ def test_planner_paper_values():
 
 
 def test_planner_static_onchip_sizes():
-    """Static on-chip size = largest power of two whose 4 arrays fit in shared
-    memory: 512 (16 KB) / 2048 (48 KB) on Table I, 8192 fp32 / 4096 fp64 on B200."""
+    """Static on-chip size = largest power of two whose 4 arrays fit in the
+    shared memory of the device's cluster: 512 (16 KB) / 2048 (48 KB) on Table
+    I (no clusters), 65536 fp32 / 32768 fp64 on B200 (8-CTA clusters)."""
     t = rplan.TABLE_I
     assert rplan.n_onchip_max(t["GeForce 8800 GTX"], rplan.F32) == 512
     assert rplan.n_onchip_max(t["GeForce GTX 280"], rplan.F32) == 512
     assert rplan.n_onchip_max(t["GeForce GTX 470"], rplan.F32) == 2048
-    assert rplan.n_onchip_max(rplan.B200, rplan.F32) == 8192
-    assert rplan.n_onchip_max(rplan.B200, rplan.F64) == 4096
+    assert rplan.n_onchip_max(rplan.B200, rplan.F32) == 65536
+    assert rplan.n_onchip_max(rplan.B200, rplan.F64) == 32768
 
 
-@pytest.mark.parametrize("dtype,n,m,k,passes,nsub", [
-    (rplan.F32, 1024, 1, 0, 0, 1024),
-    (rplan.F32, 65536, 256, 3, 1, 8192),
-    (rplan.F32, 1 << 20, 16, 7, 1, 8192),
-    (rplan.F64, 1 << 20, 16, 8, 1, 4096),
-    (rplan.F32, 16384, 4096, 1, 1, 8192),
-    (rplan.F32, 1 << 28, 1, 15, 2, 8192),
+@pytest.mark.parametrize("dtype,n,m,k,passes,nsub,cluster", [
+    (rplan.F32, 1024, 1, 0, 0, 1024, 1),
+    (rplan.F32, 65536, 256, 0, 0, 65536, 8),
+    (rplan.F32, 1 << 20, 16, 4, 1, 65536, 8),
+    (rplan.F64, 1 << 20, 16, 5, 1, 32768, 8),
+    (rplan.F32, 16384, 4096, 0, 0, 16384, 2),
+    (rplan.F32, 1 << 28, 1, 12, 2, 65536, 8),
 ])
-def test_planner_static_configs(dtype, n, m, k, passes, nsub):
-    """The STATIC plans of SURVEY.md §8(a) A1 at the BASELINE.json configs."""
+def test_planner_static_configs(dtype, n, m, k, passes, nsub, cluster):
+    """STATIC plans at the BASELINE.json configs: "switch to the on-chip kernel
+    as soon as the subsystem fits", where on B200 the on-chip
+    memory is that of one 8-CTA cluster (reading R22)."""
     p = rplan.make_plan(rplan.B200, dtype, n, m, mode=rplan.STATIC)
-    assert (p.k, p.passes, p.n_sub) == (k, passes, nsub)
+    assert (p.k, p.passes, p.n_sub, p.cluster) == (k, passes, nsub, cluster)
     assert sum(p.k_pass) == k
     assert p.k_pass[:passes] == sorted(p.k_pass[:passes], reverse=True)
     assert max(p.k_pass) - min(p.k_pass[:max(passes, 1)]) <= 1 or passes <= 1
