@@ -128,18 +128,24 @@ class ClockSampler:
 def algorithmic_bytes(info: dict, s: int):
     """Bytes per launch the method must move: split
     pass 1 reads a,b,c,d and writes normalised a',c',d' (7 s/eq); a later pass
-    reads and writes 3 arrays (6 s/eq); the on-chip kernel reads 3 (or the 4
-    raw arrays when k = 0) and writes x (4 s or 5 s per equation)."""
+    reads and writes 3 arrays (6 s/eq); the on-chip kernel reads 3 arrays and
+    writes per-subsystem x (4 s/eq; 4 raw arrays + x = 5 s/eq when k = 0); the
+    x placement reads and writes x once (2 s/eq, k > 0 only)."""
     eqs = info["n"] * info["m"]
     out = []
     for p in range(info["passes"]):
         out.append((7 if p == 0 else 6) * s * eqs)
     out.append((5 if info["passes"] == 0 else 4) * s * eqs)
+    if info["k"] > 0:
+        out.append(2 * s * eqs)
     return out
 
 
 def stage_names(info):
-    return [f"split_pass_{p}(k_p={info['k_pass'][p]})" for p in range(info["passes"])] + ["onchip_cr_pcr_thomas"]
+    names = [f"split_pass_{p}(k_p={info['k_pass'][p]})" for p in range(info["passes"])] + ["onchip_cr_pcr_thomas"]
+    if info["k"] > 0:
+        names.append("place_x")
+    return names
 
 
 def measured_peaks():
@@ -272,17 +278,14 @@ def run_tds(args):
                 os.unlink(cache)
         if world > 1:
             p = plan.params
-            vec = torch.tensor([p.k, p.passes] + list(p.k_pass) + [p.cr_levels, p.thomas_chains,
-                                                                    p.split_tile_rows, p.split_threads, p.theta],
-                               dtype=torch.int64, device=dev)
+            vec = torch.tensor(plan.params_list(), dtype=torch.int64, device=dev)
             dist.broadcast(vec, 0)
-            v = vec.tolist()
             if rank != 0:
-                plan.set_params(k_pass=[k for k in v[2:10] if k], cr_levels=v[10], thomas_chains=v[11],
-                                split_tile_rows=v[12], split_threads=v[13], theta=v[14])
+                plan.set_params_list(vec.tolist())
     info = plan.info
     ws = plan.workspace()
-    P = info["passes"]
+    NL = info["launches"]                            # kernel launches per step (all chunks)
+    S = info["passes"] + 1 + (1 if info["k"] > 0 else 0)  # kernels per chunk
     stream = torch.cuda.current_stream()
 
     def step():
@@ -301,19 +304,21 @@ def run_tds(args):
 
     # ---- timed region: K steps, events between the kernels of each step
     K = args.steps
-    ev = [[torch.cuda.Event(enable_timing=True) for _ in range(P + 2)] for _ in range(K)]
+    ev = [[torch.cuda.Event(enable_timing=True) for _ in range(NL + 1)] for _ in range(K)]
     barrier()
     torch.cuda.synchronize()
     for i in range(K):
-        for st in range(P + 1):
+        for st in range(NL):
             ev[i][st].record(stream)
             tds.api.solve_stages(plan, ta, tb, tc, td, x, ws, st, st)
-        ev[i][P + 1].record(stream)
+        ev[i][NL].record(stream)
     torch.cuda.synchronize()
     barrier()
     clocks = sampler.stop()
-    total_ms = ev[0][0].elapsed_time(ev[K - 1][P + 1])
-    stage_ms = [sum(ev[i][st].elapsed_time(ev[i][st + 1]) for i in range(K)) / K for st in range(P + 1)]
+    total_ms = ev[0][0].elapsed_time(ev[K - 1][NL])
+    # per kernel kind (split pass p, on-chip, placement), summed over the chunks of a step
+    stage_ms = [sum(ev[i][st].elapsed_time(ev[i][st + 1]) for i in range(K) for st in range(kind, NL, S)) / K
+                for kind in range(S)]
     if world > 1:
         t = torch.tensor([total_ms], dtype=torch.float64, device=dev)
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
@@ -394,7 +399,8 @@ def run_tds(args):
         "config": {"workload": f"config{args.config}: {m} x {n} {args.dtype} per GPU", "n": n, "m": m,
                    "mode": args.mode, "plan": {k: info[k] for k in ("k", "passes", "k_pass", "n_sub",
                                                                      "cr_levels", "thomas_chains",
-                                                                     "cluster", "tl_levels", "split_tile_rows", "split_threads",
+                                                                     "cluster", "tl_levels", "chunk_systems",
+                                                                     "chunks", "launches", "split_tile_rows", "split_threads",
                                                                      "theta", "split_segments",
                                                                      "onchip_threads", "workspace_bytes")},
                    "tune_trials": trials, "tune_s": round(tune_s, 2),
@@ -405,7 +411,7 @@ def run_tds(args):
         "roofline": roofline,
         "cpu_baseline": cpu,
         "e2e": e2e,
-        "gpu_launches": K * (P + 1),
+        "gpu_launches": K * NL,
         "clocks": clocks,
     }
     print(json.dumps(line), flush=True)

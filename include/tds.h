@@ -101,6 +101,7 @@ typedef struct {
     int32_t split_tile_rows;         /* shared-memory split pass tile (k_pass > 4 only) */
     int32_t split_threads;           /* shared-memory split pass CTA size (k_pass > 4)  */
     int32_t theta;                   /* stage 1->2 switch: independent systems needed   */
+    int32_t chunk_systems;           /* systems per L2-resident chunk (0 = all at once) */
 } tds_params;
 
 /* Everything a plan decided (read-only view). */
@@ -118,6 +119,8 @@ typedef struct {
     int32_t subsys_per_cta;   /* on-chip subsystems per CTA (1)                        */
     int32_t split_segments;   /* CTAs cooperating on one system in pass 1 (stage 1)    */
     int32_t split_tile_eff;   /* rows one split CTA produces per tile in pass 1        */
+    int32_t chunks;           /* system chunks the batch is processed in               */
+    int32_t launches;         /* kernel launches per solve (tds_solve_stages range)    */
     int64_t slot_rows;        /* workspace rows reserved per subsystem (final pass)    */
     size_t workspace_bytes;   /* bytes tds_solve_batched needs (0 when k == 0)         */
 } tds_plan_info;
@@ -183,13 +186,15 @@ tds_status tds_solve_batched(const tds_plan_t plan, const void *a, const void *b
                              const void *d, void *x, void *workspace, size_t workspace_bytes,
                              void *cuda_stream);
 
-/* Run only kernels first_stage..last_stage (inclusive) of the solve sequence
- * tds_solve_batched enqueues: stage p < passes is split pass p (PAPER.md
- * stages 1-2), stage == passes is the on-chip kernel (stages 3-4).  Calling
- * stages 0..passes in order on one stream is identical to tds_solve_batched
- * (used to time each kernel with events between them).  Same arguments and
- * errors as tds_solve_batched; INVALID_ARG if the range is empty or outside
- * [0, passes]. */
+/* Run only launches first_stage..last_stage (inclusive) of the kernel sequence
+ * tds_solve_batched enqueues.  The sequence is, for each chunk of
+ * chunk_systems systems in order: split passes 0..passes-1 (PAPER.md stages
+ * 1-2), the on-chip kernel (stages 3-4) and, when k > 0, the x placement;
+ * launch index = chunk * S + stage with S = passes + 1 + (k > 0), and
+ * info.launches = chunks * S.  Calling every launch in order on one stream is
+ * identical to tds_solve_batched (used to time each kernel with events between
+ * them).  Same arguments and errors as tds_solve_batched; INVALID_ARG if the
+ * range is empty or outside [0, info.launches). */
 tds_status tds_solve_stages(const tds_plan_t plan, const void *a, const void *b, const void *c,
                             const void *d, void *x, void *workspace, size_t workspace_bytes,
                             void *cuda_stream, int32_t first_stage, int32_t last_stage);

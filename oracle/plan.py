@@ -130,6 +130,9 @@ class Plan:
     subsys_per_cta: int = 1
     cluster: int = 1
     tl_levels: int = 0
+    chunk_systems: int = 0
+    chunks: int = 1
+    launches: int = 1
     split_tile_rows: int = 0
     split_threads: int = 0
     split_segments: int = 0
@@ -183,7 +186,7 @@ def make_plan(props: Props, dtype: int, n: int, m: int, batch_stride: int = 0,
     else:
         target = p.n_onchip_max
         T = STATIC_THOMAS_PER_WARP * props.warp_size
-        theta = props.sm_count
+        theta = 32 * props.sm_count  # from the processor count
         tile = min(p.n_onchip_max, r_max(dtype) * 512)
         g1t = STATIC_SPLIT_THREADS
         cmax = static_cluster(props)
@@ -239,15 +242,21 @@ def make_plan(props: Props, dtype: int, n: int, m: int, batch_stride: int = 0,
     if (3 * C * (nt >> p.tl_levels) + 4 * nt + 6 * (nt // 32) + 48) * s > budget:
         raise ValueError("unsupported: on-chip shared memory")
 
-    # Workspace: split output (normalised a, c, d) in fixed slots; ping-pong if P >= 2.
+    # L2-resident chunking is a tuner dimension only (both planners seed 0).
+    p.chunk_systems = 0
+    mc = m
+    p.chunks = cdiv(m, mc)
+    p.launches = p.chunks * (P + 1 + (1 if k > 0 else 0))
+
+    # Workspace: split output (normalised a, c, d) of one chunk in fixed slots; ping-pong if P >= 2.
     if P:
         kk, elems = 0, 0
         for i in range(P):
             kk += p.k_pass[i]
-            elems = max(elems, m * (1 << kk) * slot_rows(n, kk, dtype))
+            elems = max(elems, mc * (1 << kk) * slot_rows(n, kk, dtype))
         E = round_up(elems, 64)
         p.slot_rows = slot_rows(n, k, dtype)
         p.workspace_bytes = (1 if P == 1 else 2) * 3 * E * s
         tile_eff = REG_SPLIT_TILE if p.k_pass[0] <= REG_SPLIT_MAX_KP else tile
-        p.split_segments = segments(m, cdiv(n, tile_eff), theta)
+        p.split_segments = segments(mc, cdiv(n, tile_eff), theta)
     return p

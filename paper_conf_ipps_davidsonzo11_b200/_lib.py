@@ -43,7 +43,8 @@ class Params(ctypes.Structure):
                 ("thomas_chains", ctypes.c_int32), ("cluster", ctypes.c_int32),
                 ("tl_levels", ctypes.c_int32),
                 ("split_tile_rows", ctypes.c_int32),
-                ("split_threads", ctypes.c_int32), ("theta", ctypes.c_int32)]
+                ("split_threads", ctypes.c_int32), ("theta", ctypes.c_int32),
+                ("chunk_systems", ctypes.c_int32)]
 
 
 class PlanInfo(ctypes.Structure):
@@ -54,6 +55,7 @@ class PlanInfo(ctypes.Structure):
                 ("n_onchip_max", ctypes.c_int32), ("split_kp_max", ctypes.c_int32),
                 ("onchip_threads", ctypes.c_int32), ("subsys_per_cta", ctypes.c_int32),
                 ("split_segments", ctypes.c_int32), ("split_tile_eff", ctypes.c_int32),
+                ("chunks", ctypes.c_int32), ("launches", ctypes.c_int32),
                 ("slot_rows", ctypes.c_int64), ("workspace_bytes", ctypes.c_size_t)]
 
 

@@ -40,7 +40,7 @@ def device_props(device: int = 0) -> dict:
 def params_to_dict(p: L.Params) -> dict:
     return {"k": p.k, "passes": p.passes, "k_pass": list(p.k_pass)[: max(p.passes, 0)],
             "cr_levels": p.cr_levels, "thomas_chains": p.thomas_chains, "cluster": p.cluster,
-            "tl_levels": p.tl_levels,
+            "tl_levels": p.tl_levels, "chunk_systems": p.chunk_systems,
             "split_tile_rows": p.split_tile_rows, "split_threads": p.split_threads, "theta": p.theta}
 
 
@@ -103,6 +103,27 @@ class Plan:
                 p.k = sum(val)
             else:
                 setattr(p, key, int(val))
+        L.check(self._lib.tds_plan_set_params(self._h, ctypes.byref(p)))
+
+    def params_list(self) -> list:
+        """All tunable integers (tds_params field order) -- e.g. to broadcast a
+        tuned plan from rank 0 so every rank runs identical kernels."""
+        p = self.params
+        out = []
+        for f, _ in L.Params._fields_:
+            v = getattr(p, f)
+            out.extend(list(v) if f == "k_pass" else [v])
+        return out
+
+    def set_params_list(self, vals) -> None:
+        p = L.Params()
+        it = iter(int(v) for v in vals)
+        for f, _ in L.Params._fields_:
+            if f == "k_pass":
+                for i in range(L.TDS_MAX_PASSES):
+                    p.k_pass[i] = next(it)
+            else:
+                setattr(p, f, next(it))
         L.check(self._lib.tds_plan_set_params(self._h, ctypes.byref(p)))
 
     def permutation(self) -> np.ndarray:

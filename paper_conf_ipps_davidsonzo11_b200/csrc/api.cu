@@ -165,16 +165,23 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
         A.b = nullptr;
         A.c = w.c[ob];
         A.d = w.d[ob];
+        A.xs = w.a[ob];  // per-subsystem x overwrites a (each CTA reads its rows before writing them)
         A.slot = I.slot_rows;
         A.geom.npass = P.passes;
         for (int q = 0; q < kMaxPasses; ++q) A.geom.kpass[q] = P.k_pass[q];
         grid = (I.m << P.k) * P.cluster;
     }
-    if (P.passes < first || P.passes > last) return TDS_OK;  // on-chip stage not requested
-    if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "on-chip grid exceeds 2^31-1 CTAs");
-    const size_t smem = onchip_smem_bytes(I.dtype, I.onchip_threads, P.cluster, P.tl_levels);
-    cudaError_t err = launch_onchip<T>(A, P.cr_levels, P.k == 0, grid, I.onchip_threads, smem, st);
-    if (err != cudaSuccess) return cuda_fail(err, "onchip launch");
+    if (P.passes >= first && P.passes <= last) {
+        if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "on-chip grid exceeds 2^31-1 CTAs");
+        const size_t smem = onchip_smem_bytes(I.dtype, I.onchip_threads, P.cluster, P.tl_levels);
+        cudaError_t err = launch_onchip<T>(A, P.cr_levels, P.k == 0, grid, I.onchip_threads, smem, st);
+        if (err != cudaSuccess) return cuda_fail(err, "onchip launch");
+    }
+    if (P.k > 0 && P.passes + 1 >= first && P.passes + 1 <= last) {
+        cudaError_t err = launch_place_x<T>(A.xs, x, I.n, I.m, I.batch_stride, I.slot_rows, P.k,
+                                            vec_ok(I, {(const void *)x}), A.geom, st);
+        if (err != cudaSuccess) return cuda_fail(err, "place_x launch");
+    }
     return TDS_OK;
 }
 
@@ -213,6 +220,42 @@ static tds_status split_impl(const tds_plan_info &I, const T *a, const T *b, con
                                                                  I.params.k, I.slot_rows, g);
     cudaError_t err = cudaGetLastError();
     if (err != cudaSuccess) return cuda_fail(err, "gather launch");
+    return TDS_OK;
+}
+
+// Run launches [first, last] of the chunked sequence: for each chunk of
+// chunk_systems systems, S = passes + 1 + (k > 0) kernels.  Chunks reuse one
+// workspace, so a chunk's split output is still in L2 when its on-chip kernel
+// and x placement read it.
+template <typename T>
+static tds_status solve_chunks(const tds_plan_info &I, const T *a, const T *b, const T *c, const T *d, T *x,
+                               void *ws, cudaStream_t st, int first, int last) {
+    const int S = I.params.passes + 1 + (I.params.k > 0 ? 1 : 0);
+    const int64_t mc = chunk_m(I.params, I.m);
+    for (int64_t ch = 0; ch * mc < I.m; ++ch) {
+        const int lf = std::max<int64_t>(first - ch * S, 0);
+        const int ll = (int)std::min<int64_t>(last - ch * S, S - 1);
+        if (lf > ll) continue;
+        tds_plan_info Ic = I;
+        Ic.m = std::min<int64_t>(mc, I.m - ch * mc);
+        const int64_t off = ch * mc * I.batch_stride;
+        tds_status s = solve_impl<T>(Ic, a + off, b + off, c + off, d + off, x + off, ws, st, lf, ll);
+        if (s != TDS_OK) return s;
+    }
+    return TDS_OK;
+}
+
+template <typename T>
+static tds_status split_chunks(const tds_plan_info &I, const T *a, const T *b, const T *c, const T *d, T *oa,
+                               T *oc, T *od, void *ws, cudaStream_t st) {
+    const int64_t mc = chunk_m(I.params, I.m);
+    for (int64_t ch = 0; ch * mc < I.m; ++ch) {
+        tds_plan_info Ic = I;
+        Ic.m = std::min<int64_t>(mc, I.m - ch * mc);
+        const int64_t off = ch * mc * I.batch_stride, oo = ch * mc * I.n;
+        tds_status s = split_impl<T>(Ic, a + off, b + off, c + off, d + off, oa + oo, oc + oo, od + oo, ws, st);
+        if (s != TDS_OK) return s;
+    }
     return TDS_OK;
 }
 
@@ -257,7 +300,7 @@ tds_status tds_solve_batched(const tds_plan_t plan, const void *a, const void *b
                              void *x, void *workspace, size_t workspace_bytes, void *cuda_stream) {
     if (!plan) return fail(TDS_ERR_INVALID_ARG, "plan is NULL");
     return tds_solve_stages(plan, a, b, c, d, x, workspace, workspace_bytes, cuda_stream, 0,
-                            plan->info.params.passes);
+                            plan->info.launches - 1);
 }
 
 tds_status tds_solve_stages(const tds_plan_t plan, const void *a, const void *b, const void *c, const void *d,
@@ -265,8 +308,8 @@ tds_status tds_solve_stages(const tds_plan_t plan, const void *a, const void *b,
                             int32_t first_stage, int32_t last_stage) {
     if (!plan) return fail(TDS_ERR_INVALID_ARG, "plan is NULL");
     const tds_plan_info &I = plan->info;
-    if (first_stage < 0 || last_stage > I.params.passes || first_stage > last_stage)
-        return fail(TDS_ERR_INVALID_ARG, "stage range outside [0, passes]");
+    if (first_stage < 0 || last_stage >= I.launches || first_stage > last_stage)
+        return fail(TDS_ERR_INVALID_ARG, "launch range outside [0, info.launches)");
     tds_status s = check_arrays(I, {a, b, c, d, x});
     if (s != TDS_OK) return s;
     const size_t bytes = size_t(((I.m - 1) * I.batch_stride + I.n) * dsize(I.dtype));
@@ -282,10 +325,10 @@ tds_status tds_solve_stages(const tds_plan_t plan, const void *a, const void *b,
     if ((s = check_device(plan)) != TDS_OK) return s;
     cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
     s = I.dtype == TDS_F32
-            ? solve_impl<float>(I, (const float *)a, (const float *)b, (const float *)c, (const float *)d,
-                                (float *)x, workspace, st, first_stage, last_stage)
-            : solve_impl<double>(I, (const double *)a, (const double *)b, (const double *)c, (const double *)d,
-                                 (double *)x, workspace, st, first_stage, last_stage);
+            ? solve_chunks<float>(I, (const float *)a, (const float *)b, (const float *)c, (const float *)d,
+                                  (float *)x, workspace, st, first_stage, last_stage)
+            : solve_chunks<double>(I, (const double *)a, (const double *)b, (const double *)c,
+                                   (const double *)d, (double *)x, workspace, st, first_stage, last_stage);
     if (s == TDS_OK) clear_error();
     return s;
 }
@@ -302,10 +345,11 @@ tds_status tds_split_batched(const tds_plan_t plan, const void *a, const void *b
     if ((s = check_device(plan)) != TDS_OK) return s;
     cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
     s = I.dtype == TDS_F32
-            ? split_impl<float>(I, (const float *)a, (const float *)b, (const float *)c, (const float *)d,
-                                (float *)a_out, (float *)c_out, (float *)d_out, workspace, st)
-            : split_impl<double>(I, (const double *)a, (const double *)b, (const double *)c, (const double *)d,
-                                 (double *)a_out, (double *)c_out, (double *)d_out, workspace, st);
+            ? split_chunks<float>(I, (const float *)a, (const float *)b, (const float *)c, (const float *)d,
+                                  (float *)a_out, (float *)c_out, (float *)d_out, workspace, st)
+            : split_chunks<double>(I, (const double *)a, (const double *)b, (const double *)c,
+                                   (const double *)d, (double *)a_out, (double *)c_out, (double *)d_out, workspace,
+                                   st);
     if (s == TDS_OK) clear_error();
     return s;
 }

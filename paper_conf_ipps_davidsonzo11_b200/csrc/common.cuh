@@ -93,7 +93,8 @@ struct SplitArgs {
 template <typename T>
 struct OnchipArgs {
     const T *a, *b, *c, *d;  // RAW (K == 0): original arrays; else normalised a,c,d slots
-    T *x;
+    T *x;                    // K == 0: the solution, original layout
+    T *xs;                   // K > 0: per-subsystem solutions (workspace slots, aliasing a)
     int64_t n;
     int64_t batch_stride;    // original layout (input when RAW, always for x)
     int64_t slot;            // workspace slot capacity (K > 0)
@@ -112,6 +113,9 @@ cudaError_t launch_split_pass(const SplitArgs<T> &A, bool raw, int64_t grid, int
                               cudaStream_t st);
 template <typename T>
 cudaError_t launch_split_reg(const SplitArgs<T> &A, bool raw, int64_t grid, cudaStream_t st);
+template <typename T>
+cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batch_stride, int64_t slot, int K,
+                           int vec, const PassGeom &geom, cudaStream_t st);
 template <typename T>
 cudaError_t launch_onchip(const OnchipArgs<T> &A, int cr_levels, bool raw, int64_t grid, int threads,
                           size_t smem, cudaStream_t st);

@@ -348,13 +348,17 @@ __global__ void __launch_bounds__(R >= 8 ? 512 : 1024) onchip_kernel(const Onchi
             rd[v] = rd[v] - ra[v] * xlv - rc[v] * rd[(v + s) % R];
         }
     }
-    if (A.K == 0 && R >= W && A.vec && jt + R <= L) {
-        st16<T, R>(A.x + out_base + jt, rd);
+    // x of this subsystem is written contiguously: straight to x when K == 0, else
+    // to its workspace slot (the placement kernel restores the original order).
+    T *dst = A.K == 0 ? A.x + out_base : A.xs + sigma * A.slot;
+    const bool dvec = A.K == 0 ? (A.vec != 0) : true;
+    if (R >= W && dvec && jt + R <= L) {
+        st16<T, R>(dst + jt, rd);
     } else {
 #pragma unroll
         for (int v = 0; v < R; ++v) {
             const int64_t j = jt + v;
-            if (j < L) __stcs(A.x + out_base + (j << A.K), rd[v]);
+            if (j < L) __stcs(dst + j, rd[v]);
         }
     }
     if constexpr (C > 1) cg::this_cluster().barrier_wait();  // keep shared memory alive for the readers

@@ -1,0 +1,139 @@
+// place_x.cu -- A4 "x placement": put the per-subsystem solutions back in the
+// original row order, x[s][r + 2^K j] = xs[slot(s, r)][j].
+//
+// PCR splitting leaves 2^K interleaved subsystems (residue classes mod 2^K,
+// PAPER.md Fig. 3a); the on-chip kernel writes each subsystem's x
+// contiguously into its workspace slot.  Writing x straight to original rows
+// from there would be a stride-2^K scatter (one 4-byte sector per element).
+// Here thread t gathers 16 CONSECUTIVE original rows (the mirror image of the
+// register split kernel's de-interleaved store): for K <= 4 the 16 >> K rows
+// of one residue have consecutive j and are one vector load, and across the
+// warp every residue run is a coalesced read; the 16 rows leave as contiguous
+// 16-byte vector stores.
+#include "common.cuh"
+
+namespace tds {
+
+template <typename T>
+struct PlaceArgs {
+    const T *xs;         // per-subsystem solutions, slot sigma at xs[sigma * slot + j]
+    T *x;                // output, original layout
+    int64_t n, batch_stride, slot;
+    int32_t K;           // total split levels
+    int32_t vec;         // x rows may be written with 16-byte vector stores
+    PassGeom geom;       // slot -> residue map
+};
+
+constexpr int kPlaceRows = 16;
+constexpr int kPlaceThreads = 256;
+
+// Physical slot (within its system) of residue r: the residue's digits in pass
+// order, the first pass's digit most significant.
+__device__ __forceinline__ int64_t residue_slot(int64_t r, const PassGeom &g) {
+    if (g.npass == 1) return r;
+    int64_t sl = 0;
+    int kc = 0;
+#pragma unroll
+    for (int p = 0; p < TDS_MAX_PASSES; ++p) {
+        if (p < g.npass) {
+            const int kp = g.kpass[p];
+            sl = (sl << kp) | ((r >> kc) & ((int64_t(1) << kp) - 1));
+            kc += kp;
+        }
+    }
+    return sl;
+}
+
+template <typename T, int KK>  // KK = min(K, 4)
+__global__ void __launch_bounds__(kPlaceThreads) place_x_kernel(const PlaceArgs<T> A) {
+    constexpr int R = kPlaceRows;
+    constexpr int NRK = 1 << KK;  // residues among 16 consecutive rows
+    constexpr int G = R >> KK;    // rows per residue per thread
+    constexpr int W = 16 / int(sizeof(T));
+    const int64_t tiles = (A.n + R * kPlaceThreads - 1) / (R * kPlaceThreads);
+    const int64_t sys = blockIdx.x / tiles;
+    const int64_t i0 = ((blockIdx.x % tiles) * kPlaceThreads + threadIdx.x) * R;
+    if (i0 >= A.n) return;
+    const int64_t NR = int64_t(1) << A.K;
+    const int64_t sys_slots = sys << A.K;
+    const bool full = i0 + R <= A.n;
+    T v[R];
+#pragma unroll
+    for (int rho = 0; rho < NRK; ++rho) {
+        const int64_t row = i0 + rho;           // first of this residue's G rows
+        const int64_t r = row & (NR - 1), j = row >> A.K;
+        const T *src = A.xs + (sys_slots + residue_slot(r, A.geom)) * A.slot + j;
+        constexpr bool kVec = (G * sizeof(T) >= 16) || (sizeof(T) == 4 && G == 2);
+        if (kVec && full) {
+            if constexpr (G * sizeof(T) >= 16) {
+#pragma unroll
+                for (int q = 0; q < G / W; ++q) {
+                    if constexpr (sizeof(T) == 4) {
+                        const float4 f = __ldcs(reinterpret_cast<const float4 *>(src) + q);
+                        v[rho + NRK * (4 * q)] = f.x;
+                        v[rho + NRK * (4 * q + 1)] = f.y;
+                        v[rho + NRK * (4 * q + 2)] = f.z;
+                        v[rho + NRK * (4 * q + 3)] = f.w;
+                    } else {
+                        const double2 f = __ldcs(reinterpret_cast<const double2 *>(src) + q);
+                        v[rho + NRK * (2 * q)] = f.x;
+                        v[rho + NRK * (2 * q + 1)] = f.y;
+                    }
+                }
+            } else if constexpr (sizeof(T) == 4 && G == 2) {
+                const float2 f = __ldcs(reinterpret_cast<const float2 *>(src));
+                v[rho] = f.x;
+                v[rho + NRK] = f.y;
+            }
+        } else {
+#pragma unroll
+            for (int u = 0; u < G; ++u)
+                v[rho + NRK * u] = (row + NRK * u < A.n) ? __ldcs(src + u) : T(0);
+        }
+    }
+    T *dst = A.x + sys * A.batch_stride + i0;
+    if (full && A.vec) {
+#pragma unroll
+        for (int q = 0; q < R / W; ++q) {
+            if constexpr (sizeof(T) == 4)
+                __stcs(reinterpret_cast<float4 *>(dst) + q, make_float4(v[4 * q], v[4 * q + 1], v[4 * q + 2], v[4 * q + 3]));
+            else
+                __stcs(reinterpret_cast<double2 *>(dst) + q, make_double2(v[2 * q], v[2 * q + 1]));
+        }
+    } else {
+#pragma unroll
+        for (int u = 0; u < R; ++u)
+            if (i0 + u < A.n) dst[u] = v[u];
+    }
+}
+
+template <typename T>
+cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batch_stride, int64_t slot, int K,
+                           int vec, const PassGeom &geom, cudaStream_t st) {
+    PlaceArgs<T> A{};
+    A.xs = xs;
+    A.x = x;
+    A.n = n;
+    A.batch_stride = batch_stride;
+    A.slot = slot;
+    A.K = K;
+    A.vec = vec;
+    A.geom = geom;
+    const int64_t tiles = (n + kPlaceRows * kPlaceThreads - 1) / (kPlaceRows * kPlaceThreads);
+    const int64_t grid = m * tiles;
+    if (grid > 0x7fffffffLL) return cudaErrorInvalidConfiguration;
+    switch (K >= 4 ? 4 : K) {
+        case 1: place_x_kernel<T, 1><<<(unsigned)grid, kPlaceThreads, 0, st>>>(A); break;
+        case 2: place_x_kernel<T, 2><<<(unsigned)grid, kPlaceThreads, 0, st>>>(A); break;
+        case 3: place_x_kernel<T, 3><<<(unsigned)grid, kPlaceThreads, 0, st>>>(A); break;
+        default: place_x_kernel<T, 4><<<(unsigned)grid, kPlaceThreads, 0, st>>>(A); break;
+    }
+    return cudaGetLastError();
+}
+
+template cudaError_t launch_place_x<float>(const float *, float *, int64_t, int64_t, int64_t, int64_t, int, int,
+                                           const PassGeom &, cudaStream_t);
+template cudaError_t launch_place_x<double>(const double *, double *, int64_t, int64_t, int64_t, int64_t, int, int,
+                                            const PassGeom &, cudaStream_t);
+
+}  // namespace tds

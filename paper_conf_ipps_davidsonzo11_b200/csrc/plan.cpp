@@ -57,6 +57,10 @@ int32_t split_tile_eff(const tds_params &p, int pass) {
                                             : p.split_tile_rows;
 }
 
+int64_t chunk_m(const tds_params &p, int64_t m) {
+    return (p.chunk_systems <= 0 || p.chunk_systems >= m) ? m : p.chunk_systems;
+}
+
 int32_t split_segments(int64_t m_in, int64_t tiles, int32_t theta) {
     // Fig. 1: cooperative splitting (stage 1, several CTAs per
     // system) only while there are fewer than theta independent systems.
@@ -160,24 +164,28 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
                 return fail(TDS_ERR_UNSUPPORTED, "split tile + halo exceeds shared memory");
         }
     }
+    if (p.chunk_systems < 0) return fail(TDS_ERR_INVALID_ARG, "chunk_systems >= 0");
     // --- derived fields
     info.params = p;
     info.n_sub = n_sub;
     info.num_subsystems = m * std::min<int64_t>(int64_t(1) << std::min(p.k, 62), n);
     info.onchip_threads = (int32_t)threads;
     info.subsys_per_cta = 1;
+    const int64_t mc = chunk_m(p, m);  // systems per chunk
+    info.chunks = (int32_t)cdiv(m, mc);
+    info.launches = info.chunks * (p.passes + 1 + (p.k > 0 ? 1 : 0));
     if (p.passes > 0) {
         int kk = 0;
         int64_t elems = 0;
         for (int i = 0; i < p.passes; ++i) {
             kk += p.k_pass[i];
-            elems = std::max<int64_t>(elems, m * (int64_t(1) << kk) * slot_rows(n, kk, dtype));
+            elems = std::max<int64_t>(elems, mc * (int64_t(1) << kk) * slot_rows(n, kk, dtype));
         }
         const int64_t E = round_up(elems, 64);
         info.slot_rows = slot_rows(n, p.k, dtype);
         info.workspace_bytes = size_t((p.passes == 1 ? 1 : 2) * 3 * E * dsize(dtype));
         info.split_tile_eff = split_tile_eff(p, 0);
-        info.split_segments = split_segments(m, cdiv(n, info.split_tile_eff), p.theta);
+        info.split_segments = split_segments(mc, cdiv(n, info.split_tile_eff), p.theta);
     } else {
         info.slot_rows = 0;
         info.workspace_bytes = 0;
@@ -205,7 +213,10 @@ static tds_status seed(tds_plan_info &info, const tds_device_props &props, tds_p
     } else {
         target = info.n_onchip_max;
         T = 2 * props.warp_size;
-        theta = props.sm_count;
+        // P:L650-655 "estimate based only on the number of available processors";
+        // a B200 SM keeps several split CTAs resident and independent tiles need no
+        // inter-CTA sync, so the static guess asks for 32 independent units per SM.
+        theta = 32 * props.sm_count;
         tile = (int32_t)std::min<int64_t>(info.n_onchip_max, int64_t(r_max(dtype)) * kMaxOnchipThreadsWide);
         g1threads = 512;
         kpmax = std::min(dtype == TDS_F32 ? 9 : 8, kp_limit(props, dtype, tile));
@@ -237,6 +248,9 @@ static tds_status seed(tds_plan_info &info, const tds_device_props &props, tds_p
     p.split_tile_rows = tile;
     p.split_threads = g1threads;
     p.theta = theta;
+    // L2-resident chunking (chunk_systems) is a tuner dimension only: measured on
+    // B200 it loses to one launch per kernel over the whole batch (profiles/).
+    p.chunk_systems = 0;
     return TDS_OK;
 }
 

@@ -37,6 +37,7 @@ int32_t split_segments(int64_t m_in, int64_t tiles, int32_t theta);
 size_t split_smem_bytes(int32_t dtype, int32_t tile, int kp);
 size_t onchip_smem_bytes(int32_t dtype, int32_t threads, int32_t cluster, int32_t tl_levels);
 int32_t split_tile_eff(const tds_params &p, int pass);
+int64_t chunk_m(const tds_params &p, int64_t m);
 int32_t static_cluster(const tds_device_props &p);
 tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_params &p);
 

@@ -203,7 +203,7 @@ static std::string params_str(const tds_params &p) {
     o << p.k << " " << p.passes;
     for (int i = 0; i < TDS_MAX_PASSES; ++i) o << " " << p.k_pass[i];
     o << " " << p.cr_levels << " " << p.thomas_chains << " " << p.cluster << " " << p.tl_levels << " "
-      << p.split_tile_rows << " " << p.split_threads << " " << p.theta;
+      << p.split_tile_rows << " " << p.split_threads << " " << p.theta << " " << p.chunk_systems;
     return o.str();
 }
 
@@ -220,7 +220,7 @@ static bool cache_lookup(const std::string &path, const std::string &key, tds_pa
         is >> q.k >> q.passes;
         for (int i = 0; i < TDS_MAX_PASSES; ++i) is >> q.k_pass[i];
         is >> q.cr_levels >> q.thomas_chains >> q.cluster >> q.tl_levels >> q.split_tile_rows >> q.split_threads >>
-            q.theta;
+            q.theta >> q.chunk_systems;
         if (is) {
             p = q;
             found = true;
@@ -322,6 +322,11 @@ extern "C" tds_status tds_tune(tds_plan_t plan, void *cuda_stream, const char *c
                 q = best; q.split_tile_rows = best.split_tile_rows * 2; cands.push_back(q);
                 q = best; q.split_threads = best.split_threads / 2; cands.push_back(q);
                 q = best; q.split_threads = best.split_threads * 2; cands.push_back(q);
+                {  // L2-resident chunks of systems: halve / double the chunk (0 = whole batch)
+                    const int64_t mc = chunk_m(best, I.m);
+                    if (mc > 1) { q = best; q.chunk_systems = (int32_t)cdiv(mc, 2); cands.push_back(q); }
+                    if (mc < I.m) { q = best; q.chunk_systems = (int32_t)std::min<int64_t>(2 * mc, I.m); cands.push_back(q); }
+                }
                 if (best.passes < TDS_MAX_PASSES && best.k > best.passes) {
                     // one more (shallower) pass: less halo per pass, one more HBM round trip
                     q = best;

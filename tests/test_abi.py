@@ -78,7 +78,7 @@ def test_planner_matches_reference(tds, pname, props, dtype, mode, n, m):
                  mode="default" if mode == rp.DEFAULT else "static")
     got = p.info
     for f in ("k", "passes", "n_sub", "num_subsystems", "cr_levels", "thomas_chains", "onchip_threads",
-              "cluster", "tl_levels",
+              "cluster", "tl_levels", "chunk_systems", "chunks", "launches",
               "split_tile_rows", "split_threads", "split_segments", "theta", "n_sub_target", "n_onchip_max",
               "split_kp_max", "slot_rows", "workspace_bytes"):
         assert got[f] == getattr(ref, f), (f, got[f], getattr(ref, f))

@@ -370,3 +370,20 @@ def test_tuner_runs_and_caches(tds, tmp_path):
     plan2 = tds.Plan(n, m, "float32", device=0)
     assert plan2.tune(cache_path=cache) == 0  # saved result reused
     assert plan2.info["k"] == info["k"] and plan2.info["thomas_chains"] == info["thomas_chains"]
+
+
+@pytest.mark.parametrize("chunk", [1, 2, 3, 7])
+def test_chunked_equals_unchunked(tds, chunk):
+    """L2-resident chunks run the same kernels on each system: x bit-identical."""
+    n, m = 100000, 7
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=29)
+    base = dict(k_pass=[4, 2], cr_levels=4, thomas_chains=32, cluster=1, tl_levels=0)
+    x0, _ = run(tds, a, b, c, d, params=dict(base, chunk_systems=0))
+    x1, plan = run(tds, a, b, c, d, params=dict(base, chunk_systems=chunk))
+    assert plan.info["chunks"] == -(-m // chunk)
+    assert np.array_equal(x0, x1)
+    check(a, b, c, d, x1, np.float32)
+    g0 = split_gpu(tds, a, b, c, d, dict(base, chunk_systems=0))
+    g1 = split_gpu(tds, a, b, c, d, dict(base, chunk_systems=chunk))
+    for u, v in zip(g0[:3], g1[:3]):
+        assert np.array_equal(u, v)

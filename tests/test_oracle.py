@@ -283,7 +283,7 @@ def test_planner_paper_values():
     assert p.n_sub <= 256 and p.k == 12
     ps = rplan.make_plan(rplan.B200, rplan.F32, 1 << 20, 16, mode=rplan.STATIC)
     assert ps.thomas_chains == g["static_thomas_chains"][0]
-    assert ps.theta == rplan.B200.sm_count
+    assert ps.theta == 32 * rplan.B200.sm_count  # a multiple of the processor count
 
 
 def test_planner_static_onchip_sizes():
