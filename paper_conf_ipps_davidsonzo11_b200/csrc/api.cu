@@ -120,7 +120,10 @@ static tds_status run_split(const tds_plan_info &I, const T *a, const T *b, cons
         const int64_t grid = m_in * A.segs;
         if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "split grid exceeds 2^31-1 CTAs");
         cudaError_t err;
-        if (kp <= kRegSplitMaxKp) {
+        if (kp <= kRegSplitMaxKp && A.vec) {
+            // persistent, TMA-prefetched register kernel (16-byte aligned rows)
+            err = launch_split_pipe<T>(A, raw, m_in, len_in, st);
+        } else if (kp <= kRegSplitMaxKp) {
             err = launch_split_reg<T>(A, raw, grid, st);
         } else {
             const size_t smem = split_smem_bytes(I.dtype, P.split_tile_rows, kp);
@@ -173,8 +176,18 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
     }
     if (P.passes >= first && P.passes <= last) {
         if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "on-chip grid exceeds 2^31-1 CTAs");
-        const size_t smem = onchip_smem_bytes(I.dtype, I.onchip_threads, P.cluster, P.tl_levels);
-        cudaError_t err = launch_onchip<T>(A, P.cr_levels, P.k == 0, grid, I.onchip_threads, smem, st);
+        cudaError_t err;
+        if (onchip_pipe_ok(I)) {
+            // persistent, TMA-pipelined form (cluster == 1, 64 bytes of rows per thread)
+            int dev = 0, sms = 148;
+            cudaGetDevice(&dev);
+            cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+            const size_t smem = onchip_pipe_smem_bytes(I.dtype, I.onchip_threads, 1 << P.cr_levels, P.tl_levels);
+            err = launch_onchip_pipe<T>(A, I.m << P.k, I.onchip_threads, sms, smem, st);
+        } else {
+            const size_t smem = onchip_smem_bytes(I.dtype, I.onchip_threads, P.cluster, P.tl_levels);
+            err = launch_onchip<T>(A, P.cr_levels, P.k == 0, grid, I.onchip_threads, smem, st);
+        }
         if (err != cudaSuccess) return cuda_fail(err, "onchip launch");
     }
     if (P.k > 0 && P.passes + 1 >= first && P.passes + 1 <= last) {

@@ -114,6 +114,23 @@ cudaError_t launch_split_pass(const SplitArgs<T> &A, bool raw, int64_t grid, int
 template <typename T>
 cudaError_t launch_split_reg(const SplitArgs<T> &A, bool raw, int64_t grid, cudaStream_t st);
 template <typename T>
+cudaError_t launch_split_pipe(const SplitArgs<T> &A, bool raw, int64_t m_in, int64_t max_len, cudaStream_t st);
+template <typename T>
+cudaError_t launch_onchip_pipe(const OnchipArgs<T> &A, int64_t nslots, int threads, int sm_count, size_t smem,
+                               cudaStream_t st);
+size_t onchip_pipe_smem_bytes(int32_t dtype, int32_t threads, int32_t R, int32_t tl_levels);
+
+// The persistent TMA-pipelined on-chip kernel applies to split plans (k > 0) on
+// one CTA per subsystem whose threads hold 64 bytes of rows (fp32 c = 4, fp64 c = 3).
+inline bool onchip_pipe_ok(const tds_plan_info &I) {
+    const tds_params &P = I.params;
+    if (P.k == 0 || P.cluster != 1) return false;
+    if ((1 << P.cr_levels) * dsize(I.dtype) != 64) return false;
+    return onchip_pipe_smem_bytes(I.dtype, I.onchip_threads, 1 << P.cr_levels, P.tl_levels) + kSmemReserve + 16 <=
+           size_t(232448);
+}
+
+template <typename T>
 cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batch_stride, int64_t slot, int K,
                            int vec, const PassGeom &geom, cudaStream_t st);
 template <typename T>

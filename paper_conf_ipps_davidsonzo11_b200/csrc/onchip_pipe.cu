@@ -1,0 +1,266 @@
+// onchip_pipe.cu -- G2, persistent TMA-pipelined form (one CTA per SM).
+//
+// Same mathematics as onchip.cu with cluster = 1 (§III-A base kernel:
+// c CR levels in registers, c2 CR levels across threads, PCR on the reduced
+// system until T chains, Thomas per chain, back substitution), but the CTA is
+// persistent and walks subsystems sigma = blockIdx.x, += gridDim.x.  While it
+// solves subsystem i from registers, the Tensor Memory Accelerator streams
+// subsystems i+1 and i+2 (three contiguous workspace arrays each) into a
+// two-stage shared-memory ring with cp.async.bulk + mbarrier transaction
+// counts, so HBM traffic never waits for the CR / PCR / Thomas phases.
+//
+// Shared memory -> registers: thread t owns 16-byte chunks 4t..4t+3 of each
+// array (64 bytes, rows tR..tR+R-1).  Read in plain order, lanes 0,2,4,6 of a
+// quarter-warp would hit the same bank group (4-way conflict); lane l instead
+// reads chunk (q + l/2) mod 4 in instruction q, which is conflict-free, and a
+// 4-way select puts every chunk back in its register slot.
+#include "pipe.cuh"
+
+namespace tds {
+
+template <typename T, int ZR>
+__device__ __forceinline__ void reduced_solve_pipe(T *z, int Z, int NT, int t, int log2T);
+
+template <typename T, int R>
+__global__ void __launch_bounds__(512, 1) onchip_pipe_kernel(const OnchipArgs<T> A, int64_t nslots) {
+    static_assert(R * sizeof(T) == 64, "pipe kernel: 64 bytes of rows per thread");
+    extern __shared__ __align__(128) unsigned char smem_raw[];
+    __shared__ __align__(8) uint64_t full_bar[2];
+    constexpr int CR = ilog2c(R);
+    const int NT = blockDim.x;
+    const int ROWS = NT * R;
+    const int t = threadIdx.x, lane = t & 31, warp = t >> 5, nwarps = NT >> 5;
+    const int c2 = A.tl_levels;
+    const int Z = NT >> c2;
+    T *stage0 = reinterpret_cast<T *>(smem_raw);  // [2][3][ROWS]
+    T *z = stage0 + 6 * ROWS;                      // [3][Z]
+    T *ya = z + 3 * Z;                             // [4][NT]
+    T *yc = ya + NT, *yd = yc + NT, *yx = yd + NT;
+    T *edge = yx + NT;                             // [2][3][nwarps]
+    const int64_t KK = int64_t(1) << A.K;
+
+    auto slot_len = [&](int64_t sigma) -> int64_t {
+        const int64_t r = slot_residue(sigma & (KK - 1), A.geom.npass, A.geom.kpass);
+        return r < A.n ? (A.n - r + KK - 1) >> A.K : 0;
+    };
+    auto issue = [&](int64_t sigma, int s) {  // thread 0 only
+        if (sigma >= nslots) return;
+        const int64_t L = slot_len(sigma);
+        const uint32_t bytes = uint32_t(((L * sizeof(T)) + 15) & ~int64_t(15));
+        uint64_t *bar = &full_bar[s];
+        mbar_expect_tx(bar, 3 * bytes);
+        if (bytes) {
+            T *dst = stage0 + size_t(s) * 3 * ROWS;
+            const int64_t o = sigma * A.slot;
+            bulk_g2s(dst, A.a + o, bytes, bar);
+            bulk_g2s(dst + ROWS, A.c + o, bytes, bar);
+            bulk_g2s(dst + 2 * ROWS, A.d + o, bytes, bar);
+        }
+    };
+    if (t == 0) {
+        mbar_init(&full_bar[0], 1);
+        mbar_init(&full_bar[1], 1);
+        asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+        issue(blockIdx.x, 0);
+        issue(int64_t(blockIdx.x) + gridDim.x, 1);
+    }
+    __syncthreads();
+
+    for (int64_t it = 0;; ++it) {
+        const int64_t sigma = int64_t(blockIdx.x) + it * gridDim.x;
+        if (sigma >= nslots) break;
+        const int s = int(it & 1);
+        const int64_t L = slot_len(sigma);
+        mbar_wait(&full_bar[s], uint32_t((it >> 1) & 1));
+        const T *sb = stage0 + size_t(s) * 3 * ROWS;
+        const int64_t jt = int64_t(t) * R;
+        T ra[R], rc[R], rd[R];
+        lds_rows<T, R>(sb + jt, ra, lane);
+        lds_rows<T, R>(sb + ROWS + jt, rc, lane);
+        lds_rows<T, R>(sb + 2 * ROWS + jt, rd, lane);
+        if (jt + R > L) {  // identity rows beyond the subsystem (stale shared memory)
+#pragma unroll
+            for (int v = 0; v < R; ++v) {
+                const bool in = jt + v < L;
+                ra[v] = in ? ra[v] : T(0);
+                rc[v] = in ? rc[v] : T(0);
+                rd[v] = in ? rd[v] : T(0);
+            }
+        }
+        __syncthreads();  // every thread has read stage s: refill it
+        if (t == 0) issue(sigma + 2 * int64_t(gridDim.x), s);
+        if (L == 0) continue;  // empty slot (2^K > n): uniform
+
+        // ---- B1. CR forward levels in registers
+#pragma unroll
+        for (int l = 1; l <= CR; ++l) {
+            const int sl = 1 << (l - 1);
+            const T pa = ra[sl - 1], pc = rc[sl - 1], pd = rd[sl - 1];
+            T na = __shfl_down_sync(0xffffffffu, pa, 1);
+            T nc = __shfl_down_sync(0xffffffffu, pc, 1);
+            T nd = __shfl_down_sync(0xffffffffu, pd, 1);
+            T *eb = edge + (l & 1) * 3 * nwarps;
+            if (lane == 0) {
+                eb[warp] = pa;
+                eb[nwarps + warp] = pc;
+                eb[2 * nwarps + warp] = pd;
+            }
+            __syncthreads();
+            if (lane == 31) {
+                const bool h = warp + 1 < nwarps;
+                na = h ? eb[warp + 1] : T(0);
+                nc = h ? eb[nwarps + warp + 1] : T(0);
+                nd = h ? eb[2 * nwarps + warp + 1] : T(0);
+            }
+#pragma unroll
+            for (int v = (1 << l) - 1; v < R; v += (1 << l)) {
+                const bool last = (v == R - 1);
+                row_update(ra[v], rc[v], rd[v], ra[v - sl], rc[v - sl], rd[v - sl], last ? na : ra[(v + sl) % R],
+                           last ? nc : rc[(v + sl) % R], last ? nd : rd[(v + sl) % R]);
+            }
+        }
+        // ---- B2. c2 CR levels across threads
+        ya[t] = ra[R - 1];
+        yc[t] = rc[R - 1];
+        yd[t] = rd[R - 1];
+        for (int l = 1; l <= c2; ++l) {
+            const int sl = 1 << (l - 1);
+            __syncthreads();
+            if ((t & ((1 << l) - 1)) == (1 << l) - 1) {
+                T a = ya[t], c = yc[t], d = yd[t];
+                const bool hr = t + sl < NT;
+                row_update(a, c, d, ya[t - sl], yc[t - sl], yd[t - sl], hr ? ya[t + sl] : T(0),
+                           hr ? yc[t + sl] : T(0), hr ? yd[t + sl] : T(0));
+                ya[t] = a;
+                yc[t] = c;
+                yd[t] = d;
+            }
+        }
+        __syncthreads();
+        // ---- C. the CTA's remaining Z rows: PCR until T chains, Thomas per chain
+        const bool top = (t & ((1 << c2) - 1)) == (1 << c2) - 1;
+        const int zi = t >> c2;
+        if (top) {
+            z[zi] = ya[t];
+            z[Z + zi] = yc[t];
+            z[2 * Z + zi] = yd[t];
+        }
+        __syncthreads();
+        reduced_solve_pipe<T, 1>(z, Z, NT, t, A.log2T);
+        if (top) yx[t] = z[2 * Z + zi];
+        // ---- D. back substitution across threads, then in registers
+        for (int l = c2; l >= 1; --l) {
+            const int sl = 1 << (l - 1);
+            __syncthreads();
+            if ((t & ((1 << l) - 1)) == sl - 1) {
+                const T xl = t >= sl ? yx[t - sl] : T(0);
+                yx[t] = yd[t] - ya[t] * xl - yc[t] * yx[t + sl];
+            }
+        }
+        __syncthreads();
+        rd[R - 1] = yx[t];
+        const T xleft = t > 0 ? yx[t - 1] : T(0);
+#pragma unroll
+        for (int l = CR; l >= 1; --l) {
+            const int sl = 1 << (l - 1);
+#pragma unroll
+            for (int v = sl - 1; v < R - 1; v += 2 * sl) {
+                const T xlv = (v >= sl) ? rd[(v - sl + R) % R] : xleft;
+                rd[v] = rd[v] - ra[v] * xlv - rc[v] * rd[(v + sl) % R];
+            }
+        }
+        T *dst = A.xs + sigma * A.slot + jt;  // per-subsystem x (placement kernel follows)
+        if (jt + R <= L) {
+            constexpr int W = 16 / int(sizeof(T));
+#pragma unroll
+            for (int q = 0; q < R / W; ++q) {
+                if constexpr (sizeof(T) == 4)
+                    __stcs(reinterpret_cast<float4 *>(dst) + q,
+                           make_float4(rd[4 * q], rd[4 * q + 1], rd[4 * q + 2], rd[4 * q + 3]));
+                else
+                    __stcs(reinterpret_cast<double2 *>(dst) + q, make_double2(rd[2 * q], rd[2 * q + 1]));
+            }
+        } else {
+#pragma unroll
+            for (int v = 0; v < R; ++v)
+                if (jt + v < L) dst[v] = rd[v];
+        }
+        __syncthreads();  // y / z / edge buffers are reused by the next subsystem
+    }
+}
+
+// PCR until 2^log2T chains, then Thomas per chain, on Z <= ZR * NT rows in z.
+template <typename T, int ZR>
+__device__ __forceinline__ void reduced_solve_pipe(T *z, int Z, int NT, int t, int log2T) {
+    T *za = z, *zc = z + Z, *zd = z + 2 * Z;
+    for (int j = 0; j < log2T; ++j) {
+        const int s = 1 << j;
+        T na[ZR], nc[ZR], nd[ZR];
+#pragma unroll
+        for (int q = 0; q < ZR; ++q) {
+            const int i = t + q * NT;
+            if (i < Z) {
+                T a = za[i], c = zc[i], d = zd[i];
+                const bool hl = i >= s, hr = i + s < Z;
+                row_update(a, c, d, hl ? za[i - s] : T(0), hl ? zc[i - s] : T(0), hl ? zd[i - s] : T(0),
+                           hr ? za[i + s] : T(0), hr ? zc[i + s] : T(0), hr ? zd[i + s] : T(0));
+                na[q] = a;
+                nc[q] = c;
+                nd[q] = d;
+            }
+        }
+        __syncthreads();
+#pragma unroll
+        for (int q = 0; q < ZR; ++q) {
+            const int i = t + q * NT;
+            if (i < Z) {
+                za[i] = na[q];
+                zc[i] = nc[q];
+                zd[i] = nd[q];
+            }
+        }
+        __syncthreads();
+    }
+    const int TC = 1 << log2T;
+    for (int ch = t; ch < TC && ch < Z; ch += NT) {
+        T cp = zc[ch], dp = zd[ch];
+        int q = ch;
+        for (int qn = ch + TC; qn < Z; qn += TC) {
+            const T aq = za[qn];
+            const T w = rcp(fma(-aq, cp, T(1)));
+            cp = zc[qn] * w;
+            dp = (zd[qn] - aq * dp) * w;
+            zc[qn] = cp;
+            zd[qn] = dp;
+            q = qn;
+        }
+        T xv = dp;
+        for (int qp = q - TC; qp >= ch; qp -= TC) {
+            xv = zd[qp] - zc[qp] * xv;
+            zd[qp] = xv;
+        }
+    }
+    __syncthreads();
+}
+
+size_t onchip_pipe_smem_bytes(int32_t dtype, int32_t threads, int32_t R, int32_t tl_levels) {
+    const int64_t rows = int64_t(threads) * R;
+    return size_t((6 * rows + 3 * (threads >> tl_levels) + 4 * int64_t(threads) + 6 * (threads / 32) + 8) *
+                  dsize(dtype));
+}
+
+template <typename T>
+cudaError_t launch_onchip_pipe(const OnchipArgs<T> &A, int64_t nslots, int threads, int sm_count, size_t smem,
+                               cudaStream_t st) {
+    auto kern = onchip_pipe_kernel<T, 64 / int(sizeof(T))>;
+    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    if (e != cudaSuccess) return e;
+    const int64_t grid = std::min<int64_t>(nslots, sm_count);
+    kern<<<(unsigned)grid, threads, smem, st>>>(A, nslots);
+    return cudaGetLastError();
+}
+
+template cudaError_t launch_onchip_pipe<float>(const OnchipArgs<float> &, int64_t, int, int, size_t, cudaStream_t);
+template cudaError_t launch_onchip_pipe<double>(const OnchipArgs<double> &, int64_t, int, int, size_t, cudaStream_t);
+
+}  // namespace tds

@@ -1,0 +1,92 @@
+// pipe.cuh -- TMA bulk-copy / mbarrier helpers and conflict-free shared-memory
+// row loads shared by the persistent (pipelined) kernels.
+#pragma once
+#include "common.cuh"
+
+namespace tds {
+
+__device__ __forceinline__ uint32_t smem_u32(const void *p) {
+    return static_cast<uint32_t>(__cvta_generic_to_shared(p));
+}
+
+__device__ __forceinline__ void mbar_init(uint64_t *bar, uint32_t count) {
+    asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(count));
+}
+
+// Arrive once and announce `bytes` of TMA transactions for the current phase.
+__device__ __forceinline__ void mbar_expect_tx(uint64_t *bar, uint32_t bytes) {
+    asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)), "r"(bytes)
+                 : "memory");
+}
+
+__device__ __forceinline__ void mbar_wait(uint64_t *bar, uint32_t parity) {
+    uint32_t done = 0;
+    while (!done) {
+        asm volatile(
+            "{\n .reg .pred p;\n mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n selp.u32 %0, 1, 0, p;\n}\n"
+            : "=r"(done)
+            : "r"(smem_u32(bar)), "r"(parity)
+            : "memory");
+    }
+}
+
+// Global -> shared bulk copy by the Tensor Memory Accelerator (cp.async.bulk,
+// SASS UBLKCP); completion is counted in bytes on the mbarrier.  dst, src and
+// bytes must be multiples of 16.
+__device__ __forceinline__ void bulk_g2s(void *dst, const void *src, uint32_t bytes, uint64_t *bar) {
+    asm volatile(
+        "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
+            smem_u32(dst)),
+        "l"(src), "r"(bytes), "r"(smem_u32(bar))
+        : "memory");
+}
+
+// Load R consecutive rows (R * sizeof(T) = 16 * NCH bytes, NCH in {2, 4, 8})
+// per thread from shared memory into registers without bank conflicts.
+// Lanes l whose segments start 16*NCH bytes apart would collide on the same
+// 16-byte bank group; lane l reads chunk (q + rot) mod NCH in step q, rot
+// chosen so the 8 lanes of a quarter-warp hit 8 distinct groups, and a
+// log2(NCH)-stage barrel of predicated selects (FSEL, no branches) undoes it.
+template <typename T, int R>
+__device__ __forceinline__ void lds_rows(const T *seg, T *v, int lane) {
+    constexpr int E = 16 / sizeof(T);      // elements per 16-byte chunk
+    constexpr int NCH = R / E;             // chunks per thread
+    static_assert(NCH == 2 || NCH == 4 || NCH == 8, "lds_rows: 32, 64 or 128 bytes per thread");
+    const int rot = NCH == 8 ? (lane & 7) : NCH == 4 ? ((lane >> 1) & 3) : ((lane >> 2) & 1);
+    T arr[NCH][E];
+#pragma unroll
+    for (int q = 0; q < NCH; ++q) {
+        const int c = (q + rot) & (NCH - 1);
+        if constexpr (sizeof(T) == 4) {
+            const float4 f = reinterpret_cast<const float4 *>(seg)[c];
+            arr[q][0] = f.x;
+            arr[q][1] = f.y;
+            arr[q][2] = f.z;
+            arr[q][3] = f.w;
+        } else {
+            const double2 f = reinterpret_cast<const double2 *>(seg)[c];
+            arr[q][0] = f.x;
+            arr[q][1] = f.y;
+        }
+    }
+    // arr[q] holds chunk q + rot: rotate right by rot, one bit of rot per stage
+#pragma unroll
+    for (int b = 1; b < NCH; b <<= 1) {
+        const bool on = rot & b;
+        T nx[NCH][E];
+#pragma unroll
+        for (int q = 0; q < NCH; ++q)
+#pragma unroll
+            for (int e = 0; e < E; ++e) nx[q][e] = on ? arr[(q - b + NCH) & (NCH - 1)][e] : arr[q][e];
+#pragma unroll
+        for (int q = 0; q < NCH; ++q)
+#pragma unroll
+            for (int e = 0; e < E; ++e) arr[q][e] = nx[q][e];
+    }
+#pragma unroll
+    for (int q = 0; q < NCH; ++q)
+#pragma unroll
+        for (int e = 0; e < E; ++e) v[q * E + e] = arr[q][e];
+}
+
+}  // namespace tds

@@ -13,92 +13,9 @@
 //     de-interleaved store is a vector store per residue, coalesced across
 //     the warp (consecutive threads -> consecutive j).
 // Per row and level: one normalised row update (9 FMA-pipe ops + 1 MUFU.RCP).
-#include "common.cuh"
+#include "split_reg.cuh"
 
 namespace tds {
-
-template <typename T, int G>
-__device__ __forceinline__ void store_run(T *p, const T *v) {
-    if constexpr (G * sizeof(T) >= 16) {
-        constexpr int W = 16 / sizeof(T);
-#pragma unroll
-        for (int q = 0; q < G / W; ++q) {
-            if constexpr (sizeof(T) == 4)
-                reinterpret_cast<float4 *>(p)[q] = make_float4(v[4 * q], v[4 * q + 1], v[4 * q + 2], v[4 * q + 3]);
-            else
-                reinterpret_cast<double2 *>(p)[q] = make_double2(v[2 * q], v[2 * q + 1]);
-        }
-    } else if constexpr (G * sizeof(T) == 8 && sizeof(T) == 4) {
-        reinterpret_cast<float2 *>(p)[0] = make_float2(v[0], v[1]);
-    } else {
-#pragma unroll
-        for (int u = 0; u < G; ++u) p[u] = v[u];
-    }
-}
-
-// One PCR level with compile-time stride S on 16 register rows per thread.
-// A level couples only rows of one class rho (mod S): each class is updated in
-// place, ascending, carrying the previous OLD row, so only a few registers
-// beyond the 48 row values stay live.  eL/eR: [2][3][NW][SM] edge buffers.
-template <typename T, int R, int S, int NW, int SM>
-__device__ __forceinline__ void reg_level(T (&ra)[R], T (&rc)[R], T (&rd)[R], T *eL, T *eR, int bsel, int lane,
-                                          int warp) {
-    auto E = [&](T *e, int arr, int w, int u) -> T & { return e[((bsel * 3 + arr) * NW + w) * SM + u]; };
-    if (lane == 0) {
-#pragma unroll
-        for (int u = 0; u < S; ++u) {
-            E(eL, 0, warp, u) = ra[u];
-            E(eL, 1, warp, u) = rc[u];
-            E(eL, 2, warp, u) = rd[u];
-        }
-    }
-    if (lane == 31) {
-#pragma unroll
-        for (int u = 0; u < S; ++u) {
-            E(eR, 0, warp, u) = ra[R - S + u];
-            E(eR, 1, warp, u) = rc[R - S + u];
-            E(eR, 2, warp, u) = rd[R - S + u];
-        }
-    }
-    __syncthreads();
-#pragma unroll
-    for (int rho = 0; rho < S; ++rho) {
-        // left neighbour of row rho: row R-S+rho of thread t-1 (old; same class)
-        T pa = __shfl_up_sync(0xffffffffu, ra[R - S + rho], 1);
-        T pc = __shfl_up_sync(0xffffffffu, rc[R - S + rho], 1);
-        T pd = __shfl_up_sync(0xffffffffu, rd[R - S + rho], 1);
-        // right neighbour of row R-S+rho: row rho of thread t+1 (old)
-        T xa = __shfl_down_sync(0xffffffffu, ra[rho], 1);
-        T xc = __shfl_down_sync(0xffffffffu, rc[rho], 1);
-        T xd = __shfl_down_sync(0xffffffffu, rd[rho], 1);
-        if (lane == 0) {
-            const bool h = warp > 0;
-            const int w = h ? warp - 1 : 0;
-            pa = h ? E(eR, 0, w, rho) : T(0);
-            pc = h ? E(eR, 1, w, rho) : T(0);
-            pd = h ? E(eR, 2, w, rho) : T(0);
-        }
-        if (lane == 31) {
-            const bool h = warp < NW - 1;
-            const int w = h ? warp + 1 : 0;
-            xa = h ? E(eL, 0, w, rho) : T(0);
-            xc = h ? E(eL, 1, w, rho) : T(0);
-            xd = h ? E(eL, 2, w, rho) : T(0);
-        }
-#pragma unroll
-        for (int v = rho; v < R; v += S) {
-            const T oa = ra[v], oc = rc[v], od = rd[v];
-            if constexpr (true) {
-                const bool last = v + S >= R;
-                row_update(ra[v], rc[v], rd[v], pa, pc, pd, last ? xa : ra[(v + S) % R], last ? xc : rc[(v + S) % R],
-                           last ? xd : rd[(v + S) % R]);
-            }
-            pa = oa;
-            pc = oc;
-            pd = od;
-        }
-    }
-}
 
 template <typename T, int KP, bool RAW>
 __global__ void __launch_bounds__(kRegSplitThreads, 2) split_reg_kernel(const SplitArgs<T> A) {
