@@ -170,18 +170,18 @@ static void schedule_passes(tds_params &p, int kpmax) {
     for (int i = 0; i < p.passes; ++i) p.k_pass[i] = p.k / p.passes + (i < p.k % p.passes ? 1 : 0);
 }
 
-// Make (c, C, T) valid for a new k: grow c, then the cluster, until a CTA fits.
+// Make (c, C, T) valid for a new k: the smallest cluster (clusters cost barrier
+// latency) and the most rows per thread that fit the on-chip kernel.
 static void fit_onchip(const tds_plan_info &I, const tds_device_props &props, tds_params &p) {
     const int64_t n_sub = cdiv(I.n, int64_t(1) << p.k);
     auto cap = [](int c) { return (1 << c) >= 8 ? kMaxOnchipThreadsWide : kMaxOnchipThreads; };
     auto thr = [&](const tds_params &q) {
         return round_up(cdiv(n_sub, (int64_t(1) << q.cr_levels) * q.cluster), 32);
     };
-    while (thr(p) > cap(p.cr_levels)) {
-        if ((1 << (p.cr_levels + 1)) <= r_max(I.dtype)) ++p.cr_levels;
-        else if (p.cluster < 16 && props.cc_major >= 9) p.cluster *= 2;
-        else break;
-    }
+    p.cluster = 1;
+    p.cr_levels = ilog2i(r_max(I.dtype));
+    while (thr(p) > cap(p.cr_levels) && p.cluster < 16 && props.cc_major >= 9) p.cluster *= 2;
+    p.tl_levels = ilog2i(p.cluster);
     clamp_onchip(I, p);
 }
 
@@ -288,24 +288,40 @@ extern "C" tds_status tds_tune(tds_plan_t plan, void *cuda_stream, const char *c
     } else {
         // (1) stage 3->4 switch at the seed's subsystem size
         tune_onchip(C, best, t_best);
-        // (2) stage 2->3 switch: 2x the systems at half the size (k+1), or the reverse
+        // (2) stage 2->3 switch: 2x the systems at half the size (k+1), or the
+        // reverse.  For each k both pass schedules are tried -- register split
+        // passes (k_p <= 4) and the seed's k_p limit -- with the smallest
+        // cluster that holds the subsystem; the walk tolerates two
+        // non-improving steps (splitting and on-chip costs trade off unevenly).
         for (int dir : {+1, -1}) {
-            bool moved = true;
-            while (moved && !out_of_time(C)) {
-                moved = false;
-                tds_params cand = best;
-                cand.k += dir;
-                if (cand.k < 0 || cand.k > 30 || (int64_t(1) << cand.k) > 2 * I.n) break;
-                const int kpmax = std::max(I.split_kp_max, 1);
-                schedule_passes(cand, kpmax);
-                fit_onchip(I, plan->props, cand);
-                double t = trial(C, cand);
-                if (t >= 1e29) break;
-                tune_onchip(C, cand, t);
-                if (better(t, t_best)) {
-                    best = cand;
-                    t_best = t;
-                    moved = true;
+            tds_params walk = best;
+            int misses = 0;
+            while (misses < 3 && !out_of_time(C)) {
+                tds_params base = walk;
+                base.k += dir;
+                if (base.k < 0 || base.k > 30 || (int64_t(1) << base.k) > 2 * I.n) break;
+                double t_step = 1e30;
+                tds_params step_best = base;
+                for (int kpmax : {std::min(kRegSplitMaxKp, std::max(I.split_kp_max, 1)), std::max(I.split_kp_max, 1)}) {
+                    tds_params cand = base;
+                    schedule_passes(cand, kpmax);
+                    fit_onchip(I, plan->props, cand);
+                    double t = trial(C, cand);
+                    if (t >= 1e29) continue;
+                    tune_onchip(C, cand, t);
+                    if (t < t_step) {
+                        t_step = t;
+                        step_best = cand;
+                    }
+                }
+                if (t_step >= 1e29) break;
+                walk = step_best;
+                if (better(t_step, t_best)) {
+                    best = step_best;
+                    t_best = t_step;
+                    misses = 0;
+                } else {
+                    ++misses;
                 }
             }
         }
@@ -331,6 +347,15 @@ extern "C" tds_status tds_tune(tds_plan_t plan, void *cuda_stream, const char *c
                     // one more (shallower) pass: less halo per pass, one more HBM round trip
                     q = best;
                     schedule_passes(q, std::max(1, (best.k + best.passes) / (best.passes + 1)));
+                    cands.push_back(q);
+                }
+                if (best.passes > 1) {
+                    // one fewer (deeper) pass, and the same levels in reverse order
+                    q = best;
+                    schedule_passes(q, (best.k + best.passes - 2) / (best.passes - 1));
+                    if (q.passes < best.passes) cands.push_back(q);
+                    q = best;
+                    std::reverse(q.k_pass, q.k_pass + q.passes);
                     cands.push_back(q);
                 }
                 for (auto &cnd : cands) {
