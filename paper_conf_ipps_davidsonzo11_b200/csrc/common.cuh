@@ -38,27 +38,17 @@ __device__ __forceinline__ void row_update(T &a, T &c, T &d, T al, T cl, T dl, T
     d = nd;
 }
 
-// Original residue (mod 2^K) of workspace slot index rho after `npass`
-// passes: each pass appends its residue digit as the LOW digit of the slot
-// index, while in the original row numbering that digit has weight
-// 2^(levels of the earlier passes).
-// (Fixed-trip unrolled loops keep the kernel-parameter array in the constant
-// bank instead of copying it to local memory for dynamic indexing.)
-__device__ __forceinline__ int64_t slot_residue(int64_t rho, int npass, const int32_t *kpass) {
-    int kcum = 0;
-#pragma unroll
-    for (int p = 0; p < TDS_MAX_PASSES; ++p)
-        if (p < npass) kcum += kpass[p];
-    int64_t r = 0;
-#pragma unroll
-    for (int p = TDS_MAX_PASSES - 1; p >= 0; --p) {
-        if (p < npass) {
-            kcum -= kpass[p];
-            r += (rho & ((int64_t(1) << kpass[p]) - 1)) << kcum;
-            rho >>= kpass[p];
-        }
-    }
-    return r;
+// Workspace slots are kept in CANONICAL residue order: after K cumulative
+// levels, slot (s << K) + r holds the residue-r subsystem of system s.  Each
+// pass writes the new residue digit rho of input slot sigma (levels kprev
+// before it, kp in it) to residue r + (rho << kprev).
+__device__ __forceinline__ int64_t slot_residue(int64_t rho, int /*npass*/, const int32_t * /*kpass*/) {
+    return rho;
+}
+
+__device__ __forceinline__ int64_t out_slot_index(int64_t sigma, int kprev, int kp, int64_t rho) {
+    const int64_t sys = sigma >> kprev, r = sigma & ((int64_t(1) << kprev) - 1);
+    return (sys << (kprev + kp)) + r + (rho << kprev);
 }
 
 __device__ __forceinline__ int pass_levels(int npass, const int32_t *kpass) {

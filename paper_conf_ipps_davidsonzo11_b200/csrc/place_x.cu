@@ -27,38 +27,13 @@ struct PlaceArgs {
 constexpr int kPlaceRows = 16;
 constexpr int kPlaceThreads = 256;
 
-// Physical slot (within its system) of residue r: the residue's digits in pass
-// order, the first pass's digit most significant.
-__device__ __forceinline__ int64_t residue_slot(int64_t r, const PassGeom &g) {
-    if (g.npass == 1) return r;
-    int64_t sl = 0;
-    int kc = 0;
-#pragma unroll
-    for (int p = 0; p < TDS_MAX_PASSES; ++p) {
-        if (p < g.npass) {
-            const int kp = g.kpass[p];
-            sl = (sl << kp) | ((r >> kc) & ((int64_t(1) << kp) - 1));
-            kc += kp;
-        }
-    }
-    return sl;
-}
-
-constexpr int kPlaceTable = 4096;  // residue -> slot table in shared memory (2^K <= 4096)
-
 template <typename T, int KK>  // KK = min(K, 4)
 __global__ void __launch_bounds__(kPlaceThreads) place_x_kernel(const PlaceArgs<T> A) {
     constexpr int R = kPlaceRows;
     constexpr int NRK = 1 << KK;  // residues among 16 consecutive rows
     constexpr int G = R >> KK;    // rows per residue per thread
     constexpr int W = 16 / int(sizeof(T));
-    __shared__ int32_t slot_of[kPlaceTable];
     const int64_t NR = int64_t(1) << A.K;
-    const bool table = A.geom.npass > 1 && NR <= kPlaceTable;
-    if (table) {  // multi-pass digit reversal once per block, not once per element
-        for (int r = threadIdx.x; r < NR; r += blockDim.x) slot_of[r] = (int32_t)residue_slot(r, A.geom);
-        __syncthreads();
-    }
     const int64_t tiles = (A.n + R * kPlaceThreads - 1) / (R * kPlaceThreads);
     const int64_t sys = blockIdx.x / tiles;
     const int64_t i0 = ((blockIdx.x % tiles) * kPlaceThreads + threadIdx.x) * R;
@@ -70,8 +45,7 @@ __global__ void __launch_bounds__(kPlaceThreads) place_x_kernel(const PlaceArgs<
     for (int rho = 0; rho < NRK; ++rho) {
         const int64_t row = i0 + rho;           // first of this residue's G rows
         const int64_t r = row & (NR - 1), j = row >> A.K;
-        const int64_t sl = table ? int64_t(slot_of[r]) : residue_slot(r, A.geom);
-        const T *src = A.xs + (sys_slots + sl) * A.slot + j;
+        const T *src = A.xs + (sys_slots + r) * A.slot + j;  // slots are in canonical residue order
         constexpr bool kVec = (G * sizeof(T) >= 16) || (sizeof(T) == 4 && G == 2);
         if (kVec && full) {
             if constexpr (G * sizeof(T) >= 16) {

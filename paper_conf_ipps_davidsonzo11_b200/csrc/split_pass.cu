@@ -37,10 +37,10 @@ __global__ void __launch_bounds__(512) split_pass_kernel(const SplitArgs<T> A) {
     const int64_t sigma = int64_t(blockIdx.x) / A.segs;
     const int g = int(int64_t(blockIdx.x) % A.segs);
     int64_t L;
+    const int kprev = RAW ? 0 : pass_levels(A.geom.npass, A.geom.kpass);
     if (RAW) {
         L = A.n;
     } else {
-        const int kprev = pass_levels(A.geom.npass, A.geom.kpass);
         const int64_t rho = sigma & ((int64_t(1) << kprev) - 1);
         const int64_t r = slot_residue(rho, A.geom.npass, A.geom.kpass);
         L = r < A.n ? (A.n - r + (int64_t(1) << kprev) - 1) >> kprev : 0;
@@ -117,7 +117,7 @@ __global__ void __launch_bounds__(512) split_pass_kernel(const SplitArgs<T> A) {
             if (q < valid) {
                 const int e = H + q;
                 const int pe = e + (e >> ps);
-                const int64_t oidx = ((sigma << kp) + rr) * A.out_slot + (t0 >> kp) + jj;
+                const int64_t oidx = out_slot_index(sigma, kprev, kp, rr) * A.out_slot + (t0 >> kp) + jj;
                 A.oa[oidx] = sa[pe];
                 A.oc[oidx] = sc[pe];
                 A.od[oidx] = sd[pe];

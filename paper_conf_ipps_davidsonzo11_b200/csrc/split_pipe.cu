@@ -122,7 +122,7 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_pipe_kernel(const S
             const bool full = i0 + R <= L;
 #pragma unroll
             for (int rho = 0; rho < NR; ++rho) {
-                const int64_t o = ((sigma << KP) + rho) * A.out_slot + jb;
+                const int64_t o = out_slot_index(sigma, kprev, KP, rho) * A.out_slot + jb;
                 T va[G], vc[G], vd[G];
 #pragma unroll
                 for (int u = 0; u < G; ++u) {

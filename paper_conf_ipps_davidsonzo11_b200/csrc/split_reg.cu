@@ -34,10 +34,10 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_reg_kernel(const Sp
     const int64_t sigma = int64_t(blockIdx.x) / A.segs;
     const int g = int(int64_t(blockIdx.x) % A.segs);
     int64_t L;
+    const int kprev = RAW ? 0 : pass_levels(A.geom.npass, A.geom.kpass);
     if (RAW) {
         L = A.n;
     } else {
-        const int kprev = pass_levels(A.geom.npass, A.geom.kpass);
         const int64_t rho = sigma & ((int64_t(1) << kprev) - 1);
         const int64_t r = slot_residue(rho, A.geom.npass, A.geom.kpass);
         L = r < A.n ? (A.n - r + (int64_t(1) << kprev) - 1) >> kprev : 0;
@@ -125,7 +125,7 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_reg_kernel(const Sp
             const bool full = i0 + R <= L;
 #pragma unroll
             for (int rho = 0; rho < NR; ++rho) {
-                const int64_t o = ((sigma << KP) + rho) * A.out_slot + jb;
+                const int64_t o = out_slot_index(sigma, kprev, KP, rho) * A.out_slot + jb;
                 T va[G], vc[G], vd[G];
 #pragma unroll
                 for (int u = 0; u < G; ++u) {

@@ -1,2 +1,2 @@
-python bench.py --steps 30 --warmup 3 --no-cpu-baseline --no-e2e 2>&1 | tail -1 | python -c "
-import json,sys; d=json.loads(sys.stdin.read()); print(d['value'], d['ms_per_step'], d['config']['plan'], d['config']['tune_trials'], d['config']['tune_s']); print(json.dumps(d['roofline']['per_kernel']))"
+timeout 1200 python -m pytest tests -m gpu -x -q -p no:cacheprovider 2>&1 | tail -3
+python scripts/sweep.py --n 1048576 --m 16 --points '[{"k_pass": [4,3], "cluster": 1, "tl_levels": 0, "cr_levels": 4, "thomas_chains": 64}, {"k_pass": [3,4], "cluster": 1, "tl_levels": 0, "cr_levels": 4, "thomas_chains": 64}]' 2>&1 | cut -c260-480
