@@ -102,6 +102,8 @@ typedef struct {
     int32_t split_threads;           /* shared-memory split pass CTA size (k_pass > 4)  */
     int32_t theta;                   /* stage 1->2 switch: independent systems needed   */
     int32_t chunk_systems;           /* systems per L2-resident chunk (0 = all at once) */
+    int32_t split_only;              /* 1: plan only the split passes (tds_split_batched;
+                                        on-chip limits not checked, tds_solve_* refuse) */
 } tds_params;
 
 /* Everything a plan decided (read-only view). */

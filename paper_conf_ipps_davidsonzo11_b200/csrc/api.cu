@@ -321,6 +321,7 @@ tds_status tds_solve_stages(const tds_plan_t plan, const void *a, const void *b,
                             int32_t first_stage, int32_t last_stage) {
     if (!plan) return fail(TDS_ERR_INVALID_ARG, "plan is NULL");
     const tds_plan_info &I = plan->info;
+    if (I.params.split_only) return fail(TDS_ERR_UNSUPPORTED, "split-only plan: use tds_split_batched");
     if (first_stage < 0 || last_stage >= I.launches || first_stage > last_stage)
         return fail(TDS_ERR_INVALID_ARG, "launch range outside [0, info.launches)");
     tds_status s = check_arrays(I, {a, b, c, d, x});

@@ -133,19 +133,24 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
     const int R = 1 << p.cr_levels;
     if (p.cluster > 1 && (props.cc_major < 9 || R < 8))
         return fail(TDS_ERR_UNSUPPORTED, "clusters need compute capability >= 9.0 and 2^cr_levels >= 8");
+    if (p.split_only != 0 && p.split_only != 1) return fail(TDS_ERR_INVALID_ARG, "split_only must be 0 or 1");
+    if (p.split_only && p.k == 0) return fail(TDS_ERR_INVALID_ARG, "a split-only plan needs k >= 1");
     const int64_t n_sub = cdiv(n, int64_t(1) << std::min(p.k, 62));
     const int64_t nred = cdiv(n_sub, int64_t(R) * p.cluster);
-    const int64_t threads = std::max<int64_t>(32, round_up(nred, 32));
-    if (threads > (R >= 8 ? kMaxOnchipThreadsWide : kMaxOnchipThreads))
-        return fail(TDS_ERR_UNSUPPORTED, "subsystem too large for the on-chip kernel (n_sub / (2^c cluster) > 1024, "
-                                         "or > 512 when 2^c >= 8)");
-    if (p.tl_levels < 0 || p.tl_levels > 10 || threads % (int64_t(1) << p.tl_levels))
-        return fail(TDS_ERR_INVALID_ARG, "tl_levels must be in [0, 10] and 2^tl_levels must divide the CTA size");
-    if (p.thomas_chains > (threads >> p.tl_levels) * p.cluster)
-        return fail(TDS_ERR_INVALID_ARG, "thomas_chains > leader's reduced system (cluster x threads / 2^tl_levels)");
-    if ((int64_t)onchip_smem_bytes(dtype, (int32_t)threads, p.cluster, p.tl_levels) >
-        int64_t(props.smem_optin_bytes) - kSmemReserve)
-        return fail(TDS_ERR_UNSUPPORTED, "on-chip shared memory exceeds the device limit");
+    const int64_t threads = p.split_only ? 32 : std::max<int64_t>(32, round_up(nred, 32));
+    if (!p.split_only) {  // the on-chip stage must fit (a split-only plan never launches it)
+        if (threads > (R >= 8 ? kMaxOnchipThreadsWide : kMaxOnchipThreads))
+            return fail(TDS_ERR_UNSUPPORTED, "subsystem too large for the on-chip kernel (n_sub / (2^c cluster) > "
+                                             "1024, or > 512 when 2^c >= 8)");
+        if (p.tl_levels < 0 || p.tl_levels > 10 || threads % (int64_t(1) << p.tl_levels))
+            return fail(TDS_ERR_INVALID_ARG, "tl_levels must be in [0, 10] and 2^tl_levels must divide the CTA size");
+        if (p.thomas_chains > (threads >> p.tl_levels) * p.cluster)
+            return fail(TDS_ERR_INVALID_ARG,
+                        "thomas_chains > leader's reduced system (cluster x threads / 2^tl_levels)");
+        if ((int64_t)onchip_smem_bytes(dtype, (int32_t)threads, p.cluster, p.tl_levels) >
+            int64_t(props.smem_optin_bytes) - kSmemReserve)
+            return fail(TDS_ERR_UNSUPPORTED, "on-chip shared memory exceeds the device limit");
+    }
     if (p.passes > 0) {
         if (!is_pow2(p.split_tile_rows) || p.split_tile_rows < 32 || p.split_tile_rows > (1 << 15))
             return fail(TDS_ERR_INVALID_ARG, "split_tile_rows must be a power of two in [32, 32768]");
