@@ -120,7 +120,7 @@ static tds_status run_split(const tds_plan_info &I, const T *a, const T *b, cons
         const int64_t grid = m_in * A.segs;
         if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "split grid exceeds 2^31-1 CTAs");
         cudaError_t err;
-        if (kp <= kRegSplitMaxKp && A.vec) {
+        if (kp <= kPipeSplitMaxKp && A.vec) {
             // persistent, TMA-prefetched register kernel (16-byte aligned rows)
             err = launch_split_pipe<T>(A, raw, m_in, len_in, st);
         } else if (kp <= kRegSplitMaxKp) {

@@ -21,7 +21,131 @@ namespace tds {
 template <typename T, int ZR>
 __device__ __forceinline__ void reduced_solve_pipe(T *z, int Z, int NT, int t, int log2T);
 
+// Warp-level on-chip solve of one subsystem held as R rows per thread (x
+// returned in rd).  c = log2(R) CR levels in registers, 5 CR levels across
+// the lanes of each warp (shuffles), then the one remaining row per warp is
+// solved by warp 0 with shuffle PCR, and everything is back-substituted.  The
+// only row of a warp that reaches into the next warp is lane 31's: its chains
+// are deferred until one barrier publishes the next warp's rows (lane 0's
+// row s-1 per register level, lane s-1's row per lane level; both depend on
+// nothing beyond their own warp).  5 barriers per subsystem in total.
 template <typename T, int R>
+__device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[R], T *scr, int lane, int warp,
+                                                int nwarps) {
+    constexpr int CR = ilog2c(R);
+    constexpr unsigned FULL = 0xffffffffu;
+    T *e_in = scr;                      // [nwarps][CR][3] lane 0's row s-1, level l-1
+    T *w_in = e_in + nwarps * CR * 3;   // [nwarps][5][3]  lane s-1 at lane level l-1
+    T *lft = w_in + nwarps * 15;        // [nwarps][5][3]  lane 31-s at lane level l-1
+    T *top = lft + nwarps * 15;         // [3][32]
+    T *xtop = top + 96;                 // [32]
+    // register CR levels; lane 31 defers its row R-1 chain
+#pragma unroll
+    for (int l = 1; l <= CR; ++l) {
+        const int s = 1 << (l - 1);
+        const T pa = ra[s - 1], pc = rc[s - 1], pd = rd[s - 1];
+        const T na = __shfl_down_sync(FULL, pa, 1), nc = __shfl_down_sync(FULL, pc, 1),
+                nd = __shfl_down_sync(FULL, pd, 1);
+        if (lane == 0) {
+            T *e = e_in + (warp * CR + l - 1) * 3;
+            e[0] = pa;
+            e[1] = pc;
+            e[2] = pd;
+        }
+#pragma unroll
+        for (int v = (1 << l) - 1; v < R; v += (1 << l)) {
+            const bool last = v == R - 1;
+            if (!(last && lane == 31))
+                row_update(ra[v], rc[v], rd[v], ra[v - s], rc[v - s], rd[v - s], last ? na : ra[(v + s) % R],
+                           last ? nc : rc[(v + s) % R], last ? nd : rd[(v + s) % R]);
+        }
+    }
+    // CR across lanes; lane 31 (kept at every level) defers
+    T za = ra[R - 1], zc = rc[R - 1], zd = rd[R - 1];
+#pragma unroll
+    for (int l = 1; l <= 5; ++l) {
+        const int s = 1 << (l - 1);
+        const T la = __shfl_up_sync(FULL, za, s), lc = __shfl_up_sync(FULL, zc, s), ld = __shfl_up_sync(FULL, zd, s);
+        const T xa = __shfl_down_sync(FULL, za, s), xc = __shfl_down_sync(FULL, zc, s),
+                xd = __shfl_down_sync(FULL, zd, s);
+        if (lane == s - 1) {
+            T *w = w_in + (warp * 5 + l - 1) * 3;
+            w[0] = za;
+            w[1] = zc;
+            w[2] = zd;
+        }
+        if (lane == 31 - s) {
+            T *f = lft + (warp * 5 + l - 1) * 3;
+            f[0] = za;
+            f[1] = zc;
+            f[2] = zd;
+        }
+        if ((lane & ((1 << l) - 1)) == (1 << l) - 1 && lane != 31) row_update(za, zc, zd, la, lc, ld, xa, xc, xd);
+    }
+    __syncthreads();
+    if (lane == 31) {  // the deferred chains, with the next warp's published rows
+        const bool h = warp + 1 < nwarps;
+#pragma unroll
+        for (int l = 1; l <= CR; ++l) {
+            const int s = 1 << (l - 1);
+            const T *e = e_in + ((warp + 1) * CR + l - 1) * 3;
+            row_update(ra[R - 1], rc[R - 1], rd[R - 1], ra[R - 1 - s], rc[R - 1 - s], rd[R - 1 - s],
+                       h ? e[0] : T(0), h ? e[1] : T(0), h ? e[2] : T(0));
+        }
+        za = ra[R - 1];
+        zc = rc[R - 1];
+        zd = rd[R - 1];
+#pragma unroll
+        for (int l = 1; l <= 5; ++l) {
+            const T *f = lft + (warp * 5 + l - 1) * 3;
+            const T *w = w_in + ((warp + 1) * 5 + l - 1) * 3;
+            row_update(za, zc, zd, f[0], f[1], f[2], h ? w[0] : T(0), h ? w[1] : T(0), h ? w[2] : T(0));
+        }
+        top[warp] = za;
+        top[32 + warp] = zc;
+        top[64 + warp] = zd;
+    }
+    __syncthreads();
+    if (warp == 0) {  // one row per warp: pure PCR with shuffles (every row decouples, x = d)
+        T a = lane < nwarps ? top[lane] : T(0), c = lane < nwarps ? top[32 + lane] : T(0),
+          d = lane < nwarps ? top[64 + lane] : T(0);
+        for (int s = 1; s < nwarps; s <<= 1) {
+            const T la = __shfl_up_sync(FULL, a, s), lc = __shfl_up_sync(FULL, c, s), ld = __shfl_up_sync(FULL, d, s);
+            const T xa = __shfl_down_sync(FULL, a, s), xc = __shfl_down_sync(FULL, c, s),
+                    xd = __shfl_down_sync(FULL, d, s);
+            const bool hl = lane >= s, hr = lane + s < nwarps;
+            if (lane < nwarps)
+                row_update(a, c, d, hl ? la : T(0), hl ? lc : T(0), hl ? ld : T(0), hr ? xa : T(0), hr ? xc : T(0),
+                           hr ? xd : T(0));
+        }
+        if (lane < nwarps) xtop[lane] = d;
+    }
+    __syncthreads();
+    // back substitution across lanes, then in registers
+    T xw = lane == 31 ? xtop[warp] : T(0);
+    const T xprev = warp > 0 ? xtop[warp - 1] : T(0);  // row -1 of this warp: previous warp's lane 31
+#pragma unroll
+    for (int l = 5; l >= 1; --l) {
+        const int s = 1 << (l - 1);
+        const T xl = __shfl_up_sync(FULL, xw, s);
+        const T xr = __shfl_down_sync(FULL, xw, s);
+        if ((lane & ((1 << l) - 1)) == s - 1) xw = zd - za * (lane >= s ? xl : xprev) - zc * xr;
+    }
+    T xleft = __shfl_up_sync(FULL, xw, 1);
+    if (lane == 0) xleft = xprev;
+    rd[R - 1] = xw;
+#pragma unroll
+    for (int l = CR; l >= 1; --l) {
+        const int s = 1 << (l - 1);
+#pragma unroll
+        for (int v = s - 1; v < R - 1; v += 2 * s) {
+            const T xlv = (v >= s) ? rd[(v - s + R) % R] : xleft;
+            rd[v] = rd[v] - ra[v] * xlv - rc[v] * rd[(v + s) % R];
+        }
+    }
+}
+
+template <typename T, int R, bool WL>
 __global__ void __launch_bounds__(512, 1) onchip_pipe_kernel(const OnchipArgs<T> A, int64_t nslots) {
     static_assert(R * sizeof(T) == 64, "pipe kernel: 64 bytes of rows per thread");
     extern __shared__ __align__(128) unsigned char smem_raw[];
@@ -91,6 +215,9 @@ __global__ void __launch_bounds__(512, 1) onchip_pipe_kernel(const OnchipArgs<T>
         if (t == 0) issue(sigma + 2 * int64_t(gridDim.x), s);
         if (L == 0) continue;  // empty slot (2^K > n): uniform
 
+        if constexpr (WL) {
+            solve_item_warp<T, R>(ra, rc, rd, ya, lane, warp, nwarps);
+        } else {
         // ---- B1. CR forward levels in registers
 #pragma unroll
         for (int l = 1; l <= CR; ++l) {
@@ -169,6 +296,7 @@ __global__ void __launch_bounds__(512, 1) onchip_pipe_kernel(const OnchipArgs<T>
                 rd[v] = rd[v] - ra[v] * xlv - rc[v] * rd[(v + sl) % R];
             }
         }
+        }  // !WL
         T *dst = A.xs + sigma * A.slot + jt;  // per-subsystem x (placement kernel follows)
         if (jt + R <= L) {
             constexpr int W = 16 / int(sizeof(T));
@@ -252,10 +380,14 @@ size_t onchip_pipe_smem_bytes(int32_t dtype, int32_t threads, int32_t R, int32_t
 template <typename T>
 cudaError_t launch_onchip_pipe(const OnchipArgs<T> &A, int64_t nslots, int threads, int sm_count, size_t smem,
                                cudaStream_t st) {
-    auto kern = onchip_pipe_kernel<T, 64 / int(sizeof(T))>;
+    // tl_levels == 5 (CR across all 32 lanes) selects the warp-level shuffle path
+    auto kern = A.tl_levels == 5 ? onchip_pipe_kernel<T, 64 / int(sizeof(T)), true>
+                                 : onchip_pipe_kernel<T, 64 / int(sizeof(T)), false>;
     cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     if (e != cudaSuccess) return e;
-    const int64_t grid = std::min<int64_t>(nslots, sm_count);
+    int occ = 1;  // smaller subsystems fit two or more persistent CTAs per SM
+    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, threads, smem);
+    const int64_t grid = std::min<int64_t>(nslots, int64_t(std::max(occ, 1)) * sm_count);
     kern<<<(unsigned)grid, threads, smem, st>>>(A, nslots);
     return cudaGetLastError();
 }

@@ -1,36 +1,51 @@
-// split_pipe.cu -- G1, persistent TMA-prefetched form of the register split
-// kernel (k_p <= 4 fused PCR levels per HBM pass; §III-B/C).
+// split_pipe.cu -- G1, persistent TMA-prefetched register split kernel:
+// k_p <= 7 fused PCR levels per HBM pass (§III-B/C, P:L296-303,
+// P:L472-493), output de-interleaved into canonical residue slots.
 //
-// Work items are tiles (slot sigma, tile ti) of 16*(NT-2) output rows; a
-// resident CTA walks items w = blockIdx.x, += gridDim.x.  Each CTA owns ONE
-// shared-memory stage holding the next tile's input rows (4 raw arrays on the
-// first pass, 3 normalised ones after): as soon as every thread has copied the
-// current tile into registers the stage is refilled with cp.async.bulk (the
-// Tensor Memory Accelerator) while the CTA runs the PCR levels and the
-// de-interleaved stores -- HBM reads of tile i+1 overlap compute on tile i.
-// Levels and stores are those of split_reg.cu (reg_level / store_run), so the
-// output is bit-identical.
+// Work items are tiles (slot sigma, tile ti); a resident CTA walks items
+// w = blockIdx.x, += gridDim.x.  Thread t of the 256-thread CTA owns 16
+// consecutive rows in registers.  Levels with stride <= 8 rows exchange only
+// the first / last s rows with the neighbour threads (reg_level); levels with
+// stride 16, 32, 64 rows (k_p = 5..7) exchange whole 16-row blocks with the
+// threads 1, 2, 4 away (reg_level_far).  The first and last HT threads of a
+// CTA are the tile's halo (16*HT >= 2^k_p - 1 rows per side).
+//
+// Each CTA owns ONE shared-memory stage holding the next tile's input rows (4
+// raw arrays on the first pass, 3 normalised ones after): as soon as every
+// thread has copied the current tile into registers (conflict-free rotated
+// LDS.128) the stage is refilled by cp.async.bulk (TMA) while the CTA runs
+// the PCR levels and the de-interleaved stores.
 #include "pipe.cuh"
 #include "split_reg.cuh"
 
 namespace tds {
 
+template <int KP>
+struct SplitShape {
+    static constexpr int R = kRegSplitRows;
+    static constexpr int NT = kRegSplitThreads;
+    static constexpr int NW = NT / 32;
+    static constexpr int HT = KP <= 4 ? 1 : (1 << (KP - 4));  // halo threads per side
+    static constexpr int TV = (NT - 2 * HT) * R;               // valid rows per tile
+    static constexpr int SMN = (1 << (KP - 1)) < 8 ? (1 << (KP - 1)) : 8;
+    static constexpr int FAR = NW * kFarMaxTS * 3 * R;        // one half of a far-level edge buffer
+};
+
 template <typename T, int KP, bool RAW>
 __global__ void __launch_bounds__(kRegSplitThreads, 2) split_pipe_kernel(const SplitArgs<T> A, int64_t tps,
                                                                        int64_t nitems) {
-    constexpr int R = kRegSplitRows;
-    constexpr int NT = kRegSplitThreads;
-    constexpr int NW = NT / 32;
-    constexpr int SM = 1 << (KP - 1);
+    using S = SplitShape<KP>;
+    constexpr int R = S::R, NT = S::NT, NW = S::NW, HT = S::HT, TV = S::TV, SMN = S::SMN;
     constexpr int NR = 1 << KP;
-    constexpr int G = R >> KP;
-    constexpr int NA = RAW ? 4 : 3;         // arrays streamed
-    constexpr int ROWS = NT * R;            // rows per stage (tile + halo threads)
-    constexpr int TV = ROWS - 2 * R;        // valid rows per tile
+    constexpr int G = KP <= 4 ? (R >> KP) : 1;
+    constexpr int NA = RAW ? 4 : 3;  // arrays streamed
+    constexpr int ROWS = NT * R;     // rows per stage (tile + halo threads)
     extern __shared__ __align__(128) unsigned char smem_raw[];
     T *stage = reinterpret_cast<T *>(smem_raw);  // [NA][ROWS]
-    __shared__ T eL[2][3][NW][SM];
-    __shared__ T eR[2][3][NW][SM];
+    T *eF = stage + NA * ROWS;                   // far levels: [2][FAR] first-lane blocks
+    T *eB = eF + 2 * S::FAR;                     //             [2][FAR] last-lane blocks
+    __shared__ T eL[2][3][NW][SMN];
+    __shared__ T eR[2][3][NW][SMN];
     __shared__ __align__(8) uint64_t bar;
     const int t = threadIdx.x, lane = t & 31, warp = t >> 5;
     const int kprev = RAW ? 0 : pass_levels(A.geom.npass, A.geom.kpass);
@@ -41,16 +56,16 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_pipe_kernel(const S
         return r < A.n ? (A.n - r + (int64_t(1) << kprev) - 1) >> kprev : 0;
     };
     const T *src_arr[4] = {A.a, A.c, A.d, A.b};  // RAW also streams b
-    // rows [g0, g0 + nb) of the item go to the stage by TMA (16-byte granules)
+    // rows [g0, gt) of the item go to the stage by TMA (16-byte granules); [gt, g1) by LDG
     auto item_rows = [&](int64_t w, int64_t &sigma, int64_t &t0, int64_t &L, int64_t &g0, int64_t &g1,
                          int64_t &gt) {
         sigma = w / tps;
         t0 = (w % tps) * TV;
         L = slot_len(sigma);
-        g0 = t0 - R < 0 ? 0 : t0 - R;
-        g1 = t0 + TV + R < L ? t0 + TV + R : L;
-        gt = g0 + (((g1 - g0) * int64_t(sizeof(T))) & ~int64_t(15)) / int64_t(sizeof(T));  // TMA part end
-        if (g1 < g0) g1 = gt = g0;
+        g0 = t0 - HT * R < 0 ? 0 : t0 - HT * R;
+        g1 = t0 + TV + HT * R < L ? t0 + TV + HT * R : L;
+        if (g1 < g0) g1 = g0;
+        gt = g0 + (((g1 - g0) * int64_t(sizeof(T))) & ~int64_t(15)) / int64_t(sizeof(T));
     };
     auto issue = [&](int64_t w) {  // thread 0 only
         if (w >= nitems) return;
@@ -59,7 +74,7 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_pipe_kernel(const S
         const uint32_t bytes = uint32_t((gt - g0) * sizeof(T));
         mbar_expect_tx(&bar, NA * bytes);
         if (bytes) {
-            const int64_t so = g0 - (t0 - R);  // stage row of g0
+            const int64_t so = g0 - (t0 - HT * R);  // stage row of g0
             for (int q = 0; q < NA; ++q)
                 bulk_g2s(stage + q * ROWS + so, src_arr[q] + sigma * A.in_stride + g0, bytes, &bar);
         }
@@ -78,7 +93,7 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_pipe_kernel(const S
         int64_t sigma, t0, L, g0, g1, gt;
         item_rows(w, sigma, t0, L, g0, g1, gt);
         mbar_wait(&bar, uint32_t(it & 1));
-        const int64_t i0 = t0 - R + int64_t(t) * R;  // first row of this thread
+        const int64_t i0 = t0 - HT * R + int64_t(t) * R;  // first row of this thread
         T ra[R], rc[R], rd[R], rb[RAW ? R : 1];
         lds_rows<T, R>(stage + 0 * ROWS + t * R, ra, lane);
         lds_rows<T, R>(stage + 1 * ROWS + t * R, rc, lane);
@@ -113,35 +128,54 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_pipe_kernel(const S
                 rd[v] = rd[v] * inv;
             }
         }
-        if constexpr (KP >= 1) reg_level<T, R, 1, NW, SM>(ra, rc, rd, el, er, 0, lane, warp);
-        if constexpr (KP >= 2) reg_level<T, R, 2, NW, SM>(ra, rc, rd, el, er, 1, lane, warp);
-        if constexpr (KP >= 3) reg_level<T, R, 4, NW, SM>(ra, rc, rd, el, er, 0, lane, warp);
-        if constexpr (KP >= 4) reg_level<T, R, 8, NW, SM>(ra, rc, rd, el, er, 1, lane, warp);
-        if (t >= 1 && t <= NT - 2 && i0 < L) {
-            const int64_t jb = i0 >> KP;
+        if constexpr (KP >= 1) reg_level<T, R, 1, NW, SMN>(ra, rc, rd, el, er, 0, lane, warp);
+        if constexpr (KP >= 2) reg_level<T, R, 2, NW, SMN>(ra, rc, rd, el, er, 1, lane, warp);
+        if constexpr (KP >= 3) reg_level<T, R, 4, NW, SMN>(ra, rc, rd, el, er, 0, lane, warp);
+        if constexpr (KP >= 4) reg_level<T, R, 8, NW, SMN>(ra, rc, rd, el, er, 1, lane, warp);
+        if constexpr (KP >= 5) reg_level_far<T, R, 1, NW>(ra, rc, rd, eF, eB, 0, lane, warp);
+        if constexpr (KP >= 6) reg_level_far<T, R, 2, NW>(ra, rc, rd, eF, eB, 1, lane, warp);
+        if constexpr (KP >= 7) reg_level_far<T, R, 4, NW>(ra, rc, rd, eF, eB, 0, lane, warp);
+        if (t >= HT && t < NT - HT && i0 < L) {
             const bool full = i0 + R <= L;
+            if constexpr (KP <= 4) {
+                // residue v mod 2^KP owns G consecutive positions: one vector store each
+                const int64_t jb = i0 >> KP;
 #pragma unroll
-            for (int rho = 0; rho < NR; ++rho) {
-                const int64_t o = out_slot_index(sigma, kprev, KP, rho) * A.out_slot + jb;
-                T va[G], vc[G], vd[G];
-#pragma unroll
-                for (int u = 0; u < G; ++u) {
-                    va[u] = ra[rho + NR * u];
-                    vc[u] = rc[rho + NR * u];
-                    vd[u] = rd[rho + NR * u];
-                }
-                if (full) {
-                    store_run<T, G>(A.oa + o, va);
-                    store_run<T, G>(A.oc + o, vc);
-                    store_run<T, G>(A.od + o, vd);
-                } else {
+                for (int rho = 0; rho < NR; ++rho) {
+                    const int64_t o = out_slot_index(sigma, kprev, KP, rho) * A.out_slot + jb;
+                    T va[G], vc[G], vd[G];
 #pragma unroll
                     for (int u = 0; u < G; ++u) {
-                        if (i0 + rho + NR * u < L) {
-                            A.oa[o + u] = va[u];
-                            A.oc[o + u] = vc[u];
-                            A.od[o + u] = vd[u];
+                        va[u] = ra[rho + NR * u];
+                        vc[u] = rc[rho + NR * u];
+                        vd[u] = rd[rho + NR * u];
+                    }
+                    if (full) {
+                        store_run<T, G>(A.oa + o, va);
+                        store_run<T, G>(A.oc + o, vc);
+                        store_run<T, G>(A.od + o, vd);
+                    } else {
+#pragma unroll
+                        for (int u = 0; u < G; ++u) {
+                            if (i0 + rho + NR * u < L) {
+                                A.oa[o + u] = va[u];
+                                A.oc[o + u] = vc[u];
+                                A.od[o + u] = vd[u];
+                            }
                         }
+                    }
+                }
+            } else {
+                // 16 rows = 16 residues (16*((i0>>4) mod 2^(KP-4)) + v) at one position j
+                const int64_t j = i0 >> KP;
+                const int64_t rbase = ((i0 >> 4) & ((int64_t(1) << (KP - 4)) - 1)) << 4;
+#pragma unroll
+                for (int v = 0; v < R; ++v) {
+                    if (full || i0 + v < L) {
+                        const int64_t o = out_slot_index(sigma, kprev, KP, rbase + v) * A.out_slot + j;
+                        A.oa[o] = ra[v];
+                        A.oc[o] = rc[v];
+                        A.od[o] = rd[v];
                     }
                 }
             }
@@ -149,34 +183,46 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_pipe_kernel(const S
     }
 }
 
+template <int KP>
+constexpr int split_pipe_tv() {
+    return SplitShape<KP>::TV;
+}
+
 template <typename T, int KP, bool RAW>
-static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t tps, int64_t nitems, cudaStream_t st) {
+static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_len, cudaStream_t st) {
+    using S = SplitShape<KP>;
     auto kern = split_pipe_kernel<T, KP, RAW>;
-    const size_t smem = size_t(RAW ? 4 : 3) * kRegSplitThreads * kRegSplitRows * sizeof(T);
+    const size_t smem = size_t(RAW ? 4 : 3) * S::NT * S::R * sizeof(T) +
+                        (KP > 4 ? size_t(4) * S::FAR * sizeof(T) : 0);
     cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     if (e != cudaSuccess) return e;
+    const int64_t tps = (max_len + S::TV - 1) / S::TV;
+    const int64_t nitems = m_in * tps;
+    if (nitems <= 0) return cudaSuccess;
     int dev = 0, sms = 148, occ = 1;
     cudaGetDevice(&dev);
     cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, kRegSplitThreads, smem);
+    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, S::NT, smem);
     const int64_t grid = std::min<int64_t>(nitems, int64_t(std::max(occ, 1)) * sms);
-    kern<<<(unsigned)grid, kRegSplitThreads, smem, st>>>(A, tps, nitems);
+    kern<<<(unsigned)grid, S::NT, smem, st>>>(A, tps, nitems);
     return cudaGetLastError();
 }
 
 template <typename T>
 cudaError_t launch_split_pipe(const SplitArgs<T> &A, bool raw, int64_t m_in, int64_t max_len, cudaStream_t st) {
-    constexpr int TV = kRegSplitThreads * kRegSplitRows - 2 * kRegSplitRows;
-    const int64_t tps = (max_len + TV - 1) / TV;
-    const int64_t nitems = m_in * tps;
-    if (nitems <= 0) return cudaSuccess;
+#define TDS_SP(KPV) \
+    case KPV: return raw ? launch_sp<T, KPV, true>(A, m_in, max_len, st) : launch_sp<T, KPV, false>(A, m_in, max_len, st)
     switch (A.kp) {
-        case 1: return raw ? launch_sp<T, 1, true>(A, tps, nitems, st) : launch_sp<T, 1, false>(A, tps, nitems, st);
-        case 2: return raw ? launch_sp<T, 2, true>(A, tps, nitems, st) : launch_sp<T, 2, false>(A, tps, nitems, st);
-        case 3: return raw ? launch_sp<T, 3, true>(A, tps, nitems, st) : launch_sp<T, 3, false>(A, tps, nitems, st);
-        case 4: return raw ? launch_sp<T, 4, true>(A, tps, nitems, st) : launch_sp<T, 4, false>(A, tps, nitems, st);
+        TDS_SP(1);
+        TDS_SP(2);
+        TDS_SP(3);
+        TDS_SP(4);
+        TDS_SP(5);
+        TDS_SP(6);
+        TDS_SP(7);
         default: return cudaErrorInvalidConfiguration;
     }
+#undef TDS_SP
 }
 
 template cudaError_t launch_split_pipe<float>(const SplitArgs<float> &, bool, int64_t, int64_t, cudaStream_t);

@@ -387,3 +387,18 @@ def test_chunked_equals_unchunked(tds, chunk):
     g1 = split_gpu(tds, a, b, c, d, dict(base, chunk_systems=chunk))
     for u, v in zip(g0[:3], g1[:3]):
         assert np.array_equal(u, v)
+
+
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("n,kp", [(1 << 20, [4, 3]), (777777, [3, 4]), (300000, [5]), (70000, [3])])
+@pytest.mark.parametrize("tl,T", [(0, 64), (3, 32), (5, 16), (5, 4)])
+def test_onchip_pipe_paths(tds, dtype, n, kp, tl, T):
+    """The persistent TMA-pipelined on-chip kernel (k > 0, cluster 1, 64 bytes
+    of rows per thread), shared-memory and warp-shuffle (tl_levels = 5) forms."""
+    c_lv = 4 if dtype == np.float32 else 3
+    a, b, c, d = inputs.generate(n, 2, dtype, seed=41)
+    try:
+        x, plan = run(tds, a, b, c, d, params=dict(k_pass=kp, cr_levels=c_lv, thomas_chains=T, tl_levels=tl))
+    except tds.TdsError as e:
+        pytest.skip(f"plan rejected: {e}")
+    check(a, b, c, d, x, dtype)
