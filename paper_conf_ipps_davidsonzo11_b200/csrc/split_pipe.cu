@@ -1,20 +1,28 @@
 // split_pipe.cu -- G1, persistent TMA-prefetched register split kernel:
-// k_p <= 7 fused PCR levels per HBM pass (§III-B/C, P:L296-303,
+// k_p <= 8 fused PCR levels per HBM pass (§III-B/C, P:L296-303,
 // P:L472-493), output de-interleaved into canonical residue slots.
 //
-// Work items are tiles (slot sigma, tile ti); a resident CTA walks items
-// w = blockIdx.x, += gridDim.x.  Thread t of the 256-thread CTA owns 16
-// consecutive rows in registers.  Levels with stride <= 8 rows exchange only
-// the first / last s rows with the neighbour threads (reg_level); levels with
-// stride 16, 32, 64 rows (k_p = 5..7) exchange whole 16-row blocks with the
-// threads 1, 2, 4 away (reg_level_far).  The first and last HT threads of a
-// CTA are the tile's halo (16*HT >= 2^k_p - 1 rows per side).
+// Work items are tiles (slot sigma, tile ti); a resident CTA (256 threads)
+// walks items w = blockIdx.x, += gridDim.x.  Each CTA owns ONE shared-memory
+// stage holding the next tile's input window (4 raw arrays on the first pass,
+// 3 normalised ones after): as soon as every thread has copied the current
+// window into registers (conflict-free rotated LDS.128) the stage is refilled
+// by cp.async.bulk (TMA) while the CTA computes.
 //
-// Each CTA owns ONE shared-memory stage holding the next tile's input rows (4
-// raw arrays on the first pass, 3 normalised ones after): as soon as every
-// thread has copied the current tile into registers (conflict-free rotated
-// LDS.128) the stage is refilled by cp.async.bulk (TMA) while the CTA runs
-// the PCR levels and the de-interleaved stores.
+// Layout A (the first min(k_p, 4) levels, strides 1..8 rows): lane l of warp w
+// owns the 16 rows of A-block a = 30w + l.  Warps overlap by two lanes, so a
+// level needs no shared memory and no barrier: neighbour rows come by shuffle
+// and the two edge lanes of every warp, which see garbage, are the halo
+// (after 4 levels rows closer than 15 to a warp end are invalid: lanes 1..30
+// stay exact).  The window is 242 A-blocks; blocks 1..240 are valid.
+//   k_p <= 4: residue v mod 2^k_p of a lane's rows owns 16 >> k_p consecutive
+//     positions: one vector store per residue, coalesced across the warp.
+//   k_p = 5..8: a swizzled shared-memory transpose gives layout B -- thread
+//     (rho = t >> 4, b = t & 15) owns members m = LEFT - 16 + 16b + u, u = 0..15,
+//     of residue class rho mod 16 (member m = A-block m + 1) -- so the strides
+//     16..128 rows of the remaining k_p - 4 levels are strides 1..8 of that
+//     class (16-lane shuffles; lanes b = 0 and 15 are the halo), and the store
+//     is again one vector run per final residue from lanes b = 1..NB.
 #include "pipe.cuh"
 #include "split_reg.cuh"
 
@@ -25,45 +33,52 @@ struct SplitShape {
     static constexpr int R = kRegSplitRows;
     static constexpr int NT = kRegSplitThreads;
     static constexpr int NW = NT / 32;
-    static constexpr int HT = KP <= 4 ? 1 : (1 << (KP - 4));  // halo threads per side
-    static constexpr int TV = (NT - 2 * HT) * R;               // valid rows per tile
-    static constexpr int SMN = (1 << (KP - 1)) < 8 ? (1 << (KP - 1)) : 8;
-    static constexpr int FAR = NW * kFarMaxTS * 3 * R;        // one half of a far-level edge buffer
+    static constexpr int AV = 30 * NW;          // valid A-blocks per window
+    static constexpr int ROWS = (AV + 2) * R;   // window rows (A-blocks 0 .. AV+1)
+    static constexpr int KQ = KP > 4 ? KP - 4 : 0;
+    static constexpr int LEFT = KP > 4 ? (1 << KQ) : 0;                   // B halo members before the output
+    static constexpr int NB = KP > 4 ? (AV + 1 - (2 << KQ)) / 16 : 0;     // B blocks stored
+    static constexpr int TV = KP > 4 ? NB * 16 * R : AV * R;              // output rows per tile
+    static constexpr int HEAD = R + LEFT * R;                             // window rows before the tile
+    static_assert(TV % (1 << KP) == 0, "tile must hold whole residue periods");
 };
 
 template <typename T, int KP, bool RAW>
-__global__ void __launch_bounds__(kRegSplitThreads, 2) split_pipe_kernel(const SplitArgs<T> A, int64_t tps,
-                                                                       int64_t nitems) {
+__global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
+    split_pipe_kernel(const SplitArgs<T> A, int64_t tps, int64_t nitems) {
     using S = SplitShape<KP>;
-    constexpr int R = S::R, NT = S::NT, NW = S::NW, HT = S::HT, TV = S::TV, SMN = S::SMN;
-    constexpr int NR = 1 << KP;
-    constexpr int G = KP <= 4 ? (R >> KP) : 1;
-    constexpr int NA = RAW ? 4 : 3;  // arrays streamed
-    constexpr int ROWS = NT * R;     // rows per stage (tile + halo threads)
+    constexpr int R = S::R, AV = S::AV, TV = S::TV, HEAD = S::HEAD, ROWS = S::ROWS;
+    constexpr int NA = RAW ? 4 : 3;                            // arrays streamed
+    constexpr int NTR = KP > 4 ? (sizeof(T) == 4 ? 3 : 1) : 0;  // arrays per transpose round
     extern __shared__ __align__(128) unsigned char smem_raw[];
     T *stage = reinterpret_cast<T *>(smem_raw);  // [NA][ROWS]
-    T *eF = stage + NA * ROWS;                   // far levels: [2][FAR] first-lane blocks
-    T *eB = eF + 2 * S::FAR;                     //             [2][FAR] last-lane blocks
-    __shared__ T eL[2][3][NW][SMN];
-    __shared__ T eR[2][3][NW][SMN];
+    T *tbuf = stage + NA * ROWS;                 // [NTR][AV * 16] transpose buffer
     __shared__ __align__(8) uint64_t bar;
     const int t = threadIdx.x, lane = t & 31, warp = t >> 5;
+    const int ablk = 30 * warp + lane;  // A-block of this thread
     const int kprev = RAW ? 0 : pass_levels(A.geom.npass, A.geom.kpass);
+    const bool small_items = nitems < (int64_t(1) << 31);
 
     auto slot_len = [&](int64_t sigma) -> int64_t {
         if (RAW) return A.n;
-        const int64_t r = slot_residue(sigma & ((int64_t(1) << kprev) - 1), A.geom.npass, A.geom.kpass);
+        const int64_t r = sigma & ((int64_t(1) << kprev) - 1);
         return r < A.n ? (A.n - r + (int64_t(1) << kprev) - 1) >> kprev : 0;
     };
     const T *src_arr[4] = {A.a, A.c, A.d, A.b};  // RAW also streams b
     // rows [g0, gt) of the item go to the stage by TMA (16-byte granules); [gt, g1) by LDG
     auto item_rows = [&](int64_t w, int64_t &sigma, int64_t &t0, int64_t &L, int64_t &g0, int64_t &g1,
                          int64_t &gt) {
-        sigma = w / tps;
-        t0 = (w % tps) * TV;
+        if (small_items) {
+            const uint32_t q = uint32_t(w) / uint32_t(tps);
+            sigma = q;
+            t0 = int64_t(uint32_t(w) - q * uint32_t(tps)) * TV;
+        } else {
+            sigma = w / tps;
+            t0 = (w % tps) * TV;
+        }
         L = slot_len(sigma);
-        g0 = t0 - HT * R < 0 ? 0 : t0 - HT * R;
-        g1 = t0 + TV + HT * R < L ? t0 + TV + HT * R : L;
+        g0 = t0 - HEAD < 0 ? 0 : t0 - HEAD;
+        g1 = t0 - HEAD + ROWS < L ? t0 - HEAD + ROWS : L;
         if (g1 < g0) g1 = g0;
         gt = g0 + (((g1 - g0) * int64_t(sizeof(T))) & ~int64_t(15)) / int64_t(sizeof(T));
     };
@@ -74,7 +89,7 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_pipe_kernel(const S
         const uint32_t bytes = uint32_t((gt - g0) * sizeof(T));
         mbar_expect_tx(&bar, NA * bytes);
         if (bytes) {
-            const int64_t so = g0 - (t0 - HT * R);  // stage row of g0
+            const int64_t so = g0 - (t0 - HEAD);  // stage row of g0
             for (int q = 0; q < NA; ++q)
                 bulk_g2s(stage + q * ROWS + so, src_arr[q] + sigma * A.in_stride + g0, bytes, &bar);
         }
@@ -85,7 +100,6 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_pipe_kernel(const S
         issue(blockIdx.x);
     }
     __syncthreads();
-    T *el = &eL[0][0][0][0], *er = &eR[0][0][0][0];
 
     for (int64_t it = 0;; ++it) {
         const int64_t w = int64_t(blockIdx.x) + it * gridDim.x;
@@ -93,12 +107,12 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_pipe_kernel(const S
         int64_t sigma, t0, L, g0, g1, gt;
         item_rows(w, sigma, t0, L, g0, g1, gt);
         mbar_wait(&bar, uint32_t(it & 1));
-        const int64_t i0 = t0 - HT * R + int64_t(t) * R;  // first row of this thread
+        const int64_t i0 = t0 - HEAD + int64_t(ablk) * R;  // first row of this thread (layout A)
         T ra[R], rc[R], rd[R], rb[RAW ? R : 1];
-        lds_rows<T, R>(stage + 0 * ROWS + t * R, ra, lane);
-        lds_rows<T, R>(stage + 1 * ROWS + t * R, rc, lane);
-        lds_rows<T, R>(stage + 2 * ROWS + t * R, rd, lane);
-        if constexpr (RAW) lds_rows<T, R>(stage + 3 * ROWS + t * R, rb, lane);
+        lds_rows<T, R>(stage + 0 * ROWS + ablk * R, ra, lane);
+        lds_rows<T, R>(stage + 1 * ROWS + ablk * R, rc, lane);
+        lds_rows<T, R>(stage + 2 * ROWS + ablk * R, rd, lane);
+        if constexpr (RAW) lds_rows<T, R>(stage + 3 * ROWS + ablk * R, rb, lane);
         if (i0 < g0 || i0 + R > gt) {  // rows outside the TMA range: global tail or identity
 #pragma unroll
             for (int v = 0; v < R; ++v) {
@@ -120,29 +134,35 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_pipe_kernel(const S
         __syncthreads();  // the stage is consumed: prefetch the next tile
         if (t == 0) issue(w + gridDim.x);
         if constexpr (RAW) {
+            if (i0 <= 0 || i0 + R >= L) {  // a_0 and c_{n-1} are outside the system
+#pragma unroll
+                for (int v = 0; v < R; ++v) {
+                    if (i0 + v == 0) ra[v] = T(0);
+                    if (i0 + v == L - 1) rc[v] = T(0);
+                }
+            }
 #pragma unroll
             for (int v = 0; v < R; ++v) {
                 const T inv = rcp(rb[v]);
-                ra[v] = (i0 + v > 0 ? ra[v] : T(0)) * inv;
-                rc[v] = (i0 + v < L - 1 ? rc[v] : T(0)) * inv;
-                rd[v] = rd[v] * inv;
+                ra[v] *= inv;
+                rc[v] *= inv;
+                rd[v] *= inv;
             }
         }
-        if constexpr (KP >= 1) reg_level<T, R, 1, NW, SMN>(ra, rc, rd, el, er, 0, lane, warp);
-        if constexpr (KP >= 2) reg_level<T, R, 2, NW, SMN>(ra, rc, rd, el, er, 1, lane, warp);
-        if constexpr (KP >= 3) reg_level<T, R, 4, NW, SMN>(ra, rc, rd, el, er, 0, lane, warp);
-        if constexpr (KP >= 4) reg_level<T, R, 8, NW, SMN>(ra, rc, rd, el, er, 1, lane, warp);
-        if constexpr (KP >= 5) reg_level_far<T, R, 1, NW>(ra, rc, rd, eF, eB, 0, lane, warp);
-        if constexpr (KP >= 6) reg_level_far<T, R, 2, NW>(ra, rc, rd, eF, eB, 1, lane, warp);
-        if constexpr (KP >= 7) reg_level_far<T, R, 4, NW>(ra, rc, rd, eF, eB, 0, lane, warp);
-        if (t >= HT && t < NT - HT && i0 < L) {
-            const bool full = i0 + R <= L;
-            if constexpr (KP <= 4) {
+        if constexpr (KP >= 1) reg_level_w<T, R, 1, 32>(ra, rc, rd);
+        if constexpr (KP >= 2) reg_level_w<T, R, 2, 32>(ra, rc, rd);
+        if constexpr (KP >= 3) reg_level_w<T, R, 4, 32>(ra, rc, rd);
+        if constexpr (KP >= 4) reg_level_w<T, R, 8, 32>(ra, rc, rd);
+        if constexpr (KP <= 4) {
+            constexpr int NR = 1 << KP, G = R >> KP;
+            if (lane >= 1 && lane <= 30 && i0 < L) {
+                const bool full = i0 + R <= L;
                 // residue v mod 2^KP owns G consecutive positions: one vector store each
-                const int64_t jb = i0 >> KP;
+                const int64_t step = (int64_t(1) << kprev) * A.out_slot;
+                const int64_t o0 = out_slot_index(sigma, kprev, KP, 0) * A.out_slot + (i0 >> KP);
 #pragma unroll
                 for (int rho = 0; rho < NR; ++rho) {
-                    const int64_t o = out_slot_index(sigma, kprev, KP, rho) * A.out_slot + jb;
+                    const int64_t o = o0 + rho * step;
                     T va[G], vc[G], vd[G];
 #pragma unroll
                     for (int u = 0; u < G; ++u) {
@@ -165,17 +185,70 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_pipe_kernel(const S
                         }
                     }
                 }
-            } else {
-                // 16 rows = 16 residues (16*((i0>>4) mod 2^(KP-4)) + v) at one position j
-                const int64_t j = i0 >> KP;
-                const int64_t rbase = ((i0 >> 4) & ((int64_t(1) << (KP - 4)) - 1)) << 4;
+            }
+        } else {
+            // ---- layout B: 16 consecutive members of residue class rho mod 16
+            constexpr int KQ = S::KQ, LEFT = S::LEFT, NB = S::NB;
+            constexpr int NQ = 1 << KQ, G = R >> KQ;
+            const int rho = t >> 4, b = t & 15;
+            const int mb = LEFT - 16 + 16 * b;  // member of u = 0
+            const bool wr = lane >= 1 && lane <= 30;
+            if constexpr (NTR == 3) {  // one round: 3 buffers
+                if (wr) {
+                    tr_write<T, R>(ra, tbuf, ablk - 1);
+                    tr_write<T, R>(rc, tbuf + AV * 16, ablk - 1);
+                    tr_write<T, R>(rd, tbuf + 2 * AV * 16, ablk - 1);
+                }
+                __syncthreads();
+                tr_read<T, R, AV>(ra, tbuf, mb, rho);
+                tr_read<T, R, AV>(rc, tbuf + AV * 16, mb, rho);
+                tr_read<T, R, AV>(rd, tbuf + 2 * AV * 16, mb, rho);
+            } else {  // three rounds through one buffer
+                if (wr) tr_write<T, R>(ra, tbuf, ablk - 1);
+                __syncthreads();
+                tr_read<T, R, AV>(ra, tbuf, mb, rho);
+                __syncthreads();
+                if (wr) tr_write<T, R>(rc, tbuf, ablk - 1);
+                __syncthreads();
+                tr_read<T, R, AV>(rc, tbuf, mb, rho);
+                __syncthreads();
+                if (wr) tr_write<T, R>(rd, tbuf, ablk - 1);
+                __syncthreads();
+                tr_read<T, R, AV>(rd, tbuf, mb, rho);
+            }
+            if constexpr (KQ >= 1) reg_level_w<T, R, 1, 16>(ra, rc, rd);
+            if constexpr (KQ >= 2) reg_level_w<T, R, 2, 16>(ra, rc, rd);
+            if constexpr (KQ >= 3) reg_level_w<T, R, 4, 16>(ra, rc, rd);
+            if constexpr (KQ >= 4) reg_level_w<T, R, 8, 16>(ra, rc, rd);
+            // member LEFT + 16(b-1) + u is row t0 + 16(16(b-1) + u) + rho
+            const int64_t r0 = t0 + 256 * (b - 1) + rho;  // row of u = 0
+            if (b >= 1 && b <= NB && r0 < L) {
+                const bool full = r0 + 16 * (R - 1) < L;
+                const int64_t step = (int64_t(16) << kprev) * A.out_slot;  // residue rho + 16 mu
+                const int64_t o0 = out_slot_index(sigma, kprev, KP, rho) * A.out_slot + (r0 >> KP);
 #pragma unroll
-                for (int v = 0; v < R; ++v) {
-                    if (full || i0 + v < L) {
-                        const int64_t o = out_slot_index(sigma, kprev, KP, rbase + v) * A.out_slot + j;
-                        A.oa[o] = ra[v];
-                        A.oc[o] = rc[v];
-                        A.od[o] = rd[v];
+                for (int mu = 0; mu < NQ; ++mu) {
+                    const int64_t o = o0 + mu * step;
+                    T va[G], vc[G], vd[G];
+#pragma unroll
+                    for (int q = 0; q < G; ++q) {
+                        va[q] = ra[mu + NQ * q];
+                        vc[q] = rc[mu + NQ * q];
+                        vd[q] = rd[mu + NQ * q];
+                    }
+                    if (full) {
+                        store_run<T, G>(A.oa + o, va);
+                        store_run<T, G>(A.oc + o, vc);
+                        store_run<T, G>(A.od + o, vd);
+                    } else {
+#pragma unroll
+                        for (int q = 0; q < G; ++q) {
+                            if (r0 + 16 * (mu + NQ * q) < L) {
+                                A.oa[o + q] = va[q];
+                                A.oc[o + q] = vc[q];
+                                A.od[o + q] = vd[q];
+                            }
+                        }
                     }
                 }
             }
@@ -183,17 +256,12 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_pipe_kernel(const S
     }
 }
 
-template <int KP>
-constexpr int split_pipe_tv() {
-    return SplitShape<KP>::TV;
-}
-
 template <typename T, int KP, bool RAW>
 static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_len, cudaStream_t st) {
     using S = SplitShape<KP>;
     auto kern = split_pipe_kernel<T, KP, RAW>;
-    const size_t smem = size_t(RAW ? 4 : 3) * S::NT * S::R * sizeof(T) +
-                        (KP > 4 ? size_t(4) * S::FAR * sizeof(T) : 0);
+    constexpr int NTR = KP > 4 ? (sizeof(T) == 4 ? 3 : 1) : 0;
+    const size_t smem = (size_t((RAW ? 4 : 3)) * S::ROWS + size_t(NTR) * S::AV * 16) * sizeof(T);
     cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     if (e != cudaSuccess) return e;
     const int64_t tps = (max_len + S::TV - 1) / S::TV;
@@ -220,6 +288,7 @@ cudaError_t launch_split_pipe(const SplitArgs<T> &A, bool raw, int64_t m_in, int
         TDS_SP(5);
         TDS_SP(6);
         TDS_SP(7);
+        TDS_SP(8);
         default: return cudaErrorInvalidConfiguration;
     }
 #undef TDS_SP

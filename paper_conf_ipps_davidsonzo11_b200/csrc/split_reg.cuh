@@ -87,6 +87,62 @@ __device__ __forceinline__ void reg_level(T (&ra)[R], T (&rc)[R], T (&rd)[R], T 
     }
 }
 
+// One PCR level with stride S (in the thread's own row index) over chains of
+// W lanes (__shfl width W): the lanes of a segment hold consecutive R-row
+// blocks of one chain.  The first / last lane of a segment get their own rows
+// back as "neighbours" -- garbage that spreads 2^l - 1 rows per level from the
+// segment ends, i.e. stays inside the halo the caller discards (after l
+// levels, rows closer than 2^l - 1 to a segment end are invalid).  No shared
+// memory, no barrier, no select.
+template <typename T, int R, int S, int W>
+__device__ __forceinline__ void reg_level_w(T (&ra)[R], T (&rc)[R], T (&rd)[R]) {
+#pragma unroll
+    for (int rho = 0; rho < S; ++rho) {
+        T pa = __shfl_up_sync(0xffffffffu, ra[R - S + rho], 1, W);
+        T pc = __shfl_up_sync(0xffffffffu, rc[R - S + rho], 1, W);
+        T pd = __shfl_up_sync(0xffffffffu, rd[R - S + rho], 1, W);
+        T xa = __shfl_down_sync(0xffffffffu, ra[rho], 1, W);
+        T xc = __shfl_down_sync(0xffffffffu, rc[rho], 1, W);
+        T xd = __shfl_down_sync(0xffffffffu, rd[rho], 1, W);
+#pragma unroll
+        for (int v = rho; v < R; v += S) {
+            const T oa = ra[v], oc = rc[v], od = rd[v];
+            const bool last = v + S >= R;
+            row_update(ra[v], rc[v], rd[v], pa, pc, pd, last ? xa : ra[(v + S) % R], last ? xc : rc[(v + S) % R],
+                       last ? xd : rd[(v + S) % R]);
+            pa = oa;
+            pc = oc;
+            pd = od;
+        }
+    }
+}
+
+// Shared-memory transpose buffer of the deep split kernel: element (m, rho) =
+// row 16m + rho of the tile at 16m + (rho ^ g(m)), g(m) = ((m >> 4) + (m >> 1)) & 15.
+// Layout-A writes (fixed rho, consecutive m across lanes) and layout-B reads
+// (fixed m offset, m 16 apart across lanes, two rho per warp) both hit at most
+// two lanes per bank.
+__device__ __forceinline__ int tr_addr(int m, int rho) { return 16 * m + (rho ^ (((m >> 4) + (m >> 1)) & 15)); }
+
+// layout A -> buffer: the R rows of block m
+template <typename T, int R>
+__device__ __forceinline__ void tr_write(const T (&x)[R], T *buf, int m) {
+#pragma unroll
+    for (int v = 0; v < R; ++v) buf[tr_addr(m, v)] = x[v];
+}
+
+// buffer -> layout B: members mb .. mb+R-1 of class rho (clamped into the
+// buffer's AV blocks: the clamped members are halo garbage)
+template <typename T, int R, int AV>
+__device__ __forceinline__ void tr_read(T (&x)[R], const T *buf, int mb, int rho) {
+#pragma unroll
+    for (int u = 0; u < R; ++u) {
+        int m = mb + u;
+        m = m < 0 ? 0 : (m > AV - 1 ? AV - 1 : m);
+        x[u] = buf[tr_addr(m, rho)];
+    }
+}
+
 // One PCR level whose stride is TS whole threads (16*TS rows, TS in {1,2,4}):
 // row v of thread t needs row v of threads t-TS and t+TS.  Warp shuffles
 // carry all 16 rows; the TS edge lanes of each warp go through shared memory

@@ -19,7 +19,7 @@ constexpr int kMaxOnchipThreads = 1024;     // on-chip CTA size for R <= 4
 constexpr int kMaxOnchipThreadsWide = 512;  // ... and for R >= 8 (register budget)
 constexpr int kMaxSplitThreads = 512;
 constexpr int kRegSplitMaxKp = 4;       // split passes with k_p <= 4 use the register kernel
-constexpr int kPipeSplitMaxKp = 7;      // ... up to 7 with 16-byte aligned rows (persistent TMA kernel)
+constexpr int kPipeSplitMaxKp = 8;      // ... up to 8 with 16-byte aligned rows (persistent TMA kernel)
 constexpr int kRegSplitRows = 16;       // ... 16 rows per thread
 constexpr int kRegSplitThreads = 256;   // ... 256 threads per CTA
 

@@ -254,6 +254,56 @@ def test_split_fused_equals_multipass_and_tiles(tds):
             assert np.array_equal(u, v)
 
 
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("n,kp", [(200004, [5]), (200004, [6]), (131072, [7]), (200004, [8]),
+                                  (3588 * 3 + 4, [8]), (200004, [3, 8]), (200004, [8, 2])])
+def test_split_deep_pipe_vs_oracle(tds, dtype, n, kp):
+    """k_p = 5..8 in one pass (persistent TMA split kernel, transposed layout:
+    4 levels on consecutive rows, k_p - 4 on residue classes mod 16) vs the
+    oracle's textbook PCR, on tiles with ragged tails."""
+    a, b, c, d = inputs.generate(n, 2, dtype, seed=23)
+    ga, gc, gd, plan = split_gpu(tds, a, b, c, d, dict(k_pass=kp, split_only=1))
+    k = sum(kp)
+    perm = plan.permutation()
+    sa, sb, sc, sd = oracle.pcr_split(a, b, c, d, k)
+    ref = [v[:, perm] / sb[:, perm] for v in (sa, sc, sd)]
+    tol = 1e-5 if dtype == np.float32 else 1e-13
+    for g, r in zip((ga, gc, gd), ref):
+        assert np.abs(g - r).max() <= tol * max(1.0, np.abs(r).max())
+
+
+@pytest.mark.parametrize("n", [1 << 20, (1 << 20) + 12344, 4100])
+def test_split_deep_fused_equals_multipass(tds, n):
+    """Bit-exact: [8] == [4, 4] == [2, 2, 2, 2] and [7] == [4, 3] (the same
+    normalised row update on the same operands, whatever the layout)."""
+    a, b, c, d = inputs.generate(n, 2, np.float32, seed=5)
+    base = dict(split_only=1)
+    r8 = split_gpu(tds, a, b, c, d, dict(base, k_pass=[8]))
+    for other in ([4, 4], [2, 2, 2, 2], [5, 3]):
+        ro = split_gpu(tds, a, b, c, d, dict(base, k_pass=other))
+        for u, v in zip(r8[:3], ro[:3]):
+            assert np.array_equal(u, v)
+    r7 = split_gpu(tds, a, b, c, d, dict(base, k_pass=[7]))
+    ro = split_gpu(tds, a, b, c, d, dict(base, k_pass=[4, 3]))
+    for u, v in zip(r7[:3], ro[:3]):
+        assert np.array_equal(u, v)
+
+
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("kp", [[7], [8], [6]])
+def test_single_pass_deep_split_solve(tds, dtype, kp):
+    """Whole solve with one deep split pass + the pipelined on-chip kernel."""
+    n = (1 << 20) + 4 * 777
+    c_lv = 4 if dtype == np.float32 else 3
+    a, b, c, d = inputs.generate(n, 3, dtype, seed=44)
+    try:
+        x, plan = run(tds, a, b, c, d, params=dict(k_pass=kp, cr_levels=c_lv, thomas_chains=16, tl_levels=5,
+                                                    cluster=1))
+    except tds.TdsError as e:
+        pytest.skip(f"plan rejected: {e}")
+    check(a, b, c, d, x, dtype)
+
+
 # ------------------------------------------------ layout, aliasing, isolation
 
 def test_batch_isolation(tds):
