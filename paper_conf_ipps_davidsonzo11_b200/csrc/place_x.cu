@@ -90,6 +90,78 @@ __global__ void __launch_bounds__(kPlaceThreads) place_x_kernel(const PlaceArgs<
     }
 }
 
+// K >= 5: 32 residues x 64 positions per CTA through a shared-memory tile.
+// Reads are 32 runs of 64 consecutive positions (one per slot, 16-byte
+// vectors), writes are 64 runs of 32 consecutive original rows; the padded
+// tile (stride 33) keeps both shared-memory sides at most 2-way conflicted.
+constexpr int kTileRes = 32, kTileJ = 64;
+
+template <typename T>
+__global__ void __launch_bounds__(kPlaceThreads) place_x_tile_kernel(const PlaceArgs<T> A, int64_t jtiles,
+                                                                    int64_t lmax) {
+    constexpr int E = 16 / int(sizeof(T));                 // elements per 16-byte vector
+    constexpr int NRD = kTileRes * kTileJ / E / kPlaceThreads;  // vector reads per thread
+    constexpr int LPR = kTileJ / E;                        // lanes per residue run (read side)
+    constexpr int LPW = kTileRes / E;                      // lanes per row run (write side)
+    __shared__ T tile[kTileJ][kTileRes + 1];
+    const int t = threadIdx.x;
+    const int64_t rtiles = (int64_t(1) << A.K) / kTileRes;
+    int64_t b = blockIdx.x;
+    const int64_t jt = b % jtiles;
+    b /= jtiles;
+    const int64_t rt = b % rtiles, sys = b / rtiles;
+    const int64_t j0 = jt * kTileJ, r0 = rt * kTileRes;
+    const T *src = A.xs + ((sys << A.K) + r0) * A.slot + j0;
+#pragma unroll
+    for (int q = 0; q < NRD; ++q) {
+        const int e = q * kPlaceThreads + t;
+        const int rl = e / LPR, jj = (e % LPR) * E;
+        T v[E];
+        if (j0 + jj + E <= A.slot) {
+            if constexpr (sizeof(T) == 4) {
+                const float4 f = __ldcs(reinterpret_cast<const float4 *>(src + rl * A.slot + jj));
+                v[0] = f.x;
+                v[1] = f.y;
+                v[2] = f.z;
+                v[3] = f.w;
+            } else {
+                const double2 f = __ldcs(reinterpret_cast<const double2 *>(src + rl * A.slot + jj));
+                v[0] = f.x;
+                v[1] = f.y;
+            }
+        } else {
+#pragma unroll
+            for (int u = 0; u < E; ++u) v[u] = j0 + jj + u < A.slot ? src[rl * A.slot + jj + u] : T(0);
+        }
+#pragma unroll
+        for (int u = 0; u < E; ++u) tile[jj + u][rl] = v[u];
+    }
+    __syncthreads();
+    T *dst = A.x + sys * A.batch_stride + r0;
+#pragma unroll
+    for (int q = 0; q < NRD; ++q) {
+        const int e = q * kPlaceThreads + t;
+        const int jj = e / LPW, rl = (e % LPW) * E;
+        const int64_t j = j0 + jj;
+        if (j >= lmax) continue;
+        const int64_t row = (j << A.K) + r0 + rl;  // original row of residue r0 + rl
+        T v[E];
+#pragma unroll
+        for (int u = 0; u < E; ++u) v[u] = tile[jj][rl + u];
+        T *p = dst + (j << A.K) + rl;
+        if (A.vec && row + E <= A.n) {
+            if constexpr (sizeof(T) == 4)
+                __stcs(reinterpret_cast<float4 *>(p), make_float4(v[0], v[1], v[2], v[3]));
+            else
+                __stcs(reinterpret_cast<double2 *>(p), make_double2(v[0], v[1]));
+        } else {
+#pragma unroll
+            for (int u = 0; u < E; ++u)
+                if (row + u < A.n) p[u] = v[u];
+        }
+    }
+}
+
 template <typename T>
 cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batch_stride, int64_t slot, int K,
                            int vec, const PassGeom &geom, cudaStream_t st) {
@@ -102,6 +174,14 @@ cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batc
     A.K = K;
     A.vec = vec;
     A.geom = geom;
+    if (K >= 5) {
+        const int64_t lmax = (n + (int64_t(1) << K) - 1) >> K;
+        const int64_t jtiles = (lmax + kTileJ - 1) / kTileJ;
+        const int64_t grid = m * ((int64_t(1) << K) / kTileRes) * jtiles;
+        if (grid > 0x7fffffffLL) return cudaErrorInvalidConfiguration;
+        place_x_tile_kernel<T><<<(unsigned)grid, kPlaceThreads, 0, st>>>(A, jtiles, lmax);
+        return cudaGetLastError();
+    }
     const int64_t tiles = (n + kPlaceRows * kPlaceThreads - 1) / (kPlaceRows * kPlaceThreads);
     const int64_t grid = m * tiles;
     if (grid > 0x7fffffffLL) return cudaErrorInvalidConfiguration;

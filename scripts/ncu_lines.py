@@ -1,7 +1,7 @@
 #!/usr/bin/env python
 """Attribute ncu per-SASS warp-stall samples to CUDA source lines.
 
-    python scripts/ncu_lines.py gpurun_out/prof.ncu-rep [kernel-substring] [top]
+    python scripts/ncu_lines.py gpurun_out/prof.ncu-rep [mangled-substring] [top] [ncu-kernel-regex]
 
 ncu's SASS page gives samples per instruction address; the cubin's line table
 (nvdisasm -g over the cubin extracted from libtds.so) maps each address to a
@@ -20,15 +20,22 @@ ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 LIB = os.path.join(ROOT, "paper_conf_ipps_davidsonzo11_b200", "libtds.so")
 
 
-def sass_samples(rep):
-    out = subprocess.run(["ncu", "-i", rep, "--page", "source", "--csv", "--print-source", "sass"],
-                         capture_output=True, text=True).stdout
+def sass_samples(rep, kfilter=""):
+    cmd = ["ncu", "-i", rep, "--page", "source", "--csv", "--print-source", "sass"]
+    if kfilter:
+        cmd += ["-k", "regex:" + kfilter]
+    out = subprocess.run(cmd, capture_output=True, text=True).stdout
     rows = list(csv.reader(io.StringIO(out)))
     name = rows[0][1] if rows and rows[0][0] == "Kernel Name" else ""
     hi = [i for i, r in enumerate(rows) if r and r[0] == "Address"][0]
     h = rows[hi]
     si = h.index("Warp Stall Sampling (All Samples)")
-    body = [r for r in rows[hi + 1:] if len(r) > si and r[si].isdigit()]
+    body = []
+    for r in rows[hi + 1:]:
+        if r and r[0] == "Kernel Name":
+            break
+        if len(r) > si and r[si].isdigit():
+            body.append(r)
     base = int(body[0][0], 16)
     return name, [(int(r[0], 16) - base, int(r[si]), r[h.index("Source")].strip()) for r in body]
 
@@ -62,7 +69,7 @@ def main():
     rep = sys.argv[1]
     sub = sys.argv[2] if len(sys.argv) > 2 else ""
     top = int(sys.argv[3]) if len(sys.argv) > 3 else 30
-    name, samples = sass_samples(rep)
+    name, samples = sass_samples(rep, sys.argv[4] if len(sys.argv) > 4 else "")
     # pick the mangled function whose instruction count best matches
     table = line_table(sub)
     funcs = collections.defaultdict(dict)
