@@ -38,6 +38,22 @@ __device__ __forceinline__ void row_update(T &a, T &c, T &d, T al, T cl, T dl, T
     d = nd;
 }
 
+// The same update on two independent rows at once with the packed fp32x2
+// instructions of sm_100 (FFMA2 / FMUL2): per lane bit-identical to
+// row_update<float> (same fused operations, same rounding), half the issue slots.
+__device__ __forceinline__ float2 neg2(float2 a) { return make_float2(-a.x, -a.y); }
+__device__ __forceinline__ void row_update2(float2 &a, float2 &c, float2 &d, float2 al, float2 cl, float2 dl, float2 ar,
+                                            float2 cr, float2 dr) {
+    const float2 den = __ffma2_rn(neg2(c), ar, __ffma2_rn(neg2(a), cl, make_float2(1.f, 1.f)));
+    const float2 r = make_float2(rcp(den.x), rcp(den.y));
+    const float2 ma = __fmul2_rn(neg2(a), r);
+    const float2 mc = __fmul2_rn(neg2(c), r);
+    const float2 nd = __ffma2_rn(ma, dl, __ffma2_rn(mc, dr, __fmul2_rn(d, r)));
+    a = __fmul2_rn(ma, al);
+    c = __fmul2_rn(mc, cr);
+    d = nd;
+}
+
 // Workspace slots are kept in CANONICAL residue order: after K cumulative
 // levels, slot (s << K) + r holds the residue-r subsystem of system s.  Each
 // pass writes the new residue digit rho of input slot sigma (levels kprev

@@ -141,12 +141,28 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
                     if (i0 + v == L - 1) rc[v] = T(0);
                 }
             }
+            if constexpr (sizeof(T) == 4) {
 #pragma unroll
-            for (int v = 0; v < R; ++v) {
-                const T inv = rcp(rb[v]);
-                ra[v] *= inv;
-                rc[v] *= inv;
-                rd[v] *= inv;
+                for (int v = 0; v < R; v += 2) {
+                    const float2 inv = make_float2(rcp(rb[v]), rcp(rb[v + 1]));
+                    const float2 a = __fmul2_rn(make_float2(ra[v], ra[v + 1]), inv);
+                    const float2 c = __fmul2_rn(make_float2(rc[v], rc[v + 1]), inv);
+                    const float2 d = __fmul2_rn(make_float2(rd[v], rd[v + 1]), inv);
+                    ra[v] = a.x;
+                    ra[v + 1] = a.y;
+                    rc[v] = c.x;
+                    rc[v + 1] = c.y;
+                    rd[v] = d.x;
+                    rd[v + 1] = d.y;
+                }
+            } else {
+#pragma unroll
+                for (int v = 0; v < R; ++v) {
+                    const T inv = rcp(rb[v]);
+                    ra[v] *= inv;
+                    rc[v] *= inv;
+                    rd[v] *= inv;
+                }
             }
         }
         if constexpr (KP >= 1) reg_level_w<T, R, 1, 32>(ra, rc, rd);

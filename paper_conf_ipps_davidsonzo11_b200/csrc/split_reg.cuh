@@ -96,6 +96,45 @@ __device__ __forceinline__ void reg_level(T (&ra)[R], T (&rc)[R], T (&rd)[R], T 
 // memory, no barrier, no select.
 template <typename T, int R, int S, int W>
 __device__ __forceinline__ void reg_level_w(T (&ra)[R], T (&rc)[R], T (&rd)[R]) {
+    if constexpr (sizeof(T) == 4 && S % 2 == 0) {
+        // fp32, even stride: classes rho and rho + 1 move together as row pairs
+        // (v, v+1), whose neighbours (v -+ S, v+1 -+ S) are again aligned pairs
+        auto P = [](const T *r, int v) { return make_float2(r[v], r[v + 1]); };
+#pragma unroll
+        for (int rho = 0; rho < S; rho += 2) {
+            float2 pa, pc, pd, xa, xc, xd;
+            pa.x = __shfl_up_sync(0xffffffffu, ra[R - S + rho], 1, W);
+            pa.y = __shfl_up_sync(0xffffffffu, ra[R - S + rho + 1], 1, W);
+            pc.x = __shfl_up_sync(0xffffffffu, rc[R - S + rho], 1, W);
+            pc.y = __shfl_up_sync(0xffffffffu, rc[R - S + rho + 1], 1, W);
+            pd.x = __shfl_up_sync(0xffffffffu, rd[R - S + rho], 1, W);
+            pd.y = __shfl_up_sync(0xffffffffu, rd[R - S + rho + 1], 1, W);
+            xa.x = __shfl_down_sync(0xffffffffu, ra[rho], 1, W);
+            xa.y = __shfl_down_sync(0xffffffffu, ra[rho + 1], 1, W);
+            xc.x = __shfl_down_sync(0xffffffffu, rc[rho], 1, W);
+            xc.y = __shfl_down_sync(0xffffffffu, rc[rho + 1], 1, W);
+            xd.x = __shfl_down_sync(0xffffffffu, rd[rho], 1, W);
+            xd.y = __shfl_down_sync(0xffffffffu, rd[rho + 1], 1, W);
+#pragma unroll
+            for (int v = rho; v < R; v += S) {
+                float2 a = P(ra, v), c = P(rc, v), d = P(rd, v);
+                const float2 oa = a, oc = c, od = d;
+                const bool last = v + S >= R;
+                row_update2(a, c, d, pa, pc, pd, last ? xa : P(ra, (v + S) % R), last ? xc : P(rc, (v + S) % R),
+                            last ? xd : P(rd, (v + S) % R));
+                ra[v] = a.x;
+                ra[v + 1] = a.y;
+                rc[v] = c.x;
+                rc[v + 1] = c.y;
+                rd[v] = d.x;
+                rd[v + 1] = d.y;
+                pa = oa;
+                pc = oc;
+                pd = od;
+            }
+        }
+        return;
+    }
 #pragma unroll
     for (int rho = 0; rho < S; ++rho) {
         T pa = __shfl_up_sync(0xffffffffu, ra[R - S + rho], 1, W);
