@@ -1,6 +1,8 @@
 // pipe.cuh -- TMA bulk-copy / mbarrier helpers and conflict-free shared-memory
 // row loads shared by the persistent (pipelined) kernels.
 #pragma once
+#include <cuda.h>
+
 #include "common.cuh"
 
 namespace tds {
@@ -40,6 +42,64 @@ __device__ __forceinline__ void bulk_g2s(void *dst, const void *src, uint32_t by
         "l"(src), "r"(bytes), "r"(smem_u32(bar))
         : "memory");
 }
+
+// ---- TMA tensor tiles with the 128-byte swizzle --------------------------
+// A batch of row slots viewed as a 3-D tensor {ELINE rows per 128-byte line,
+// lines per slot, slots}; a box of BL lines lands in shared memory with the
+// 16-byte chunks of line L permuted by chunk ^ (L & 7) (the stage must be
+// 1024-byte aligned).  A thread reading the 64 or 128 consecutive bytes of its
+// rows then hits 8 distinct bank groups per quarter-warp with no register
+// rotation.  Coordinates are signed: lines before 0 or past the tensor are
+// zero-filled (their bytes still count on the mbarrier).
+struct TmapSet {
+    CUtensorMap m[4];
+};
+
+__device__ __forceinline__ void tma_load_lines(void *dst, const CUtensorMap *map, int line, int slot, uint64_t *bar) {
+    asm volatile(
+        "cp.async.bulk.tensor.3d.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1, {%2, %3, %4}], [%5];" ::
+            "r"(smem_u32(dst)),
+        "l"(map), "r"(0), "r"(line), "r"(slot), "r"(smem_u32(bar))
+        : "memory");
+}
+
+// Element offset of stage row s in a swizzled stage.
+template <typename T>
+__device__ __forceinline__ int sw_off(int s) {
+    constexpr int CH = 16 / int(sizeof(T)), ELINE = 128 / int(sizeof(T));
+    const int line = s / ELINE, within = s % ELINE;
+    return line * ELINE + (((within / CH) ^ (line & 7)) * CH) + within % CH;
+}
+
+// R consecutive rows starting at stage row s0 (a multiple of R) of a swizzled stage.
+template <typename T, int R>
+__device__ __forceinline__ void lds_rows_sw(const T *stage, int s0, T *v) {
+    constexpr int CH = 16 / int(sizeof(T));     // rows per 16-byte chunk
+    constexpr int ELINE = 128 / int(sizeof(T));  // rows per line
+    const unsigned char *base = reinterpret_cast<const unsigned char *>(stage);
+#pragma unroll
+    for (int q = 0; q < R / CH; ++q) {
+        const int row = s0 + q * CH;
+        const int line = row / ELINE, chunk = (row % ELINE) / CH;
+        const unsigned char *p = base + line * 128 + ((chunk ^ (line & 7)) << 4);
+        if constexpr (sizeof(T) == 4) {
+            const float4 f = *reinterpret_cast<const float4 *>(p);
+            v[4 * q] = f.x;
+            v[4 * q + 1] = f.y;
+            v[4 * q + 2] = f.z;
+            v[4 * q + 3] = f.w;
+        } else {
+            const double2 f = *reinterpret_cast<const double2 *>(p);
+            v[2 * q] = f.x;
+            v[2 * q + 1] = f.y;
+        }
+    }
+}
+
+// Host: encode the tensor map of `slots` row slots of `lines` full 128-byte
+// lines each, slot stride `stride` elements, box of `box_lines` lines.
+bool encode_rows_tmap(CUtensorMap *out, const void *base, int dsize, int64_t lines, int64_t slots, int64_t stride,
+                      int box_lines);
 
 // Load R consecutive rows (R * sizeof(T) = 16 * NCH bytes, NCH in {2, 4, 8})
 // per thread from shared memory into registers without bank conflicts.

@@ -41,33 +41,52 @@ struct SplitShape {
     static constexpr int TV = KP > 4 ? NB * 16 * R : AV * R;              // output rows per tile
     static constexpr int HEAD = R + LEFT * R;                             // window rows before the tile
     static_assert(TV % (1 << KP) == 0, "tile must hold whole residue periods");
+    // TMA view: the tensor starts TOFF rows into each slot so that every
+    // window starts on a 128-byte line (then the 8 lanes of a quarter-warp read
+    // 4 whole swizzled lines: no bank conflict); rows [0, TOFF) come by LDG.
+    template <typename T>
+    __host__ __device__ static constexpr int toff() {
+        return (128 / int(sizeof(T)) - HEAD % (128 / int(sizeof(T)))) % (128 / int(sizeof(T)));
+    }
+    template <typename T>
+    __host__ __device__ static constexpr int box_lines() { return ROWS / (128 / int(sizeof(T))); }
+    template <typename T>
+    __host__ __device__ static constexpr int stage_elems() { return (box_lines<T>() * 128 + 1023) / 1024 * 1024 / int(sizeof(T)); }
+    template <typename T>
+    static constexpr size_t smem_bytes(bool raw) {
+        return 1024 + (size_t(raw ? 4 : 3) * stage_elems<T>() +
+                       size_t(KP > 4 ? (sizeof(T) == 4 ? 3 : 1) : 0) * AV * 16) * sizeof(T);
+    }
 };
 
 template <typename T, int KP, bool RAW>
 __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
-    split_pipe_kernel(const SplitArgs<T> A, int64_t tps, int64_t nitems) {
+    split_pipe_kernel(const SplitArgs<T> A, int64_t tps, int64_t nitems, const __grid_constant__ TmapSet tm,
+                      int32_t tma_lines) {
     using S = SplitShape<KP>;
     constexpr int R = S::R, AV = S::AV, TV = S::TV, HEAD = S::HEAD, ROWS = S::ROWS;
+    constexpr int TOFF = S::template toff<T>(), BL = S::template box_lines<T>(), ELINE = 128 / int(sizeof(T));
+    static_assert(ROWS % ELINE == 0, "window of whole lines");
+    constexpr int STG = S::template stage_elems<T>();          // elements per array stage (1024-byte multiple)
     constexpr int NA = RAW ? 4 : 3;                            // arrays streamed
     constexpr int NTR = KP > 4 ? (sizeof(T) == 4 ? 3 : 1) : 0;  // arrays per transpose round
-    extern __shared__ __align__(128) unsigned char smem_raw[];
-    T *stage = reinterpret_cast<T *>(smem_raw);  // [NA][ROWS]
-    T *tbuf = stage + NA * ROWS;                 // [NTR][AV * 16] transpose buffer
+    extern __shared__ __align__(1024) unsigned char smem_raw[];
+    T *stage = reinterpret_cast<T *>(smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u));  // 1024-aligned
+    T *tbuf = stage + NA * STG;                                // [NTR][AV * 16] transpose buffer
     __shared__ __align__(8) uint64_t bar;
     const int t = threadIdx.x, lane = t & 31, warp = t >> 5;
     const int ablk = 30 * warp + lane;  // A-block of this thread
     const int kprev = RAW ? 0 : pass_levels(A.geom.npass, A.geom.kpass);
     const bool small_items = nitems < (int64_t(1) << 31);
+    const int64_t tma_end = TOFF + int64_t(tma_lines) * ELINE;  // rows [TOFF, tma_end) of every slot are TMA lines
 
     auto slot_len = [&](int64_t sigma) -> int64_t {
         if (RAW) return A.n;
         const int64_t r = sigma & ((int64_t(1) << kprev) - 1);
         return r < A.n ? (A.n - r + (int64_t(1) << kprev) - 1) >> kprev : 0;
     };
-    const T *src_arr[4] = {A.a, A.c, A.d, A.b};  // RAW also streams b
-    // rows [g0, gt) of the item go to the stage by TMA (16-byte granules); [gt, g1) by LDG
-    auto item_rows = [&](int64_t w, int64_t &sigma, int64_t &t0, int64_t &L, int64_t &g0, int64_t &g1,
-                         int64_t &gt) {
+    // window rows [ws, ws + ROWS); rows [g0, gt) come from the TMA box, the rest by LDG / identity
+    auto item_rows = [&](int64_t w, int64_t &sigma, int64_t &t0, int64_t &L, int64_t &g0, int64_t &gt) {
         if (small_items) {
             const uint32_t q = uint32_t(w) / uint32_t(tps);
             sigma = q;
@@ -77,22 +96,21 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
             t0 = (w % tps) * TV;
         }
         L = slot_len(sigma);
-        g0 = t0 - HEAD < 0 ? 0 : t0 - HEAD;
-        g1 = t0 - HEAD + ROWS < L ? t0 - HEAD + ROWS : L;
-        if (g1 < g0) g1 = g0;
-        gt = g0 + (((g1 - g0) * int64_t(sizeof(T))) & ~int64_t(15)) / int64_t(sizeof(T));
+        g0 = t0 - HEAD < TOFF ? TOFF : t0 - HEAD;
+        gt = t0 - HEAD + ROWS < tma_end ? t0 - HEAD + ROWS : tma_end;
     };
     auto issue = [&](int64_t w) {  // thread 0 only
         if (w >= nitems) return;
-        int64_t sigma, t0, L, g0, g1, gt;
-        item_rows(w, sigma, t0, L, g0, g1, gt);
-        const uint32_t bytes = uint32_t((gt - g0) * sizeof(T));
-        mbar_expect_tx(&bar, NA * bytes);
-        if (bytes) {
-            const int64_t so = g0 - (t0 - HEAD);  // stage row of g0
-            for (int q = 0; q < NA; ++q)
-                bulk_g2s(stage + q * ROWS + so, src_arr[q] + sigma * A.in_stride + g0, bytes, &bar);
+        if (tma_lines == 0) {  // slots shorter than one line: everything by LDG
+            mbar_expect_tx(&bar, 0);
+            return;
         }
+        int64_t sigma, t0, L, g0, gt;
+        item_rows(w, sigma, t0, L, g0, gt);
+        mbar_expect_tx(&bar, NA * BL * 128);
+        const int line0 = int((t0 - HEAD - TOFF) / ELINE);  // exact: TV and HEAD + TOFF are whole lines
+#pragma unroll
+        for (int q = 0; q < NA; ++q) tma_load_lines(stage + q * STG, &tm.m[q], line0, int(sigma), &bar);
     };
     if (t == 0) {
         mbar_init(&bar, 1);
@@ -104,43 +122,48 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
     for (int64_t it = 0;; ++it) {
         const int64_t w = int64_t(blockIdx.x) + it * gridDim.x;
         if (w >= nitems) break;
-        int64_t sigma, t0, L, g0, g1, gt;
-        item_rows(w, sigma, t0, L, g0, g1, gt);
+        int64_t sigma, t0, L, g0, gt;
+        item_rows(w, sigma, t0, L, g0, gt);
         mbar_wait(&bar, uint32_t(it & 1));
-        const int64_t i0 = t0 - HEAD + int64_t(ablk) * R;  // first row of this thread (layout A)
-        T ra[R], rc[R], rd[R], rb[RAW ? R : 1];
-        lds_rows<T, R>(stage + 0 * ROWS + ablk * R, ra, lane);
-        lds_rows<T, R>(stage + 1 * ROWS + ablk * R, rc, lane);
-        lds_rows<T, R>(stage + 2 * ROWS + ablk * R, rd, lane);
-        if constexpr (RAW) lds_rows<T, R>(stage + 3 * ROWS + ablk * R, rb, lane);
-        if (i0 < g0 || i0 + R > gt) {  // rows outside the TMA range: global tail or identity
-#pragma unroll
-            for (int v = 0; v < R; ++v) {
-                const int64_t row = i0 + v;
-                if (row < 0 || row >= L) {
-                    ra[v] = T(0);
-                    rc[v] = T(0);
-                    rd[v] = T(0);
-                    if constexpr (RAW) rb[v] = T(1);
-                } else if (row >= gt) {
-                    const int64_t o = sigma * A.in_stride + row;
-                    ra[v] = A.a[o];
-                    rc[v] = A.c[o];
-                    rd[v] = A.d[o];
-                    if constexpr (RAW) rb[v] = A.b[o];
+        const int64_t ws = t0 - HEAD;  // window start row
+        if (ws <= 0 || ws + ROWS >= L || g0 > ws || gt < ws + ROWS) {
+            // CTA-uniform: patch the stage where the window leaves the TMA range --
+            // identity rows outside [0, L), the tail rows by LDG, and (first pass)
+            // a_0 = c_{n-1} = 0 -- so the register loads below need no branch
+            for (int s = t; s < ROWS; s += S::NT) {
+                const int64_t row = ws + s;
+                const bool ident = row < 0 || row >= L, tail = !ident && (row < g0 || row >= gt);
+                if (!(ident || tail || (RAW && (row == 0 || row == L - 1)))) continue;
+                const int o = sw_off<T>(s);
+                T va = stage[o], vc = stage[STG + o], vd = stage[2 * STG + o], vb = RAW ? stage[3 * STG + o] : T(1);
+                if (ident) {
+                    va = vc = vd = T(0);
+                    vb = T(1);
+                } else if (tail) {
+                    const int64_t g = sigma * A.in_stride + row;
+                    va = A.a[g];
+                    vc = A.c[g];
+                    vd = A.d[g];
+                    if constexpr (RAW) vb = A.b[g];
                 }
+                if (RAW && row == 0) va = T(0);
+                if (RAW && row == L - 1) vc = T(0);
+                stage[o] = va;
+                stage[STG + o] = vc;
+                stage[2 * STG + o] = vd;
+                if constexpr (RAW) stage[3 * STG + o] = vb;
             }
+            asm volatile("fence.proxy.async.shared::cta;" ::: "memory");  // before the next TMA refill
+            __syncthreads();
         }
-        __syncthreads();  // the stage is consumed: prefetch the next tile
-        if (t == 0) issue(w + gridDim.x);
+        const int64_t i0 = ws + int64_t(ablk) * R;  // first row of this thread (layout A)
+        T ra[R], rc[R], rd[R];
+        lds_rows_sw<T, R>(stage + 0 * STG, ablk * R, ra);
+        lds_rows_sw<T, R>(stage + 1 * STG, ablk * R, rc);
+        lds_rows_sw<T, R>(stage + 2 * STG, ablk * R, rd);
         if constexpr (RAW) {
-            if (i0 <= 0 || i0 + R >= L) {  // a_0 and c_{n-1} are outside the system
-#pragma unroll
-                for (int v = 0; v < R; ++v) {
-                    if (i0 + v == 0) ra[v] = T(0);
-                    if (i0 + v == L - 1) rc[v] = T(0);
-                }
-            }
+            T rb[R];
+            lds_rows_sw<T, R>(stage + 3 * STG, ablk * R, rb);
             if constexpr (sizeof(T) == 4) {
 #pragma unroll
                 for (int v = 0; v < R; v += 2) {
@@ -165,6 +188,8 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
                 }
             }
         }
+        __syncthreads();  // the stage is consumed: prefetch the next tile
+        if (t == 0) issue(w + gridDim.x);
         if constexpr (KP >= 1) reg_level_w<T, R, 1, 32>(ra, rc, rd);
         if constexpr (KP >= 2) reg_level_w<T, R, 2, 32>(ra, rc, rd);
         if constexpr (KP >= 3) reg_level_w<T, R, 4, 32>(ra, rc, rd);
@@ -276,19 +301,36 @@ template <typename T, int KP, bool RAW>
 static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_len, cudaStream_t st) {
     using S = SplitShape<KP>;
     auto kern = split_pipe_kernel<T, KP, RAW>;
-    constexpr int NTR = KP > 4 ? (sizeof(T) == 4 ? 3 : 1) : 0;
-    const size_t smem = (size_t((RAW ? 4 : 3)) * S::ROWS + size_t(NTR) * S::AV * 16) * sizeof(T);
+    const size_t smem = S::template smem_bytes<T>(RAW);
     cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     if (e != cudaSuccess) return e;
     const int64_t tps = (max_len + S::TV - 1) / S::TV;
     const int64_t nitems = m_in * tps;
     if (nitems <= 0) return cudaSuccess;
+    // every input slot holds at least n >> kprev rows: that many full lines go by TMA
+    const int kprev = RAW ? 0 : [&] {
+        int k = 0;
+        for (int p = 0; p < A.geom.npass; ++p) k += A.geom.kpass[p];
+        return k;
+    }();
+    constexpr int TOFF = S::template toff<T>();
+    const int64_t lmin = A.n >> kprev;
+    const int64_t tma_lines = lmin > TOFF ? (lmin - TOFF) / (128 / int64_t(sizeof(T))) : 0;
+    if (tma_lines > 0x7fffffffLL || m_in > 0x7fffffffLL) return cudaErrorInvalidConfiguration;
+    TmapSet tm{};
+    if (tma_lines > 0) {
+        const T *arrs[4] = {A.a, A.c, A.d, A.b};
+        for (int q = 0; q < (RAW ? 4 : 3); ++q)
+            if (!encode_rows_tmap(&tm.m[q], arrs[q] + TOFF, int(sizeof(T)), tma_lines, m_in, A.in_stride,
+                                  S::template box_lines<T>()))
+                return cudaErrorInvalidValue;
+    }
     int dev = 0, sms = 148, occ = 1;
     cudaGetDevice(&dev);
     cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
     cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, S::NT, smem);
     const int64_t grid = std::min<int64_t>(nitems, int64_t(std::max(occ, 1)) * sms);
-    kern<<<(unsigned)grid, S::NT, smem, st>>>(A, tps, nitems);
+    kern<<<(unsigned)grid, S::NT, smem, st>>>(A, tps, nitems, tm, int32_t(tma_lines));
     return cudaGetLastError();
 }
 

@@ -133,8 +133,7 @@ __device__ __forceinline__ void reg_level_w(T (&ra)[R], T (&rc)[R], T (&rd)[R]) 
                 pd = od;
             }
         }
-        return;
-    }
+    } else {
 #pragma unroll
     for (int rho = 0; rho < S; ++rho) {
         T pa = __shfl_up_sync(0xffffffffu, ra[R - S + rho], 1, W);
@@ -153,6 +152,7 @@ __device__ __forceinline__ void reg_level_w(T (&ra)[R], T (&rc)[R], T (&rd)[R]) 
             pc = oc;
             pd = od;
         }
+    }
     }
 }
 

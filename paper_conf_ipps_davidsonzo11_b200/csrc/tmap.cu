@@ -1,0 +1,37 @@
+// tmap.cu -- host-side encoding of the TMA tensor maps used by the persistent
+// kernels (pipe.cuh).  The driver entry point is resolved through the runtime
+// (cudaGetDriverEntryPoint), so libtds.so needs no link against libcuda.
+#include <cudaTypedefs.h>
+
+#include "pipe.cuh"
+
+namespace tds {
+
+static PFN_cuTensorMapEncodeTiled_v12000 encode_fn() {
+    static const PFN_cuTensorMapEncodeTiled_v12000 fn = [] {
+        void *p = nullptr;
+        cudaDriverEntryPointQueryResult q{};
+        if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &p, cudaEnableDefault, &q) != cudaSuccess ||
+            q != cudaDriverEntryPointSuccess)
+            return static_cast<PFN_cuTensorMapEncodeTiled_v12000>(nullptr);
+        return reinterpret_cast<PFN_cuTensorMapEncodeTiled_v12000>(p);
+    }();
+    return fn;
+}
+
+bool encode_rows_tmap(CUtensorMap *out, const void *base, int dsize, int64_t lines, int64_t slots, int64_t stride,
+                      int box_lines) {
+    const PFN_cuTensorMapEncodeTiled_v12000 fn = encode_fn();
+    if (!fn || lines < 1 || slots < 1 || box_lines < 1 || box_lines > 256) return false;
+    const cuuint64_t dims[3] = {cuuint64_t(128 / dsize), cuuint64_t(lines), cuuint64_t(slots)};
+    const cuuint64_t strides[2] = {128, cuuint64_t(stride) * cuuint64_t(dsize)};
+    const cuuint32_t box[3] = {cuuint32_t(128 / dsize), cuuint32_t(box_lines), 1};
+    const cuuint32_t estr[3] = {1, 1, 1};
+    const CUresult r = fn(out, dsize == 4 ? CU_TENSOR_MAP_DATA_TYPE_FLOAT32 : CU_TENSOR_MAP_DATA_TYPE_FLOAT64, 3,
+                          const_cast<void *>(base), dims, strides, box, estr, CU_TENSOR_MAP_INTERLEAVE_NONE,
+                          CU_TENSOR_MAP_SWIZZLE_128B, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
+                          CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+    return r == CUDA_SUCCESS;
+}
+
+}  // namespace tds
