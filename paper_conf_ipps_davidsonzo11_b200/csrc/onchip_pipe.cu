@@ -146,9 +146,11 @@ __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[
 }
 
 template <typename T, int R, bool WL>
-__global__ void __launch_bounds__(512, 1) onchip_pipe_kernel(const OnchipArgs<T> A, int64_t nslots) {
+__global__ void __launch_bounds__(512, 1)
+    onchip_pipe_kernel(const OnchipArgs<T> A, int64_t nslots, const __grid_constant__ TmapSet tm, int32_t tma_lines) {
     static_assert(R * sizeof(T) == 64, "pipe kernel: 64 bytes of rows per thread");
-    extern __shared__ __align__(128) unsigned char smem_raw[];
+    constexpr int ELINE = 128 / int(sizeof(T));
+    extern __shared__ __align__(1024) unsigned char smem_raw[];
     __shared__ __align__(8) uint64_t full_bar[2];
     constexpr int CR = ilog2c(R);
     const int NT = blockDim.x;
@@ -156,7 +158,7 @@ __global__ void __launch_bounds__(512, 1) onchip_pipe_kernel(const OnchipArgs<T>
     const int t = threadIdx.x, lane = t & 31, warp = t >> 5, nwarps = NT >> 5;
     const int c2 = A.tl_levels;
     const int Z = NT >> c2;
-    T *stage0 = reinterpret_cast<T *>(smem_raw);  // [2][3][ROWS]
+    T *stage0 = reinterpret_cast<T *>(smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u));  // [2][3][ROWS]
     T *z = stage0 + 6 * ROWS;                      // [3][Z]
     T *ya = z + 3 * Z;                             // [4][NT]
     T *yc = ya + NT, *yd = yc + NT, *yx = yd + NT;
@@ -167,19 +169,19 @@ __global__ void __launch_bounds__(512, 1) onchip_pipe_kernel(const OnchipArgs<T>
         const int64_t r = slot_residue(sigma & (KK - 1), A.geom.npass, A.geom.kpass);
         return r < A.n ? (A.n - r + KK - 1) >> A.K : 0;
     };
+    const int64_t tma_rows = int64_t(tma_lines) * ELINE;  // rows of every slot in whole TMA lines
     auto issue = [&](int64_t sigma, int s) {  // thread 0 only
         if (sigma >= nslots) return;
-        const int64_t L = slot_len(sigma);
-        const uint32_t bytes = uint32_t(((L * sizeof(T)) + 15) & ~int64_t(15));
         uint64_t *bar = &full_bar[s];
-        mbar_expect_tx(bar, 3 * bytes);
-        if (bytes) {
-            T *dst = stage0 + size_t(s) * 3 * ROWS;
-            const int64_t o = sigma * A.slot;
-            bulk_g2s(dst, A.a + o, bytes, bar);
-            bulk_g2s(dst + ROWS, A.c + o, bytes, bar);
-            bulk_g2s(dst + 2 * ROWS, A.d + o, bytes, bar);
+        if (tma_lines == 0) {
+            mbar_expect_tx(bar, 0);
+            return;
         }
+        // one swizzled box of ROWS rows per array; lines past the slot are zero-filled
+        mbar_expect_tx(bar, 3 * uint32_t(ROWS) * sizeof(T));
+        T *dst = stage0 + size_t(s) * 3 * ROWS;
+#pragma unroll
+        for (int q = 0; q < 3; ++q) tma_load_lines(dst + q * ROWS, &tm.m[q], 0, int(sigma), bar);
     };
     if (t == 0) {
         mbar_init(&full_bar[0], 1);
@@ -196,21 +198,26 @@ __global__ void __launch_bounds__(512, 1) onchip_pipe_kernel(const OnchipArgs<T>
         const int s = int(it & 1);
         const int64_t L = slot_len(sigma);
         mbar_wait(&full_bar[s], uint32_t((it >> 1) & 1));
-        const T *sb = stage0 + size_t(s) * 3 * ROWS;
+        T *sb = stage0 + size_t(s) * 3 * ROWS;
+        if (L > tma_rows || tma_lines == 0) {
+            // CTA-uniform: rows [tma_rows, L) by LDG; with no TMA at all also zero the rest
+            const int64_t hi = tma_lines == 0 ? ROWS : L;
+            for (int64_t j = tma_rows + t; j < hi; j += NT) {
+                const int o = sw_off<T>(int(j));
+                const bool in = j < L;
+                const int64_t g = sigma * A.slot + j;
+                sb[o] = in ? A.a[g] : T(0);
+                sb[ROWS + o] = in ? A.c[g] : T(0);
+                sb[2 * ROWS + o] = in ? A.d[g] : T(0);
+            }
+            asm volatile("fence.proxy.async.shared::cta;" ::: "memory");  // before the next TMA refill
+            __syncthreads();
+        }
         const int64_t jt = int64_t(t) * R;
         T ra[R], rc[R], rd[R];
-        lds_rows<T, R>(sb + jt, ra, lane);
-        lds_rows<T, R>(sb + ROWS + jt, rc, lane);
-        lds_rows<T, R>(sb + 2 * ROWS + jt, rd, lane);
-        if (jt + R > L) {  // identity rows beyond the subsystem (stale shared memory)
-#pragma unroll
-            for (int v = 0; v < R; ++v) {
-                const bool in = jt + v < L;
-                ra[v] = in ? ra[v] : T(0);
-                rc[v] = in ? rc[v] : T(0);
-                rd[v] = in ? rd[v] : T(0);
-            }
-        }
+        lds_rows_sw<T, R>(sb, t * R, ra);
+        lds_rows_sw<T, R>(sb + ROWS, t * R, rc);
+        lds_rows_sw<T, R>(sb + 2 * ROWS, t * R, rd);
         __syncthreads();  // every thread has read stage s: refill it
         if (t == 0) issue(sigma + 2 * int64_t(gridDim.x), s);
         if (L == 0) continue;  // empty slot (2^K > n): uniform
@@ -373,8 +380,8 @@ __device__ __forceinline__ void reduced_solve_pipe(T *z, int Z, int NT, int t, i
 
 size_t onchip_pipe_smem_bytes(int32_t dtype, int32_t threads, int32_t R, int32_t tl_levels) {
     const int64_t rows = int64_t(threads) * R;
-    return size_t((6 * rows + 3 * (threads >> tl_levels) + 4 * int64_t(threads) + 6 * (threads / 32) + 8) *
-                  dsize(dtype));
+    return 1024 + size_t((6 * rows + 3 * (threads >> tl_levels) + 4 * int64_t(threads) + 6 * (threads / 32) + 8) *
+                         dsize(dtype));
 }
 
 template <typename T>
@@ -388,7 +395,19 @@ cudaError_t launch_onchip_pipe(const OnchipArgs<T> &A, int64_t nslots, int threa
     int occ = 1;  // smaller subsystems fit two or more persistent CTAs per SM
     cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, threads, smem);
     const int64_t grid = std::min<int64_t>(nslots, int64_t(std::max(occ, 1)) * sm_count);
-    kern<<<(unsigned)grid, threads, smem, st>>>(A, nslots);
+    // every slot holds at least n >> K rows: that many whole 128-byte lines go by TMA
+    constexpr int R = 64 / int(sizeof(T)), ELINE = 128 / int(sizeof(T));
+    const int64_t rows = int64_t(threads) * R;
+    const int64_t tma_lines = std::min<int64_t>((A.n >> A.K) / ELINE, rows / ELINE);
+    if (nslots > 0x7fffffffLL) return cudaErrorInvalidConfiguration;
+    TmapSet tm{};
+    if (tma_lines > 0) {
+        const T *arrs[3] = {A.a, A.c, A.d};
+        for (int q = 0; q < 3; ++q)
+            if (!encode_rows_tmap(&tm.m[q], arrs[q], int(sizeof(T)), tma_lines, nslots, A.slot, int(rows / ELINE)))
+                return cudaErrorInvalidValue;
+    }
+    kern<<<(unsigned)grid, threads, smem, st>>>(A, nslots, tm, int32_t(tma_lines));
     return cudaGetLastError();
 }
 
