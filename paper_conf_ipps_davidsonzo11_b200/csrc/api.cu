@@ -183,7 +183,7 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
             cudaGetDevice(&dev);
             cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
             const size_t smem = onchip_pipe_smem_bytes(I.dtype, I.onchip_threads, 1 << P.cr_levels, P.tl_levels);
-            err = launch_onchip_pipe<T>(A, I.m << P.k, I.onchip_threads, sms, smem, st);
+            err = launch_onchip_pipe<T>(A, I.m << P.k, I.onchip_threads, P.cr_levels, sms, smem, st);
         } else {
             const size_t smem = onchip_smem_bytes(I.dtype, I.onchip_threads, P.cluster, P.tl_levels);
             err = launch_onchip<T>(A, P.cr_levels, P.k == 0, grid, I.onchip_threads, smem, st);

@@ -122,16 +122,19 @@ cudaError_t launch_split_reg(const SplitArgs<T> &A, bool raw, int64_t grid, cuda
 template <typename T>
 cudaError_t launch_split_pipe(const SplitArgs<T> &A, bool raw, int64_t m_in, int64_t max_len, cudaStream_t st);
 template <typename T>
-cudaError_t launch_onchip_pipe(const OnchipArgs<T> &A, int64_t nslots, int threads, int sm_count, size_t smem,
-                               cudaStream_t st);
+cudaError_t launch_onchip_pipe(const OnchipArgs<T> &A, int64_t nslots, int threads, int cr_levels, int sm_count,
+                               size_t smem, cudaStream_t st);
 size_t onchip_pipe_smem_bytes(int32_t dtype, int32_t threads, int32_t R, int32_t tl_levels);
 
 // The persistent TMA-pipelined on-chip kernel applies to split plans (k > 0) on
-// one CTA per subsystem whose threads hold 64 bytes of rows (fp32 c = 4, fp64 c = 3).
+// one CTA per subsystem whose threads hold 64 bytes of rows per array (fp32
+// c = 4, fp64 c = 3; up to 512 threads) or 32 bytes (fp32 c = 3, fp64 c = 2;
+// up to 1024 threads).
 inline bool onchip_pipe_ok(const tds_plan_info &I) {
     const tds_params &P = I.params;
     if (P.k == 0 || P.cluster != 1) return false;
-    if ((1 << P.cr_levels) * dsize(I.dtype) != 64) return false;
+    const int rb = (1 << P.cr_levels) * dsize(I.dtype);
+    if (rb != 64 && rb != 32) return false;
     return onchip_pipe_smem_bytes(I.dtype, I.onchip_threads, 1 << P.cr_levels, P.tl_levels) + kSmemReserve + 16 <=
            size_t(232448);
 }

@@ -137,7 +137,7 @@ __device__ __forceinline__ void cluster_or_cta_sync() {
 }
 
 template <typename T, int R, int C, bool RAW>
-__global__ void __launch_bounds__(R >= 8 ? 512 : 1024) onchip_kernel(const OnchipArgs<T> A) {
+__global__ void __launch_bounds__(R * sizeof(T) >= 64 ? 512 : 1024) onchip_kernel(const OnchipArgs<T> A) {
     extern __shared__ __align__(16) unsigned char smem_raw[];
     constexpr int CR = ilog2c(R);
     constexpr int W = 16 / int(sizeof(T));  // elements per 16-byte vector

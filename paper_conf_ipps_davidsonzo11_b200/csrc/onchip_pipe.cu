@@ -146,9 +146,9 @@ __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[
 }
 
 template <typename T, int R, bool WL>
-__global__ void __launch_bounds__(512, 1)
+__global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
     onchip_pipe_kernel(const OnchipArgs<T> A, int64_t nslots, const __grid_constant__ TmapSet tm, int32_t tma_lines) {
-    static_assert(R * sizeof(T) == 64, "pipe kernel: 64 bytes of rows per thread");
+    static_assert(R * sizeof(T) == 64 || R * sizeof(T) == 32, "pipe kernel: 32 or 64 bytes of rows per thread");
     constexpr int ELINE = 128 / int(sizeof(T));
     extern __shared__ __align__(1024) unsigned char smem_raw[];
     __shared__ __align__(8) uint64_t full_bar[2];
@@ -385,19 +385,21 @@ size_t onchip_pipe_smem_bytes(int32_t dtype, int32_t threads, int32_t R, int32_t
 }
 
 template <typename T>
-cudaError_t launch_onchip_pipe(const OnchipArgs<T> &A, int64_t nslots, int threads, int sm_count, size_t smem,
-                               cudaStream_t st) {
+cudaError_t launch_onchip_pipe(const OnchipArgs<T> &A, int64_t nslots, int threads, int cr_levels, int sm_count,
+                               size_t smem, cudaStream_t st) {
     // tl_levels == 5 (CR across all 32 lanes) selects the warp-level shuffle path
-    auto kern = A.tl_levels == 5 ? onchip_pipe_kernel<T, 64 / int(sizeof(T)), true>
-                                 : onchip_pipe_kernel<T, 64 / int(sizeof(T)), false>;
+    constexpr int RW = 64 / int(sizeof(T)), RN = 32 / int(sizeof(T));
+    const bool wide = (1 << cr_levels) == RW;
+    auto kern = wide ? (A.tl_levels == 5 ? onchip_pipe_kernel<T, RW, true> : onchip_pipe_kernel<T, RW, false>)
+                     : (A.tl_levels == 5 ? onchip_pipe_kernel<T, RN, true> : onchip_pipe_kernel<T, RN, false>);
     cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     if (e != cudaSuccess) return e;
     int occ = 1;  // smaller subsystems fit two or more persistent CTAs per SM
     cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, threads, smem);
     const int64_t grid = std::min<int64_t>(nslots, int64_t(std::max(occ, 1)) * sm_count);
     // every slot holds at least n >> K rows: that many whole 128-byte lines go by TMA
-    constexpr int R = 64 / int(sizeof(T)), ELINE = 128 / int(sizeof(T));
-    const int64_t rows = int64_t(threads) * R;
+    constexpr int ELINE = 128 / int(sizeof(T));
+    const int64_t rows = int64_t(threads) * (wide ? RW : RN);
     const int64_t tma_lines = std::min<int64_t>((A.n >> A.K) / ELINE, rows / ELINE);
     if (nslots > 0x7fffffffLL) return cudaErrorInvalidConfiguration;
     TmapSet tm{};
@@ -411,7 +413,9 @@ cudaError_t launch_onchip_pipe(const OnchipArgs<T> &A, int64_t nslots, int threa
     return cudaGetLastError();
 }
 
-template cudaError_t launch_onchip_pipe<float>(const OnchipArgs<float> &, int64_t, int, int, size_t, cudaStream_t);
-template cudaError_t launch_onchip_pipe<double>(const OnchipArgs<double> &, int64_t, int, int, size_t, cudaStream_t);
+template cudaError_t launch_onchip_pipe<float>(const OnchipArgs<float> &, int64_t, int, int, int, size_t,
+                                               cudaStream_t);
+template cudaError_t launch_onchip_pipe<double>(const OnchipArgs<double> &, int64_t, int, int, int, size_t,
+                                                cudaStream_t);
 
 }  // namespace tds

@@ -139,9 +139,9 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
     const int64_t nred = cdiv(n_sub, int64_t(R) * p.cluster);
     const int64_t threads = p.split_only ? 32 : std::max<int64_t>(32, round_up(nred, 32));
     if (!p.split_only) {  // the on-chip stage must fit (a split-only plan never launches it)
-        if (threads > (R >= 8 ? kMaxOnchipThreadsWide : kMaxOnchipThreads))
+        if (threads > onchip_max_threads(R, dsize(dtype)))
             return fail(TDS_ERR_UNSUPPORTED, "subsystem too large for the on-chip kernel (n_sub / (2^c cluster) > "
-                                             "1024, or > 512 when 2^c >= 8)");
+                                             "1024, or > 512 when 2^c * sizeof(T) >= 64)");
         if (p.tl_levels < 0 || p.tl_levels > 10 || threads % (int64_t(1) << p.tl_levels))
             return fail(TDS_ERR_INVALID_ARG, "tl_levels must be in [0, 10] and 2^tl_levels must divide the CTA size");
         if (p.thomas_chains > (threads >> p.tl_levels) * p.cluster)

@@ -15,8 +15,8 @@ namespace tds {
 // Kernel limits the planner validates against.
 constexpr int kSplitQMax = 24;        // rows per thread held in registers by the split pass
 constexpr int kSmemReserve = 1024;    // per-CTA shared memory reserved by the runtime
-constexpr int kMaxOnchipThreads = 1024;     // on-chip CTA size for R <= 4
-constexpr int kMaxOnchipThreadsWide = 512;  // ... and for R >= 8 (register budget)
+constexpr int kMaxOnchipThreads = 1024;     // on-chip CTA size while R rows take <= 32 bytes per array
+constexpr int kMaxOnchipThreadsWide = 512;  // ... and with 64 bytes (register budget)
 constexpr int kMaxSplitThreads = 512;
 constexpr int kRegSplitMaxKp = 4;       // split passes with k_p <= 4 use the register kernel
 constexpr int kPipeSplitMaxKp = 8;      // ... up to 8 with 16-byte aligned rows (persistent TMA kernel)
@@ -27,6 +27,7 @@ inline int dsize(int32_t dtype) { return dtype == TDS_F64 ? 8 : 4; }
 inline int r_max(int32_t dtype) { return dtype == TDS_F64 ? 8 : 16; }
 inline int64_t cdiv(int64_t a, int64_t b) { return (a + b - 1) / b; }
 inline int64_t round_up(int64_t a, int64_t b) { return cdiv(a, b) * b; }
+inline int onchip_max_threads(int R, int ds) { return R * ds >= 64 ? kMaxOnchipThreadsWide : kMaxOnchipThreads; }
 
 // Thread-local error detail (tds_last_error).
 tds_status fail(tds_status st, const std::string &msg);

@@ -174,7 +174,7 @@ static void schedule_passes(tds_params &p, int kpmax) {
 // latency) and the most rows per thread that fit the on-chip kernel.
 static void fit_onchip(const tds_plan_info &I, const tds_device_props &props, tds_params &p) {
     const int64_t n_sub = cdiv(I.n, int64_t(1) << p.k);
-    auto cap = [](int c) { return (1 << c) >= 8 ? kMaxOnchipThreadsWide : kMaxOnchipThreads; };
+    auto cap = [&](int c) { return onchip_max_threads(1 << c, dsize(I.dtype)); };
     auto thr = [&](const tds_params &q) {
         return round_up(cdiv(n_sub, (int64_t(1) << q.cr_levels) * q.cluster), 32);
     };

@@ -1,7 +1,9 @@
 timeout 900 python -m pytest tests/test_gpu_parity.py -m gpu -x -q 2>&1 | tail -3 > gpurun_out/t_all.txt
 P='[{"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16},
-{"k_pass": [4,3], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16},
-{"k_pass": [8], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 8}]'
+{"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 3, "thomas_chains": 32},
+{"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 3, "thomas_chains": 16},
+{"k_pass": [8], "cluster": 1, "tl_levels": 5, "cr_levels": 3, "thomas_chains": 16},
+{"k_pass": [6], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16}]'
 timeout 300 python scripts/sweep.py --n 1048576 --m 16 --reps 20 --points "$P" > gpurun_out/sweep_a.txt 2>&1
-timeout 300 ncu --set full --clock-control none --import-source on -s 3 -c 1 -o gpurun_out/prof_k7d python scripts/sweep.py --n 1048576 --m 16 --reps 1 --points '[{"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16}]' > /dev/null 2>&1
+timeout 300 python scripts/sweep.py --dtype float64 --n 1048576 --m 16 --reps 10 --points '[{"k_pass": [8], "cluster": 1, "tl_levels": 5, "cr_levels": 3, "thomas_chains": 16}, {"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 2, "thomas_chains": 16}, {"k_pass": [4,4], "cluster": 1, "tl_levels": 5, "cr_levels": 3, "thomas_chains": 16}]' >> gpurun_out/sweep_a.txt 2>&1
 cat gpurun_out/t_all.txt gpurun_out/sweep_a.txt
