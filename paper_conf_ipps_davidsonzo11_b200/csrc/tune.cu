@@ -138,8 +138,11 @@ static void tune_onchip(TuneCtx &C, tds_params &best, double &t_best) {
     bool improved = true;
     while (improved && !out_of_time(C)) {
         improved = false;
-        tds_params cand[8];
+        tds_params cand[10];
         int nc = 0;
+        // the warp-level form (CR across all 32 lanes, shuffles only) is a
+        // different kernel path, not a neighbour of tl_levels = 4: try it directly
+        if (best.cluster == 1 && best.tl_levels != 5) { cand[nc] = best; cand[nc++].tl_levels = 5; }
         if (best.thomas_chains > 1) { cand[nc] = best; cand[nc++].thomas_chains /= 2; }
         cand[nc] = best; cand[nc++].thomas_chains *= 2;
         if (best.tl_levels > 0) { cand[nc] = best; cand[nc++].tl_levels -= 1; }
@@ -290,7 +293,8 @@ extern "C" tds_status tds_tune(tds_plan_t plan, void *cuda_stream, const char *c
         tune_onchip(C, best, t_best);
         // (2) stage 2->3 switch: 2x the systems at half the size (k+1), or the
         // reverse.  For each k both pass schedules are tried -- register split
-        // passes (k_p <= 4) and the seed's k_p limit -- with the smallest
+        // passes (k_p <= 4), the persistent TMA split kernel's limit (k_p <= 8)
+        // and the seed's k_p limit -- with the smallest
         // cluster that holds the subsystem; the walk tolerates two
         // non-improving steps (splitting and on-chip costs trade off unevenly).
         for (int dir : {+1, -1}) {
@@ -302,7 +306,11 @@ extern "C" tds_status tds_tune(tds_plan_t plan, void *cuda_stream, const char *c
                 if (base.k < 0 || base.k > 30 || (int64_t(1) << base.k) > 2 * I.n) break;
                 double t_step = 1e30;
                 tds_params step_best = base;
-                for (int kpmax : {std::min(kRegSplitMaxKp, std::max(I.split_kp_max, 1)), std::max(I.split_kp_max, 1)}) {
+                const int spk = std::max(I.split_kp_max, 1);
+                int kps[3] = {std::min(kRegSplitMaxKp, spk), std::min(kPipeSplitMaxKp, spk), spk};
+                for (int ki = 0; ki < 3; ++ki) {
+                    const int kpmax = kps[ki];
+                    if (ki > 0 && kpmax == kps[ki - 1]) continue;
                     tds_params cand = base;
                     schedule_passes(cand, kpmax);
                     fit_onchip(I, plan->props, cand);

@@ -1,9 +1,17 @@
-timeout 900 python -m pytest tests/test_gpu_parity.py -m gpu -x -q 2>&1 | tail -3 > gpurun_out/t_all.txt
-P='[{"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16},
-{"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 3, "thomas_chains": 32},
-{"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 3, "thomas_chains": 16},
-{"k_pass": [8], "cluster": 1, "tl_levels": 5, "cr_levels": 3, "thomas_chains": 16},
-{"k_pass": [6], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16}]'
-timeout 300 python scripts/sweep.py --n 1048576 --m 16 --reps 20 --points "$P" > gpurun_out/sweep_a.txt 2>&1
-timeout 300 python scripts/sweep.py --dtype float64 --n 1048576 --m 16 --reps 10 --points '[{"k_pass": [8], "cluster": 1, "tl_levels": 5, "cr_levels": 3, "thomas_chains": 16}, {"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 2, "thomas_chains": 16}, {"k_pass": [4,4], "cluster": 1, "tl_levels": 5, "cr_levels": 3, "thomas_chains": 16}]' >> gpurun_out/sweep_a.txt 2>&1
-cat gpurun_out/t_all.txt gpurun_out/sweep_a.txt
+P='[{"k_pass": [], "cluster": 2, "tl_levels": 2, "cr_levels": 3, "thomas_chains": 64},
+{"k_pass": [1], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16},
+{"k_pass": [2], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 8},
+{"k_pass": [3], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 4},
+{"k_pass": [2], "cluster": 1, "tl_levels": 5, "cr_levels": 3, "thomas_chains": 16}]'
+timeout 300 python scripts/sweep.py --n 16384 --m 4096 --reps 10 --points "$P" > gpurun_out/sweep_c4.txt 2>&1
+P='[{"k_pass": [3], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16},
+{"k_pass": [4], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 8},
+{"k_pass": [2], "cluster": 1, "tl_levels": 5, "cr_levels": 3, "thomas_chains": 32},
+{"k_pass": [], "cluster": 8, "tl_levels": 3, "cr_levels": 4, "thomas_chains": 64}]'
+timeout 300 python scripts/sweep.py --n 65536 --m 256 --reps 10 --points "$P" >> gpurun_out/sweep_c4.txt 2>&1
+python -c "
+import json
+for l in open('gpurun_out/sweep_c4.txt'):
+    d=json.loads(l)
+    print(d['params'], d.get('error') or (d['stage_ms'], d['total_ms'], d['geq_per_s']))
+"
