@@ -302,8 +302,19 @@ def run_tds(args):
             step()
         torch.cuda.synchronize()
 
-    # ---- timed region: K steps, events between the kernels of each step
+    # ---- timed region: K steps back to back (value, ms_per_step)
     K = args.steps
+    e_start, e_stop = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    barrier()
+    torch.cuda.synchronize()
+    e_start.record(stream)
+    for _ in range(K):
+        step()
+    e_stop.record(stream)
+    torch.cuda.synchronize()
+    barrier()
+    total_ms = e_start.elapsed_time(e_stop)
+    # ---- kernel breakdown: K more steps with events between the kernels (roofline)
     ev = [[torch.cuda.Event(enable_timing=True) for _ in range(NL + 1)] for _ in range(K)]
     barrier()
     torch.cuda.synchronize()
@@ -315,7 +326,7 @@ def run_tds(args):
     torch.cuda.synchronize()
     barrier()
     clocks = sampler.stop()
-    total_ms = ev[0][0].elapsed_time(ev[K - 1][NL])
+    breakdown_ms = ev[0][0].elapsed_time(ev[K - 1][NL]) / K
     # per kernel kind (split pass p, on-chip, placement), summed over the chunks of a step
     stage_ms = [sum(ev[i][st].elapsed_time(ev[i][st + 1]) for i in range(K) for st in range(kind, NL, S)) / K
                 for kind in range(S)]
@@ -341,6 +352,9 @@ def run_tds(args):
         "algorithmic_bytes_per_launch": abytes[dom], "share_of_step": stage_ms[dom] / sum(stage_ms),
         "per_kernel": [{"kernel": nm, "ms": ms_, "algorithmic_bytes": ab, "gbs": ab / (ms_ / 1e3) / 1e9}
                        for nm, ms_, ab in zip(names, stage_ms, abytes)],
+        "kernel_timing": "CUDA events between the kernels of K extra steps right after the timed region "
+                         f"(that region: {breakdown_ms:.4f} ms/step; timed region back to back: "
+                         f"{total_ms / K:.4f} ms/step)",
         "step": {"algorithmic_bytes": sum(abytes), "bytes_per_eq": sum(abytes) / eqs_per_step,
                  "gbs": sum(abytes) / (total_ms / K / 1e3) / 1e9,
                  "frac": sum(abytes) / (total_ms / K / 1e3) / 1e9 / hbm_peak,
