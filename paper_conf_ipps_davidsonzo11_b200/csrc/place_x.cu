@@ -90,11 +90,11 @@ __global__ void __launch_bounds__(kPlaceThreads) place_x_kernel(const PlaceArgs<
     }
 }
 
-// K >= 5: 32 residues x 64 positions per CTA through a shared-memory tile.
-// Reads are 32 runs of 64 consecutive positions (one per slot, 16-byte
-// vectors), writes are 64 runs of 32 consecutive original rows; the padded
+// K >= 5: 32 residues x 128 positions per CTA through a shared-memory tile.
+// Reads are 32 runs of 128 consecutive positions (one per slot, 16-byte
+// vectors), writes are 128 runs of 32 consecutive original rows; the padded
 // tile (stride 33) keeps both shared-memory sides at most 2-way conflicted.
-constexpr int kTileRes = 32, kTileJ = 64;
+constexpr int kTileRes = 32, kTileJ = 128;
 
 template <typename T>
 __global__ void __launch_bounds__(kPlaceThreads) place_x_tile_kernel(const PlaceArgs<T> A, int64_t jtiles,
@@ -105,10 +105,10 @@ __global__ void __launch_bounds__(kPlaceThreads) place_x_tile_kernel(const Place
     constexpr int LPW = kTileRes / E;                      // lanes per row run (write side)
     __shared__ T tile[kTileJ][kTileRes + 1];
     const int t = threadIdx.x;
-    const int64_t rtiles = (int64_t(1) << A.K) / kTileRes;
-    int64_t b = blockIdx.x;
-    const int64_t jt = b % jtiles;
-    b /= jtiles;
+    const uint32_t rtiles = uint32_t((int64_t(1) << A.K) / kTileRes);
+    uint32_t b = blockIdx.x;  // grid < 2^31: 32-bit index arithmetic
+    const uint32_t jt = b % uint32_t(jtiles);
+    b /= uint32_t(jtiles);
     const int64_t rt = b % rtiles, sys = b / rtiles;
     const int64_t j0 = jt * kTileJ, r0 = rt * kTileRes;
     const T *src = A.xs + ((sys << A.K) + r0) * A.slot + j0;

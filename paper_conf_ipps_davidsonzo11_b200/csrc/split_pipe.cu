@@ -234,6 +234,8 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
             const int rho = t >> 4, b = t & 15;
             const int mb = LEFT - 16 + 16 * b;  // member of u = 0
             const bool wr = lane >= 1 && lane <= 30;
+            int ad[R];
+            tr_read_addrs<R, AV, (LEFT - 16) & 15>(mb, rho, ad);
             if constexpr (NTR == 3) {  // one round: 3 buffers
                 if (wr) {
                     tr_write<T, R>(ra, tbuf, ablk - 1);
@@ -241,21 +243,21 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
                     tr_write<T, R>(rd, tbuf + 2 * AV * 16, ablk - 1);
                 }
                 __syncthreads();
-                tr_read<T, R, AV>(ra, tbuf, mb, rho);
-                tr_read<T, R, AV>(rc, tbuf + AV * 16, mb, rho);
-                tr_read<T, R, AV>(rd, tbuf + 2 * AV * 16, mb, rho);
+                tr_read<T, R>(ra, tbuf, ad);
+                tr_read<T, R>(rc, tbuf + AV * 16, ad);
+                tr_read<T, R>(rd, tbuf + 2 * AV * 16, ad);
             } else {  // three rounds through one buffer
                 if (wr) tr_write<T, R>(ra, tbuf, ablk - 1);
                 __syncthreads();
-                tr_read<T, R, AV>(ra, tbuf, mb, rho);
+                tr_read<T, R>(ra, tbuf, ad);
                 __syncthreads();
                 if (wr) tr_write<T, R>(rc, tbuf, ablk - 1);
                 __syncthreads();
-                tr_read<T, R, AV>(rc, tbuf, mb, rho);
+                tr_read<T, R>(rc, tbuf, ad);
                 __syncthreads();
                 if (wr) tr_write<T, R>(rd, tbuf, ablk - 1);
                 __syncthreads();
-                tr_read<T, R, AV>(rd, tbuf, mb, rho);
+                tr_read<T, R>(rd, tbuf, ad);
             }
             if constexpr (KQ >= 1) reg_level_w<T, R, 1, 16>(ra, rc, rd);
             if constexpr (KQ >= 2) reg_level_w<T, R, 2, 16>(ra, rc, rd);

@@ -170,69 +170,25 @@ __device__ __forceinline__ void tr_write(const T (&x)[R], T *buf, int m) {
     for (int v = 0; v < R; ++v) buf[tr_addr(m, v)] = x[v];
 }
 
-// buffer -> layout B: members mb .. mb+R-1 of class rho (clamped into the
-// buffer's AV blocks: the clamped members are halo garbage)
-template <typename T, int R, int AV>
-__device__ __forceinline__ void tr_read(T (&x)[R], const T *buf, int mb, int rho) {
+// buffer -> layout B: the addresses of members mb .. mb+R-1 of class rho
+// (mb even, mb mod 16 = MBLOW known at compile time, so g(mb + u) =
+// (g0 + K(u)) & 15 with a compile-time K); members outside [0, AV) -- the
+// halo lanes b = 0 / 15 -- are clamped to a valid address (halo garbage).
+template <int R, int AV, int MBLOW>
+__device__ __forceinline__ void tr_read_addrs(int mb, int rho, int (&ad)[R]) {
+    const int g0 = (mb >> 4) + (mb >> 1);
 #pragma unroll
     for (int u = 0; u < R; ++u) {
-        int m = mb + u;
-        m = m < 0 ? 0 : (m > AV - 1 ? AV - 1 : m);
-        x[u] = buf[tr_addr(m, rho)];
+        const int k = ((MBLOW + u) >> 4) + (u >> 1);
+        const int a = 16 * (mb + u) + (rho ^ ((g0 + k) & 15));
+        ad[u] = int(min(unsigned(a), unsigned(16 * AV - 1)));
     }
 }
 
-// One PCR level whose stride is TS whole threads (16*TS rows, TS in {1,2,4}):
-// row v of thread t needs row v of threads t-TS and t+TS.  Warp shuffles
-// carry all 16 rows; the TS edge lanes of each warp go through shared memory
-// (eF: [2][NW*4*3*R] first TS lanes, eB: last TS lanes; the two halves
-// alternate between levels).  In place: every neighbour value is read
-// (shuffle / smem) before the lane updates that row.
-constexpr int kFarMaxTS = 4;
-template <typename T, int R, int TS, int NW>
-__device__ __forceinline__ void reg_level_far(T (&ra)[R], T (&rc)[R], T (&rd)[R], T *eF, T *eB, int bsel, int lane,
-                                              int warp) {
-    static_assert(TS <= kFarMaxTS, "far level: thread stride <= 4");
-    auto E = [&](T *e, int w, int l, int arr, int v) -> T & {
-        return e[bsel * (NW * kFarMaxTS * 3 * R) + (((w * TS + l) * 3) + arr) * R + v];
-    };
-    if (lane < TS) {
+template <typename T, int R>
+__device__ __forceinline__ void tr_read(T (&x)[R], const T *buf, const int (&ad)[R]) {
 #pragma unroll
-        for (int v = 0; v < R; ++v) {
-            E(eF, warp, lane, 0, v) = ra[v];
-            E(eF, warp, lane, 1, v) = rc[v];
-            E(eF, warp, lane, 2, v) = rd[v];
-        }
-    }
-    if (lane >= 32 - TS) {
-#pragma unroll
-        for (int v = 0; v < R; ++v) {
-            E(eB, warp, lane - (32 - TS), 0, v) = ra[v];
-            E(eB, warp, lane - (32 - TS), 1, v) = rc[v];
-            E(eB, warp, lane - (32 - TS), 2, v) = rd[v];
-        }
-    }
-    __syncthreads();
-    const bool hp = warp > 0, hn = warp < NW - 1;
-    const int wp = hp ? warp - 1 : 0, wn = hn ? warp + 1 : 0;
-#pragma unroll
-    for (int v = 0; v < R; ++v) {
-        T al = __shfl_up_sync(0xffffffffu, ra[v], TS), cl = __shfl_up_sync(0xffffffffu, rc[v], TS),
-          dl = __shfl_up_sync(0xffffffffu, rd[v], TS);
-        T ar = __shfl_down_sync(0xffffffffu, ra[v], TS), cr = __shfl_down_sync(0xffffffffu, rc[v], TS),
-          dr = __shfl_down_sync(0xffffffffu, rd[v], TS);
-        if (lane < TS) {  // thread t-TS is lane 32-TS+lane of the previous warp
-            al = hp ? E(eB, wp, lane, 0, v) : T(0);
-            cl = hp ? E(eB, wp, lane, 1, v) : T(0);
-            dl = hp ? E(eB, wp, lane, 2, v) : T(0);
-        }
-        if (lane >= 32 - TS) {  // thread t+TS is lane lane+TS-32 of the next warp
-            ar = hn ? E(eF, wn, lane - (32 - TS), 0, v) : T(0);
-            cr = hn ? E(eF, wn, lane - (32 - TS), 1, v) : T(0);
-            dr = hn ? E(eF, wn, lane - (32 - TS), 2, v) : T(0);
-        }
-        row_update(ra[v], rc[v], rd[v], al, cl, dl, ar, cr, dr);
-    }
+    for (int u = 0; u < R; ++u) x[u] = buf[ad[u]];
 }
 
 }  // namespace tds

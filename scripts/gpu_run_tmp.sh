@@ -1,7 +1,11 @@
-nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm,power.draw --format=csv > gpurun_out/gpu_info.txt
-bash scripts/gpu_prof.sh r01c3 --config 3
-python bench.py --impl reference --steps 3 --warmup 1 > gpurun_out/bench_ref.json 2>&1
-python bench.py --config 2 --steps 30 --warmup 3 --no-cpu-baseline > gpurun_out/bench_cfg2.json 2>&1
-python bench.py --config 4 --steps 20 --warmup 3 --no-cpu-baseline > gpurun_out/bench_cfg4.json 2>&1
-python bench.py --config 1 --steps 200 --warmup 10 --no-cpu-baseline > gpurun_out/bench_cfg1.json 2>&1
-python bench.py --config 3 --dtype f64 --steps 20 --warmup 3 --no-cpu-baseline > gpurun_out/bench_cfg3_f64.json 2>&1
+timeout 900 python -m pytest tests/test_gpu_parity.py -m gpu -x -q 2>&1 | tail -2 > gpurun_out/t_all.txt
+P='[{"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16},
+{"k_pass": [8], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 8},
+{"k_pass": [6], "cluster": 2, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16}]'
+timeout 300 python scripts/sweep.py --n 1048576 --m 16 --reps 20 --points "$P" > gpurun_out/sweep_a.txt 2>&1
+cat gpurun_out/t_all.txt; python -c "
+import json
+for l in open('gpurun_out/sweep_a.txt'):
+    d=json.loads(l)
+    print(d['params'], d.get('error') or (d['stage_ms'], d['total_ms'], d['geq_per_s']))
+"
