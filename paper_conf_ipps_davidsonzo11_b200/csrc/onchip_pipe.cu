@@ -55,9 +55,13 @@ __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[
 #pragma unroll
         for (int v = (1 << l) - 1; v < R; v += (1 << l)) {
             const bool last = v == R - 1;
-            if (!(last && lane == 31))
-                row_update(ra[v], rc[v], rd[v], ra[v - s], rc[v - s], rd[v - s], last ? na : ra[(v + s) % R],
-                           last ? nc : rc[(v + s) % R], last ? nd : rd[(v + s) % R]);
+            T a = ra[v], c = rc[v], d = rd[v];
+            row_update(a, c, d, ra[v - s], rc[v - s], rd[v - s], last ? na : ra[(v + s) % R],
+                       last ? nc : rc[(v + s) % R], last ? nd : rd[(v + s) % R]);
+            const bool keep = last && lane == 31;  // select, not branch: no divergence
+            ra[v] = keep ? ra[v] : a;
+            rc[v] = keep ? rc[v] : c;
+            rd[v] = keep ? rd[v] : d;
         }
     }
     // CR across lanes; lane 31 (kept at every level) defers
@@ -80,7 +84,12 @@ __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[
             f[1] = zc;
             f[2] = zd;
         }
-        if ((lane & ((1 << l) - 1)) == (1 << l) - 1 && lane != 31) row_update(za, zc, zd, la, lc, ld, xa, xc, xd);
+        T na2 = za, nc2 = zc, nd2 = zd;
+        row_update(na2, nc2, nd2, la, lc, ld, xa, xc, xd);
+        const bool upd = (lane & ((1 << l) - 1)) == (1 << l) - 1 && lane != 31;
+        za = upd ? na2 : za;
+        zc = upd ? nc2 : zc;
+        zd = upd ? nd2 : zd;
     }
     __syncthreads();
     if (lane == 31) {  // the deferred chains, with the next warp's published rows
@@ -129,7 +138,8 @@ __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[
         const int s = 1 << (l - 1);
         const T xl = __shfl_up_sync(FULL, xw, s);
         const T xr = __shfl_down_sync(FULL, xw, s);
-        if ((lane & ((1 << l) - 1)) == s - 1) xw = zd - za * (lane >= s ? xl : xprev) - zc * xr;
+        const T xn = zd - za * (lane >= s ? xl : xprev) - zc * xr;
+        xw = (lane & ((1 << l) - 1)) == s - 1 ? xn : xw;
     }
     T xleft = __shfl_up_sync(FULL, xw, 1);
     if (lane == 0) xleft = xprev;
