@@ -36,8 +36,10 @@ struct SplitShape {
     static constexpr int AV = 30 * NW;          // valid A-blocks per window
     static constexpr int ROWS = (AV + 2) * R;   // window rows (A-blocks 0 .. AV+1)
     static constexpr int KQ = KP > 4 ? KP - 4 : 0;
-    static constexpr int LEFT = KP > 4 ? (1 << KQ) : 0;                   // B halo members before the output
-    static constexpr int NB = KP > 4 ? (AV + 1 - (2 << KQ)) / 16 : 0;     // B blocks stored
+    // B halo members before the output (>= 2^KQ - 1 rows of garbage reach; a
+    // multiple of 4 so layout-B reads are whole 16-byte chunks)
+    static constexpr int LEFT = KP > 4 ? ((1 << KQ) > 4 ? (1 << KQ) : 4) : 0;
+    static constexpr int NB = KP > 4 ? (AV + 1 - LEFT - (1 << KQ)) / 16 : 0;  // B blocks stored
     static constexpr int TV = KP > 4 ? NB * 16 * R : AV * R;              // output rows per tile
     static constexpr int HEAD = R + LEFT * R;                             // window rows before the tile
     static_assert(TV % (1 << KP) == 0, "tile must hold whole residue periods");
@@ -234,19 +236,22 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
             const int rho = t >> 4, b = t & 15;
             const int mb = LEFT - 16 + 16 * b;  // member of u = 0
             const bool wr = lane >= 1 && lane <= 30;
-            int ad[R];
-            tr_read_addrs<R, AV, (LEFT - 16) & 15>(mb, rho, ad);
-            if constexpr (NTR == 3) {  // one round: 3 buffers
+            if constexpr (NTR == 3) {  // fp32, one round: 3 class-major buffers [rho][m]
                 if (wr) {
-                    tr_write<T, R>(ra, tbuf, ablk - 1);
-                    tr_write<T, R>(rc, tbuf + AV * 16, ablk - 1);
-                    tr_write<T, R>(rd, tbuf + 2 * AV * 16, ablk - 1);
+                    const int pm = trc_phys(ablk - 1);
+                    trc_write<T, R, AV>(ra, tbuf + pm);
+                    trc_write<T, R, AV>(rc, tbuf + AV * 16 + pm);
+                    trc_write<T, R, AV>(rd, tbuf + 2 * AV * 16 + pm);
                 }
                 __syncthreads();
-                tr_read<T, R>(ra, tbuf, ad);
-                tr_read<T, R>(rc, tbuf + AV * 16, ad);
-                tr_read<T, R>(rd, tbuf + 2 * AV * 16, ad);
-            } else {  // three rounds through one buffer
+                int ch[R / 4];
+                trc_read_chunks<R, AV>(mb, ch);
+                trc_read<R>(ra, tbuf + rho * AV, ch);
+                trc_read<R>(rc, tbuf + AV * 16 + rho * AV, ch);
+                trc_read<R>(rd, tbuf + 2 * AV * 16 + rho * AV, ch);
+            } else {
+                int ad[R];
+                tr_read_addrs<R, AV, (LEFT - 16) & 15>(mb, rho, ad);  // three rounds through one buffer
                 if (wr) tr_write<T, R>(ra, tbuf, ablk - 1);
                 __syncthreads();
                 tr_read<T, R>(ra, tbuf, ad);

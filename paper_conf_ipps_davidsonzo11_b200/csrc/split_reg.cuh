@@ -185,6 +185,41 @@ __device__ __forceinline__ void tr_read_addrs(int mb, int rho, int (&ad)[R]) {
     }
 }
 
+// fp32 class-major transpose buffer [rho][m] (row stride AV): member m of
+// class rho at rho*AV + 4*((m >> 2) ^ ((m >> 5) & 3)) + (m & 3).  Layout-A
+// writes are 16 scalar stores at immediate offsets (consecutive m across the
+// warp, <= 2-way conflicts); layout-B reads are 4 LDS.128 of 4 consecutive
+// members each, conflict-free across the 16 lanes of a class.
+__device__ __forceinline__ int trc_phys(int m) { return (((m >> 2) ^ ((m >> 5) & 3)) << 2) | (m & 3); }
+
+template <typename T, int R, int AV>
+__device__ __forceinline__ void trc_write(const T (&x)[R], T *p) {  // p = buf + trc_phys(m)
+#pragma unroll
+    for (int v = 0; v < R; ++v) p[v * AV] = x[v];
+}
+
+// chunk offsets of members mb + 4q (mb a multiple of 4), clamped into [0, AV)
+template <int R, int AV>
+__device__ __forceinline__ void trc_read_chunks(int mb, int (&ch)[R / 4]) {
+#pragma unroll
+    for (int q = 0; q < R / 4; ++q) {
+        const int c = min(unsigned(mb / 4 + q), unsigned(AV / 4 - 1));  // halo lanes: clamp
+        ch[q] = (c ^ ((c >> 3) & 3)) << 2;
+    }
+}
+
+template <int R>
+__device__ __forceinline__ void trc_read(float (&x)[R], const float *row, const int (&ch)[R / 4]) {
+#pragma unroll
+    for (int q = 0; q < R / 4; ++q) {
+        const float4 f = *reinterpret_cast<const float4 *>(row + ch[q]);
+        x[4 * q] = f.x;
+        x[4 * q + 1] = f.y;
+        x[4 * q + 2] = f.z;
+        x[4 * q + 3] = f.w;
+    }
+}
+
 template <typename T, int R>
 __device__ __forceinline__ void tr_read(T (&x)[R], const T *buf, const int (&ad)[R]) {
 #pragma unroll

@@ -1,11 +1,3 @@
-timeout 900 python -m pytest tests/test_gpu_parity.py -m gpu -x -q 2>&1 | tail -2 > gpurun_out/t_all.txt
-P='[{"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16},
-{"k_pass": [8], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 8},
-{"k_pass": [6], "cluster": 2, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16}]'
-timeout 300 python scripts/sweep.py --n 1048576 --m 16 --reps 20 --points "$P" > gpurun_out/sweep_a.txt 2>&1
-cat gpurun_out/t_all.txt; python -c "
-import json
-for l in open('gpurun_out/sweep_a.txt'):
-    d=json.loads(l)
-    print(d['params'], d.get('error') or (d['stage_ms'], d['total_ms'], d['geq_per_s']))
-"
+P='[{"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16}]'
+timeout 300 ncu --set full --clock-control none --import-source on -s 3 -c 3 -o gpurun_out/prof_cur python scripts/sweep.py --n 1048576 --m 16 --reps 1 --points "$P" > /dev/null 2>&1
+ls gpurun_out

@@ -37,7 +37,12 @@ def sass_samples(rep, kfilter=""):
         if len(r) > si and r[si].isdigit():
             body.append(r)
     base = int(body[0][0], 16)
-    return name, [(int(r[0], 16) - base, int(r[si]), r[h.index("Source")].strip()) for r in body]
+    stall_cols = [(i, c[len("stall_"):]) for i, c in enumerate(h) if c.startswith("stall_") and "Not Issued" not in c]
+    out = []
+    for r in body:
+        st = {nm: int(r[i]) for i, nm in stall_cols if i < len(r) and r[i].isdigit() and int(r[i]) > 0}
+        out.append((int(r[0], 16) - base, int(r[si]), r[h.index("Source")].strip(), st))
+    return name, out
 
 
 def line_table(mangled_substr):
@@ -75,14 +80,18 @@ def main():
     funcs = collections.defaultdict(dict)
     for (fn, off), ln in table.items():
         funcs[fn][off] = ln
-    best = max(funcs, key=lambda fn: sum(1 for off, _, _ in samples if off in funcs[fn])) if funcs else None
+    best = max(funcs, key=lambda fn: sum(1 for off, _, _, _ in samples if off in funcs[fn])) if funcs else None
     agg = collections.Counter()
-    tot = sum(s for _, s, _ in samples) or 1
-    for off, s, _ in samples:
-        agg[funcs[best].get(off, "?") if best else "?"] += s
+    why = collections.defaultdict(collections.Counter)
+    tot = sum(s for _, s, _, _ in samples) or 1
+    for off, s, _, st in samples:
+        ln = funcs[best].get(off, "?") if best else "?"
+        agg[ln] += s
+        why[ln].update(st)
     print(f"{name[:90]}  ({best})")
     for ln, s in agg.most_common(top):
-        print(f"  {s / tot * 100:5.1f}%  {ln}")
+        w = ", ".join(f"{k} {v * 100 // max(s, 1)}%" for k, v in why[ln].most_common(3))
+        print(f"  {s / tot * 100:5.1f}%  {ln:28s} {w}")
 
 
 if __name__ == "__main__":
