@@ -96,6 +96,26 @@ __device__ __forceinline__ void lds_rows_sw(const T *stage, int s0, T *v) {
     }
 }
 
+// TMA tensor store (shared -> global, bulk-group completion) of a 4-D box.
+__device__ __forceinline__ void tma_store_4d(const CUtensorMap *map, const void *src, int c0, int c1, int c2, int c3) {
+    asm volatile("cp.async.bulk.tensor.4d.global.shared::cta.bulk_group [%0, {%2, %3, %4, %5}], [%1];" ::"l"(map),
+                 "r"(smem_u32(src)), "r"(c0), "r"(c1), "r"(c2), "r"(c3)
+                 : "memory");
+}
+__device__ __forceinline__ void bulk_commit() { asm volatile("cp.async.bulk.commit_group;" ::: "memory"); }
+// the committed bulk stores have finished READING shared memory
+__device__ __forceinline__ void bulk_wait_read0() { asm volatile("cp.async.bulk.wait_group.read 0;" ::: "memory"); }
+__device__ __forceinline__ void bulk_wait_all() { asm volatile("cp.async.bulk.wait_group 0;" ::: "memory"); }
+__device__ __forceinline__ void fence_proxy_async_smem() {
+    asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+}
+
+// Host: encode the output view of a split pass -- slot (sys << (kprev + kp)) +
+// (rho << kprev) + r as the 4-D tensor {position < slot, r < nr, rho < nrho,
+// sys < msys} -- with a box of {box_pos, 1, nrho, 1}.
+bool encode_out_tmap(CUtensorMap *out, const void *base, int dsize, int64_t slot, int64_t nr, int64_t nrho,
+                     int64_t msys, int box_pos);
+
 // Host: encode the tensor map of `slots` row slots of `lines` full 128-byte
 // lines each, slot stride `stride` elements, box of `box_lines` lines.
 bool encode_rows_tmap(CUtensorMap *out, const void *base, int dsize, int64_t lines, int64_t slots, int64_t stride,

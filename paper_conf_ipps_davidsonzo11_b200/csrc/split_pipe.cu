@@ -54,17 +54,30 @@ struct SplitShape {
     __host__ __device__ static constexpr int box_lines() { return ROWS / (128 / int(sizeof(T))); }
     template <typename T>
     __host__ __device__ static constexpr int stage_elems() { return (box_lines<T>() * 128 + 1023) / 1024 * 1024 / int(sizeof(T)); }
+    // output staging for the TMA tensor store: [array][residue][position], PT
+    // positions per residue per tile (rows of PT * sizeof(T) bytes, a 16-byte multiple)
+    static constexpr int PT = TV >> KP;
+    static constexpr int BOXP = PT <= 256 ? PT : 240;  // TMA box dims are <= 256: KP <= 3 stores PT / 240 boxes
+    static constexpr int NBOX = PT / BOXP;
+    static_assert(PT % BOXP == 0, "whole boxes");
+    template <typename T>
+    __host__ __device__ static constexpr bool tstore() { return (PT * int(sizeof(T))) % 16 == 0; }
+    template <typename T>
+    __host__ __device__ static constexpr int tbuf_elems() {
+        const int tr = KP > 4 ? (sizeof(T) == 4 ? 3 : 1) * AV * 16 : 0;
+        const int so = tstore<T>() ? 3 * TV : 0;
+        return tr > so ? tr : so;
+    }
     template <typename T>
     static constexpr size_t smem_bytes(bool raw) {
-        return 1024 + (size_t(raw ? 4 : 3) * stage_elems<T>() +
-                       size_t(KP > 4 ? (sizeof(T) == 4 ? 3 : 1) : 0) * AV * 16) * sizeof(T);
+        return 1024 + (size_t(raw ? 4 : 3) * stage_elems<T>() + size_t(tbuf_elems<T>())) * sizeof(T);
     }
 };
 
 template <typename T, int KP, bool RAW>
 __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
     split_pipe_kernel(const SplitArgs<T> A, int64_t tps, int64_t nitems, const __grid_constant__ TmapSet tm,
-                      int32_t tma_lines) {
+                      int32_t tma_lines, const __grid_constant__ TmapSet tmo) {
     using S = SplitShape<KP>;
     constexpr int R = S::R, AV = S::AV, TV = S::TV, HEAD = S::HEAD, ROWS = S::ROWS;
     constexpr int TOFF = S::template toff<T>(), BL = S::template box_lines<T>(), ELINE = 128 / int(sizeof(T));
@@ -74,7 +87,11 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
     constexpr int NTR = KP > 4 ? (sizeof(T) == 4 ? 3 : 1) : 0;  // arrays per transpose round
     extern __shared__ __align__(1024) unsigned char smem_raw[];
     T *stage = reinterpret_cast<T *>(smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u));  // 1024-aligned
-    T *tbuf = stage + NA * STG;                                // [NTR][AV * 16] transpose buffer
+    T *tbuf = stage + NA * STG;  // [NTR][AV * 16] transpose buffer / [3][TV] output staging
+    constexpr bool TSTORE = S::template tstore<T>();
+    constexpr int PT = S::PT, BOXP = S::BOXP, NBOX = S::NBOX, NRES = 1 << KP;
+    // staging index of (residue rr, tile position p): [box][residue][BOXP]
+    auto sidx = [](int rr, int p) { return (p / BOXP) * (NRES * BOXP) + rr * BOXP + p % BOXP; };
     __shared__ __align__(8) uint64_t bar;
     const int t = threadIdx.x, lane = t & 31, warp = t >> 5;
     const int ablk = 30 * warp + lane;  // A-block of this thread
@@ -113,6 +130,22 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
         const int line0 = int((t0 - HEAD - TOFF) / ELINE);  // exact: TV and HEAD + TOFF are whole lines
 #pragma unroll
         for (int q = 0; q < NA; ++q) tma_load_lines(stage + q * STG, &tm.m[q], line0, int(sigma), &bar);
+    };
+    // the tile's outputs, staged in tbuf as [array][residue][position], leave by one
+    // TMA tensor store per array: box {PT positions, 1, 2^KP residues, 1} of the
+    // output view {position, r < 2^kprev, rho < 2^KP, system}
+    auto tma_store_tile = [&](int64_t sigma, int64_t t0, int kp_prev) {
+        fence_proxy_async_smem();  // generic-proxy smem writes -> visible to the TMA
+        __syncthreads();
+        if (t == 0) {
+            const int j0 = int(t0 >> KP), r = int(sigma & ((int64_t(1) << kp_prev) - 1)), sys = int(sigma >> kp_prev);
+#pragma unroll
+            for (int q = 0; q < 3; ++q)
+#pragma unroll
+                for (int bx = 0; bx < NBOX; ++bx)
+                    tma_store_4d(&tmo.m[q], tbuf + q * TV + bx * NRES * BOXP, j0 + bx * BOXP, r, 0, sys);
+            bulk_commit();
+        }
     };
     if (t == 0) {
         mbar_init(&bar, 1);
@@ -190,13 +223,36 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
                 }
             }
         }
+        if constexpr (TSTORE) {
+            if (t == 0) bulk_wait_read0();  // the previous tile's TMA store has read tbuf
+        }
         __syncthreads();  // the stage is consumed: prefetch the next tile
         if (t == 0) issue(w + gridDim.x);
         if constexpr (KP >= 1) reg_level_w<T, R, 1, 32>(ra, rc, rd);
         if constexpr (KP >= 2) reg_level_w<T, R, 2, 32>(ra, rc, rd);
         if constexpr (KP >= 3) reg_level_w<T, R, 4, 32>(ra, rc, rd);
         if constexpr (KP >= 4) reg_level_w<T, R, 8, 32>(ra, rc, rd);
-        if constexpr (KP <= 4) {
+        if constexpr (KP <= 4 && TSTORE) {
+            constexpr int NR = 1 << KP, G = R >> KP;
+            if (lane >= 1 && lane <= 30) {  // residue rr, positions 16(a-1)/2^KP + u
+                const int p0 = (16 * (ablk - 1)) >> KP;
+#pragma unroll
+                for (int rr = 0; rr < NR; ++rr) {
+                    T va[G], vc[G], vd[G];
+#pragma unroll
+                    for (int u = 0; u < G; ++u) {
+                        va[u] = ra[rr + NR * u];
+                        vc[u] = rc[rr + NR * u];
+                        vd[u] = rd[rr + NR * u];
+                    }
+                    const int o = sidx(rr, p0);  // G | BOXP: a run never crosses a box
+                    store_run<T, G>(tbuf + o, va);
+                    store_run<T, G>(tbuf + TV + o, vc);
+                    store_run<T, G>(tbuf + 2 * TV + o, vd);
+                }
+            }
+            tma_store_tile(sigma, t0, kprev);
+        } else if constexpr (KP <= 4) {
             constexpr int NR = 1 << KP, G = R >> KP;
             if (lane >= 1 && lane <= 30 && i0 < L) {
                 const bool full = i0 + R <= L;
@@ -269,6 +325,27 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
             if constexpr (KQ >= 3) reg_level_w<T, R, 4, 16>(ra, rc, rd);
             if constexpr (KQ >= 4) reg_level_w<T, R, 8, 16>(ra, rc, rd);
             // member LEFT + 16(b-1) + u is row t0 + 16(16(b-1) + u) + rho
+            if constexpr (TSTORE) {
+                __syncthreads();  // every layout-B read of tbuf is done: reuse it as the staging buffer
+                if (b >= 1 && b <= NB) {
+#pragma unroll
+                    for (int mu = 0; mu < NQ; ++mu) {  // residue rho + 16 mu, positions G(b-1) + q
+                        T va[G], vc[G], vd[G];
+#pragma unroll
+                        for (int q = 0; q < G; ++q) {
+                            va[q] = ra[mu + NQ * q];
+                            vc[q] = rc[mu + NQ * q];
+                            vd[q] = rd[mu + NQ * q];
+                        }
+                        const int o = sidx(rho + 16 * mu, G * (b - 1));
+                        store_run<T, G>(tbuf + o, va);
+                        store_run<T, G>(tbuf + TV + o, vc);
+                        store_run<T, G>(tbuf + 2 * TV + o, vd);
+                    }
+                }
+                tma_store_tile(sigma, t0, kprev);
+                continue;
+            }
             const int64_t r0 = t0 + 256 * (b - 1) + rho;  // row of u = 0
             if (b >= 1 && b <= NB && r0 < L) {
                 const bool full = r0 + 16 * (R - 1) < L;
@@ -302,6 +379,9 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
             }
         }
     }
+    if constexpr (TSTORE) {
+        if (t == 0) bulk_wait_all();
+    }
 }
 
 template <typename T, int KP, bool RAW>
@@ -332,12 +412,21 @@ static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_le
                                   S::template box_lines<T>()))
                 return cudaErrorInvalidValue;
     }
+    TmapSet tmo{};
+    if constexpr (S::template tstore<T>()) {  // output view {position, r, rho, system}
+        T *outs[3] = {A.oa, A.oc, A.od};
+        const int64_t msys = m_in >> kprev;
+        for (int q = 0; q < 3; ++q)
+            if (!encode_out_tmap(&tmo.m[q], outs[q], int(sizeof(T)), A.out_slot, int64_t(1) << kprev, int64_t(1) << KP,
+                                 msys, S::BOXP))
+                return cudaErrorInvalidValue;
+    }
     int dev = 0, sms = 148, occ = 1;
     cudaGetDevice(&dev);
     cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
     cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, S::NT, smem);
     const int64_t grid = std::min<int64_t>(nitems, int64_t(std::max(occ, 1)) * sms);
-    kern<<<(unsigned)grid, S::NT, smem, st>>>(A, tps, nitems, tm, int32_t(tma_lines));
+    kern<<<(unsigned)grid, S::NT, smem, st>>>(A, tps, nitems, tm, int32_t(tma_lines), tmo);
     return cudaGetLastError();
 }
 

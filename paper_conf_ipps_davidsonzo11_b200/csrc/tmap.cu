@@ -34,4 +34,20 @@ bool encode_rows_tmap(CUtensorMap *out, const void *base, int dsize, int64_t lin
     return r == CUDA_SUCCESS;
 }
 
+bool encode_out_tmap(CUtensorMap *out, const void *base, int dsize, int64_t slot, int64_t nr, int64_t nrho,
+                     int64_t msys, int box_pos) {
+    const PFN_cuTensorMapEncodeTiled_v12000 fn = encode_fn();
+    if (!fn || slot < 1 || nr < 1 || nrho < 1 || nrho > 256 || msys < 1 || box_pos < 1 || box_pos > 256) return false;
+    const cuuint64_t ds = cuuint64_t(dsize);
+    const cuuint64_t dims[4] = {cuuint64_t(slot), cuuint64_t(nr), cuuint64_t(nrho), cuuint64_t(msys)};
+    const cuuint64_t strides[3] = {cuuint64_t(slot) * ds, cuuint64_t(slot * nr) * ds, cuuint64_t(slot * nr * nrho) * ds};
+    const cuuint32_t box[4] = {cuuint32_t(box_pos), 1, cuuint32_t(nrho), 1};
+    const cuuint32_t estr[4] = {1, 1, 1, 1};
+    const CUresult r = fn(out, dsize == 4 ? CU_TENSOR_MAP_DATA_TYPE_FLOAT32 : CU_TENSOR_MAP_DATA_TYPE_FLOAT64, 4,
+                          const_cast<void *>(base), dims, strides, box, estr, CU_TENSOR_MAP_INTERLEAVE_NONE,
+                          CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_NONE,
+                          CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+    return r == CUDA_SUCCESS;
+}
+
 }  // namespace tds
