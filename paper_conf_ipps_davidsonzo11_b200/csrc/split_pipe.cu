@@ -223,15 +223,16 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
                 }
             }
         }
-        if constexpr (TSTORE) {
-            if (t == 0) bulk_wait_read0();  // the previous tile's TMA store has read tbuf
-        }
         __syncthreads();  // the stage is consumed: prefetch the next tile
         if (t == 0) issue(w + gridDim.x);
         if constexpr (KP >= 1) reg_level_w<T, R, 1, 32>(ra, rc, rd);
         if constexpr (KP >= 2) reg_level_w<T, R, 2, 32>(ra, rc, rd);
         if constexpr (KP >= 3) reg_level_w<T, R, 4, 32>(ra, rc, rd);
         if constexpr (KP >= 4) reg_level_w<T, R, 8, 32>(ra, rc, rd);
+        if constexpr (TSTORE) {  // tbuf is written next: the previous tile's TMA store must have read it
+            if (t == 0) bulk_wait_read0();
+            __syncthreads();
+        }
         if constexpr (KP <= 4 && TSTORE) {
             constexpr int NR = 1 << KP, G = R >> KP;
             if (lane >= 1 && lane <= 30) {  // residue rr, positions 16(a-1)/2^KP + u
