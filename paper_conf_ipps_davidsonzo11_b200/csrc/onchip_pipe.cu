@@ -180,8 +180,11 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
         return r < A.n ? (A.n - r + KK - 1) >> A.K : 0;
     };
     const int64_t tma_rows = int64_t(tma_lines) * ELINE;  // rows of every slot in whole TMA lines
-    auto issue = [&](int64_t sigma, int s) {  // thread 0 only
-        if (sigma >= nslots) return;
+    // work item q solves slot nslots-1-q: the split pass wrote the last slots
+    // last, so the first items a CTA waits for are still in L2
+    auto issue = [&](int64_t q, int s) {  // thread 0 only
+        if (q >= nslots) return;
+        const int64_t sigma = nslots - 1 - q;
         uint64_t *bar = &full_bar[s];
         if (tma_lines == 0) {
             mbar_expect_tx(bar, 0);
@@ -203,8 +206,9 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
     __syncthreads();
 
     for (int64_t it = 0;; ++it) {
-        const int64_t sigma = int64_t(blockIdx.x) + it * gridDim.x;
-        if (sigma >= nslots) break;
+        const int64_t q = int64_t(blockIdx.x) + it * gridDim.x;
+        if (q >= nslots) break;
+        const int64_t sigma = nslots - 1 - q;
         const int s = int(it & 1);
         const int64_t L = slot_len(sigma);
         mbar_wait(&full_bar[s], uint32_t((it >> 1) & 1));
@@ -229,7 +233,7 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
         lds_rows_sw<T, R>(sb + ROWS, t * R, rc);
         lds_rows_sw<T, R>(sb + 2 * ROWS, t * R, rd);
         __syncthreads();  // every thread has read stage s: refill it
-        if (t == 0) issue(sigma + 2 * int64_t(gridDim.x), s);
+        if (t == 0) issue(q + 2 * int64_t(gridDim.x), s);
         if (L == 0) continue;  // empty slot (2^K > n): uniform
 
         if constexpr (WL) {
@@ -330,7 +334,8 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
             for (int v = 0; v < R; ++v)
                 if (jt + v < L) dst[v] = rd[v];
         }
-        __syncthreads();  // y / z / edge buffers are reused by the next subsystem
+        // no barrier here: the next item's first shared-scratch write follows its
+        // stage-consumed barrier, which every thread reaches only after this item
     }
 }
 
