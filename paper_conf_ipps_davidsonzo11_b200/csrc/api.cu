@@ -122,7 +122,7 @@ static tds_status run_split(const tds_plan_info &I, const T *a, const T *b, cons
         cudaError_t err;
         if (kp <= kPipeSplitMaxKp && A.vec) {
             // persistent, TMA-prefetched register kernel (16-byte aligned rows)
-            err = launch_split_pipe<T>(A, raw, m_in, len_in, st);
+            err = launch_split_pipe<T>(A, raw, m_in, len_in, I.params.split_threads, st);
         } else if (kp <= kRegSplitMaxKp) {
             err = launch_split_reg<T>(A, raw, grid, st);
         } else {

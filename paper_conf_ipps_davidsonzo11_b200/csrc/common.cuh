@@ -120,7 +120,8 @@ cudaError_t launch_split_pass(const SplitArgs<T> &A, bool raw, int64_t grid, int
 template <typename T>
 cudaError_t launch_split_reg(const SplitArgs<T> &A, bool raw, int64_t grid, cudaStream_t st);
 template <typename T>
-cudaError_t launch_split_pipe(const SplitArgs<T> &A, bool raw, int64_t m_in, int64_t max_len, cudaStream_t st);
+cudaError_t launch_split_pipe(const SplitArgs<T> &A, bool raw, int64_t m_in, int64_t max_len, int threads,
+                              cudaStream_t st);
 template <typename T>
 cudaError_t launch_onchip_pipe(const OnchipArgs<T> &A, int64_t nslots, int threads, int cr_levels, int sm_count,
                                size_t smem, cudaStream_t st);

@@ -28,10 +28,11 @@
 
 namespace tds {
 
-template <int KP>
+template <int KP, int NT_>
 struct SplitShape {
     static constexpr int R = kRegSplitRows;
-    static constexpr int NT = kRegSplitThreads;
+    static constexpr int NT = NT_;                      // 256 (2 CTAs/SM) or 512 (1 CTA/SM, less halo)
+    static constexpr int CH = NT / 16;                  // lanes per layout-B chain (shuffle width)
     static constexpr int NW = NT / 32;
     static constexpr int AV = 30 * NW;          // valid A-blocks per window
     static constexpr int ROWS = (AV + 2) * R;   // window rows (A-blocks 0 .. AV+1)
@@ -39,7 +40,11 @@ struct SplitShape {
     // B halo members before the output (>= 2^KQ - 1 rows of garbage reach; a
     // multiple of 4 so layout-B reads are whole 16-byte chunks)
     static constexpr int LEFT = KP > 4 ? ((1 << KQ) > 4 ? (1 << KQ) : 4) : 0;
-    static constexpr int NB = KP > 4 ? (AV + 1 - LEFT - (1 << KQ)) / 16 : 0;  // B blocks stored
+    static constexpr int NBMAX = KP > 4 ? (AV + 1 - LEFT - (1 << KQ)) / 16 : 0;
+    // B blocks stored; with 512 threads rounded so a residue's positions per tile
+    // (NB * 256 / 2^KP) stay a 16-byte multiple (TMA store rows)
+    static constexpr int NBQ = (KP >= 8 ? 4 : KP == 7 ? 2 : 1);
+    static constexpr int NB = NT == 512 ? NBMAX - NBMAX % NBQ : NBMAX;
     static constexpr int TV = KP > 4 ? NB * 16 * R : AV * R;              // output rows per tile
     static constexpr int HEAD = R + LEFT * R;                             // window rows before the tile
     static_assert(TV % (1 << KP) == 0, "tile must hold whole residue periods");
@@ -74,12 +79,12 @@ struct SplitShape {
     }
 };
 
-template <typename T, int KP, bool RAW>
-__global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
+template <typename T, int KP, bool RAW, int NT>
+__global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
     split_pipe_kernel(const SplitArgs<T> A, int64_t tps, int64_t nitems, const __grid_constant__ TmapSet tm,
                       int32_t tma_lines, const __grid_constant__ TmapSet tmo) {
-    using S = SplitShape<KP>;
-    constexpr int R = S::R, AV = S::AV, TV = S::TV, HEAD = S::HEAD, ROWS = S::ROWS;
+    using S = SplitShape<KP, NT>;
+    constexpr int R = S::R, AV = S::AV, TV = S::TV, HEAD = S::HEAD, ROWS = S::ROWS, CH = S::CH;
     constexpr int TOFF = S::template toff<T>(), BL = S::template box_lines<T>(), ELINE = 128 / int(sizeof(T));
     static_assert(ROWS % ELINE == 0, "window of whole lines");
     constexpr int STG = S::template stage_elems<T>();          // elements per array stage (1024-byte multiple)
@@ -290,7 +295,7 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
             // ---- layout B: 16 consecutive members of residue class rho mod 16
             constexpr int KQ = S::KQ, LEFT = S::LEFT, NB = S::NB;
             constexpr int NQ = 1 << KQ, G = R >> KQ;
-            const int rho = t >> 4, b = t & 15;
+            const int rho = t / CH, b = t % CH;
             const int mb = LEFT - 16 + 16 * b;  // member of u = 0
             const bool wr = lane >= 1 && lane <= 30;
             if constexpr (NTR == 3) {  // fp32, one round: 3 class-major buffers [rho][m]
@@ -321,10 +326,10 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
                 __syncthreads();
                 tr_read<T, R>(rd, tbuf, ad);
             }
-            if constexpr (KQ >= 1) reg_level_w<T, R, 1, 16>(ra, rc, rd);
-            if constexpr (KQ >= 2) reg_level_w<T, R, 2, 16>(ra, rc, rd);
-            if constexpr (KQ >= 3) reg_level_w<T, R, 4, 16>(ra, rc, rd);
-            if constexpr (KQ >= 4) reg_level_w<T, R, 8, 16>(ra, rc, rd);
+            if constexpr (KQ >= 1) reg_level_w<T, R, 1, CH>(ra, rc, rd);
+            if constexpr (KQ >= 2) reg_level_w<T, R, 2, CH>(ra, rc, rd);
+            if constexpr (KQ >= 3) reg_level_w<T, R, 4, CH>(ra, rc, rd);
+            if constexpr (KQ >= 4) reg_level_w<T, R, 8, CH>(ra, rc, rd);
             // member LEFT + 16(b-1) + u is row t0 + 16(16(b-1) + u) + rho
             if constexpr (TSTORE) {
                 __syncthreads();  // every layout-B read of tbuf is done: reuse it as the staging buffer
@@ -385,10 +390,10 @@ __global__ void __launch_bounds__(kRegSplitThreads, sizeof(T) == 4 ? 2 : 1)
     }
 }
 
-template <typename T, int KP, bool RAW>
+template <typename T, int KP, bool RAW, int NT>
 static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_len, cudaStream_t st) {
-    using S = SplitShape<KP>;
-    auto kern = split_pipe_kernel<T, KP, RAW>;
+    using S = SplitShape<KP, NT>;
+    auto kern = split_pipe_kernel<T, KP, RAW, NT>;
     const size_t smem = S::template smem_bytes<T>(RAW);
     cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     if (e != cudaSuccess) return e;
@@ -432,9 +437,17 @@ static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_le
 }
 
 template <typename T>
-cudaError_t launch_split_pipe(const SplitArgs<T> &A, bool raw, int64_t m_in, int64_t max_len, cudaStream_t st) {
-#define TDS_SP(KPV) \
-    case KPV: return raw ? launch_sp<T, KPV, true>(A, m_in, max_len, st) : launch_sp<T, KPV, false>(A, m_in, max_len, st)
+cudaError_t launch_split_pipe(const SplitArgs<T> &A, bool raw, int64_t m_in, int64_t max_len, int threads,
+                              cudaStream_t st) {
+    // fp32: 512 threads (1 CTA/SM, 7.7K-row windows, less halo) when split_threads >= 512; fp64 always 256
+    constexpr int NTW = sizeof(T) == 4 ? 512 : 256;
+    const bool wide = threads >= 512;
+#define TDS_SP(KPV)                                                                                       \
+    case KPV:                                                                                             \
+        if (wide)                                                                                         \
+            return raw ? launch_sp<T, KPV, true, NTW>(A, m_in, max_len, st)                               \
+                       : launch_sp<T, KPV, false, NTW>(A, m_in, max_len, st);                             \
+        return raw ? launch_sp<T, KPV, true, 256>(A, m_in, max_len, st) : launch_sp<T, KPV, false, 256>(A, m_in, max_len, st)
     switch (A.kp) {
         TDS_SP(1);
         TDS_SP(2);
@@ -449,7 +462,7 @@ cudaError_t launch_split_pipe(const SplitArgs<T> &A, bool raw, int64_t m_in, int
 #undef TDS_SP
 }
 
-template cudaError_t launch_split_pipe<float>(const SplitArgs<float> &, bool, int64_t, int64_t, cudaStream_t);
-template cudaError_t launch_split_pipe<double>(const SplitArgs<double> &, bool, int64_t, int64_t, cudaStream_t);
+template cudaError_t launch_split_pipe<float>(const SplitArgs<float> &, bool, int64_t, int64_t, int, cudaStream_t);
+template cudaError_t launch_split_pipe<double>(const SplitArgs<double> &, bool, int64_t, int64_t, int, cudaStream_t);
 
 }  // namespace tds

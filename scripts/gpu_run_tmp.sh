@@ -1,3 +1,5 @@
-P='[{"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16}]'
-timeout 300 ncu --set full --clock-control none --import-source on -s 3 -c 3 -o gpurun_out/prof_cur python scripts/sweep.py --n 1048576 --m 16 --reps 1 --points "$P" > /dev/null 2>&1
-ls gpurun_out
+P='[{"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16, "split_threads": 256, "split_tile_rows": 4096},
+{"k_pass": [7], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 16, "split_threads": 512},
+{"k_pass": [8], "cluster": 1, "tl_levels": 5, "cr_levels": 4, "thomas_chains": 8, "split_threads": 512},
+{"k_pass": [8], "cluster": 1, "tl_levels": 5, "cr_levels": 3, "thomas_chains": 16, "split_threads": 512}]'
+SWEEP_POINTS="$P" bash scripts/gpu_test_sweep.sh

@@ -254,15 +254,20 @@ def test_split_fused_equals_multipass_and_tiles(tds):
             assert np.array_equal(u, v)
 
 
+PIPE_THREADS = [dict(split_threads=512), dict(split_threads=256, split_tile_rows=4096)]
+
+
 @pytest.mark.parametrize("dtype", [np.float32, np.float64])
 @pytest.mark.parametrize("n,kp", [(200004, [5]), (200004, [6]), (131072, [7]), (200004, [8]),
-                                  (3588 * 3 + 4, [8]), (200004, [3, 8]), (200004, [8, 2])])
-def test_split_deep_pipe_vs_oracle(tds, dtype, n, kp):
-    """k_p = 5..8 in one pass (persistent TMA split kernel, transposed layout:
-    4 levels on consecutive rows, k_p - 4 on residue classes mod 16) vs the
-    oracle's textbook PCR, on tiles with ragged tails."""
+                                  (3588 * 3 + 4, [8]), (200004, [3, 8]), (200004, [8, 2]), (300000, [2]),
+                                  (7424 * 2 + 36, [7]), (100000, [4, 4])])
+@pytest.mark.parametrize("geom", PIPE_THREADS, ids=["t512", "t256"])
+def test_split_deep_pipe_vs_oracle(tds, dtype, n, kp, geom):
+    """k_p <= 8 in one pass (persistent TMA split kernel: 4 levels on
+    consecutive rows, k_p - 4 on residue classes mod 16; 256- and 512-thread
+    tiles) vs the oracle's textbook PCR, on tiles with ragged tails."""
     a, b, c, d = inputs.generate(n, 2, dtype, seed=23)
-    ga, gc, gd, plan = split_gpu(tds, a, b, c, d, dict(k_pass=kp, split_only=1))
+    ga, gc, gd, plan = split_gpu(tds, a, b, c, d, dict(geom, k_pass=kp, split_only=1))
     k = sum(kp)
     perm = plan.permutation()
     sa, sb, sc, sd = oracle.pcr_split(a, b, c, d, k)
@@ -273,11 +278,12 @@ def test_split_deep_pipe_vs_oracle(tds, dtype, n, kp):
 
 
 @pytest.mark.parametrize("n", [1 << 20, (1 << 20) + 12344, 4100])
-def test_split_deep_fused_equals_multipass(tds, n):
+@pytest.mark.parametrize("geom", PIPE_THREADS, ids=["t512", "t256"])
+def test_split_deep_fused_equals_multipass(tds, n, geom):
     """Bit-exact: [8] == [4, 4] == [2, 2, 2, 2] and [7] == [4, 3] (the same
     normalised row update on the same operands, whatever the layout)."""
     a, b, c, d = inputs.generate(n, 2, np.float32, seed=5)
-    base = dict(split_only=1)
+    base = dict(geom, split_only=1)
     r8 = split_gpu(tds, a, b, c, d, dict(base, k_pass=[8]))
     for other in ([4, 4], [2, 2, 2, 2], [5, 3]):
         ro = split_gpu(tds, a, b, c, d, dict(base, k_pass=other))
