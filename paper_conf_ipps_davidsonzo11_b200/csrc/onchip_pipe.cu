@@ -29,9 +29,9 @@ __device__ __forceinline__ void reduced_solve_pipe(T *z, int Z, int NT, int t, i
 // are deferred until one barrier publishes the next warp's rows (lane 0's
 // row s-1 per register level, lane s-1's row per lane level; both depend on
 // nothing beyond their own warp).  5 barriers per subsystem in total.
-template <typename T, int R>
+template <typename T, int R, typename Hook>
 __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[R], T *scr, int lane, int warp,
-                                                int nwarps) {
+                                                int nwarps, Hook &&after_barrier) {
     constexpr int CR = ilog2c(R);
     constexpr unsigned FULL = 0xffffffffu;
     T *e_in = scr;                      // [nwarps][CR][3] lane 0's row s-1, level l-1
@@ -92,6 +92,7 @@ __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[
         zd = upd ? nd2 : zd;
     }
     __syncthreads();
+    after_barrier();
     if (lane == 31) {  // the deferred chains, with the next warp's published rows
         const bool h = warp + 1 < nwarps;
 #pragma unroll
@@ -182,7 +183,12 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
     const int64_t tma_rows = int64_t(tma_lines) * ELINE;  // rows of every slot in whole TMA lines
     // work item q solves slot nslots-1-q: the split pass wrote the last slots
     // last, so the first items a CTA waits for are still in L2
-    auto issue = [&](int64_t q, int s) {  // thread 0 only
+    // One swizzled box of ROWS rows per array (lines past the slot are
+    // zero-filled).  The a-region of a consumed stage first holds the item's x
+    // for the TMA store (x overwrites a in the workspace), so a stage is
+    // refilled in two steps: c and d as soon as the stage is in registers,
+    // a once the previous x store has read it.
+    auto issue_cd = [&](int64_t q, int s) {  // thread 0 only; announces all three arrays
         if (q >= nslots) return;
         const int64_t sigma = nslots - 1 - q;
         uint64_t *bar = &full_bar[s];
@@ -190,20 +196,26 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
             mbar_expect_tx(bar, 0);
             return;
         }
-        // one swizzled box of ROWS rows per array; lines past the slot are zero-filled
         mbar_expect_tx(bar, 3 * uint32_t(ROWS) * sizeof(T));
         T *dst = stage0 + size_t(s) * 3 * ROWS;
-#pragma unroll
-        for (int q = 0; q < 3; ++q) tma_load_lines(dst + q * ROWS, &tm.m[q], 0, int(sigma), bar);
+        tma_load_lines(dst + ROWS, &tm.m[1], 0, int(sigma), bar);
+        tma_load_lines(dst + 2 * ROWS, &tm.m[2], 0, int(sigma), bar);
+    };
+    auto issue_a = [&](int64_t q, int s) {  // thread 0 only
+        if (q >= nslots || tma_lines == 0) return;
+        tma_load_lines(stage0 + size_t(s) * 3 * ROWS, &tm.m[0], 0, int(nslots - 1 - q), &full_bar[s]);
     };
     if (t == 0) {
         mbar_init(&full_bar[0], 1);
         mbar_init(&full_bar[1], 1);
         asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
-        issue(blockIdx.x, 0);
-        issue(int64_t(blockIdx.x) + gridDim.x, 1);
+        issue_cd(blockIdx.x, 0);
+        issue_a(blockIdx.x, 0);
+        issue_cd(int64_t(blockIdx.x) + gridDim.x, 1);
+        issue_a(int64_t(blockIdx.x) + gridDim.x, 1);
     }
     __syncthreads();
+    int64_t pend = -1;  // slot whose x waits in the a-region of stage 1-s for its TMA store
 
     for (int64_t it = 0;; ++it) {
         const int64_t q = int64_t(blockIdx.x) + it * gridDim.x;
@@ -232,13 +244,33 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
         lds_rows_sw<T, R>(sb, t * R, ra);
         lds_rows_sw<T, R>(sb + ROWS, t * R, rc);
         lds_rows_sw<T, R>(sb + 2 * ROWS, t * R, rd);
-        __syncthreads();  // every thread has read stage s: refill it
-        if (t == 0) issue(q + 2 * int64_t(gridDim.x), s);
-        if (L == 0) continue;  // empty slot (2^K > n): uniform
+        __syncthreads();  // every thread has read stage s (and written the previous item's x)
+        if (t == 0) {
+            issue_cd(q + 2 * int64_t(gridDim.x), s);
+            if (pend >= 0) {  // the previous item's x: one tensor store from the a-region of stage 1-s
+                tma_store_lines(&tm.m[0], stage0 + size_t(1 - s) * 3 * ROWS, 0, int(pend));
+                bulk_commit();
+            }
+        }
+        const bool had_pend = pend >= 0;
+        pend = -1;
+        // once the store has read the region (checked after the solve's first
+        // barrier), stage 1-s gets its a-array for item q + G
+        auto refill_a = [&]() {
+            if (t == 0 && had_pend) {
+                bulk_wait_read0();
+                issue_a(q + int64_t(gridDim.x), 1 - s);
+            }
+        };
+        if (L == 0) {  // empty slot (2^K > n): uniform
+            refill_a();
+            continue;
+        }
 
         if constexpr (WL) {
-            solve_item_warp<T, R>(ra, rc, rd, ya, lane, warp, nwarps);
+            solve_item_warp<T, R>(ra, rc, rd, ya, lane, warp, nwarps, refill_a);
         } else {
+        refill_a();
         // ---- B1. CR forward levels in registers
 #pragma unroll
         for (int l = 1; l <= CR; ++l) {
@@ -319,7 +351,19 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
         }
         }  // !WL
         T *dst = A.xs + sigma * A.slot + jt;  // per-subsystem x (placement kernel follows)
-        if (jt + R <= L) {
+        if (tma_lines > 0) {
+            // x to the a-region of stage s (swizzled like the loads); the next
+            // item's first barrier makes it complete, then thread 0 stores it.
+            // Rows past the tensor's whole lines go straight to global memory.
+            sts_rows_sw<T, R>(sb, t * R, rd);
+            fence_proxy_async_smem();
+            if (jt + R > tma_rows) {
+#pragma unroll
+                for (int v = 0; v < R; ++v)
+                    if (jt + v >= tma_rows && jt + v < L) dst[v] = rd[v];
+            }
+            pend = sigma;
+        } else if (jt + R <= L) {
             constexpr int W = 16 / int(sizeof(T));
 #pragma unroll
             for (int q = 0; q < R / W; ++q) {
@@ -336,6 +380,16 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
         }
         // no barrier here: the next item's first shared-scratch write follows its
         // stage-consumed barrier, which every thread reaches only after this item
+    }
+    __syncthreads();  // the last item's x is complete in shared memory
+    if (t == 0) {
+        if (pend >= 0) {
+            // the stage index of the last item: it = number of items - 1
+            const int64_t nit = (nslots - int64_t(blockIdx.x) + gridDim.x - 1) / gridDim.x;
+            tma_store_lines(&tm.m[0], stage0 + size_t((nit - 1) & 1) * 3 * ROWS, 0, int(pend));
+            bulk_commit();
+        }
+        bulk_wait_all();
     }
 }
 

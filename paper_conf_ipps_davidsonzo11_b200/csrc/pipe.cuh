@@ -116,6 +116,31 @@ __device__ __forceinline__ void fence_proxy_async_smem() {
 bool encode_out_tmap(CUtensorMap *out, const void *base, int dsize, int64_t slot, int64_t nr, int64_t nrho,
                      int64_t msys, int box_pos);
 
+// R consecutive rows to stage row s0 of a swizzled stage (the inverse of lds_rows_sw).
+template <typename T, int R>
+__device__ __forceinline__ void sts_rows_sw(T *stage, int s0, const T *v) {
+    constexpr int CH = 16 / int(sizeof(T));
+    constexpr int ELINE = 128 / int(sizeof(T));
+    unsigned char *base = reinterpret_cast<unsigned char *>(stage);
+#pragma unroll
+    for (int q = 0; q < R / CH; ++q) {
+        const int row = s0 + q * CH;
+        const int line = row / ELINE, chunk = (row % ELINE) / CH;
+        unsigned char *p = base + line * 128 + ((chunk ^ (line & 7)) << 4);
+        if constexpr (sizeof(T) == 4)
+            *reinterpret_cast<float4 *>(p) = make_float4(v[4 * q], v[4 * q + 1], v[4 * q + 2], v[4 * q + 3]);
+        else
+            *reinterpret_cast<double2 *>(p) = make_double2(v[2 * q], v[2 * q + 1]);
+    }
+}
+
+// TMA tensor store of a 3-D row box (the inverse of tma_load_lines).
+__device__ __forceinline__ void tma_store_lines(const CUtensorMap *map, const void *src, int line, int slot) {
+    asm volatile("cp.async.bulk.tensor.3d.global.shared::cta.bulk_group [%0, {%2, %3, %4}], [%1];" ::"l"(map),
+                 "r"(smem_u32(src)), "r"(0), "r"(line), "r"(slot)
+                 : "memory");
+}
+
 // Host: encode the tensor map of `slots` row slots of `lines` full 128-byte
 // lines each, slot stride `stride` elements, box of `box_lines` lines.
 bool encode_rows_tmap(CUtensorMap *out, const void *base, int dsize, int64_t lines, int64_t slots, int64_t stride,
