@@ -141,6 +141,24 @@ __device__ __forceinline__ void tma_store_lines(const CUtensorMap *map, const vo
                  : "memory");
 }
 
+// 3-D box load / store with explicit coordinates (generic views).
+__device__ __forceinline__ void tma_load_box3(void *dst, const CUtensorMap *map, int c0, int c1, int c2, uint64_t *bar) {
+    asm volatile(
+        "cp.async.bulk.tensor.3d.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1, {%2, %3, %4}], [%5];" ::
+            "r"(smem_u32(dst)),
+        "l"(map), "r"(c0), "r"(c1), "r"(c2), "r"(smem_u32(bar))
+        : "memory");
+}
+__device__ __forceinline__ void tma_store_box3(const CUtensorMap *map, const void *src, int c0, int c1, int c2) {
+    asm volatile("cp.async.bulk.tensor.3d.global.shared::cta.bulk_group [%0, {%2, %3, %4}], [%1];" ::"l"(map),
+                 "r"(smem_u32(src)), "r"(c0), "r"(c1), "r"(c2)
+                 : "memory");
+}
+
+// Host: a 3-D view with the 128-byte swizzle (box inner dimension = 128 bytes).
+bool encode_box3_tmap(CUtensorMap *out, const void *base, int dsize, const uint64_t dims[3], const uint64_t strides[2],
+                      const uint32_t box[3]);
+
 // Host: encode the tensor map of `slots` row slots of `lines` full 128-byte
 // lines each, slot stride `stride` elements, box of `box_lines` lines.
 bool encode_rows_tmap(CUtensorMap *out, const void *base, int dsize, int64_t lines, int64_t slots, int64_t stride,

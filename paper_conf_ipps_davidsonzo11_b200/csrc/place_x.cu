@@ -10,7 +10,9 @@
 // of one residue have consecutive j and are one vector load, and across the
 // warp every residue run is a coalesced read; the 16 rows leave as contiguous
 // 16-byte vector stores.
-#include "common.cuh"
+#include <algorithm>
+
+#include "pipe.cuh"
 
 namespace tds {
 
@@ -162,6 +164,107 @@ __global__ void __launch_bounds__(kPlaceThreads) place_x_tile_kernel(const Place
     }
 }
 
+// K >= 5 (fp32) / 4 (fp64), 16-byte aligned rows: a persistent TMA transposer.
+// A box is E x E elements (E = 128 bytes / sizeof(T)): E positions of E
+// consecutive residue slots in (tensor view {positions, slots} of xs), E
+// residues of E consecutive j out (view {2^K, floor(n / 2^K), m} of x), both
+// with the 128-byte swizzle so the shared-memory transpose (one LDS.128 of a
+// slot's chunk, CH scalar STS into the j rows) is conflict-free.  NBX boxes
+// along j per tile; loads run two tiles ahead; stores are TMA tensor stores.
+// Rows past floor(n / 2^K) * 2^K (fewer than 2^K per system) are copied last
+// with plain loads and stores.
+constexpr int kTpBoxes = 4, kTpThreads = 256;
+
+template <typename T>
+__global__ void __launch_bounds__(kTpThreads) place_x_tma_kernel(const PlaceArgs<T> A, const __grid_constant__ TmapSet tm,
+                                                                int64_t ntiles, int64_t jtiles, int64_t lfull,
+                                                                int64_t msys) {
+    constexpr int E = 128 / int(sizeof(T)), CH = 16 / int(sizeof(T)), NBX = kTpBoxes;
+    constexpr int BOX = E * E;  // elements per box
+    extern __shared__ __align__(1024) unsigned char smem_raw[];
+    T *base = reinterpret_cast<T *>(smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u));
+    T *sin = base;                   // [2][NBX][E slots][E positions]
+    T *sout = base + 2 * NBX * BOX;  // [NBX][E j][E residues]
+    __shared__ __align__(8) uint64_t full[2];
+    const int t = threadIdx.x;
+    const int64_t rtiles = (int64_t(1) << A.K) / E;
+    auto coords = [&](int64_t w, int64_t &sys, int64_t &rt, int64_t &jt) {
+        jt = w % jtiles;
+        const int64_t q = w / jtiles;
+        rt = q % rtiles;
+        sys = q / rtiles;
+    };
+    auto issue = [&](int64_t w, int s) {  // thread 0
+        if (w >= ntiles) return;
+        int64_t sys, rt, jt;
+        coords(w, sys, rt, jt);
+        mbar_expect_tx(&full[s], NBX * BOX * sizeof(T));
+        const int slot0 = int((sys << A.K) + rt * E);
+#pragma unroll
+        for (int bx = 0; bx < NBX; ++bx)
+            tma_load_box3(sin + (s * NBX + bx) * BOX, &tm.m[0], int((jt * NBX + bx) * E), slot0, 0, &full[s]);
+    };
+    if (t == 0) {
+        mbar_init(&full[0], 1);
+        mbar_init(&full[1], 1);
+        asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+        issue(blockIdx.x, 0);
+        issue(int64_t(blockIdx.x) + gridDim.x, 1);
+    }
+    __syncthreads();
+    for (int64_t it = 0;; ++it) {
+        const int64_t w = int64_t(blockIdx.x) + it * gridDim.x;
+        if (w >= ntiles) break;
+        const int s = int(it & 1);
+        mbar_wait(&full[s], uint32_t((it >> 1) & 1));
+        if (t == 0) bulk_wait_read0();  // the previous tile's stores have read sout
+        __syncthreads();
+        // transpose: task = (box, slot r, chunk jq); LDS.128 of slot r's chunk jq,
+        // CH scalar stores into rows j = jq*CH + e of the output box
+        for (int task = t; task < NBX * E * 8; task += kTpThreads) {
+            const int bx = task / (E * 8), rem = task % (E * 8), r = rem % E, jq = rem / E;
+            const T *in = sin + (s * NBX + bx) * BOX + r * E + ((jq ^ (r & 7)) * CH);
+            T v[CH];
+            if constexpr (sizeof(T) == 4) {
+                const float4 f = *reinterpret_cast<const float4 *>(in);
+                v[0] = f.x;
+                v[1] = f.y;
+                v[2] = f.z;
+                v[3] = f.w;
+            } else {
+                const double2 f = *reinterpret_cast<const double2 *>(in);
+                v[0] = f.x;
+                v[1] = f.y;
+            }
+            T *out = sout + bx * BOX;
+#pragma unroll
+            for (int e = 0; e < CH; ++e) {
+                const int j = jq * CH + e;
+                out[j * E + (((r / CH) ^ (j & 7)) * CH) + r % CH] = v[e];
+            }
+        }
+        fence_proxy_async_smem();
+        __syncthreads();
+        if (t == 0) {
+            int64_t sys, rt, jt;
+            coords(w, sys, rt, jt);
+#pragma unroll
+            for (int bx = 0; bx < NBX; ++bx)
+                tma_store_box3(&tm.m[1], sout + bx * BOX, int(rt * E), int((jt * NBX + bx) * E), int(sys));
+            bulk_commit();
+            issue(w + 2 * int64_t(gridDim.x), s);  // stage s is free: every thread passed the barrier
+        }
+    }
+    if (t == 0) bulk_wait_all();
+    // rows [lfull * 2^K, n) of every system (fewer than 2^K): position lfull of slot r
+    const int64_t tail = A.n - (lfull << A.K);
+    for (int64_t idx = int64_t(blockIdx.x) * kTpThreads + t; idx < msys * tail;
+         idx += int64_t(gridDim.x) * kTpThreads) {
+        const int64_t sys = idx / tail, r = idx % tail;
+        A.x[sys * A.batch_stride + (lfull << A.K) + r] = A.xs[((sys << A.K) + r) * A.slot + lfull];
+    }
+}
+
 template <typename T>
 cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batch_stride, int64_t slot, int K,
                            int vec, const PassGeom &geom, cudaStream_t st) {
@@ -174,6 +277,37 @@ cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batc
     A.K = K;
     A.vec = vec;
     A.geom = geom;
+    constexpr int E = 128 / int(sizeof(T));
+    const int64_t lfull = n >> K;  // whole j rows of 2^K residues
+    if ((int64_t(1) << K) >= E && vec && lfull > 0 && n > 0 && m > 0) {
+        const int64_t rtiles = (int64_t(1) << K) / E;
+        const int64_t jtiles = (lfull + kTpBoxes * E - 1) / (kTpBoxes * E);
+        const int64_t ntiles = m * rtiles * jtiles;
+        TmapSet tm{};
+        // xs: {positions, slots, 1}, box {E positions, E slots, 1}
+        const uint64_t din[3] = {uint64_t(slot), uint64_t(m << K), 1};
+        const uint64_t sin_[2] = {uint64_t(slot) * sizeof(T), uint64_t(slot) * sizeof(T) * uint64_t(m << K)};
+        const uint32_t bin[3] = {uint32_t(E), uint32_t(E), 1};
+        // x: {2^K residues, lfull j, m systems}, box {E residues, E j, 1}
+        const uint64_t dout[3] = {uint64_t(1) << K, uint64_t(lfull), uint64_t(m)};
+        const uint64_t sout_[2] = {(uint64_t(1) << K) * sizeof(T), uint64_t(batch_stride) * sizeof(T)};
+        const uint32_t bout[3] = {uint32_t(E), uint32_t(E), 1};
+        if ((m << K) < (int64_t(1) << 31) &&
+            encode_box3_tmap(&tm.m[0], xs, int(sizeof(T)), din, sin_, bin) &&
+            encode_box3_tmap(&tm.m[1], x, int(sizeof(T)), dout, sout_, bout)) {
+            const size_t smem = 1024 + size_t(3 * kTpBoxes * E * E) * sizeof(T);
+            auto kern = place_x_tma_kernel<T>;
+            cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+            if (e != cudaSuccess) return e;
+            int dev = 0, sms = 148, occ = 1;
+            cudaGetDevice(&dev);
+            cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, kTpThreads, smem);
+            const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(ntiles, int64_t(std::max(occ, 1)) * sms));
+            kern<<<(unsigned)grid, kTpThreads, smem, st>>>(A, tm, ntiles, jtiles, lfull, m);
+            return cudaGetLastError();
+        }
+    }
     if (K >= 5) {
         const int64_t lmax = (n + (int64_t(1) << K) - 1) >> K;
         const int64_t jtiles = (lmax + kTileJ - 1) / kTileJ;
