@@ -145,6 +145,7 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
     A.n = I.n;
     A.batch_stride = I.batch_stride;
     A.K = P.k;
+    A.m_systems = I.m;
     int t = P.thomas_chains, l2 = 0;
     while ((1 << l2) < t) ++l2;
     A.log2T = l2;
@@ -177,7 +178,13 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
     if (P.passes >= first && P.passes <= last) {
         if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "on-chip grid exceeds 2^31-1 CTAs");
         cudaError_t err;
-        if (onchip_pipe_ok(I)) {
+        if (P.k == 0 && onchip_cpipe_ok(I) && A.vec) {
+            // persistent, TMA-fed warp-form kernel on one CTA or a 2-CTA cluster per system
+            int dev = 0, sms = 148;
+            cudaGetDevice(&dev);
+            cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+            err = launch_onchip_cpipe<T>(A, I.onchip_threads, sms, st);
+        } else if (onchip_pipe_ok(I)) {
             // persistent, TMA-pipelined form (cluster == 1, 64 bytes of rows per thread)
             int dev = 0, sms = 148;
             cudaGetDevice(&dev);

@@ -104,6 +104,7 @@ struct OnchipArgs {
     int64_t n;
     int64_t batch_stride;    // original layout (input when RAW, always for x)
     int64_t slot;            // workspace slot capacity (K > 0)
+    int64_t m_systems;       // number of systems (K == 0 persistent kernel)
     int32_t K;               // total split levels
     int32_t log2T;           // PCR levels on the reduced system (T = 2^log2T chains)
     int32_t cluster;         // CTAs per subsystem (thread-block cluster size)
@@ -138,6 +139,20 @@ inline bool onchip_pipe_ok(const tds_plan_info &I) {
     if (rb != 64 && rb != 32) return false;
     return onchip_pipe_smem_bytes(I.dtype, I.onchip_threads, 1 << P.cr_levels, P.tl_levels) + kSmemReserve + 16 <=
            size_t(232448);
+}
+
+template <typename T>
+cudaError_t launch_onchip_cpipe(const OnchipArgs<T> &A, int threads, int sm_count, cudaStream_t st);
+size_t onchip_cpipe_smem_bytes(int32_t dtype, int32_t threads);
+
+// k = 0 systems on chip straight from a, b, c, d: persistent TMA kernel, warp
+// form, one CTA or a 2-CTA cluster per system, 64 bytes of rows per thread.
+inline bool onchip_cpipe_ok(const tds_plan_info &I) {
+    const tds_params &P = I.params;
+    if (P.k != 0 || (P.cluster != 1 && P.cluster != 2) || P.tl_levels != 5) return false;
+    if ((1 << P.cr_levels) * dsize(I.dtype) != 64) return false;
+    if (I.onchip_threads % 32 || I.onchip_threads > 512 || P.cluster * (I.onchip_threads / 32) > 32) return false;
+    return onchip_cpipe_smem_bytes(I.dtype, I.onchip_threads) + kSmemReserve + 16 <= size_t(232448);
 }
 
 template <typename T>

@@ -1,0 +1,362 @@
+// onchip_cpipe.cu -- G2 for k = 0 (no split pass): persistent, TMA-fed,
+// optionally spread over a 2-CTA thread-block cluster (§III-A base
+// kernel, §III-D Stage 1 "several processors on one system" mapped to a
+// cluster with distributed shared memory).
+//
+// Every system of n rows is solved on chip straight from the caller's a, b,
+// c, d: 20 bytes per equation instead of the 52 of a split pass + on-chip +
+// placement.  A cluster of C CTAs (C = 1 or 2) x NT threads x R rows per
+// thread holds one system (n <= C * NT * R: 16384 fp32 / 8192 fp64 rows for
+// C = 2); clusters walk systems sys = cluster id, += clusters.  Per CTA one
+// shared-memory stage holds the next system's 4 raw arrays (one swizzled TMA
+// box each); it is refilled as soon as the rows are in registers.
+//
+// The solve is the warp form of onchip_pipe.cu (CR in registers, CR across
+// the 32 lanes of each warp by shuffles, one row per warp left, PCR over
+// those rows by one warp, back substitution) with the CTA boundary handled
+// like the warp boundary: the last warp's lane-31 chain reads the next CTA's
+// published rows through DSMEM, the per-warp top rows are gathered in CTA 0,
+// and x of the top rows is scattered back -- three cluster barriers per
+// system.  x is written in original order (k = 0: no placement).
+#include <cooperative_groups.h>
+
+#include "pipe.cuh"
+
+namespace cg = cooperative_groups;
+
+namespace tds {
+
+template <int C>
+__device__ __forceinline__ void csync() {
+    if constexpr (C > 1) cg::this_cluster().sync(); else __syncthreads();
+}
+
+template <typename T>
+__device__ __forceinline__ T *peer(T *p, int rank) {  // DSMEM address of p in cluster CTA `rank`
+    return cg::this_cluster().map_shared_rank(p, rank);
+}
+
+template <typename T, int R, int C>
+__global__ void __launch_bounds__(512, 1)
+    onchip_cpipe_kernel(const OnchipArgs<T> A, const __grid_constant__ TmapSet tm, int32_t tma_lines) {
+    static_assert(R * sizeof(T) == 64, "64 bytes of rows per thread");
+    constexpr int CR = ilog2c(R), ELINE = 128 / int(sizeof(T));
+    constexpr unsigned FULL = 0xffffffffu;
+    extern __shared__ __align__(1024) unsigned char smem_raw[];
+    __shared__ __align__(8) uint64_t full_bar;
+    const int NT = blockDim.x, ROWS = NT * R;
+    const int t = threadIdx.x, lane = t & 31, warp = t >> 5, nwarps = NT >> 5;
+    const int rank = C > 1 ? int(cg::this_cluster().block_rank()) : 0;
+    const int64_t cid = int64_t(blockIdx.x) / C, ncl = int64_t(gridDim.x) / C;
+    T *stage = reinterpret_cast<T *>(smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u));  // [4][ROWS]
+    T *e_in = stage + 4 * ROWS;        // [nwarps][CR][3]  lane 0's row s-1 before register level l
+    T *w_in = e_in + nwarps * CR * 3;  // [nwarps][5][3]   lane s-1 before lane level l
+    T *lft = w_in + nwarps * 15;       // [nwarps][5][3]   lane 31-s before lane level l
+    T *top = lft + nwarps * 15;        // [3][32]          per-warp top rows (CTA 0: all C*nwarps)
+    T *xtop = top + 96;                // [33]             x of this CTA's top rows; [32] = previous CTA's last
+    const int64_t n = A.n;
+    const int64_t tma_rows = int64_t(tma_lines) * ELINE;  // rows of every system in whole TMA lines
+    const int64_t row0 = int64_t(rank) * ROWS;              // this CTA's first row of the system
+
+    auto issue = [&](int64_t sys) {  // thread 0
+        if (sys >= A.m_systems) return;
+        if (tma_lines == 0 || row0 >= tma_rows) {
+            mbar_expect_tx(&full_bar, 0);
+            return;
+        }
+        mbar_expect_tx(&full_bar, 4 * uint32_t(ROWS) * sizeof(T));
+#pragma unroll
+        for (int q = 0; q < 4; ++q)
+            tma_load_lines(stage + q * ROWS, &tm.m[q], int(row0 / ELINE), int(sys), &full_bar);
+    };
+    if (t == 0) {
+        mbar_init(&full_bar, 1);
+        asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+        issue(cid);
+    }
+    csync<C>();  // every CTA of the cluster runs before any DSMEM access
+
+    for (int64_t it = 0;; ++it) {
+        const int64_t sys = cid + it * ncl;
+        if (sys >= A.m_systems) break;
+        mbar_wait(&full_bar, uint32_t(it & 1));
+        const int64_t i0 = row0 + int64_t(t) * R;  // first row of this thread
+        if (row0 + ROWS > tma_rows) {
+            // CTA-uniform: rows past the TMA lines are patched into the stage --
+            // the tail by LDG, identity rows (0, 1, 0, 0) past n
+            for (int j = t; j < ROWS; j += NT) {
+                const int64_t i = row0 + j;
+                if (i < tma_rows) continue;
+                const int o = sw_off<T>(j);
+                T va = T(0), vb = T(1), vc = T(0), vd = T(0);
+                if (i < n) {
+                    const int64_t g = sys * A.batch_stride + i;
+                    va = A.a[g];
+                    vb = A.b[g];
+                    vc = A.c[g];
+                    vd = A.d[g];
+                }
+                stage[o] = va;
+                stage[ROWS + o] = vb;
+                stage[2 * ROWS + o] = vc;
+                stage[3 * ROWS + o] = vd;
+            }
+            fence_proxy_async_smem();  // before the TMA refill of the stage
+            __syncthreads();
+        }
+        // normalise while loading (b = 1): only 1/b and the three arrays stay live
+        T ra[R], rc[R], rd[R];
+        {
+            T inv[R];
+            lds_rows_sw<T, R>(stage + ROWS, t * R, inv);
+#pragma unroll
+            for (int v = 0; v < R; ++v) inv[v] = rcp(inv[v]);
+            lds_rows_sw<T, R>(stage, t * R, ra);
+            lds_rows_sw<T, R>(stage + 2 * ROWS, t * R, rc);
+            lds_rows_sw<T, R>(stage + 3 * ROWS, t * R, rd);
+#pragma unroll
+            for (int v = 0; v < R; ++v) {
+                ra[v] *= inv[v];
+                rc[v] *= inv[v];
+                rd[v] *= inv[v];
+            }
+        }
+        __syncthreads();  // the stage is in registers: prefetch the next system
+        if (t == 0) issue(sys + ncl);
+        if (i0 <= 0 || i0 + R >= n) {  // a_0 and c_{n-1} are outside the system
+#pragma unroll
+            for (int v = 0; v < R; ++v) {
+                if (i0 + v == 0) ra[v] = T(0);
+                if (i0 + v == n - 1) rc[v] = T(0);
+            }
+        }
+        // ---- register CR levels; lane 31 defers its row R-1 chain
+#pragma unroll
+        for (int l = 1; l <= CR; ++l) {
+            const int s = 1 << (l - 1);
+            const T pa = ra[s - 1], pc = rc[s - 1], pd = rd[s - 1];
+            const T na = __shfl_down_sync(FULL, pa, 1), nc = __shfl_down_sync(FULL, pc, 1),
+                    nd = __shfl_down_sync(FULL, pd, 1);
+            if (lane == 0) {
+                T *e = e_in + (warp * CR + l - 1) * 3;
+                e[0] = pa;
+                e[1] = pc;
+                e[2] = pd;
+            }
+#pragma unroll
+            for (int v = (1 << l) - 1; v < R; v += (1 << l)) {
+                const bool last = v == R - 1;
+                T a = ra[v], c = rc[v], d = rd[v];
+                row_update(a, c, d, ra[v - s], rc[v - s], rd[v - s], last ? na : ra[(v + s) % R],
+                           last ? nc : rc[(v + s) % R], last ? nd : rd[(v + s) % R]);
+                const bool keep = last && lane == 31;
+                ra[v] = keep ? ra[v] : a;
+                rc[v] = keep ? rc[v] : c;
+                rd[v] = keep ? rd[v] : d;
+            }
+        }
+        // ---- CR across lanes; lane 31 (kept at every level) defers
+        T za = ra[R - 1], zc = rc[R - 1], zd = rd[R - 1];
+#pragma unroll
+        for (int l = 1; l <= 5; ++l) {
+            const int s = 1 << (l - 1);
+            const T la = __shfl_up_sync(FULL, za, s), lc = __shfl_up_sync(FULL, zc, s),
+                    ld = __shfl_up_sync(FULL, zd, s);
+            const T xa = __shfl_down_sync(FULL, za, s), xc = __shfl_down_sync(FULL, zc, s),
+                    xd = __shfl_down_sync(FULL, zd, s);
+            if (lane == s - 1) {
+                T *w = w_in + (warp * 5 + l - 1) * 3;
+                w[0] = za;
+                w[1] = zc;
+                w[2] = zd;
+            }
+            if (lane == 31 - s) {
+                T *f = lft + (warp * 5 + l - 1) * 3;
+                f[0] = za;
+                f[1] = zc;
+                f[2] = zd;
+            }
+            T a = za, c = zc, d = zd;
+            row_update(a, c, d, la, lc, ld, xa, xc, xd);
+            const bool upd = (lane & ((1 << l) - 1)) == (1 << l) - 1 && lane != 31;
+            za = upd ? a : za;
+            zc = upd ? c : zc;
+            zd = upd ? d : zd;
+        }
+        csync<C>();  // (1) every warp's (and CTA's) first rows are published
+        if (lane == 31) {  // the deferred chains; the last warp reads the next CTA's rows by DSMEM
+            const bool last_warp = warp == nwarps - 1;
+            const bool h = !last_warp || rank + 1 < C;
+            const T *en = e_in, *wn = w_in;
+            int wsrc = warp + 1;
+            if constexpr (C > 1) {
+                if (last_warp && rank + 1 < C) {
+                    en = peer(e_in, rank + 1);
+                    wn = peer(w_in, rank + 1);
+                    wsrc = 0;
+                }
+            }
+#pragma unroll
+            for (int l = 1; l <= CR; ++l) {
+                const int s = 1 << (l - 1);
+                const T *e = en + (wsrc * CR + l - 1) * 3;
+                row_update(ra[R - 1], rc[R - 1], rd[R - 1], ra[R - 1 - s], rc[R - 1 - s], rd[R - 1 - s],
+                           h ? e[0] : T(0), h ? e[1] : T(0), h ? e[2] : T(0));
+            }
+            za = ra[R - 1];
+            zc = rc[R - 1];
+            zd = rd[R - 1];
+#pragma unroll
+            for (int l = 1; l <= 5; ++l) {
+                const T *f = lft + (warp * 5 + l - 1) * 3;
+                const T *w = wn + (wsrc * 5 + l - 1) * 3;
+                row_update(za, zc, zd, f[0], f[1], f[2], h ? w[0] : T(0), h ? w[1] : T(0), h ? w[2] : T(0));
+            }
+            T *tp = top;
+            if constexpr (C > 1) tp = peer(top, 0);
+            const int z = rank * nwarps + warp;
+            tp[z] = za;
+            tp[32 + z] = zc;
+            tp[64 + z] = zd;
+        }
+        csync<C>();  // (2) CTA 0 holds every top row
+        if (rank == 0 && warp == 0) {  // C * nwarps <= 32 rows: pure PCR with shuffles, x = d
+            const int Z = C * nwarps;
+            T a = lane < Z ? top[lane] : T(0), c = lane < Z ? top[32 + lane] : T(0),
+              d = lane < Z ? top[64 + lane] : T(0);
+            for (int s = 1; s < Z; s <<= 1) {
+                const T la = __shfl_up_sync(FULL, a, s), lc = __shfl_up_sync(FULL, c, s),
+                        ld = __shfl_up_sync(FULL, d, s);
+                const T xa = __shfl_down_sync(FULL, a, s), xc = __shfl_down_sync(FULL, c, s),
+                        xd = __shfl_down_sync(FULL, d, s);
+                const bool hl = lane >= s, hr = lane + s < Z;
+                T na = a, nc = c, nd = d;
+                row_update(na, nc, nd, hl ? la : T(0), hl ? lc : T(0), hl ? ld : T(0), hr ? xa : T(0),
+                           hr ? xc : T(0), hr ? xd : T(0));
+                a = lane < Z ? na : a;
+                c = lane < Z ? nc : c;
+                d = lane < Z ? nd : d;
+            }
+            if (lane < Z) {  // x of top row z to its CTA; the last one of a CTA also to the next CTA
+                const int r = lane / nwarps, w = lane % nwarps;
+                T *xt = xtop;
+                if constexpr (C > 1) xt = peer(xtop, r);
+                xt[w] = d;
+                if (w == nwarps - 1 && r + 1 < C) {
+                    T *xn = xtop;
+                    if constexpr (C > 1) xn = peer(xtop, r + 1);
+                    xn[32] = d;
+                }
+            }
+        }
+        csync<C>();  // (3) x of the top rows is in every CTA
+        // ---- back substitution across lanes, then in registers
+        T xw = lane == 31 ? xtop[warp] : T(0);
+        const T xprev = warp > 0 ? xtop[warp - 1] : (rank > 0 ? xtop[32] : T(0));
+#pragma unroll
+        for (int l = 5; l >= 1; --l) {
+            const int s = 1 << (l - 1);
+            const T xl = __shfl_up_sync(FULL, xw, s);
+            const T xr = __shfl_down_sync(FULL, xw, s);
+            const T xn = zd - za * (lane >= s ? xl : xprev) - zc * xr;
+            xw = (lane & ((1 << l) - 1)) == s - 1 ? xn : xw;
+        }
+        T xleft = __shfl_up_sync(FULL, xw, 1);
+        if (lane == 0) xleft = xprev;
+        rd[R - 1] = xw;
+#pragma unroll
+        for (int l = CR; l >= 1; --l) {
+            const int s = 1 << (l - 1);
+#pragma unroll
+            for (int v = s - 1; v < R - 1; v += 2 * s) {
+                const T xlv = (v >= s) ? rd[(v - s + R) % R] : xleft;
+                rd[v] = rd[v] - ra[v] * xlv - rc[v] * rd[(v + s) % R];
+            }
+        }
+        // ---- x in original order (k = 0): contiguous rows, 16-byte stores
+        T *dst = A.x + sys * A.batch_stride + i0;
+        if (i0 + R <= n) {
+            constexpr int W = 16 / int(sizeof(T));
+#pragma unroll
+            for (int q = 0; q < R / W; ++q) {
+                if constexpr (sizeof(T) == 4)
+                    __stcs(reinterpret_cast<float4 *>(dst) + q,
+                           make_float4(rd[4 * q], rd[4 * q + 1], rd[4 * q + 2], rd[4 * q + 3]));
+                else
+                    __stcs(reinterpret_cast<double2 *>(dst) + q, make_double2(rd[2 * q], rd[2 * q + 1]));
+            }
+        } else if (i0 < n) {
+#pragma unroll
+            for (int v = 0; v < R; ++v)
+                if (i0 + v < n) dst[v] = rd[v];
+        }
+        // the next system's first scratch writes follow its stage barrier and the
+        // cluster barrier (1) orders every cross-CTA read of this system's scratch
+    }
+    csync<C>();  // no CTA leaves while a peer may still read its shared memory
+}
+
+size_t onchip_cpipe_smem_bytes(int32_t dtype, int32_t threads) {
+    const int64_t R = 64 / dsize(dtype);
+    const int64_t nw = threads / 32;
+    return 1024 + size_t((4 * int64_t(threads) * R + nw * (4 + 5 + 5) * 3 + 96 + 33) * dsize(dtype));
+}
+
+template <typename T>
+cudaError_t launch_onchip_cpipe(const OnchipArgs<T> &A, int threads, int sm_count, cudaStream_t st) {
+    constexpr int R = 64 / int(sizeof(T)), ELINE = 128 / int(sizeof(T));
+    const int C = A.cluster;
+    if (C != 1 && C != 2) return cudaErrorInvalidConfiguration;
+    if (threads % 32 || threads > 512 || C * (threads / 32) > 32) return cudaErrorInvalidConfiguration;
+    const int64_t rows = int64_t(threads) * R;
+    const size_t smem = onchip_cpipe_smem_bytes(sizeof(T) == 4 ? TDS_F32 : TDS_F64, threads);
+    auto kern = C == 2 ? onchip_cpipe_kernel<T, R, 2> : onchip_cpipe_kernel<T, R, 1>;
+    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    if (e != cudaSuccess) return e;
+    if (C > 1) {
+        e = cudaFuncSetAttribute(kern, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
+        if (e != cudaSuccess) return e;
+    }
+    // whole 128-byte lines of every system go by TMA (rows past them: LDG)
+    const int64_t tma_lines = A.n / ELINE;
+    if (tma_lines > 0x7fffffffLL || A.m_systems > 0x7fffffffLL) return cudaErrorInvalidConfiguration;
+    TmapSet tm{};
+    if (tma_lines > 0) {
+        const T *arrs[4] = {A.a, A.b, A.c, A.d};
+        for (int q = 0; q < 4; ++q)
+            if (!encode_rows_tmap(&tm.m[q], arrs[q], int(sizeof(T)), tma_lines, A.m_systems, A.batch_stride,
+                                  int(rows / ELINE)))
+                return cudaErrorInvalidValue;
+    }
+    cudaLaunchConfig_t cfg{};
+    cfg.blockDim = dim3(threads, 1, 1);
+    cfg.dynamicSmemBytes = smem;
+    cfg.stream = st;
+    cudaLaunchAttribute attr[1];
+    int nclusters = 0;
+    if (C > 1) {
+        attr[0].id = cudaLaunchAttributeClusterDimension;
+        attr[0].val.clusterDim.x = C;
+        attr[0].val.clusterDim.y = 1;
+        attr[0].val.clusterDim.z = 1;
+        cfg.attrs = attr;
+        cfg.numAttrs = 1;
+        cfg.gridDim = dim3(unsigned(C), 1, 1);
+        e = cudaOccupancyMaxActiveClusters(&nclusters, kern, &cfg);
+        if (e != cudaSuccess) return e;
+    } else {
+        int occ = 1;
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, threads, smem);
+        nclusters = std::max(occ, 1) * sm_count;
+    }
+    nclusters = int(std::min<int64_t>(std::max(nclusters, 1), A.m_systems));
+    cfg.gridDim = dim3(unsigned(nclusters * C), 1, 1);
+    e = cudaLaunchKernelEx(&cfg, kern, A, tm, int32_t(tma_lines));
+    if (e != cudaSuccess) return e;
+    return cudaGetLastError();
+}
+
+template cudaError_t launch_onchip_cpipe<float>(const OnchipArgs<float> &, int, int, cudaStream_t);
+template cudaError_t launch_onchip_cpipe<double>(const OnchipArgs<double> &, int, int, cudaStream_t);
+
+}  // namespace tds

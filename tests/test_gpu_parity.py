@@ -112,6 +112,21 @@ def test_onchip_cluster(tds, dtype, n, cl, T, tl):
     check(a, b, c, d, x, dtype)
 
 
+@pytest.mark.parametrize("dtype,n,cl", [(np.float32, 16384, 2), (np.float32, 16383, 2), (np.float32, 9001, 2),
+                                        (np.float32, 8192, 1), (np.float32, 5000, 1), (np.float32, 1000, 1),
+                                        (np.float32, 33, 1), (np.float64, 8192, 2), (np.float64, 6007, 2),
+                                        (np.float64, 4096, 1), (np.float64, 777, 1)])
+def test_onchip_k0_persistent(tds, dtype, n, cl):
+    """k = 0 straight from a, b, c, d: the persistent TMA warp-form kernel on
+    one CTA or a 2-CTA cluster (DSMEM for the CTA boundary), ragged sizes."""
+    c_lv = 4 if dtype == np.float32 else 3
+    a, b, c, d = inputs.generate(n, 5, dtype, seed=29)
+    x, plan = run(tds, a, b, c, d, params=dict(k_pass=[], cr_levels=c_lv, thomas_chains=1, cluster=cl,
+                                               tl_levels=5))
+    assert plan.info["k"] == 0 and plan.info["cluster"] == cl
+    check(a, b, c, d, x, dtype)
+
+
 @pytest.mark.parametrize("n,tl,T", [(8192, 9, 1), (8192, 4, 32), (5000, 3, 8), (1000, 5, 1), (100, 5, 1)])
 def test_onchip_thread_level_cr(tds, n, tl, T):
     """CR across threads inside one CTA (C = 1, c2 > 0) down to a tiny leader system."""
