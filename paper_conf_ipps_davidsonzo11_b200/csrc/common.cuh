@@ -143,16 +143,20 @@ inline bool onchip_pipe_ok(const tds_plan_info &I) {
 
 template <typename T>
 cudaError_t launch_onchip_cpipe(const OnchipArgs<T> &A, int threads, int sm_count, cudaStream_t st);
-size_t onchip_cpipe_smem_bytes(int32_t dtype, int32_t threads);
+size_t onchip_cpipe_smem_bytes(int32_t dtype, int32_t threads, int32_t cluster);
 
 // k = 0 systems on chip straight from a, b, c, d: persistent TMA kernel, warp
-// form, one CTA or a 2-CTA cluster per system, 64 bytes of rows per thread.
+// form, one CTA or a cluster of 2, 4 or 8 CTAs per system, 64 bytes of rows
+// per thread.
 inline bool onchip_cpipe_ok(const tds_plan_info &I) {
     const tds_params &P = I.params;
-    if (P.k != 0 || (P.cluster != 1 && P.cluster != 2) || P.tl_levels != 5) return false;
+    const int C = P.cluster;
+    if (P.k != 0 || (C != 1 && C != 2 && C != 4 && C != 8) || P.tl_levels != 5) return false;
     if ((1 << P.cr_levels) * dsize(I.dtype) != 64) return false;
-    if (I.onchip_threads % 32 || I.onchip_threads > 512 || P.cluster * (I.onchip_threads / 32) > 32) return false;
-    return onchip_cpipe_smem_bytes(I.dtype, I.onchip_threads) + kSmemReserve + 16 <= size_t(232448);
+    const int nw = I.onchip_threads / 32;
+    if (I.onchip_threads % 32 || I.onchip_threads > 512) return false;
+    if (C * nw > 32 && I.onchip_threads < C * 16) return false;  // CTA 0 solves the C*nw top rows
+    return onchip_cpipe_smem_bytes(I.dtype, I.onchip_threads, C) + kSmemReserve + 16 <= size_t(232448);
 }
 
 template <typename T>

@@ -1,5 +1,5 @@
 // onchip_cpipe.cu -- G2 for k = 0 (no split pass): persistent, TMA-fed,
-// optionally spread over a 2-CTA thread-block cluster (§III-A base
+// optionally spread over a thread-block cluster of 2-8 CTAs (§III-A base
 // kernel, §III-D Stage 1 "several processors on one system" mapped to a
 // cluster with distributed shared memory).
 //
@@ -7,7 +7,8 @@
 // c, d: 20 bytes per equation instead of the 52 of a split pass + on-chip +
 // placement.  A cluster of C CTAs (C = 1 or 2) x NT threads x R rows per
 // thread holds one system (n <= C * NT * R: 16384 fp32 / 8192 fp64 rows for
-// C = 2); clusters walk systems sys = cluster id, += clusters.  Per CTA one
+// C = 2, up to 65536 / 32768 for C = 8); clusters walk systems sys = cluster
+// id, += clusters.  Per CTA one
 // shared-memory stage holds the next system's 4 raw arrays (one swizzled TMA
 // box each); it is refilled as soon as the rows are in registers.
 //
@@ -15,9 +16,10 @@
 // the 32 lanes of each warp by shuffles, one row per warp left, PCR over
 // those rows by one warp, back substitution) with the CTA boundary handled
 // like the warp boundary: the last warp's lane-31 chain reads the next CTA's
-// published rows through DSMEM, the per-warp top rows are gathered in CTA 0,
-// and x of the top rows is scattered back -- three cluster barriers per
-// system.  x is written in original order (k = 0: no placement).
+// published rows through DSMEM, the per-warp top rows are gathered in CTA 0
+// (solved by one warp's shuffles up to 32 rows, else by CTA 0 in shared
+// memory), and x of the top rows is scattered back -- three cluster barriers
+// per system.  x is written in original order (k = 0: no placement).
 #include <cooperative_groups.h>
 
 #include "pipe.cuh"
@@ -41,6 +43,7 @@ __global__ void __launch_bounds__(512, 1)
     onchip_cpipe_kernel(const OnchipArgs<T> A, const __grid_constant__ TmapSet tm, int32_t tma_lines) {
     static_assert(R * sizeof(T) == 64, "64 bytes of rows per thread");
     constexpr int CR = ilog2c(R), ELINE = 128 / int(sizeof(T));
+    constexpr int ZMAX = 16 * C > 32 ? 16 * C : 32;  // top rows of a cluster (<= 16 warps per CTA)
     constexpr unsigned FULL = 0xffffffffu;
     extern __shared__ __align__(1024) unsigned char smem_raw[];
     __shared__ __align__(8) uint64_t full_bar;
@@ -52,8 +55,8 @@ __global__ void __launch_bounds__(512, 1)
     T *e_in = stage + 4 * ROWS;        // [nwarps][CR][3]  lane 0's row s-1 before register level l
     T *w_in = e_in + nwarps * CR * 3;  // [nwarps][5][3]   lane s-1 before lane level l
     T *lft = w_in + nwarps * 15;       // [nwarps][5][3]   lane 31-s before lane level l
-    T *top = lft + nwarps * 15;        // [3][32]          per-warp top rows (CTA 0: all C*nwarps)
-    T *xtop = top + 96;                // [33]             x of this CTA's top rows; [32] = previous CTA's last
+    T *top = lft + nwarps * 15;        // [3][ZMAX]        per-warp top rows (CTA 0: all C*nwarps)
+    T *xtop = top + 3 * ZMAX;          // [33]             x of this CTA's top rows; [32] = previous CTA's last
     const int64_t n = A.n;
     const int64_t tma_rows = int64_t(tma_lines) * ELINE;  // rows of every system in whole TMA lines
     const int64_t row0 = int64_t(rank) * ROWS;              // this CTA's first row of the system
@@ -216,14 +219,43 @@ __global__ void __launch_bounds__(512, 1)
             if constexpr (C > 1) tp = peer(top, 0);
             const int z = rank * nwarps + warp;
             tp[z] = za;
-            tp[32 + z] = zc;
-            tp[64 + z] = zd;
+            tp[ZMAX + z] = zc;
+            tp[2 * ZMAX + z] = zd;
         }
         csync<C>();  // (2) CTA 0 holds every top row
-        if (rank == 0 && warp == 0) {  // C * nwarps <= 32 rows: pure PCR with shuffles, x = d
+        if (C * nwarps > 32 && rank == 0) {
+            // CTA 0: PCR over the Z = C * nwarps top rows in shared memory (every row decouples, x = d)
             const int Z = C * nwarps;
-            T a = lane < Z ? top[lane] : T(0), c = lane < Z ? top[32 + lane] : T(0),
-              d = lane < Z ? top[64 + lane] : T(0);
+            T *za2 = top, *zc2 = top + ZMAX, *zd2 = top + 2 * ZMAX;
+            for (int s = 1; s < Z; s <<= 1) {
+                T a = T(0), c = T(0), d = T(0);
+                if (t < Z) {
+                    a = za2[t];
+                    c = zc2[t];
+                    d = zd2[t];
+                    const bool hl = t >= s, hr = t + s < Z;
+                    row_update(a, c, d, hl ? za2[t - s] : T(0), hl ? zc2[t - s] : T(0), hl ? zd2[t - s] : T(0),
+                               hr ? za2[t + s] : T(0), hr ? zc2[t + s] : T(0), hr ? zd2[t + s] : T(0));
+                }
+                __syncthreads();
+                if (t < Z) {
+                    za2[t] = a;
+                    zc2[t] = c;
+                    zd2[t] = d;
+                }
+                __syncthreads();
+            }
+            if (t < Z) {
+                const T d = zd2[t];
+                const int r = t / nwarps, w = t % nwarps;
+                T *xt = peer(xtop, r);
+                xt[w] = d;
+                if (w == nwarps - 1 && r + 1 < C) peer(xtop, r + 1)[32] = d;
+            }
+        } else if (C * nwarps <= 32 && rank == 0 && warp == 0) {  // <= 32 rows: PCR with shuffles, x = d
+            const int Z = C * nwarps;
+            T a = lane < Z ? top[lane] : T(0), c = lane < Z ? top[ZMAX + lane] : T(0),
+              d = lane < Z ? top[2 * ZMAX + lane] : T(0);
             for (int s = 1; s < Z; s <<= 1) {
                 const T la = __shfl_up_sync(FULL, a, s), lc = __shfl_up_sync(FULL, c, s),
                         ld = __shfl_up_sync(FULL, d, s);
@@ -296,21 +328,26 @@ __global__ void __launch_bounds__(512, 1)
     csync<C>();  // no CTA leaves while a peer may still read its shared memory
 }
 
-size_t onchip_cpipe_smem_bytes(int32_t dtype, int32_t threads) {
+size_t onchip_cpipe_smem_bytes(int32_t dtype, int32_t threads, int32_t cluster) {
     const int64_t R = 64 / dsize(dtype);
     const int64_t nw = threads / 32;
-    return 1024 + size_t((4 * int64_t(threads) * R + nw * (4 + 5 + 5) * 3 + 96 + 33) * dsize(dtype));
+    const int64_t zmax = std::max<int64_t>(32, 16 * cluster);
+    return 1024 + size_t((4 * int64_t(threads) * R + nw * (4 + 5 + 5) * 3 + 3 * zmax + 33) * dsize(dtype));
 }
 
 template <typename T>
 cudaError_t launch_onchip_cpipe(const OnchipArgs<T> &A, int threads, int sm_count, cudaStream_t st) {
     constexpr int R = 64 / int(sizeof(T)), ELINE = 128 / int(sizeof(T));
     const int C = A.cluster;
-    if (C != 1 && C != 2) return cudaErrorInvalidConfiguration;
-    if (threads % 32 || threads > 512 || C * (threads / 32) > 32) return cudaErrorInvalidConfiguration;
+    if (C != 1 && C != 2 && C != 4 && C != 8) return cudaErrorInvalidConfiguration;
+    if (threads % 32 || threads > 512 || (C * (threads / 32) > 32 && threads < C * 16))
+        return cudaErrorInvalidConfiguration;
     const int64_t rows = int64_t(threads) * R;
-    const size_t smem = onchip_cpipe_smem_bytes(sizeof(T) == 4 ? TDS_F32 : TDS_F64, threads);
-    auto kern = C == 2 ? onchip_cpipe_kernel<T, R, 2> : onchip_cpipe_kernel<T, R, 1>;
+    const size_t smem = onchip_cpipe_smem_bytes(sizeof(T) == 4 ? TDS_F32 : TDS_F64, threads, C);
+    auto kern = C == 8   ? onchip_cpipe_kernel<T, R, 8>
+                : C == 4 ? onchip_cpipe_kernel<T, R, 4>
+                : C == 2 ? onchip_cpipe_kernel<T, R, 2>
+                         : onchip_cpipe_kernel<T, R, 1>;
     cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     if (e != cudaSuccess) return e;
     if (C > 1) {

@@ -138,11 +138,17 @@ static void tune_onchip(TuneCtx &C, tds_params &best, double &t_best) {
     bool improved = true;
     while (improved && !out_of_time(C)) {
         improved = false;
-        tds_params cand[10];
+        tds_params cand[12];
         int nc = 0;
         // the warp-level form (CR across all 32 lanes, shuffles only) is a
         // different kernel path, not a neighbour of tl_levels = 4: try it directly
         if (best.cluster == 1 && best.tl_levels != 5) { cand[nc] = best; cand[nc++].tl_levels = 5; }
+        // ... and for k = 0 on one CTA or a cluster of <= 8, the persistent kernel's shape (64 bytes of rows per thread)
+        if (best.k == 0 && best.cluster <= 8 && !(best.tl_levels == 5 && (1 << best.cr_levels) == r_max(I.dtype))) {
+            cand[nc] = best;
+            cand[nc].tl_levels = 5;
+            cand[nc++].cr_levels = ilog2i(r_max(I.dtype));
+        }
         if (best.thomas_chains > 1) { cand[nc] = best; cand[nc++].thomas_chains /= 2; }
         cand[nc] = best; cand[nc++].thomas_chains *= 2;
         if (best.tl_levels > 0) { cand[nc] = best; cand[nc++].tl_levels -= 1; }

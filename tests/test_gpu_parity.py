@@ -115,10 +115,13 @@ def test_onchip_cluster(tds, dtype, n, cl, T, tl):
 @pytest.mark.parametrize("dtype,n,cl", [(np.float32, 16384, 2), (np.float32, 16383, 2), (np.float32, 9001, 2),
                                         (np.float32, 8192, 1), (np.float32, 5000, 1), (np.float32, 1000, 1),
                                         (np.float32, 33, 1), (np.float64, 8192, 2), (np.float64, 6007, 2),
-                                        (np.float64, 4096, 1), (np.float64, 777, 1)])
+                                        (np.float64, 4096, 1), (np.float64, 777, 1), (np.float32, 65536, 8),
+                                        (np.float32, 50001, 8), (np.float32, 32768, 4), (np.float32, 20000, 4),
+                                        (np.float64, 32768, 8), (np.float64, 16000, 4)])
 def test_onchip_k0_persistent(tds, dtype, n, cl):
     """k = 0 straight from a, b, c, d: the persistent TMA warp-form kernel on
-    one CTA or a 2-CTA cluster (DSMEM for the CTA boundary), ragged sizes."""
+    one CTA or a cluster of 2, 4 or 8 CTAs (DSMEM for the CTA boundaries, the
+    top rows solved by one warp or by CTA 0 in shared memory), ragged sizes."""
     c_lv = 4 if dtype == np.float32 else 3
     a, b, c, d = inputs.generate(n, 5, dtype, seed=29)
     x, plan = run(tds, a, b, c, d, params=dict(k_pass=[], cr_levels=c_lv, thomas_chains=1, cluster=cl,
