@@ -40,7 +40,8 @@ __device__ __forceinline__ T *peer(T *p, int rank) {  // DSMEM address of p in c
 
 template <typename T, int R, int C>
 __global__ void __launch_bounds__(512, 1)
-    onchip_cpipe_kernel(const OnchipArgs<T> A, const __grid_constant__ TmapSet tm, int32_t tma_lines) {
+    onchip_cpipe_kernel(const OnchipArgs<T> A, const __grid_constant__ TmapSet tm, int32_t tma_lines,
+                        const __grid_constant__ TmapSet tmx) {
     static_assert(R * sizeof(T) == 64, "64 bytes of rows per thread");
     constexpr int CR = ilog2c(R), ELINE = 128 / int(sizeof(T));
     constexpr int ZMAX = 16 * C > 32 ? 16 * C : 32;  // top rows of a cluster (<= 16 warps per CTA)
@@ -52,7 +53,8 @@ __global__ void __launch_bounds__(512, 1)
     const int rank = C > 1 ? int(cg::this_cluster().block_rank()) : 0;
     const int64_t cid = int64_t(blockIdx.x) / C, ncl = int64_t(gridDim.x) / C;
     T *stage = reinterpret_cast<T *>(smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u));  // [4][ROWS]
-    T *e_in = stage + 4 * ROWS;        // [nwarps][CR][3]  lane 0's row s-1 before register level l
+    T *xst = stage + 4 * ROWS;         // [ROWS]           x of the previous system, for its TMA store
+    T *e_in = xst + ROWS;              // [nwarps][CR][3]  lane 0's row s-1 before register level l
     T *w_in = e_in + nwarps * CR * 3;  // [nwarps][5][3]   lane s-1 before lane level l
     T *lft = w_in + nwarps * 15;       // [nwarps][5][3]   lane 31-s before lane level l
     T *top = lft + nwarps * 15;        // [3][ZMAX]        per-warp top rows (CTA 0: all C*nwarps)
@@ -124,8 +126,14 @@ __global__ void __launch_bounds__(512, 1)
                 rd[v] *= inv[v];
             }
         }
-        __syncthreads();  // the stage is in registers: prefetch the next system
-        if (t == 0) issue(sys + ncl);
+        __syncthreads();  // the stage is in registers (and the previous x is in xst)
+        if (t == 0) {
+            issue(sys + ncl);
+            if (it > 0 && tma_lines > 0 && row0 < tma_rows) {  // the previous system's x: one TMA store
+                tma_store_lines(&tmx.m[0], xst, int(row0 / ELINE), int(sys - ncl));
+                bulk_commit();
+            }
+        }
         if (i0 <= 0 || i0 + R >= n) {  // a_0 and c_{n-1} are outside the system
 #pragma unroll
             for (int v = 0; v < R; ++v) {
@@ -186,6 +194,7 @@ __global__ void __launch_bounds__(512, 1)
             zc = upd ? c : zc;
             zd = upd ? d : zd;
         }
+        if (t == 0) bulk_wait_read0();  // xst is rewritten at the end of this system
         csync<C>();  // (1) every warp's (and CTA's) first rows are published
         if (lane == 31) {  // the deferred chains; the last warp reads the next CTA's rows by DSMEM
             const bool last_warp = warp == nwarps - 1;
@@ -305,9 +314,19 @@ __global__ void __launch_bounds__(512, 1)
                 rd[v] = rd[v] - ra[v] * xlv - rc[v] * rd[(v + s) % R];
             }
         }
-        // ---- x in original order (k = 0): contiguous rows, 16-byte stores
+        // ---- x in original order (k = 0): staged (swizzled) for the next
+        // iteration's TMA store -- no global stores pending at the cluster
+        // barriers -- except rows past the TMA lines
         T *dst = A.x + sys * A.batch_stride + i0;
-        if (i0 + R <= n) {
+        if (tma_lines > 0 && row0 < tma_rows) {
+            sts_rows_sw<T, R>(xst, t * R, rd);
+            fence_proxy_async_smem();
+            if (i0 + R > tma_rows) {
+#pragma unroll
+                for (int v = 0; v < R; ++v)
+                    if (i0 + v >= tma_rows && i0 + v < n) dst[v] = rd[v];
+            }
+        } else if (i0 + R <= n) {
             constexpr int W = 16 / int(sizeof(T));
 #pragma unroll
             for (int q = 0; q < R / W; ++q) {
@@ -325,6 +344,15 @@ __global__ void __launch_bounds__(512, 1)
         // the next system's first scratch writes follow its stage barrier and the
         // cluster barrier (1) orders every cross-CTA read of this system's scratch
     }
+    __syncthreads();
+    if (t == 0) {  // the last system's x
+        const int64_t nit = (A.m_systems - cid + ncl - 1) / ncl;
+        if (nit > 0 && tma_lines > 0 && row0 < tma_rows) {
+            tma_store_lines(&tmx.m[0], xst, int(row0 / ELINE), int(cid + (nit - 1) * ncl));
+            bulk_commit();
+        }
+        bulk_wait_all();
+    }
     csync<C>();  // no CTA leaves while a peer may still read its shared memory
 }
 
@@ -332,7 +360,7 @@ size_t onchip_cpipe_smem_bytes(int32_t dtype, int32_t threads, int32_t cluster) 
     const int64_t R = 64 / dsize(dtype);
     const int64_t nw = threads / 32;
     const int64_t zmax = std::max<int64_t>(32, 16 * cluster);
-    return 1024 + size_t((4 * int64_t(threads) * R + nw * (4 + 5 + 5) * 3 + 3 * zmax + 33) * dsize(dtype));
+    return 1024 + size_t((5 * int64_t(threads) * R + nw * (4 + 5 + 5) * 3 + 3 * zmax + 33) * dsize(dtype));
 }
 
 template <typename T>
@@ -357,12 +385,12 @@ cudaError_t launch_onchip_cpipe(const OnchipArgs<T> &A, int threads, int sm_coun
     // whole 128-byte lines of every system go by TMA (rows past them: LDG)
     const int64_t tma_lines = A.n / ELINE;
     if (tma_lines > 0x7fffffffLL || A.m_systems > 0x7fffffffLL) return cudaErrorInvalidConfiguration;
-    TmapSet tm{};
+    TmapSet tm{}, tmx{};
     if (tma_lines > 0) {
-        const T *arrs[4] = {A.a, A.b, A.c, A.d};
-        for (int q = 0; q < 4; ++q)
-            if (!encode_rows_tmap(&tm.m[q], arrs[q], int(sizeof(T)), tma_lines, A.m_systems, A.batch_stride,
-                                  int(rows / ELINE)))
+        const T *arrs[5] = {A.a, A.b, A.c, A.d, A.x};
+        for (int q = 0; q < 5; ++q)
+            if (!encode_rows_tmap(q < 4 ? &tm.m[q] : &tmx.m[0], arrs[q], int(sizeof(T)), tma_lines, A.m_systems,
+                                  A.batch_stride, int(rows / ELINE)))
                 return cudaErrorInvalidValue;
     }
     cudaLaunchConfig_t cfg{};
@@ -388,7 +416,7 @@ cudaError_t launch_onchip_cpipe(const OnchipArgs<T> &A, int threads, int sm_coun
     }
     nclusters = int(std::min<int64_t>(std::max(nclusters, 1), A.m_systems));
     cfg.gridDim = dim3(unsigned(nclusters * C), 1, 1);
-    e = cudaLaunchKernelEx(&cfg, kern, A, tm, int32_t(tma_lines));
+    e = cudaLaunchKernelEx(&cfg, kern, A, tm, int32_t(tma_lines), tmx);
     if (e != cudaSuccess) return e;
     return cudaGetLastError();
 }
