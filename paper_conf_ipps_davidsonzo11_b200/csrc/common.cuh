@@ -11,13 +11,22 @@ constexpr int kMaxPasses = TDS_MAX_PASSES;
 
 // Reciprocal.  fp32: the SFU approximation (MUFU.RCP, <= 1 ulp) -- the
 // north_star's fp32 tolerance (1e-4 error, 1e-5 residual) leaves room for it
-// (reading R16).  fp64: IEEE division.
+// (reading R16).  fp64: the SFU seed (MUFU.RCP64H) refined by two
+// Newton steps (relative error ~1 ulp, R16) instead of IEEE
+// division, whose special-case slow path costs a call per row update.
 __device__ __forceinline__ float rcp(float x) {
     float r;
     asm("rcp.approx.ftz.f32 %0, %1;" : "=f"(r) : "f"(x));
     return r;
 }
-__device__ __forceinline__ double rcp(double x) { return 1.0 / x; }
+__device__ __forceinline__ double rcp(double x) {
+    double r;
+    asm("rcp.approx.ftz.f64 %0, %1;" : "=d"(r) : "d"(x));
+    double e = fma(-x, r, 1.0);
+    r = fma(r, e, r);
+    e = fma(-x, r, 1.0);
+    return fma(r, e, r);
+}
 
 // One PCR/CR row update in NORMALISED form (every row scaled so b = 1).
 // With the textbook update (Hockney & Jesshope [11], cited
