@@ -18,8 +18,9 @@
 // like the warp boundary: the last warp's lane-31 chain reads the next CTA's
 // published rows through DSMEM, the per-warp top rows are gathered in CTA 0
 // (solved by one warp's shuffles up to 32 rows, else by CTA 0 in shared
-// memory), and x of the top rows is scattered back -- three cluster barriers
-// per system.  x is written in original order (k = 0: no placement).
+// memory), and x of the top rows is scattered back.  The three cross-CTA
+// hand-offs are point-to-point: st.async stores into the peer's shared memory
+// counted on the peer's mbarrier (no cluster barrier inside the loop).  x is written in original order (k = 0: no placement).
 #include <cooperative_groups.h>
 
 #include "pipe.cuh"
@@ -59,6 +60,10 @@ __global__ void __launch_bounds__(512, 1)
     T *lft = w_in + nwarps * 15;       // [nwarps][5][3]   lane 31-s before lane level l
     T *top = lft + nwarps * 15;        // [3][ZMAX]        per-warp top rows (CTA 0: all C*nwarps)
     T *xtop = top + 3 * ZMAX;          // [33]             x of this CTA's top rows; [32] = previous CTA's last
+    T *rnext = xtop + 33;              // [CR+5][3]        the next CTA's warp-0 rows (e_in, w_in) for our last warp
+    // mbarriers of the cluster hand-offs (one phase per system): rnext filled,
+    // top rows gathered (CTA 0), x of the top rows delivered
+    __shared__ __align__(8) uint64_t mb_next, mb_top, mb_x;
     const int64_t n = A.n;
     const int64_t tma_rows = int64_t(tma_lines) * ELINE;  // rows of every system in whole TMA lines
     const int64_t row0 = int64_t(rank) * ROWS;              // this CTA's first row of the system
@@ -76,10 +81,23 @@ __global__ void __launch_bounds__(512, 1)
     };
     if (t == 0) {
         mbar_init(&full_bar, 1);
+        mbar_init(&mb_next, 1);
+        mbar_init(&mb_top, 1);
+        mbar_init(&mb_x, 1);
         asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
         issue(cid);
     }
-    csync<C>();  // every CTA of the cluster runs before any DSMEM access
+    csync<C>();  // every CTA of the cluster runs (and has its mbarriers) before any DSMEM access
+    // peer addresses of the hand-off buffers
+    uint32_t prev_rnext = 0, prev_mb_next = 0, top0 = 0, mb_top0 = 0;
+    if constexpr (C > 1) {
+        if (rank > 0) {
+            prev_rnext = cluster_addr(rnext, rank - 1);
+            prev_mb_next = cluster_addr(&mb_next, rank - 1);
+        }
+        top0 = cluster_addr(top, 0);
+        mb_top0 = cluster_addr(&mb_top, 0);
+    }
 
     for (int64_t it = 0;; ++it) {
         const int64_t sys = cid + it * ncl;
@@ -128,6 +146,11 @@ __global__ void __launch_bounds__(512, 1)
         }
         __syncthreads();  // the stage is in registers (and the previous x is in xst)
         if (t == 0) {
+            if constexpr (C > 1) {  // announce this system's incoming hand-off bytes
+                mbar_expect_tx(&mb_x, uint32_t((nwarps + (rank > 0 ? 1 : 0)) * sizeof(T)));
+                if (rank + 1 < C) mbar_expect_tx(&mb_next, uint32_t((CR + 5) * 3 * sizeof(T)));
+                if (rank == 0) mbar_expect_tx(&mb_top, uint32_t(C * nwarps * 3 * sizeof(T)));
+            }
             issue(sys + ncl);
             if (it > 0 && tma_lines > 0 && row0 < tma_rows) {  // the previous system's x: one TMA store
                 tma_store_lines(&tmx.m[0], xst, int(row0 / ELINE), int(sys - ncl));
@@ -153,6 +176,14 @@ __global__ void __launch_bounds__(512, 1)
                 e[0] = pa;
                 e[1] = pc;
                 e[2] = pd;
+                if constexpr (C > 1) {
+                    if (warp == 0 && rank > 0) {  // the previous CTA's last warp needs them
+                        const uint32_t o = prev_rnext + uint32_t((l - 1) * 3 * sizeof(T));
+                        st_async(o, pa, prev_mb_next);
+                        st_async(o + sizeof(T), pc, prev_mb_next);
+                        st_async(o + 2 * sizeof(T), pd, prev_mb_next);
+                    }
+                }
             }
 #pragma unroll
             for (int v = (1 << l) - 1; v < R; v += (1 << l)) {
@@ -180,6 +211,14 @@ __global__ void __launch_bounds__(512, 1)
                 w[0] = za;
                 w[1] = zc;
                 w[2] = zd;
+                if constexpr (C > 1) {
+                    if (warp == 0 && rank > 0) {
+                        const uint32_t o = prev_rnext + uint32_t((CR + l - 1) * 3 * sizeof(T));
+                        st_async(o, za, prev_mb_next);
+                        st_async(o + sizeof(T), zc, prev_mb_next);
+                        st_async(o + 2 * sizeof(T), zd, prev_mb_next);
+                    }
+                }
             }
             if (lane == 31 - s) {
                 T *f = lft + (warp * 5 + l - 1) * 3;
@@ -195,23 +234,22 @@ __global__ void __launch_bounds__(512, 1)
             zd = upd ? d : zd;
         }
         if (t == 0) bulk_wait_read0();  // xst is rewritten at the end of this system
-        csync<C>();  // (1) every warp's (and CTA's) first rows are published
-        if (lane == 31) {  // the deferred chains; the last warp reads the next CTA's rows by DSMEM
+        __syncthreads();  // (1) every warp's first rows are published (this CTA)
+        if (lane == 31) {  // the deferred chains; the last warp uses the next CTA's pushed rows
             const bool last_warp = warp == nwarps - 1;
             const bool h = !last_warp || rank + 1 < C;
-            const T *en = e_in, *wn = w_in;
-            int wsrc = warp + 1;
+            const T *en = e_in + (warp + 1) * CR * 3, *wn = w_in + (warp + 1) * 15;
             if constexpr (C > 1) {
                 if (last_warp && rank + 1 < C) {
-                    en = peer(e_in, rank + 1);
-                    wn = peer(w_in, rank + 1);
-                    wsrc = 0;
+                    mbar_wait(&mb_next, uint32_t(it & 1));
+                    en = rnext;
+                    wn = rnext + CR * 3;
                 }
             }
 #pragma unroll
             for (int l = 1; l <= CR; ++l) {
                 const int s = 1 << (l - 1);
-                const T *e = en + (wsrc * CR + l - 1) * 3;
+                const T *e = en + (l - 1) * 3;
                 row_update(ra[R - 1], rc[R - 1], rd[R - 1], ra[R - 1 - s], rc[R - 1 - s], rd[R - 1 - s],
                            h ? e[0] : T(0), h ? e[1] : T(0), h ? e[2] : T(0));
             }
@@ -221,17 +259,24 @@ __global__ void __launch_bounds__(512, 1)
 #pragma unroll
             for (int l = 1; l <= 5; ++l) {
                 const T *f = lft + (warp * 5 + l - 1) * 3;
-                const T *w = wn + (wsrc * 5 + l - 1) * 3;
+                const T *w = wn + (l - 1) * 3;
                 row_update(za, zc, zd, f[0], f[1], f[2], h ? w[0] : T(0), h ? w[1] : T(0), h ? w[2] : T(0));
             }
-            T *tp = top;
-            if constexpr (C > 1) tp = peer(top, 0);
             const int z = rank * nwarps + warp;
-            tp[z] = za;
-            tp[ZMAX + z] = zc;
-            tp[2 * ZMAX + z] = zd;
+            if constexpr (C > 1) {  // to CTA 0 (itself included), counted on its mb_top
+                st_async(top0 + uint32_t(z * sizeof(T)), za, mb_top0);
+                st_async(top0 + uint32_t((ZMAX + z) * sizeof(T)), zc, mb_top0);
+                st_async(top0 + uint32_t((2 * ZMAX + z) * sizeof(T)), zd, mb_top0);
+            } else {
+                top[z] = za;
+                top[ZMAX + z] = zc;
+                top[2 * ZMAX + z] = zd;
+            }
         }
-        csync<C>();  // (2) CTA 0 holds every top row
+        if constexpr (C == 1) __syncthreads();  // (2) every top row is in top[]
+        if constexpr (C > 1) {
+            if (rank == 0 && (C * nwarps > 32 || warp == 0)) mbar_wait(&mb_top, uint32_t(it & 1));
+        }
         if (C * nwarps > 32 && rank == 0) {
             // CTA 0: PCR over the Z = C * nwarps top rows in shared memory (every row decouples, x = d)
             const int Z = C * nwarps;
@@ -254,12 +299,11 @@ __global__ void __launch_bounds__(512, 1)
                 }
                 __syncthreads();
             }
-            if (t < Z) {
+            if (t < Z) {  // x of top row t to its CTA (and the next CTA's xprev), counted on their mb_x
                 const T d = zd2[t];
                 const int r = t / nwarps, w = t % nwarps;
-                T *xt = peer(xtop, r);
-                xt[w] = d;
-                if (w == nwarps - 1 && r + 1 < C) peer(xtop, r + 1)[32] = d;
+                st_async(cluster_addr(xtop + w, r), d, cluster_addr(&mb_x, r));
+                if (w == nwarps - 1 && r + 1 < C) st_async(cluster_addr(xtop + 32, r + 1), d, cluster_addr(&mb_x, r + 1));
             }
         } else if (C * nwarps <= 32 && rank == 0 && warp == 0) {  // <= 32 rows: PCR with shuffles, x = d
             const int Z = C * nwarps;
@@ -280,17 +324,17 @@ __global__ void __launch_bounds__(512, 1)
             }
             if (lane < Z) {  // x of top row z to its CTA; the last one of a CTA also to the next CTA
                 const int r = lane / nwarps, w = lane % nwarps;
-                T *xt = xtop;
-                if constexpr (C > 1) xt = peer(xtop, r);
-                xt[w] = d;
-                if (w == nwarps - 1 && r + 1 < C) {
-                    T *xn = xtop;
-                    if constexpr (C > 1) xn = peer(xtop, r + 1);
-                    xn[32] = d;
+                if constexpr (C > 1) {
+                    st_async(cluster_addr(xtop + w, r), d, cluster_addr(&mb_x, r));
+                    if (w == nwarps - 1 && r + 1 < C)
+                        st_async(cluster_addr(xtop + 32, r + 1), d, cluster_addr(&mb_x, r + 1));
+                } else {
+                    xtop[w] = d;
                 }
             }
         }
-        csync<C>();  // (3) x of the top rows is in every CTA
+        // (3) x of the top rows is in every CTA
+        if constexpr (C > 1) mbar_wait(&mb_x, uint32_t(it & 1)); else __syncthreads();
         // ---- back substitution across lanes, then in registers
         T xw = lane == 31 ? xtop[warp] : T(0);
         const T xprev = warp > 0 ? xtop[warp - 1] : (rank > 0 ? xtop[32] : T(0));
@@ -360,7 +404,7 @@ size_t onchip_cpipe_smem_bytes(int32_t dtype, int32_t threads, int32_t cluster) 
     const int64_t R = 64 / dsize(dtype);
     const int64_t nw = threads / 32;
     const int64_t zmax = std::max<int64_t>(32, 16 * cluster);
-    return 1024 + size_t((5 * int64_t(threads) * R + nw * (4 + 5 + 5) * 3 + 3 * zmax + 33) * dsize(dtype));
+    return 1024 + size_t((5 * int64_t(threads) * R + nw * (4 + 5 + 5) * 3 + 3 * zmax + 33 + 27) * dsize(dtype));
 }
 
 template <typename T>

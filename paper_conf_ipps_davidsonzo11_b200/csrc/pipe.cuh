@@ -159,6 +159,25 @@ __device__ __forceinline__ void tma_store_box3(const CUtensorMap *map, const voi
 bool encode_box3_tmap(CUtensorMap *out, const void *base, int dsize, const uint64_t dims[3], const uint64_t strides[2],
                       const uint32_t box[3]);
 
+// ---- cluster point-to-point transfers (DSMEM): st.async stores into a peer
+// CTA's shared memory that count down the peer's mbarrier transaction bytes,
+// so a consumer waits on its own mbarrier instead of a cluster barrier.
+__device__ __forceinline__ uint32_t cluster_addr(const void *p, int rank) {
+    uint32_t r;
+    asm volatile("mapa.shared::cluster.u32 %0, %1, %2;" : "=r"(r) : "r"(smem_u32(p)), "r"(rank));
+    return r;
+}
+__device__ __forceinline__ void st_async(uint32_t raddr, float v, uint32_t rbar) {
+    asm volatile("st.async.shared::cluster.mbarrier::complete_tx::bytes.b32 [%0], %1, [%2];" ::"r"(raddr),
+                 "r"(__float_as_uint(v)), "r"(rbar)
+                 : "memory");
+}
+__device__ __forceinline__ void st_async(uint32_t raddr, double v, uint32_t rbar) {
+    asm volatile("st.async.shared::cluster.mbarrier::complete_tx::bytes.b64 [%0], %1, [%2];" ::"r"(raddr),
+                 "l"(__double_as_longlong(v)), "r"(rbar)
+                 : "memory");
+}
+
 // Host: encode the tensor map of `slots` row slots of `lines` full 128-byte
 // lines each, slot stride `stride` elements, box of `box_lines` lines.
 bool encode_rows_tmap(CUtensorMap *out, const void *base, int dsize, int64_t lines, int64_t slots, int64_t stride,
