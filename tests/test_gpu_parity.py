@@ -357,6 +357,46 @@ def test_inplace_and_stride(tds):
     check(a, b, c, d, xs[:, :n], np.float32)
 
 
+STRIDE_PLANS = [dict(k_pass=[], cr_levels=4, thomas_chains=16, cluster=2, tl_levels=5),   # k = 0 cluster kernel
+                dict(k_pass=[2], cr_levels=4, thomas_chains=1, cluster=1, tl_levels=5),  # TMA split + pipe
+                dict(k_pass=[7], cr_levels=2, thomas_chains=1, cluster=1, tl_levels=5),  # deep split, 4-D store
+                dict(k_pass=[3, 2], cr_levels=4, thomas_chains=1, cluster=1, tl_levels=5)]
+
+
+@pytest.mark.parametrize("plan_kw", STRIDE_PLANS, ids=["k0c2", "k2", "k7", "k3+2"])
+@pytest.mark.parametrize("inplace", [False, True])
+def test_tma_paths_stride_inplace(tds, plan_kw, inplace):
+    """16-byte aligned batch stride > n (TMA tensor maps with a slot stride)
+    in place and out of place: the padding between systems stays untouched."""
+    import torch
+    n, m, stride = 10000, 3, 10012
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=10)
+    pad = lambda v: np.pad(v, ((0, 0), (0, stride - n)), constant_values=7.0)
+    A, B, C, D = (pad(v).reshape(-1) for v in (a, b, c, d))
+    plan = tds.Plan(n, m, "float32", device=0, batch_stride=stride)
+    plan.set_params(**plan_kw)
+    ta, tb, tc, td = to_dev(A, B, C, D)
+    out = td if inplace else torch.full_like(td, 7.0)
+    x = tds.solve_batched(plan, ta, tb, tc, td, out=out)
+    torch.cuda.synchronize()
+    xs = x.cpu().numpy().reshape(m, stride)
+    assert np.all(xs[:, n:] == 7.0)
+    check(a, b, c, d, xs[:, :n], np.float32)
+
+
+def test_batch_isolation_k0_cluster(tds):
+    """A poisoned neighbour system leaves the others bit-identical (k = 0 cluster kernel)."""
+    n, m = 16000, 4
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=8)
+    kw = dict(k_pass=[], cr_levels=4, thomas_chains=16, cluster=2, tl_levels=5)
+    x0, _ = run(tds, a, b, c, d, params=kw)
+    d2 = d.copy(); b2 = b.copy()
+    d2[2] *= 1e6; b2[2] += 5
+    x1, _ = run(tds, a, b2, c, d2, params=kw)
+    for s in (0, 1, 3):
+        assert np.array_equal(x0[s], x1[s])
+
+
 def test_workspace_errors(tds):
     import torch
     n, m = 4096, 2
