@@ -25,8 +25,19 @@
 //     is again one vector run per final residue from lanes b = 1..NB.
 #include "pipe.cuh"
 #include "split_reg.cuh"
+#include <cstdlib>
 
 namespace tds {
+
+// Ablation build (-DTDS_SPLIT_ABLATION, diagnostics only -- results are wrong
+// when a bit is set): env TDS_SPLIT_ABLATION = 1 skip the PCR levels, 2 skip
+// the TMA loads, 4 skip the TMA stores.  Product builds compile TDS_ABL to false.
+#ifdef TDS_SPLIT_ABLATION
+__constant__ int tds_split_ablation;
+#define TDS_ABL(bit) ((tds_split_ablation & (bit)) != 0)
+#else
+#define TDS_ABL(bit) false
+#endif
 
 template <int KP, int NT_>
 struct SplitShape {
@@ -124,7 +135,7 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
         gt = t0 - HEAD + ROWS < tma_end ? t0 - HEAD + ROWS : tma_end;
     };
     auto issue = [&](int64_t w) {  // thread 0 only
-        if (w >= nitems) return;
+        if (w >= nitems || TDS_ABL(2)) return;
         if (tma_lines == 0) {  // slots shorter than one line: everything by LDG
             mbar_expect_tx(&bar, 0);
             return;
@@ -142,7 +153,7 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
     auto tma_store_tile = [&](int64_t sigma, int64_t t0, int kp_prev) {
         fence_proxy_async_smem();  // generic-proxy smem writes -> visible to the TMA
         __syncthreads();
-        if (t == 0) {
+        if (t == 0 && !TDS_ABL(4)) {
             const int j0 = int(t0 >> KP), r = int(sigma & ((int64_t(1) << kp_prev) - 1)), sys = int(sigma >> kp_prev);
 #pragma unroll
             for (int q = 0; q < 3; ++q)
@@ -164,9 +175,9 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
         if (w >= nitems) break;
         int64_t sigma, t0, L, g0, gt;
         item_rows(w, sigma, t0, L, g0, gt);
-        mbar_wait(&bar, uint32_t(it & 1));
+        if (!TDS_ABL(2)) mbar_wait(&bar, uint32_t(it & 1));
         const int64_t ws = t0 - HEAD;  // window start row
-        if (ws <= 0 || ws + ROWS >= L || g0 > ws || gt < ws + ROWS) {
+        if (!TDS_ABL(2) && (ws <= 0 || ws + ROWS >= L || g0 > ws || gt < ws + ROWS)) {
             // CTA-uniform: patch the stage where the window leaves the TMA range --
             // identity rows outside [0, L), the tail rows by LDG, and (first pass)
             // a_0 = c_{n-1} = 0 -- so the register loads below need no branch
@@ -230,10 +241,12 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
         }
         __syncthreads();  // the stage is consumed: prefetch the next tile
         if (t == 0) issue(w + gridDim.x);
+        if (!TDS_ABL(1)) {
         if constexpr (KP >= 1) reg_level_w<T, R, 1, 32>(ra, rc, rd);
         if constexpr (KP >= 2) reg_level_w<T, R, 2, 32>(ra, rc, rd);
         if constexpr (KP >= 3) reg_level_w<T, R, 4, 32>(ra, rc, rd);
         if constexpr (KP >= 4) reg_level_w<T, R, 8, 32>(ra, rc, rd);
+        }
         if constexpr (TSTORE) {  // tbuf is written next: the previous tile's TMA store must have read it
             if (t == 0) bulk_wait_read0();
             __syncthreads();
@@ -326,10 +339,12 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
                 __syncthreads();
                 tr_read<T, R>(rd, tbuf, ad);
             }
+            if (!TDS_ABL(1)) {
             if constexpr (KQ >= 1) reg_level_w<T, R, 1, CH>(ra, rc, rd);
             if constexpr (KQ >= 2) reg_level_w<T, R, 2, CH>(ra, rc, rd);
             if constexpr (KQ >= 3) reg_level_w<T, R, 4, CH>(ra, rc, rd);
             if constexpr (KQ >= 4) reg_level_w<T, R, 8, CH>(ra, rc, rd);
+            }
             // member LEFT + 16(b-1) + u is row t0 + 16(16(b-1) + u) + rho
             if constexpr (TSTORE) {
                 __syncthreads();  // every layout-B read of tbuf is done: reuse it as the staging buffer
@@ -432,6 +447,13 @@ static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_le
     cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
     cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, S::NT, smem);
     const int64_t grid = std::min<int64_t>(nitems, int64_t(std::max(occ, 1)) * sms);
+#ifdef TDS_SPLIT_ABLATION
+    {
+        const char *ab = std::getenv("TDS_SPLIT_ABLATION");
+        const int v = ab ? std::atoi(ab) : 0;
+        cudaMemcpyToSymbolAsync(tds_split_ablation, &v, sizeof(int), 0, cudaMemcpyHostToDevice, st);
+    }
+#endif
     kern<<<(unsigned)grid, S::NT, smem, st>>>(A, tps, nitems, tm, int32_t(tma_lines), tmo);
     return cudaGetLastError();
 }

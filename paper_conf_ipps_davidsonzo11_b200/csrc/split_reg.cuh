@@ -198,12 +198,18 @@ __device__ __forceinline__ void trc_write(const T (&x)[R], T *p) {  // p = buf +
     for (int v = 0; v < R; ++v) p[v * AV] = x[v];
 }
 
-// chunk offsets of members mb + 4q (mb a multiple of 4), clamped into [0, AV)
+// chunk offsets of members mb + 4q (mb a multiple of 4).  Chunks outside
+// [0, AV) (halo lanes, garbage anyway) are moved by whole lanes (4 chunks) onto
+// the chunk a neighbouring lane of the same quarter-warp reads in the same
+// instruction: a broadcast, so the halo lanes add no extra wavefront.
 template <int R, int AV>
 __device__ __forceinline__ void trc_read_chunks(int mb, int (&ch)[R / 4]) {
 #pragma unroll
     for (int q = 0; q < R / 4; ++q) {
-        const int c = min(unsigned(mb / 4 + q), unsigned(AV / 4 - 1));  // halo lanes: clamp
+        int c = mb / 4 + q;
+        c = c < 0 ? c + 4 : c;
+        c = c > AV / 4 - 1 ? c - 4 : c;
+        c = c > AV / 4 - 1 ? c - 4 : c;
         ch[q] = (c ^ ((c >> 3) & 3)) << 2;
     }
 }
