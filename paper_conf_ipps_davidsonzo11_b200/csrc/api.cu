@@ -171,6 +171,10 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
         A.d = w.d[ob];
         A.xs = w.a[ob];  // per-subsystem x overwrites a (each CTA reads its rows before writing them)
         A.slot = I.slot_rows;
+        // the on-chip kernel is the last reader of c', d': their whole 128-byte
+        // lines are dropped from L2 once loaded (no write-back of dead scratch)
+        A.l2_discard = (I.slot_rows * int64_t(sizeof(T))) % 128 == 0 && uintptr_t(A.c) % 128 == 0 &&
+                       uintptr_t(A.d) % 128 == 0;
         A.geom.npass = P.passes;
         for (int q = 0; q < kMaxPasses; ++q) A.geom.kpass[q] = P.k_pass[q];
         grid = (I.m << P.k) * P.cluster;

@@ -120,6 +120,7 @@ struct OnchipArgs {
     int32_t tl_levels;       // CR levels across threads before the leader's solve
     int32_t vec;             // 16-byte vector loads/stores allowed
     PassGeom geom;           // passes applied (for the slot -> residue map)
+    int32_t l2_discard;      // K > 0: slots are 128-byte aligned, c/d lines may be discarded once loaded
 };
 
 __host__ __device__ constexpr int ilog2c(int v) { return v <= 1 ? 0 : 1 + ilog2c(v / 2); }

@@ -181,6 +181,19 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
         return r < A.n ? (A.n - r + KK - 1) >> A.K : 0;
     };
     const int64_t tma_rows = int64_t(tma_lines) * ELINE;  // rows of every slot in whole TMA lines
+    // workspace slots are read once (evict first); x slots are re-read by place_x (evict last)
+    auto ld_ws = [&](T *dst, const CUtensorMap *map, int slot, uint64_t *bar) {
+        if constexpr ((TDS_L2HINT & 1) != 0)
+            tma_load_lines_hint(dst, map, 0, slot, bar, l2_evict_first());
+        else
+            tma_load_lines(dst, map, 0, slot, bar);
+    };
+    auto st_x = [&](const T *src, int slot) {
+        if constexpr ((TDS_L2HINT & 2) != 0)
+            tma_store_lines_hint(&tm.m[0], src, 0, slot, l2_evict_last());
+        else
+            tma_store_lines(&tm.m[0], src, 0, slot);
+    };
     // work item q solves slot nslots-1-q: the split pass wrote the last slots
     // last, so the first items a CTA waits for are still in L2
     // One swizzled box of ROWS rows per array (lines past the slot are
@@ -198,12 +211,12 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
         }
         mbar_expect_tx(bar, 3 * uint32_t(ROWS) * sizeof(T));
         T *dst = stage0 + size_t(s) * 3 * ROWS;
-        tma_load_lines(dst + ROWS, &tm.m[1], 0, int(sigma), bar);
-        tma_load_lines(dst + 2 * ROWS, &tm.m[2], 0, int(sigma), bar);
+        ld_ws(dst + ROWS, &tm.m[1], int(sigma), bar);
+        ld_ws(dst + 2 * ROWS, &tm.m[2], int(sigma), bar);
     };
     auto issue_a = [&](int64_t q, int s) {  // thread 0 only
         if (q >= nslots || tma_lines == 0) return;
-        tma_load_lines(stage0 + size_t(s) * 3 * ROWS, &tm.m[0], 0, int(nslots - 1 - q), &full_bar[s]);
+        ld_ws(stage0 + size_t(s) * 3 * ROWS, &tm.m[0], int(nslots - 1 - q), &full_bar[s]);
     };
     if (t == 0) {
         mbar_init(&full_bar[0], 1);
@@ -239,6 +252,11 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
             asm volatile("fence.proxy.async.shared::cta;" ::: "memory");  // before the next TMA refill
             __syncthreads();
         }
+        if (A.l2_discard) {  // c', d' of this slot are dead once in shared memory
+            const int nl = int(min(L, tma_rows) / ELINE);
+            for (int li = t; li < 2 * nl; li += NT)
+                l2_discard_line((li < nl ? A.c : A.d) + sigma * A.slot + int64_t(li < nl ? li : li - nl) * ELINE);
+        }
         const int64_t jt = int64_t(t) * R;
         T ra[R], rc[R], rd[R];
         lds_rows_sw<T, R>(sb, t * R, ra);
@@ -248,7 +266,7 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
         if (t == 0) {
             issue_cd(q + 2 * int64_t(gridDim.x), s);
             if (pend >= 0) {  // the previous item's x: one tensor store from the a-region of stage 1-s
-                tma_store_lines(&tm.m[0], stage0 + size_t(1 - s) * 3 * ROWS, 0, int(pend));
+                st_x(stage0 + size_t(1 - s) * 3 * ROWS, int(pend));
                 bulk_commit();
             }
         }
@@ -386,7 +404,7 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
         if (pend >= 0) {
             // the stage index of the last item: it = number of items - 1
             const int64_t nit = (nslots - int64_t(blockIdx.x) + gridDim.x - 1) / gridDim.x;
-            tma_store_lines(&tm.m[0], stage0 + size_t((nit - 1) & 1) * 3 * ROWS, 0, int(pend));
+            st_x(stage0 + size_t((nit - 1) & 1) * 3 * ROWS, int(pend));
             bulk_commit();
         }
         bulk_wait_all();

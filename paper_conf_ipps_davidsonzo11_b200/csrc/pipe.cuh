@@ -63,6 +63,47 @@ __device__ __forceinline__ void tma_load_lines(void *dst, const CUtensorMap *map
         : "memory");
 }
 
+// L2 eviction-priority policies for TMA (createpolicy): streamed-once inputs
+// evict first, data a later kernel re-reads evicts last.
+// TDS_L2HINT bits (default 7): 1 on-chip workspace loads evict-first, 2 on-chip
+// x-slot stores evict-last, 4 placement loads evict-first, 8 split input loads
+// evict-first, 16 split output stores evict-last (8 and 16 measured neutral /
+// slower, profiles/r01g_l2.md).
+#ifndef TDS_L2HINT
+#define TDS_L2HINT 7
+#endif
+// Drop a dead 128-byte line from L2 without writing it back (scratch data
+// whose last reader has it in shared memory).  p must be 128-byte aligned.
+__device__ __forceinline__ void l2_discard_line(const void *p) {
+    asm volatile("discard.global.L2 [%0], 128;" ::"l"(p) : "memory");
+}
+__device__ __forceinline__ uint64_t l2_evict_first() {
+    uint64_t p;
+    asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(p));
+    return p;
+}
+__device__ __forceinline__ uint64_t l2_evict_last() {
+    uint64_t p;
+    asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(p));
+    return p;
+}
+__device__ __forceinline__ void tma_load_lines_hint(void *dst, const CUtensorMap *map, int line, int slot, uint64_t *bar,
+                                                    uint64_t pol) {
+    asm volatile(
+        "cp.async.bulk.tensor.3d.shared::cluster.global.mbarrier::complete_tx::bytes.L2::cache_hint [%0], [%1, {%2, %3, "
+        "%4}], [%5], %6;" ::"r"(smem_u32(dst)),
+        "l"(map), "r"(0), "r"(line), "r"(slot), "r"(smem_u32(bar)), "l"(pol)
+        : "memory");
+}
+__device__ __forceinline__ void tma_load_box3_hint(void *dst, const CUtensorMap *map, int c0, int c1, int c2,
+                                                   uint64_t *bar, uint64_t pol) {
+    asm volatile(
+        "cp.async.bulk.tensor.3d.shared::cluster.global.mbarrier::complete_tx::bytes.L2::cache_hint [%0], [%1, {%2, %3, "
+        "%4}], [%5], %6;" ::"r"(smem_u32(dst)),
+        "l"(map), "r"(c0), "r"(c1), "r"(c2), "r"(smem_u32(bar)), "l"(pol)
+        : "memory");
+}
+
 // Element offset of stage row s in a swizzled stage.
 template <typename T>
 __device__ __forceinline__ int sw_off(int s) {
@@ -138,6 +179,20 @@ __device__ __forceinline__ void sts_rows_sw(T *stage, int s0, const T *v) {
 __device__ __forceinline__ void tma_store_lines(const CUtensorMap *map, const void *src, int line, int slot) {
     asm volatile("cp.async.bulk.tensor.3d.global.shared::cta.bulk_group [%0, {%2, %3, %4}], [%1];" ::"l"(map),
                  "r"(smem_u32(src)), "r"(0), "r"(line), "r"(slot)
+                 : "memory");
+}
+
+__device__ __forceinline__ void tma_store_lines_hint(const CUtensorMap *map, const void *src, int line, int slot,
+                                                     uint64_t pol) {
+    asm volatile("cp.async.bulk.tensor.3d.global.shared::cta.bulk_group.L2::cache_hint [%0, {%2, %3, %4}], [%1], %5;" ::"l"(map),
+                 "r"(smem_u32(src)), "r"(0), "r"(line), "r"(slot), "l"(pol)
+                 : "memory");
+}
+
+__device__ __forceinline__ void tma_store_4d_hint(const CUtensorMap *map, const void *src, int c0, int c1, int c2,
+                                                  int c3, uint64_t pol) {
+    asm volatile("cp.async.bulk.tensor.4d.global.shared::cta.bulk_group.L2::cache_hint [%0, {%2, %3, %4, %5}], [%1], %6;" ::"l"(map),
+                 "r"(smem_u32(src)), "r"(c0), "r"(c1), "r"(c2), "r"(c3), "l"(pol)
                  : "memory");
 }
 

@@ -178,7 +178,7 @@ constexpr int kTpBoxes = 4, kTpThreads = 256;
 template <typename T>
 __global__ void __launch_bounds__(kTpThreads) place_x_tma_kernel(const PlaceArgs<T> A, const __grid_constant__ TmapSet tm,
                                                                 int64_t ntiles, int64_t jtiles, int64_t lfull,
-                                                                int64_t msys) {
+                                                                int64_t msys, int32_t l2_discard) {
     constexpr int E = 128 / int(sizeof(T)), CH = 16 / int(sizeof(T)), NBX = kTpBoxes;
     constexpr int BOX = E * E;  // elements per box
     extern __shared__ __align__(1024) unsigned char smem_raw[];
@@ -202,7 +202,11 @@ __global__ void __launch_bounds__(kTpThreads) place_x_tma_kernel(const PlaceArgs
         const int slot0 = int((sys << A.K) + rt * E);
 #pragma unroll
         for (int bx = 0; bx < NBX; ++bx)
-            tma_load_box3(sin + (s * NBX + bx) * BOX, &tm.m[0], int((jt * NBX + bx) * E), slot0, 0, &full[s]);
+            if constexpr ((TDS_L2HINT & 4) != 0)
+                tma_load_box3_hint(sin + (s * NBX + bx) * BOX, &tm.m[0], int((jt * NBX + bx) * E), slot0, 0, &full[s],
+                                   l2_evict_first());
+            else
+                tma_load_box3(sin + (s * NBX + bx) * BOX, &tm.m[0], int((jt * NBX + bx) * E), slot0, 0, &full[s]);
     };
     if (t == 0) {
         mbar_init(&full[0], 1);
@@ -217,6 +221,12 @@ __global__ void __launch_bounds__(kTpThreads) place_x_tma_kernel(const PlaceArgs
         if (w >= ntiles) break;
         const int s = int(it & 1);
         mbar_wait(&full[s], uint32_t((it >> 1) & 1));
+        if (l2_discard && t < NBX * E) {  // the x-slot lines of this tile are dead once in shared memory
+            int64_t sys, rt, jt;
+            coords(w, sys, rt, jt);
+            const int64_t pos = (jt * NBX + t / E) * E;
+            if (pos + E <= lfull) l2_discard_line(A.xs + ((sys << A.K) + rt * E + t % E) * A.slot + pos);
+        }
         if (t == 0) bulk_wait_read0();  // the previous tile's stores have read sout
         __syncthreads();
         // transpose: task = (box, slot r, chunk jq); LDS.128 of slot r's chunk jq,
@@ -304,7 +314,9 @@ cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batc
             cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
             cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, kTpThreads, smem);
             const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(ntiles, int64_t(std::max(occ, 1)) * sms));
-            kern<<<(unsigned)grid, kTpThreads, smem, st>>>(A, tm, ntiles, jtiles, lfull, m);
+            // x slots are scratch whose last reader is this kernel: drop their lines from L2 once loaded
+            const int32_t disc = (slot * int64_t(sizeof(T))) % 128 == 0 && uintptr_t(xs) % 128 == 0;
+            kern<<<(unsigned)grid, kTpThreads, smem, st>>>(A, tm, ntiles, jtiles, lfull, m, disc);
             return cudaGetLastError();
         }
     }

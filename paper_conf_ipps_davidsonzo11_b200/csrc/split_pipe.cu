@@ -145,7 +145,12 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
         mbar_expect_tx(&bar, NA * BL * 128);
         const int line0 = int((t0 - HEAD - TOFF) / ELINE);  // exact: TV and HEAD + TOFF are whole lines
 #pragma unroll
-        for (int q = 0; q < NA; ++q) tma_load_lines(stage + q * STG, &tm.m[q], line0, int(sigma), &bar);
+        for (int q = 0; q < NA; ++q) {
+            if constexpr ((TDS_L2HINT & 8) != 0)
+                tma_load_lines_hint(stage + q * STG, &tm.m[q], line0, int(sigma), &bar, l2_evict_first());
+            else
+                tma_load_lines(stage + q * STG, &tm.m[q], line0, int(sigma), &bar);
+        }
     };
     // the tile's outputs, staged in tbuf as [array][residue][position], leave by one
     // TMA tensor store per array: box {PT positions, 1, 2^KP residues, 1} of the
@@ -159,7 +164,11 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
             for (int q = 0; q < 3; ++q)
 #pragma unroll
                 for (int bx = 0; bx < NBOX; ++bx)
-                    tma_store_4d(&tmo.m[q], tbuf + q * TV + bx * NRES * BOXP, j0 + bx * BOXP, r, 0, sys);
+                    if constexpr ((TDS_L2HINT & 16) != 0)
+                        tma_store_4d_hint(&tmo.m[q], tbuf + q * TV + bx * NRES * BOXP, j0 + bx * BOXP, r, 0, sys,
+                                          l2_evict_last());
+                    else
+                        tma_store_4d(&tmo.m[q], tbuf + q * TV + bx * NRES * BOXP, j0 + bx * BOXP, r, 0, sys);
             bulk_commit();
         }
     };
