@@ -181,9 +181,11 @@ tds_status tds_plan_tune_trials(const tds_plan_t plan, int32_t *trials);
 /* x = A^{-1} d for every system.  a, b, c, d: device, dtype, m x batch_stride.
  * x: device, same layout; may alias d exactly (in-place), must not otherwise
  * overlap a, b, c or d.  workspace: device, >= info.workspace_bytes bytes,
- * 256-byte aligned (may be NULL when info.workspace_bytes == 0).  Enqueued on
- * cuda_stream; returns immediately.  Errors (nothing enqueued): INVALID_ARG,
- * WORKSPACE, DEVICE_MISMATCH, UNSUPPORTED; CUDA on a launch failure. */
+ * 256-byte aligned (may be NULL when info.workspace_bytes == 0); its contents
+ * are scratch, undefined after the call (the kernels drop dead workspace lines
+ * from L2 without writing them back).  Enqueued on cuda_stream; returns
+ * immediately.  Errors (nothing enqueued): INVALID_ARG, WORKSPACE,
+ * DEVICE_MISMATCH, UNSUPPORTED; CUDA on a launch failure. */
 tds_status tds_solve_batched(const tds_plan_t plan, const void *a, const void *b, const void *c,
                              const void *d, void *x, void *workspace, size_t workspace_bytes,
                              void *cuda_stream);
@@ -195,7 +197,8 @@ tds_status tds_solve_batched(const tds_plan_t plan, const void *a, const void *b
  * launch index = chunk * S + stage with S = passes + 1 + (k > 0), and
  * info.launches = chunks * S.  Calling every launch in order on one stream is
  * identical to tds_solve_batched (used to time each kernel with events between
- * them).  Same arguments and errors as tds_solve_batched; INVALID_ARG if the
+ * them); each launch consumes what the previous one left in the workspace, so a
+ * stage re-run without its predecessors reads undefined data.  Same arguments and errors as tds_solve_batched; INVALID_ARG if the
  * range is empty or outside [0, info.launches). */
 tds_status tds_solve_stages(const tds_plan_t plan, const void *a, const void *b, const void *c,
                             const void *d, void *x, void *workspace, size_t workspace_bytes,
