@@ -79,6 +79,7 @@ __global__ void __launch_bounds__(512, 1)
         for (int q = 0; q < 4; ++q)
             tma_load_lines(stage + q * ROWS, &tm.m[q], int(row0 / ELINE), int(sys), &full_bar);
     };
+    pdl_wait();  // the previous kernel on the stream is complete before any global access
     if (t == 0) {
         mbar_init(&full_bar, 1);
         mbar_init(&mb_next, 1);
@@ -459,8 +460,7 @@ cudaError_t launch_onchip_cpipe(const OnchipArgs<T> &A, int threads, int sm_coun
         nclusters = std::max(occ, 1) * sm_count;
     }
     nclusters = int(std::min<int64_t>(std::max(nclusters, 1), A.m_systems));
-    cfg.gridDim = dim3(unsigned(nclusters * C), 1, 1);
-    e = cudaLaunchKernelEx(&cfg, kern, A, tm, int32_t(tma_lines), tmx);
+    e = launch_pdl(kern, dim3(unsigned(nclusters * C)), dim3(threads), smem, st, C, A, tm, int32_t(tma_lines), tmx);
     if (e != cudaSuccess) return e;
     return cudaGetLastError();
 }

@@ -15,8 +15,19 @@
 // reads chunk (q + l/2) mod 4 in instruction q, which is conflict-free, and a
 // 4-way select puts every chunk back in its register slot.
 #include "pipe.cuh"
+#include <cstdlib>
 
 namespace tds {
+
+// Ablation build (-DTDS_ONCHIP_ABLATION, diagnostics only -- results are wrong
+// when a bit is set): env TDS_ONCHIP_ABLATION = 1 skip the solve, 2 skip the
+// TMA loads, 4 skip the x stores.  Product builds compile TDS_OABL to false.
+#ifdef TDS_ONCHIP_ABLATION
+__constant__ int tds_onchip_ablation;
+#define TDS_OABL(bit) ((tds_onchip_ablation & (bit)) != 0)
+#else
+#define TDS_OABL(bit) false
+#endif
 
 template <typename T, int ZR>
 __device__ __forceinline__ void reduced_solve_pipe(T *z, int Z, int NT, int t, int log2T);
@@ -189,6 +200,7 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
             tma_load_lines(dst, map, 0, slot, bar);
     };
     auto st_x = [&](const T *src, int slot) {
+        if (TDS_OABL(4)) return;
         if constexpr ((TDS_L2HINT & 2) != 0)
             tma_store_lines_hint(&tm.m[0], src, 0, slot, l2_evict_last());
         else
@@ -202,7 +214,7 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
     // refilled in two steps: c and d as soon as the stage is in registers,
     // a once the previous x store has read it.
     auto issue_cd = [&](int64_t q, int s) {  // thread 0 only; announces all three arrays
-        if (q >= nslots) return;
+        if (q >= nslots || TDS_OABL(2)) return;
         const int64_t sigma = nslots - 1 - q;
         uint64_t *bar = &full_bar[s];
         if (tma_lines == 0) {
@@ -215,9 +227,10 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
         ld_ws(dst + 2 * ROWS, &tm.m[2], int(sigma), bar);
     };
     auto issue_a = [&](int64_t q, int s) {  // thread 0 only
-        if (q >= nslots || tma_lines == 0) return;
+        if (q >= nslots || tma_lines == 0 || TDS_OABL(2)) return;
         ld_ws(stage0 + size_t(s) * 3 * ROWS, &tm.m[0], int(nslots - 1 - q), &full_bar[s]);
     };
+    pdl_wait();  // the previous kernel on the stream is complete before any global access
     if (t == 0) {
         mbar_init(&full_bar[0], 1);
         mbar_init(&full_bar[1], 1);
@@ -236,7 +249,7 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
         const int64_t sigma = nslots - 1 - q;
         const int s = int(it & 1);
         const int64_t L = slot_len(sigma);
-        mbar_wait(&full_bar[s], uint32_t((it >> 1) & 1));
+        if (!TDS_OABL(2)) mbar_wait(&full_bar[s], uint32_t((it >> 1) & 1));
         T *sb = stage0 + size_t(s) * 3 * ROWS;
         if (L > tma_rows || tma_lines == 0) {
             // CTA-uniform: rows [tma_rows, L) by LDG; with no TMA at all also zero the rest
@@ -286,7 +299,10 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
         }
 
         if constexpr (WL) {
-            solve_item_warp<T, R>(ra, rc, rd, ya, lane, warp, nwarps, refill_a);
+            if (!TDS_OABL(1))
+                solve_item_warp<T, R>(ra, rc, rd, ya, lane, warp, nwarps, refill_a);
+            else
+                refill_a();
         } else {
         refill_a();
         // ---- B1. CR forward levels in registers
@@ -496,7 +512,16 @@ cudaError_t launch_onchip_pipe(const OnchipArgs<T> &A, int64_t nslots, int threa
             if (!encode_rows_tmap(&tm.m[q], arrs[q], int(sizeof(T)), tma_lines, nslots, A.slot, int(rows / ELINE)))
                 return cudaErrorInvalidValue;
     }
-    kern<<<(unsigned)grid, threads, smem, st>>>(A, nslots, tm, int32_t(tma_lines));
+#ifdef TDS_ONCHIP_ABLATION
+    {
+        const char *ab = std::getenv("TDS_ONCHIP_ABLATION");
+        const int v = ab ? std::atoi(ab) : 0;
+        cudaMemcpyToSymbolAsync(tds_onchip_ablation, &v, sizeof(int), 0, cudaMemcpyHostToDevice, st);
+    }
+#endif
+    cudaError_t le = launch_pdl(kern, dim3(unsigned(grid)), dim3(threads), smem, st, 1, A, nslots, tm,
+                                int32_t(tma_lines));
+    if (le != cudaSuccess) return le;
     return cudaGetLastError();
 }
 

@@ -208,6 +208,7 @@ __global__ void __launch_bounds__(kTpThreads) place_x_tma_kernel(const PlaceArgs
             else
                 tma_load_box3(sin + (s * NBX + bx) * BOX, &tm.m[0], int((jt * NBX + bx) * E), slot0, 0, &full[s]);
     };
+    pdl_wait();  // the previous kernel on the stream is complete before any global access
     if (t == 0) {
         mbar_init(&full[0], 1);
         mbar_init(&full[1], 1);
@@ -316,7 +317,9 @@ cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batc
             const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(ntiles, int64_t(std::max(occ, 1)) * sms));
             // x slots are scratch whose last reader is this kernel: drop their lines from L2 once loaded
             const int32_t disc = (slot * int64_t(sizeof(T))) % 128 == 0 && uintptr_t(xs) % 128 == 0;
-            kern<<<(unsigned)grid, kTpThreads, smem, st>>>(A, tm, ntiles, jtiles, lfull, m, disc);
+            e = launch_pdl(kern, dim3(unsigned(grid)), dim3(kTpThreads), smem, st, 1, A, tm, ntiles, jtiles, lfull, m,
+                           disc);
+            if (e != cudaSuccess) return e;
             return cudaGetLastError();
         }
     }

@@ -172,6 +172,7 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
             bulk_commit();
         }
     };
+    pdl_wait();  // the previous kernel on the stream is complete before any global access
     if (t == 0) {
         mbar_init(&bar, 1);
         asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
@@ -463,7 +464,9 @@ static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_le
         cudaMemcpyToSymbolAsync(tds_split_ablation, &v, sizeof(int), 0, cudaMemcpyHostToDevice, st);
     }
 #endif
-    kern<<<(unsigned)grid, S::NT, smem, st>>>(A, tps, nitems, tm, int32_t(tma_lines), tmo);
+    cudaError_t le = launch_pdl(kern, dim3(unsigned(grid)), dim3(S::NT), smem, st, 1, A, tps, nitems, tm,
+                                int32_t(tma_lines), tmo);
+    if (le != cudaSuccess) return le;
     return cudaGetLastError();
 }
 

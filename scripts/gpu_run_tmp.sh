@@ -1,5 +1,5 @@
-bash scripts/gpu_prof.sh r01g --config 3
-for c in 1 2 4 5; do timeout 600 python bench.py --config $c > gpurun_out/bench_r01g_cfg$c.json 2> gpurun_out/bench_r01g_cfg$c.err; done
-timeout 600 python bench.py --config 3 --dtype f64 > gpurun_out/bench_r01g_cfg3_f64.json 2> gpurun_out/bench_r01g_cfg3_f64.err
-timeout 600 python bench.py --impl reference > gpurun_out/bench_r01g_ref.json 2> gpurun_out/bench_r01g_ref.err
-ls gpurun_out
+timeout 300 python bench.py --steps 30 --warmup 5 --no-e2e --no-cpu-baseline --soak-s 0 --tune-cache gpurun_out/tc.txt > gpurun_out/pdl3.json 2>gpurun_out/pdl3.err
+for c in 2 4; do timeout 300 python bench.py --config $c --steps 30 --warmup 5 --no-e2e --no-cpu-baseline --soak-s 0 > gpurun_out/pdl$c.json 2>gpurun_out/pdl$c.err; done
+for c in 3 2 4; do python -c "
+import json; d=json.load(open('gpurun_out/pdl$c.json')); print($c, round(d['ms_per_step'],4), '%.3e'%d['value'], [(k['kernel'], round(k['ms'],4)) for k in d['roofline']['per_kernel']])"; done
+timeout 1200 python -m pytest tests -m gpu -x -q -p no:cacheprovider 2>&1 | tail -3
