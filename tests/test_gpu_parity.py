@@ -516,3 +516,53 @@ def test_onchip_pipe_paths(tds, dtype, n, kp, tl, T):
     except tds.TdsError as e:
         pytest.skip(f"plan rejected: {e}")
     check(a, b, c, d, x, dtype)
+
+
+# ------------------------------------------- back-to-back solves on one stream
+
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+def test_back_to_back_shared_workspace(tds, dtype):
+    """Several solves of different plans enqueued back to back on one stream with
+    no host synchronisation, all through ONE workspace buffer and some writing x
+    over the previous solve's input: the programmatic-dependent-launch waits
+    (griddepcontrol.wait before any global access) and the L2 discards of dead
+    scratch lines must leave every result equal to its own solve run alone."""
+    import torch
+    dt = "float32" if dtype == np.float32 else "float64"
+    cases = [(1 << 17, 4, {"k_pass": [5], "cr_levels": 4 if dtype == np.float32 else 3, "thomas_chains": 4,
+                           "tl_levels": 5}),
+             (65536, 6, {"k_pass": [4], "cr_levels": 3 if dtype == np.float32 else 2, "thomas_chains": 32,
+                         "tl_levels": 0}),
+             (8192, 8, None),                      # k = 0, static
+             ((1 << 16) + 1000, 3, {"k_pass": [4, 2], "cr_levels": 2, "thomas_chains": 32, "tl_levels": 0})]
+    plans, data, refs, wbytes = [], [], [], 0
+    for i, (n, m, params) in enumerate(cases):
+        a, b, c, d = inputs.generate(n, m, dtype, seed=40 + i)
+        plan = tds.Plan(n, m, dt, device=0, mode="static")
+        if params:
+            plan.set_params(**dict({"cluster": 1}, **params))
+        plans.append(plan)
+        data.append(to_dev(a, b, c, d))
+        refs.append((a, b, c, d))
+        wbytes = max(wbytes, plan.workspace_bytes)
+    ws = torch.empty(max(wbytes, 1), dtype=torch.uint8, device="cuda")
+    outs = [torch.empty_like(dv[3]) for dv in data]
+    torch.cuda.synchronize()
+    for rep in range(3):
+        for plan, (ta, tb, tc, td), x in zip(plans, data, outs):
+            tds.solve_batched(plan, ta, tb, tc, td, out=x, workspace=ws)
+    torch.cuda.synchronize()
+    for (a, b, c, d), x in zip(refs, outs):
+        check(a, b, c, d, x.cpu().numpy(), dtype)
+
+
+@pytest.mark.parametrize("n", [8192 * 5 + 1, 8192 * 5 + 32])
+def test_unaligned_slots_no_discard(tds, n):
+    """Slots that are not whole 128-byte lines (ceil(n / 2^k) not a multiple of
+    32 floats) disable the L2 discards; the result must not depend on it."""
+    a, b, c, d = inputs.generate(n, 6, np.float32, seed=n)
+    x, plan = run(tds, a, b, c, d, params={"k_pass": [3], "cr_levels": 4, "thomas_chains": 4, "tl_levels": 5})
+    assert plan.info["slot_rows"] * 4 % 128 != 0
+    check(a, b, c, d, x, np.float32)
+    x2, _ = run(tds, a, b, c, d, params={"k_pass": [3], "cr_levels": 4, "thomas_chains": 4, "tl_levels": 5})
+    assert np.array_equal(x, x2)
