@@ -23,9 +23,11 @@ def _dtype_code(dtype) -> int:
     return _DTYPES[name]
 
 
-def _stream_ptr(stream) -> Optional[int]:
+def _stream_ptr(stream, device: Optional[int] = None) -> Optional[int]:
     import torch
     if stream is None:
+        if device is not None:  # the raw current-stream handle, without building a Stream object
+            return torch._C._cuda_getCurrentRawStream(device)
         stream = torch.cuda.current_stream()
     return stream.cuda_stream
 
@@ -76,6 +78,18 @@ class Plan:
         L.check(self._lib.tds_plan_info_get(self._h, ctypes.byref(info)))
         return info
 
+    def _solve_info(self):
+        """(info, required elements, torch dtype, device), cached per plan state
+        (set_params / set_params_list / tune drop it)."""
+        c = getattr(self, "_cache", None)
+        if c is None:
+            import torch
+            info = self.info_struct()
+            c = (info, (info.m - 1) * info.batch_stride + info.n,
+                 torch.float32 if info.dtype == L.TDS_F32 else torch.float64, int(info.device))
+            self._cache = c
+        return c
+
     @property
     def info(self) -> dict:
         s = self.info_struct()
@@ -103,6 +117,7 @@ class Plan:
                 p.k = sum(val)
             else:
                 setattr(p, key, int(val))
+        self._cache = None
         L.check(self._lib.tds_plan_set_params(self._h, ctypes.byref(p)))
 
     def params_list(self) -> list:
@@ -124,6 +139,7 @@ class Plan:
                     p.k_pass[i] = next(it)
             else:
                 setattr(p, f, next(it))
+        self._cache = None
         L.check(self._lib.tds_plan_set_params(self._h, ctypes.byref(p)))
 
     def permutation(self) -> np.ndarray:
@@ -135,6 +151,7 @@ class Plan:
     def tune(self, stream=None, cache_path: Optional[str] = None) -> int:
         """tds_tune; returns the number of timed trials (0 on a cache hit)."""
         cp = cache_path.encode() if cache_path else None
+        self._cache = None
         L.check(self._lib.tds_tune(self._h, _stream_ptr(stream), cp))
         t = ctypes.c_int32()
         L.check(self._lib.tds_plan_tune_trials(self._h, ctypes.byref(t)))
@@ -154,12 +171,17 @@ def _ptr(t) -> int:
 
 def _check_tensor(t, plan_info, name):
     import torch
-    if not isinstance(t, torch.Tensor) or not t.is_cuda:
-        raise TypeError(f"{name} must be a CUDA tensor")
     want = torch.float32 if plan_info.dtype == L.TDS_F32 else torch.float64
+    need = (plan_info.m - 1) * plan_info.batch_stride + plan_info.n
+    _check_fast(t, need, want, name)
+
+
+def _check_fast(t, need, want, name):
+    """Argument checks of the Python face (the C ABI re-checks pointers / sizes)."""
+    if getattr(t, "is_cuda", False) is not True:
+        raise TypeError(f"{name} must be a CUDA tensor")
     if t.dtype != want:
         raise TypeError(f"{name} has dtype {t.dtype}, plan expects {want}")
-    need = (plan_info.m - 1) * plan_info.batch_stride + plan_info.n
     if t.numel() < need or not t.is_contiguous():
         raise ValueError(f"{name} must be contiguous with >= {need} elements")
 
@@ -168,18 +190,21 @@ def solve_batched(plan: Plan, a, b, c, d, out=None, workspace=None, stream=None)
     """x = A^{-1} d for every system (tds_solve_batched).  a, b, c, d: CUDA
     tensors laid out as the plan says (m x batch_stride).  Returns x."""
     import torch
-    info = plan.info_struct()
-    for name, t in (("a", a), ("b", b), ("c", c), ("d", d)):
-        _check_tensor(t, info, name)
+    info, need, want, dev = plan._solve_info()
+    _check_fast(a, need, want, "a")
+    _check_fast(b, need, want, "b")
+    _check_fast(c, need, want, "c")
+    _check_fast(d, need, want, "d")
     if out is None:
         out = torch.empty_like(d)
-    _check_tensor(out, info, "out")
-    if workspace is None:
+    else:
+        _check_fast(out, need, want, "out")
+    if workspace is None and info.workspace_bytes > 0:
         workspace = plan.workspace()
-    wptr = _ptr(workspace) if workspace is not None else None
+    wptr = workspace.data_ptr() if workspace is not None else None
     wbytes = workspace.numel() * workspace.element_size() if workspace is not None else 0
-    L.check(plan._lib.tds_solve_batched(plan.handle, _ptr(a), _ptr(b), _ptr(c), _ptr(d), _ptr(out), wptr,
-                                        wbytes, _stream_ptr(stream)))
+    L.check(plan._lib.tds_solve_batched(plan.handle, a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
+                                        out.data_ptr(), wptr, wbytes, _stream_ptr(stream, dev)))
     return out
 
 

@@ -6,6 +6,7 @@
 #include <string>
 
 #include "common.cuh"
+#include "pipe.cuh"
 
 namespace tds {
 
@@ -184,15 +185,10 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
         cudaError_t err;
         if (P.k == 0 && onchip_cpipe_ok(I) && A.vec) {
             // persistent, TMA-fed warp-form kernel on one CTA or a 2-CTA cluster per system
-            int dev = 0, sms = 148;
-            cudaGetDevice(&dev);
-            cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-            err = launch_onchip_cpipe<T>(A, I.onchip_threads, sms, st);
+            err = launch_onchip_cpipe<T>(A, I.onchip_threads, sm_count_current(), st);
         } else if (onchip_pipe_ok(I)) {
             // persistent, TMA-pipelined form (cluster == 1, 64 bytes of rows per thread)
-            int dev = 0, sms = 148;
-            cudaGetDevice(&dev);
-            cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+            const int sms = sm_count_current();
             const size_t smem = onchip_pipe_smem_bytes(I.dtype, I.onchip_threads, 1 << P.cr_levels, P.tl_levels);
             err = launch_onchip_pipe<T>(A, I.m << P.k, I.onchip_threads, P.cr_levels, sms, smem, st);
         } else {

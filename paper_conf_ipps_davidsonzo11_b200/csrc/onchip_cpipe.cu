@@ -421,12 +421,9 @@ cudaError_t launch_onchip_cpipe(const OnchipArgs<T> &A, int threads, int sm_coun
                 : C == 4 ? onchip_cpipe_kernel<T, R, 4>
                 : C == 2 ? onchip_cpipe_kernel<T, R, 2>
                          : onchip_cpipe_kernel<T, R, 1>;
-    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    int occ = 1;  // CTAs per SM (C == 1) or clusters per device (C > 1)
+    cudaError_t e = kernel_setup((const void *)kern, threads, smem, C, &occ);
     if (e != cudaSuccess) return e;
-    if (C > 1) {
-        e = cudaFuncSetAttribute(kern, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
-        if (e != cudaSuccess) return e;
-    }
     // whole 128-byte lines of every system go by TMA (rows past them: LDG)
     const int64_t tma_lines = A.n / ELINE;
     if (tma_lines > 0x7fffffffLL || A.m_systems > 0x7fffffffLL) return cudaErrorInvalidConfiguration;
@@ -438,27 +435,7 @@ cudaError_t launch_onchip_cpipe(const OnchipArgs<T> &A, int threads, int sm_coun
                                   A.batch_stride, int(rows / ELINE)))
                 return cudaErrorInvalidValue;
     }
-    cudaLaunchConfig_t cfg{};
-    cfg.blockDim = dim3(threads, 1, 1);
-    cfg.dynamicSmemBytes = smem;
-    cfg.stream = st;
-    cudaLaunchAttribute attr[1];
-    int nclusters = 0;
-    if (C > 1) {
-        attr[0].id = cudaLaunchAttributeClusterDimension;
-        attr[0].val.clusterDim.x = C;
-        attr[0].val.clusterDim.y = 1;
-        attr[0].val.clusterDim.z = 1;
-        cfg.attrs = attr;
-        cfg.numAttrs = 1;
-        cfg.gridDim = dim3(unsigned(C), 1, 1);
-        e = cudaOccupancyMaxActiveClusters(&nclusters, kern, &cfg);
-        if (e != cudaSuccess) return e;
-    } else {
-        int occ = 1;
-        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, threads, smem);
-        nclusters = std::max(occ, 1) * sm_count;
-    }
+    int nclusters = C > 1 ? occ : std::max(occ, 1) * sm_count;
     nclusters = int(std::min<int64_t>(std::max(nclusters, 1), A.m_systems));
     e = launch_pdl(kern, dim3(unsigned(nclusters * C)), dim3(threads), smem, st, C, A, tm, int32_t(tma_lines), tmx);
     if (e != cudaSuccess) return e;

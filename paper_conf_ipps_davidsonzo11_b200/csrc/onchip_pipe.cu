@@ -495,10 +495,9 @@ cudaError_t launch_onchip_pipe(const OnchipArgs<T> &A, int64_t nslots, int threa
     const bool wide = (1 << cr_levels) == RW;
     auto kern = wide ? (A.tl_levels == 5 ? onchip_pipe_kernel<T, RW, true> : onchip_pipe_kernel<T, RW, false>)
                      : (A.tl_levels == 5 ? onchip_pipe_kernel<T, RN, true> : onchip_pipe_kernel<T, RN, false>);
-    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-    if (e != cudaSuccess) return e;
     int occ = 1;  // smaller subsystems fit two or more persistent CTAs per SM
-    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, threads, smem);
+    cudaError_t e = kernel_setup((const void *)kern, threads, smem, 1, &occ);
+    if (e != cudaSuccess) return e;
     const int64_t grid = std::min<int64_t>(nslots, int64_t(std::max(occ, 1)) * sm_count);
     // every slot holds at least n >> K rows: that many whole 128-byte lines go by TMA
     constexpr int ELINE = 128 / int(sizeof(T));

@@ -3,6 +3,9 @@
 #pragma once
 #include <cuda.h>
 
+#include <map>
+#include <mutex>
+#include <tuple>
 #include <utility>
 
 #include "common.cuh"
@@ -15,6 +18,71 @@ namespace tds {
 // on the stream drains; every thread waits here for that kernel's completion
 // and memory before its first global-memory access.  A no-op for a normal launch.
 __device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
+
+// Host: per-launch setup that does not change between solves -- the dynamic
+// shared-memory opt-in, the non-portable cluster opt-in and the occupancy
+// query -- done once per (kernel, device, block, smem, cluster) and cached
+// (they cost several microseconds of host time per launch otherwise).
+// Returns the resident CTAs per SM (cluster == 1) or the resident clusters
+// per device (cluster > 1) through *occ.
+inline cudaError_t kernel_setup(const void *kern, int threads, size_t smem, int cluster, int *occ) {
+    static std::mutex mu;
+    static std::map<std::tuple<const void *, int, int, size_t, int>, int> cache;  // -> occupancy
+    static std::map<std::pair<const void *, int>, size_t> smem_set;              // opt-in granted so far
+    int dev = 0;
+    cudaError_t e = cudaGetDevice(&dev);
+    if (e != cudaSuccess) return e;
+    const auto key = std::make_tuple(kern, dev, threads, smem, cluster);
+    std::lock_guard<std::mutex> lock(mu);
+    const auto it = cache.find(key);
+    if (it != cache.end()) {
+        *occ = it->second;
+        return cudaSuccess;
+    }
+    // the opt-in only ever grows: a smaller request must not revoke a larger one
+    size_t &granted = smem_set[std::make_pair(kern, dev)];
+    if (smem > granted) {
+        e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, int(smem));
+        if (e != cudaSuccess) return e;
+        granted = smem;
+    }
+    int v = 1;
+    if (cluster > 1) {
+        e = cudaFuncSetAttribute(kern, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
+        if (e != cudaSuccess) return e;
+        cudaLaunchConfig_t cfg{};
+        cfg.blockDim = dim3(unsigned(threads));
+        cfg.gridDim = dim3(unsigned(cluster));
+        cfg.dynamicSmemBytes = smem;
+        cudaLaunchAttribute attr[1];
+        attr[0].id = cudaLaunchAttributeClusterDimension;
+        attr[0].val.clusterDim.x = unsigned(cluster);
+        attr[0].val.clusterDim.y = 1;
+        attr[0].val.clusterDim.z = 1;
+        cfg.attrs = attr;
+        cfg.numAttrs = 1;
+        e = cudaOccupancyMaxActiveClusters(&v, kern, &cfg);
+    } else {
+        e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&v, kern, threads, smem);
+    }
+    if (e != cudaSuccess) return e;
+    cache.emplace(key, v);
+    *occ = v;
+    return cudaSuccess;
+}
+
+// Host: SM count of the current device (cached).
+inline int sm_count_current() {
+    static int sms[64] = {0};
+    int dev = 0;
+    if (cudaGetDevice(&dev) != cudaSuccess || dev < 0 || dev >= 64) return 148;
+    if (sms[dev] == 0) {
+        int v = 0;
+        cudaDeviceGetAttribute(&v, cudaDevAttrMultiProcessorCount, dev);
+        sms[dev] = v > 0 ? v : 148;
+    }
+    return sms[dev];
+}
 
 // Host: launch with programmatic stream serialisation (plus an optional cluster).
 template <typename... KArgs, typename... Args>

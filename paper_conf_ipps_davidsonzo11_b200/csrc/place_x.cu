@@ -308,13 +308,11 @@ cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batc
             encode_box3_tmap(&tm.m[1], x, int(sizeof(T)), dout, sout_, bout)) {
             const size_t smem = 1024 + size_t(3 * kTpBoxes * E * E) * sizeof(T);
             auto kern = place_x_tma_kernel<T>;
-            cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+            int occ = 1;
+            cudaError_t e = kernel_setup((const void *)kern, kTpThreads, smem, 1, &occ);
             if (e != cudaSuccess) return e;
-            int dev = 0, sms = 148, occ = 1;
-            cudaGetDevice(&dev);
-            cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, kTpThreads, smem);
-            const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(ntiles, int64_t(std::max(occ, 1)) * sms));
+            const int64_t grid =
+                std::max<int64_t>(1, std::min<int64_t>(ntiles, int64_t(std::max(occ, 1)) * sm_count_current()));
             // x slots are scratch whose last reader is this kernel: drop their lines from L2 once loaded
             const int32_t disc = (slot * int64_t(sizeof(T))) % 128 == 0 && uintptr_t(xs) % 128 == 0;
             e = launch_pdl(kern, dim3(unsigned(grid)), dim3(kTpThreads), smem, st, 1, A, tm, ntiles, jtiles, lfull, m,

@@ -420,7 +420,8 @@ static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_le
     using S = SplitShape<KP, NT>;
     auto kern = split_pipe_kernel<T, KP, RAW, NT>;
     const size_t smem = S::template smem_bytes<T>(RAW);
-    cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    int occ = 1;
+    cudaError_t e = kernel_setup((const void *)kern, S::NT, smem, 1, &occ);
     if (e != cudaSuccess) return e;
     const int64_t tps = (max_len + S::TV - 1) / S::TV;
     const int64_t nitems = m_in * tps;
@@ -452,11 +453,7 @@ static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_le
                                  msys, S::BOXP))
                 return cudaErrorInvalidValue;
     }
-    int dev = 0, sms = 148, occ = 1;
-    cudaGetDevice(&dev);
-    cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, kern, S::NT, smem);
-    const int64_t grid = std::min<int64_t>(nitems, int64_t(std::max(occ, 1)) * sms);
+    const int64_t grid = std::min<int64_t>(nitems, int64_t(std::max(occ, 1)) * sm_count_current());
 #ifdef TDS_SPLIT_ABLATION
     {
         const char *ab = std::getenv("TDS_SPLIT_ABLATION");
