@@ -130,20 +130,21 @@ def algorithmic_bytes(info: dict, s: int):
     pass 1 reads a,b,c,d and writes normalised a',c',d' (7 s/eq); a later pass
     reads and writes 3 arrays (6 s/eq); the on-chip kernel reads 3 arrays and
     writes per-subsystem x (4 s/eq; 4 raw arrays + x = 5 s/eq when k = 0); the
-    x placement reads and writes x once (2 s/eq, k > 0 only)."""
+    x placement reads and writes x once (2 s/eq, k > 0 and x_group == 0 only;
+    with x_group > 0 the on-chip kernel writes x in place: still 4 s/eq)."""
     eqs = info["n"] * info["m"]
     out = []
     for p in range(info["passes"]):
         out.append((7 if p == 0 else 6) * s * eqs)
     out.append((5 if info["passes"] == 0 else 4) * s * eqs)
-    if info["k"] > 0:
+    if info["k"] > 0 and info["x_group"] == 0:
         out.append(2 * s * eqs)
     return out
 
 
 def stage_names(info):
     names = [f"split_pass_{p}(k_p={info['k_pass'][p]})" for p in range(info["passes"])] + ["onchip_cr_pcr_thomas"]
-    if info["k"] > 0:
+    if info["k"] > 0 and info["x_group"] == 0:
         names.append("place_x")
     return names
 
@@ -285,7 +286,7 @@ def run_tds(args):
     info = plan.info
     ws = plan.workspace()
     NL = info["launches"]                            # kernel launches per step (all chunks)
-    S = info["passes"] + 1 + (1 if info["k"] > 0 else 0)  # kernels per chunk
+    S = info["passes"] + 1 + (1 if info["k"] > 0 and info["x_group"] == 0 else 0)  # kernels per chunk
     stream = torch.cuda.current_stream()
 
     def step():
@@ -440,7 +441,7 @@ def run_tds(args):
                                                                      "cr_levels", "thomas_chains",
                                                                      "cluster", "tl_levels", "chunk_systems",
                                                                      "chunks", "launches", "split_tile_rows", "split_threads",
-                                                                     "theta", "split_segments",
+                                                                     "theta", "split_segments", "x_group",
                                                                      "onchip_threads", "workspace_bytes")},
                    "tune_trials": trials, "tune_s": round(tune_s, 2),
                    "l2": f"no flush: per-step working set {(5 * eqs_per_step * s + info['workspace_bytes']) / 2**20:.0f} MiB > L2 126 MiB"

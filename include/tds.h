@@ -104,6 +104,14 @@ typedef struct {
     int32_t chunk_systems;           /* systems per L2-resident chunk (0 = all at once) */
     int32_t split_only;              /* 1: plan only the split passes (tds_split_batched;
                                         on-chip limits not checked, tds_solve_* refuse) */
+    int32_t x_group;                 /* 0: x placed by a separate kernel (k > 0).  G = 2, 4
+                                        or 8: a cluster of G on-chip CTAs solves G adjacent
+                                        residue classes (Fig. 3a) and stores x
+                                        straight to rows r + 2^k j in G-element runs; needs
+                                        k > 0, 2^k | n, G <= 2^k, one subsystem per CTA
+                                        (n / 2^k = threads x 2^c), tl_levels = 5,
+                                        2^c sizeof(T) = 64, G sizeof(T) >= 16, and
+                                        2^k sizeof(T), batch_stride sizeof(T) multiples of 16 */
 } tds_params;
 
 /* Everything a plan decided (read-only view). */
@@ -193,8 +201,8 @@ tds_status tds_solve_batched(const tds_plan_t plan, const void *a, const void *b
 /* Run only launches first_stage..last_stage (inclusive) of the kernel sequence
  * tds_solve_batched enqueues.  The sequence is, for each chunk of
  * chunk_systems systems in order: split passes 0..passes-1 (PAPER.md stages
- * 1-2), the on-chip kernel (stages 3-4) and, when k > 0, the x placement;
- * launch index = chunk * S + stage with S = passes + 1 + (k > 0), and
+ * 1-2), the on-chip kernel (stages 3-4) and, when k > 0 and x_group == 0, the x placement;
+ * launch index = chunk * S + stage with S = passes + 1 + (k > 0 && x_group == 0), and
  * info.launches = chunks * S.  Calling every launch in order on one stream is
  * identical to tds_solve_batched (used to time each kernel with events between
  * them); each launch consumes what the previous one left in the workspace, so a

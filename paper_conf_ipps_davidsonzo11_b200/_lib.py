@@ -44,7 +44,8 @@ class Params(ctypes.Structure):
                 ("tl_levels", ctypes.c_int32),
                 ("split_tile_rows", ctypes.c_int32),
                 ("split_threads", ctypes.c_int32), ("theta", ctypes.c_int32),
-                ("chunk_systems", ctypes.c_int32), ("split_only", ctypes.c_int32)]
+                ("chunk_systems", ctypes.c_int32), ("split_only", ctypes.c_int32),
+                ("x_group", ctypes.c_int32)]
 
 
 class PlanInfo(ctypes.Structure):

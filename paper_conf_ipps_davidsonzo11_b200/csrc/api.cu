@@ -152,6 +152,7 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
     A.log2T = l2;
     A.cluster = P.cluster;
     A.tl_levels = P.tl_levels;
+    A.x_group = P.x_group;
     int64_t grid;
     if (P.k == 0) {
         A.a = a;
@@ -186,6 +187,9 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
         if (P.k == 0 && onchip_cpipe_ok(I) && A.vec) {
             // persistent, TMA-fed warp-form kernel on one CTA or a 2-CTA cluster per system
             err = launch_onchip_cpipe<T>(A, I.onchip_threads, sm_count_current(), st);
+        } else if (P.x_group > 0 && uintptr_t(x) % 16 == 0) {
+            // cluster of x_group CTAs on adjacent residue classes, x stored in place (no placement kernel)
+            err = launch_onchip_gpipe<T>(A, I.m << P.k, I.onchip_threads, sm_count_current(), st);
         } else if (onchip_pipe_ok(I)) {
             // persistent, TMA-pipelined form (cluster == 1, 64 bytes of rows per thread)
             const int sms = sm_count_current();
@@ -197,7 +201,11 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
         }
         if (err != cudaSuccess) return cuda_fail(err, "onchip launch");
     }
-    if (P.k > 0 && P.passes + 1 >= first && P.passes + 1 <= last) {
+    // x_group plans place x inside the on-chip stage (a misaligned x falls back
+    // to the slot kernel + placement, both counted as that one stage)
+    const bool place = P.x_group == 0 ? P.passes + 1 >= first && P.passes + 1 <= last
+                                      : uintptr_t(x) % 16 != 0 && P.passes >= first && P.passes <= last;
+    if (P.k > 0 && place) {
         cudaError_t err = launch_place_x<T>(A.xs, x, I.n, I.m, I.batch_stride, I.slot_rows, P.k,
                                             vec_ok(I, {(const void *)x}), A.geom, st);
         if (err != cudaSuccess) return cuda_fail(err, "place_x launch");
@@ -244,13 +252,13 @@ static tds_status split_impl(const tds_plan_info &I, const T *a, const T *b, con
 }
 
 // Run launches [first, last] of the chunked sequence: for each chunk of
-// chunk_systems systems, S = passes + 1 + (k > 0) kernels.  Chunks reuse one
+// chunk_systems systems, S = passes + 1 + (k > 0 && x_group == 0) kernels.  Chunks reuse one
 // workspace, so a chunk's split output is still in L2 when its on-chip kernel
 // and x placement read it.
 template <typename T>
 static tds_status solve_chunks(const tds_plan_info &I, const T *a, const T *b, const T *c, const T *d, T *x,
                                void *ws, cudaStream_t st, int first, int last) {
-    const int S = I.params.passes + 1 + (I.params.k > 0 ? 1 : 0);
+    const int S = I.params.passes + 1 + (I.params.k > 0 && I.params.x_group == 0 ? 1 : 0);
     const int64_t mc = chunk_m(I.params, I.m);
     for (int64_t ch = 0; ch * mc < I.m; ++ch) {
         const int lf = std::max<int64_t>(first - ch * S, 0);

@@ -121,6 +121,7 @@ struct OnchipArgs {
     int32_t vec;             // 16-byte vector loads/stores allowed
     PassGeom geom;           // passes applied (for the slot -> residue map)
     int32_t l2_discard;      // K > 0: slots are 128-byte aligned, c/d lines may be discarded once loaded
+    int32_t x_group;         // K > 0: CTAs (one cluster) storing x of adjacent residue classes together
 };
 
 __host__ __device__ constexpr int ilog2c(int v) { return v <= 1 ? 0 : 1 + ilog2c(v / 2); }
@@ -142,6 +143,9 @@ size_t onchip_pipe_smem_bytes(int32_t dtype, int32_t threads, int32_t R, int32_t
 // one CTA per subsystem whose threads hold 64 bytes of rows per array (fp32
 // c = 4, fp64 c = 3; up to 512 threads) or 32 bytes (fp32 c = 3, fp64 c = 2;
 // up to 1024 threads).
+template <typename T>
+cudaError_t launch_onchip_gpipe(const OnchipArgs<T> &A, int64_t nslots, int threads, int sm_count, cudaStream_t st);
+
 inline bool onchip_pipe_ok(const tds_plan_info &I) {
     const tds_params &P = I.params;
     if (P.k == 0 || P.cluster != 1) return false;

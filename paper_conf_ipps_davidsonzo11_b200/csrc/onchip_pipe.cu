@@ -14,8 +14,13 @@
 // quarter-warp would hit the same bank group (4-way conflict); lane l instead
 // reads chunk (q + l/2) mod 4 in instruction q, which is conflict-free, and a
 // 4-way select puts every chunk back in its register slot.
-#include "pipe.cuh"
+#include <cooperative_groups.h>
+
 #include <cstdlib>
+
+#include "pipe.cuh"
+
+namespace cg = cooperative_groups;
 
 namespace tds {
 
@@ -480,6 +485,197 @@ __device__ __forceinline__ void reduced_solve_pipe(T *z, int Z, int NT, int t, i
     }
     __syncthreads();
 }
+
+// ---- fused x placement (plan x_group = G > 0): a cluster of G persistent
+// CTAs walks groups of G adjacent residue classes r0 .. r0+G-1 of one system
+// (slots sys 2^K + r, Fig. 3a) in lock step, one class per CTA.
+// Row j of class r0+q is original row r0 + q + 2^K j, so the G classes
+// together own G-element runs of x.  After the solve, every thread pushes its
+// R rows of x (st.async, 16 bytes each) into the a-region of the consumed stage
+// of the CTA that stores rows [p SEG, (p+1) SEG) of the group (SEG = rows/G),
+// class-major; that CTA transposes the block in place to [row][class] and
+// writes it with TMA tensor stores of {G classes x box_rows rows} boxes of the
+// x view {2^K, n/2^K, m}: whole G-element runs, no placement kernel, no x-slot
+// round trip.  Hand-offs are point-to-point mbarriers (no cluster barrier in
+// the loop): x_full counts the bytes pushed into this CTA, ready[p] tells a
+// pusher that CTA p has consumed its stage for this item.
+// Measured on B200 (profiles/r01h_xgroup.md): bit-identical to the separate
+// placement but SLOWER (config 3: 193 us vs 159 us per solve) -- DSMEM moves
+// ~20 B/clk per SM, so pushing 32 KB of x per item costs more than place_x's
+// L2 round trip, and 1-CTA/SM clusters of 4 / 8 fit only 132 / 120 of the 148
+// SMs.  Kept as a tuner dimension (tds_tune tries it; it does not win).
+// Direct G-element STG runs instead of the TMA boxes measured slower still.
+template <typename T, int R, int G>
+__global__ void __launch_bounds__(512, 1)
+    onchip_gpipe_kernel(const OnchipArgs<T> A, int64_t ngroups, const __grid_constant__ TmapSet tm,
+                        const __grid_constant__ TmapSet tmx, int32_t box_rows) {
+    static_assert(R * sizeof(T) == 64, "gpipe kernel: 64 bytes of rows per thread");
+    static_assert(R % G == 0 && G * sizeof(T) >= 16, "gpipe kernel: whole 16-byte runs");
+    constexpr int ELINE = 128 / int(sizeof(T));
+    constexpr int E16 = 16 / int(sizeof(T));  // elements per 16-byte push
+    constexpr int PER = R / G;                 // segment rows per thread in the transpose
+    extern __shared__ __align__(1024) unsigned char smem_raw[];
+    __shared__ __align__(8) uint64_t full_bar[2];
+    __shared__ __align__(8) uint64_t x_full;    // x runs of this item pushed into this CTA (bytes)
+    __shared__ __align__(8) uint64_t ready[G];  // ready[p]: CTA p consumed its stage (this item)
+    const int NT = blockDim.x;
+    const int ROWS = NT * R, SEG = ROWS / G;
+    const int t = threadIdx.x, lane = t & 31, warp = t >> 5, nwarps = NT >> 5;
+    const int rank = int(blockIdx.x % G);
+    const int64_t cid = blockIdx.x / G, ncl = gridDim.x / G;
+    T *stage0 = reinterpret_cast<T *>(smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u));  // [2][3][ROWS]
+    T *scr = stage0 + 6 * ROWS;
+    const int64_t KK = int64_t(1) << A.K;
+    auto slot_of = [&](int64_t it) -> int64_t {  // groups walked last-first (the split wrote them last)
+        const int64_t g = cid + it * ncl;
+        return g < ngroups ? (ngroups - 1 - g) * G + rank : -1;
+    };
+    auto ld_ws = [&](T *dst, const CUtensorMap *map, int64_t slot, uint64_t *bar) {
+        if constexpr ((TDS_L2HINT & 1) != 0)
+            tma_load_lines_hint(dst, map, 0, int(slot), bar, l2_evict_first());
+        else
+            tma_load_lines(dst, map, 0, int(slot), bar);
+    };
+    auto issue_cd = [&](int64_t it, int s) {  // thread 0; announces all three arrays
+        const int64_t sl = slot_of(it);
+        if (sl < 0) return;
+        mbar_expect_tx(&full_bar[s], 3 * uint32_t(ROWS) * sizeof(T));
+        T *dst = stage0 + size_t(s) * 3 * ROWS;
+        ld_ws(dst + ROWS, &tm.m[1], sl, &full_bar[s]);
+        ld_ws(dst + 2 * ROWS, &tm.m[2], sl, &full_bar[s]);
+    };
+    auto issue_a = [&](int64_t it, int s) {  // thread 0
+        const int64_t sl = slot_of(it);
+        if (sl >= 0) ld_ws(stage0 + size_t(s) * 3 * ROWS, &tm.m[0], sl, &full_bar[s]);
+    };
+    pdl_wait();  // the split pass is complete before any global access
+    if (t == 0) {
+        mbar_init(&full_bar[0], 1);
+        mbar_init(&full_bar[1], 1);
+        mbar_init(&x_full, 1);
+#pragma unroll
+        for (int q = 0; q < G; ++q) mbar_init(&ready[q], 1);
+        asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+        issue_cd(0, 0);
+        issue_a(0, 0);
+        issue_cd(1, 1);
+        issue_a(1, 1);
+    }
+    cg::this_cluster().sync();  // every CTA runs (mbarriers initialised) before any DSMEM access
+    const int own = (t * R) / SEG;  // CTA storing this thread's rows
+    const uint32_t r_xfull = cluster_addr(&x_full, own);
+    const uint32_t r_ready = t < G ? cluster_addr(&ready[rank], t) : 0u;
+
+    for (int64_t it = 0;; ++it) {
+        const int64_t sigma = slot_of(it);
+        if (sigma < 0) break;
+        const int s = int(it & 1);
+        const uint32_t ph = uint32_t(it & 1);
+        if (t == 0) mbar_expect_tx(&x_full, uint32_t(ROWS) * sizeof(T));
+        mbar_wait(&full_bar[s], uint32_t((it >> 1) & 1));
+        T *sb = stage0 + size_t(s) * 3 * ROWS;
+        if (A.l2_discard) {  // c', d' of this slot are dead once in shared memory
+            const int nl = ROWS / ELINE;
+            for (int li = t; li < 2 * nl; li += NT)
+                l2_discard_line((li < nl ? A.c : A.d) + sigma * A.slot + int64_t(li < nl ? li : li - nl) * ELINE);
+        }
+        T ra[R], rc[R], rd[R];
+        lds_rows_sw<T, R>(sb, t * R, ra);
+        lds_rows_sw<T, R>(sb + ROWS, t * R, rc);
+        lds_rows_sw<T, R>(sb + 2 * ROWS, t * R, rd);
+        __syncthreads();  // stage s consumed: its a-region now takes this item's x runs
+        if (t == 0) issue_cd(it + 2, s);
+        if (t < G) mbar_arrive_remote(r_ready);  // relaxed: the stage's reads are complete (barrier above)
+        // the previous item's x store (stage 1-s) has read its region before the a-refill
+        auto refill_a = [&]() {
+            if (t == 0 && it > 0) {
+                bulk_wait_read0();
+                issue_a(it + 1, 1 - s);
+            }
+        };
+        solve_item_warp<T, R>(ra, rc, rd, scr, lane, warp, nwarps, refill_a);
+        // push rows tR .. tR+R-1 of class rank+r0 to CTA `own`, block [G][SEG]
+        mbar_wait(&ready[own], ph);  // CTA scope: no L1 invalidation (CCTL.IVALL) per item
+        const uint32_t dst = cluster_addr(sb + rank * SEG + (t * R - own * SEG), own);
+#pragma unroll
+        for (int q = 0; q < R / E16; ++q) st_async16(dst + 16 * q, rd + q * E16, r_xfull);
+        mbar_wait(&x_full, ph);  // the G classes' runs of this CTA's segment (st.async complete_tx)
+        T v[PER][G];
+#pragma unroll
+        for (int i = 0; i < PER; ++i)
+#pragma unroll
+            for (int q = 0; q < G; ++q) v[i][q] = sb[q * SEG + t + i * NT];
+        __syncthreads();  // in place: every read precedes every write
+#pragma unroll
+        for (int i = 0; i < PER; ++i) {
+            T *row = sb + (t + i * NT) * G;
+#pragma unroll
+            for (int q = 0; q < G; q += E16) {
+                if constexpr (sizeof(T) == 4)
+                    *reinterpret_cast<float4 *>(row + q) = make_float4(v[i][q], v[i][q + 1], v[i][q + 2], v[i][q + 3]);
+                else
+                    *reinterpret_cast<double2 *>(row + q) = make_double2(v[i][q], v[i][q + 1]);
+            }
+        }
+        fence_proxy_async_smem();
+        __syncthreads();
+        if (t == 0) {
+            const int sys = int(sigma >> A.K), r0 = int((sigma & (KK - 1)) - rank);
+            for (int b = 0; b * box_rows < SEG; ++b)
+                tma_store_box3(&tmx.m[0], sb + size_t(b) * box_rows * G, r0, rank * SEG + b * box_rows, sys);
+            bulk_commit();
+        }
+    }
+    if (t == 0) bulk_wait_all();
+    cg::this_cluster().sync();  // no CTA leaves while a peer may still push into it
+}
+
+size_t onchip_gpipe_smem_bytes(int32_t dtype, int32_t threads) {
+    const int64_t R = 64 / dsize(dtype), nw = threads / 32;
+    return 1024 + size_t((6 * int64_t(threads) * R + nw * (3 * ilog2c(int(R)) + 30) + 128 + 8) * dsize(dtype));
+}
+
+template <typename T>
+cudaError_t launch_onchip_gpipe(const OnchipArgs<T> &A, int64_t nslots, int threads, int sm_count, cudaStream_t st) {
+    constexpr int R = 64 / int(sizeof(T)), ELINE = 128 / int(sizeof(T));
+    (void)sm_count;
+    const int G = A.x_group;
+    const int64_t rows = int64_t(threads) * R, L = A.n >> A.K;
+    if ((G != 2 && G != 4 && G != 8) || G * int(sizeof(T)) < 16 || L != rows || rows % (G * ELINE) || nslots % G ||
+        threads % 32 || threads > 512)
+        return cudaErrorInvalidConfiguration;
+    const int64_t seg = rows / G;
+    const int box_rows = int(std::min<int64_t>(seg, 256));
+    if (seg % box_rows || nslots > 0x7fffffffLL || A.m_systems > 0x7fffffffLL || A.K > 30)
+        return cudaErrorInvalidConfiguration;
+    const size_t smem = onchip_gpipe_smem_bytes(sizeof(T) == 4 ? TDS_F32 : TDS_F64, threads);
+    void (*kern)(const OnchipArgs<T>, int64_t, const TmapSet, const TmapSet, int32_t) = nullptr;
+    if (G == 8) kern = onchip_gpipe_kernel<T, R, 8>;
+    else if (G == 4) kern = onchip_gpipe_kernel<T, R, 4>;
+    else if constexpr (sizeof(T) == 8) kern = onchip_gpipe_kernel<T, R, 2>;
+    if (!kern) return cudaErrorInvalidConfiguration;
+    int occ = 1;  // resident clusters per device
+    cudaError_t e = kernel_setup((const void *)kern, threads, smem, G, &occ);
+    if (e != cudaSuccess) return e;
+    TmapSet tm{}, tmx{};
+    const T *arrs[3] = {A.a, A.c, A.d};
+    for (int q = 0; q < 3; ++q)
+        if (!encode_rows_tmap(&tm.m[q], arrs[q], int(sizeof(T)), rows / ELINE, nslots, A.slot, int(rows / ELINE)))
+            return cudaErrorInvalidValue;
+    const uint64_t dims[3] = {uint64_t(1) << A.K, uint64_t(L), uint64_t(A.m_systems)};
+    const uint64_t strides[2] = {(uint64_t(1) << A.K) * sizeof(T), uint64_t(A.batch_stride) * sizeof(T)};
+    const uint32_t box[3] = {uint32_t(G), uint32_t(box_rows), 1};
+    if (!encode_box3_tmap_plain(&tmx.m[0], A.x, int(sizeof(T)), dims, strides, box)) return cudaErrorInvalidValue;
+    const int64_t ngroups = nslots / G;
+    const int64_t ncl = std::min<int64_t>(std::max(occ, 1), ngroups);
+    e = launch_pdl(kern, dim3(unsigned(ncl * G)), dim3(threads), smem, st, G, A, ngroups, tm, tmx,
+                   int32_t(box_rows));
+    if (e != cudaSuccess) return e;
+    return cudaGetLastError();
+}
+
+template cudaError_t launch_onchip_gpipe<float>(const OnchipArgs<float> &, int64_t, int, int, cudaStream_t);
+template cudaError_t launch_onchip_gpipe<double>(const OnchipArgs<double> &, int64_t, int, int, cudaStream_t);
 
 size_t onchip_pipe_smem_bytes(int32_t dtype, int32_t threads, int32_t R, int32_t tl_levels) {
     const int64_t rows = int64_t(threads) * R;

@@ -336,6 +336,42 @@ __device__ __forceinline__ void st_async(uint32_t raddr, double v, uint32_t rbar
                  : "memory");
 }
 
+// 16 bytes (4 fp32 / 2 fp64) into a peer CTA's shared memory, counted on its mbarrier.
+__device__ __forceinline__ void st_async16(uint32_t raddr, const float *v, uint32_t rbar) {
+    asm volatile("st.async.shared::cluster.mbarrier::complete_tx::bytes.v4.b32 [%0], {%1, %2, %3, %4}, [%5];" ::"r"(
+                     raddr),
+                 "r"(__float_as_uint(v[0])), "r"(__float_as_uint(v[1])), "r"(__float_as_uint(v[2])),
+                 "r"(__float_as_uint(v[3])), "r"(rbar)
+                 : "memory");
+}
+__device__ __forceinline__ void st_async16(uint32_t raddr, const double *v, uint32_t rbar) {
+    asm volatile("st.async.shared::cluster.mbarrier::complete_tx::bytes.v2.b64 [%0], {%1, %2}, [%3];" ::"r"(raddr),
+                 "l"(__double_as_longlong(v[0])), "l"(__double_as_longlong(v[1])), "r"(rbar)
+                 : "memory");
+}
+// Arrive (count 1) on an mbarrier of a cluster peer (address from cluster_addr).
+// Relaxed: used only as a "this buffer may be overwritten" signal after a CTA
+// barrier that completed every read of the buffer (no data is published).
+__device__ __forceinline__ void mbar_arrive_remote(uint32_t rbar) {
+    asm volatile("mbarrier.arrive.relaxed.cluster.shared::cluster.b64 _, [%0];" ::"r"(rbar) : "memory");
+}
+// Wait for a phase completed by cluster peers (acquire at cluster scope).
+__device__ __forceinline__ void mbar_wait_cluster(uint64_t *bar, uint32_t parity) {
+    uint32_t done = 0;
+    while (!done) {
+        asm volatile(
+            "{\n .reg .pred p;\n mbarrier.try_wait.parity.acquire.cluster.shared::cta.b64 p, [%1], %2;\n selp.u32 %0, "
+            "1, 0, p;\n}\n"
+            : "=r"(done)
+            : "r"(smem_u32(bar)), "r"(parity)
+            : "memory");
+    }
+}
+
+// Host: a 3-D view without swizzle (box inner dimension: any multiple of 16 bytes).
+bool encode_box3_tmap_plain(CUtensorMap *out, const void *base, int dsize, const uint64_t dims[3],
+                            const uint64_t strides[2], const uint32_t box[3]);
+
 // Host: encode the tensor map of `slots` row slots of `lines` full 128-byte
 // lines each, slot stride `stride` elements, box of `box_lines` lines.
 bool encode_rows_tmap(CUtensorMap *out, const void *base, int dsize, int64_t lines, int64_t slots, int64_t stride,

@@ -170,6 +170,20 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
         }
     }
     if (p.chunk_systems < 0) return fail(TDS_ERR_INVALID_ARG, "chunk_systems >= 0");
+    if (p.x_group != 0) {  // fused x placement (onchip_pipe.cu, gpipe kernel)
+        const int G = p.x_group, ds = dsize(dtype);
+        if (G != 2 && G != 4 && G != 8) return fail(TDS_ERR_INVALID_ARG, "x_group must be 0, 2, 4 or 8");
+        if (p.split_only) return fail(TDS_ERR_INVALID_ARG, "x_group needs an on-chip stage");
+        if (p.k == 0 || p.k > 30 || (int64_t(1) << p.k) < G || n % (int64_t(1) << p.k) != 0)
+            return fail(TDS_ERR_UNSUPPORTED, "x_group needs k >= log2(x_group) and 2^k dividing n");
+        const int64_t L = n >> p.k, seg = L / G;
+        if (p.cluster != 1 || p.tl_levels != 5 || R * ds != 64 || L != threads * R || L % G ||
+            (L * ds) % 128 || (seg > 256 && seg % 256))
+            return fail(TDS_ERR_UNSUPPORTED, "x_group needs cluster 1, tl_levels 5, 64 bytes of rows per thread, "
+                                             "n / 2^k = threads x 2^c in whole 128-byte lines");
+        if (G * ds < 16 || ((int64_t(1) << p.k) * ds) % 16 || (info.batch_stride * ds) % 16)
+            return fail(TDS_ERR_UNSUPPORTED, "x_group needs 16-byte runs, 2^k and batch_stride in 16-byte units");
+    }
     // --- derived fields
     info.params = p;
     info.n_sub = n_sub;
@@ -178,7 +192,7 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
     info.subsys_per_cta = 1;
     const int64_t mc = chunk_m(p, m);  // systems per chunk
     info.chunks = (int32_t)cdiv(m, mc);
-    info.launches = info.chunks * (p.passes + 1 + (p.k > 0 ? 1 : 0));
+    info.launches = info.chunks * (p.passes + 1 + (p.k > 0 && p.x_group == 0 ? 1 : 0));
     if (p.passes > 0) {
         int kk = 0;
         int64_t elems = 0;

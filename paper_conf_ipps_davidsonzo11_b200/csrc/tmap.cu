@@ -67,4 +67,21 @@ bool encode_box3_tmap(CUtensorMap *out, const void *base, int dsize, const uint6
     return r == CUDA_SUCCESS;
 }
 
+bool encode_box3_tmap_plain(CUtensorMap *out, const void *base, int dsize, const uint64_t dims[3],
+                            const uint64_t strides[2], const uint32_t box[3]) {
+    const PFN_cuTensorMapEncodeTiled_v12000 fn = encode_fn();
+    if (!fn) return false;
+    for (int i = 0; i < 3; ++i)
+        if (dims[i] < 1 || box[i] < 1 || box[i] > 256) return false;
+    const cuuint64_t d[3] = {dims[0], dims[1], dims[2]};
+    const cuuint64_t st[2] = {strides[0], strides[1]};
+    const cuuint32_t b[3] = {box[0], box[1], box[2]};
+    const cuuint32_t estr[3] = {1, 1, 1};
+    const CUresult r = fn(out, dsize == 4 ? CU_TENSOR_MAP_DATA_TYPE_FLOAT32 : CU_TENSOR_MAP_DATA_TYPE_FLOAT64, 3,
+                          const_cast<void *>(base), d, st, b, estr, CU_TENSOR_MAP_INTERLEAVE_NONE,
+                          CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_NONE,
+                          CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+    return r == CUDA_SUCCESS;
+}
+
 }  // namespace tds

@@ -138,7 +138,7 @@ static void tune_onchip(TuneCtx &C, tds_params &best, double &t_best) {
     bool improved = true;
     while (improved && !out_of_time(C)) {
         improved = false;
-        tds_params cand[12];
+        tds_params cand[16];
         int nc = 0;
         // the warp-level form (CR across all 32 lanes, shuffles only) is a
         // different kernel path, not a neighbour of tl_levels = 4: try it directly
@@ -158,6 +158,20 @@ static void tune_onchip(TuneCtx &C, tds_params &best, double &t_best) {
         if (best.cluster > 1) { cand[nc] = best; cand[nc].cluster /= 2; cand[nc++].tl_levels -= best.tl_levels > 0; }
         if (best.cluster < 16 && C.plan->props.cc_major >= 9) {
             cand[nc] = best; cand[nc].cluster *= 2; cand[nc++].tl_levels += 1;
+        }
+        // fused x placement (k > 0, warp form, 64 bytes of rows per thread): off, or
+        // clusters of G CTAs on adjacent residue classes; G halves / doubles
+        if (best.k > 0 && best.cluster == 1 && best.tl_levels == 5 &&
+            (1 << best.cr_levels) * dsize(I.dtype) == 64) {
+            const int gmin = 16 / dsize(I.dtype);
+            if (best.x_group == 0) {
+                cand[nc] = best; cand[nc++].x_group = 8;
+                cand[nc] = best; cand[nc++].x_group = 4;
+            } else {
+                cand[nc] = best; cand[nc++].x_group = 0;
+                if (best.x_group / 2 >= gmin) { cand[nc] = best; cand[nc++].x_group = best.x_group / 2; }
+                if (best.x_group < 8) { cand[nc] = best; cand[nc++].x_group = best.x_group * 2; }
+            }
         }
         for (int i = 0; i < nc; ++i) {
             clamp_onchip(I, cand[i]);
@@ -191,6 +205,7 @@ static void fit_onchip(const tds_plan_info &I, const tds_device_props &props, td
     p.cr_levels = ilog2i(r_max(I.dtype));
     while (thr(p) > cap(p.cr_levels) && p.cluster < 16 && props.cc_major >= 9) p.cluster *= 2;
     p.tl_levels = ilog2i(p.cluster);
+    p.x_group = 0;  // re-enabled by tune_onchip where the new subsystem size allows it
     clamp_onchip(I, p);
 }
 
@@ -212,7 +227,8 @@ static std::string params_str(const tds_params &p) {
     o << p.k << " " << p.passes;
     for (int i = 0; i < TDS_MAX_PASSES; ++i) o << " " << p.k_pass[i];
     o << " " << p.cr_levels << " " << p.thomas_chains << " " << p.cluster << " " << p.tl_levels << " "
-      << p.split_tile_rows << " " << p.split_threads << " " << p.theta << " " << p.chunk_systems;
+      << p.split_tile_rows << " " << p.split_threads << " " << p.theta << " " << p.chunk_systems << " "
+      << p.x_group;
     return o.str();
 }
 
@@ -231,6 +247,7 @@ static bool cache_lookup(const std::string &path, const std::string &key, tds_pa
         is >> q.cr_levels >> q.thomas_chains >> q.cluster >> q.tl_levels >> q.split_tile_rows >> q.split_threads >>
             q.theta >> q.chunk_systems;
         if (is) {
+            if (!(is >> q.x_group)) q.x_group = 0;  // lines written before x_group existed
             p = q;
             found = true;
         }

@@ -154,3 +154,31 @@ def test_solve_argument_errors_before_launch(tds):
     assert f(A, B, C, D, X, A, ws_need) == 1                    # workspace overlaps an array
     assert f(A, B, C, D, D, W, ws_need) in (5, 7)               # valid (x == d): no device here
     assert nbytes < (1 << 30)
+
+
+def test_x_group_validation(tds):
+    """Fused x placement (x_group): accepted only where the gpipe kernel can
+    store whole G-element runs of x (include/tds.h tds_params.x_group)."""
+    p = tds.Plan(1 << 20, 16, props=_props(rp.B200))
+    base = dict(k_pass=[7], cr_levels=4, thomas_chains=16, cluster=1, tl_levels=5)
+    p.set_params(**base, x_group=8)
+    i = p.info
+    assert i["x_group"] == 8 and i["launches"] == 2  # split + on-chip, no placement kernel
+    p.set_params(**base, x_group=0)
+    assert p.info["launches"] == 3
+    bad = [dict(x_group=3), dict(x_group=16), dict(x_group=2),          # fp32 runs need >= 4 elements
+           dict(x_group=8, tl_levels=3), dict(x_group=8, cluster=2),
+           dict(x_group=8, cr_levels=3),                                  # 32 bytes of rows per thread
+           dict(x_group=8, k_pass=[], cr_levels=4)]                       # k = 0
+    for kw in bad:
+        with pytest.raises(tds.TdsError):
+            p.set_params(**dict(base, **kw))
+    q = tds.Plan((1 << 20) + 128, 2, props=_props(rp.B200))             # 2^7 does not divide n
+    with pytest.raises(tds.TdsError):
+        q.set_params(**base, x_group=8)
+    q = tds.Plan(98304, 2, props=_props(rp.B200))                        # 768-row slots: 48 rows short of 64 x 16
+    with pytest.raises(tds.TdsError):
+        q.set_params(**dict(base, thomas_chains=1), x_group=8)
+    r = tds.Plan(1 << 20, 2, "float64", props=_props(rp.B200))
+    r.set_params(k_pass=[8], cr_levels=3, thomas_chains=16, cluster=1, tl_levels=5, x_group=2)
+    assert r.info["launches"] == 2

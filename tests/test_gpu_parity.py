@@ -566,3 +566,108 @@ def test_unaligned_slots_no_discard(tds, n):
     check(a, b, c, d, x, np.float32)
     x2, _ = run(tds, a, b, c, d, params={"k_pass": [3], "cr_levels": 4, "thomas_chains": 4, "tl_levels": 5})
     assert np.array_equal(x, x2)
+
+
+# ------------------------------- fused x placement (x_group: clusters of G CTAs)
+
+XG_CASES = [  # (dtype, n, m, k_pass, G)
+    (np.float32, 1 << 20, 3, [7], 8), (np.float32, 1 << 20, 2, [7], 4), (np.float32, 1 << 17, 5, [4], 8),
+    (np.float32, 1 << 16, 3, [3], 8),           # 2^k == G: one group per system
+    (np.float32, 1 << 15, 4, [2], 4),           # 2^k == G == 4
+    (np.float32, 1 << 20, 2, [4, 3], 8),        # two split passes
+    (np.float32, 24576, 3, [4], 8),             # 96 threads: 1536-row slots, 192-row segments (one box)
+    (np.float32, 1 << 21, 1, [8], 8),           # 256 threads, m = 1
+    (np.float64, 1 << 20, 2, [8], 2), (np.float64, 1 << 20, 2, [8], 4), (np.float64, 1 << 20, 2, [8], 8),
+    (np.float64, 1 << 16, 3, [4], 4), (np.float64, 1 << 18, 2, [3, 3], 8)]
+
+
+def _xg_params(dtype, kp, G):
+    return dict(k_pass=kp, cr_levels=4 if dtype == np.float32 else 3, thomas_chains=1, tl_levels=5, x_group=G)
+
+
+@pytest.mark.parametrize("dtype,n,m,kp,G", XG_CASES)
+def test_fused_placement_vs_oracle_and_unfused(tds, dtype, n, m, kp, G):
+    """x_group = G stores x straight from a cluster of G on-chip CTAs: the
+    result is the oracle's within tolerance and BIT-identical to the same plan
+    with the separate placement kernel (same arithmetic, different data path)."""
+    a, b, c, d = inputs.generate(n, m, dtype, seed=60 + G)
+    x, plan = run(tds, a, b, c, d, params=_xg_params(dtype, kp, G))
+    assert plan.info["x_group"] == G and plan.info["launches"] == len(kp) + 1
+    check(a, b, c, d, x, dtype)
+    x0, _ = run(tds, a, b, c, d, params=_xg_params(dtype, kp, 0))
+    assert np.array_equal(x, x0)
+
+
+@pytest.mark.parametrize("inplace", [False, True])
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+def test_fused_placement_stride_inplace(tds, inplace, dtype):
+    """Padded 16-byte batch stride, in and out of place: the padding between
+    systems is never written by the G-element TMA runs."""
+    import torch
+    n, m, stride = 1 << 17, 3, (1 << 17) + 16
+    a, b, c, d = inputs.generate(n, m, dtype, seed=70)
+    pad = lambda v: np.pad(v, ((0, 0), (0, stride - n)), constant_values=7.0)
+    A, B, C, D = (pad(v).reshape(-1) for v in (a, b, c, d))
+    dt = "float32" if dtype == np.float32 else "float64"
+    plan = tds.Plan(n, m, dt, device=0, batch_stride=stride)
+    plan.set_params(cluster=1, **_xg_params(dtype, [4] if dtype == np.float32 else [5], 8))
+    ta, tb, tc, td = to_dev(A, B, C, D)
+    out = td if inplace else torch.full_like(td, 7.0)
+    x = tds.solve_batched(plan, ta, tb, tc, td, out=out)
+    torch.cuda.synchronize()
+    xs = x.cpu().numpy().reshape(m, stride)
+    assert np.all(xs[:, n:] == 7.0)
+    check(a, b, c, d, xs[:, :n], dtype)
+
+
+def test_fused_placement_misaligned_x_falls_back(tds):
+    """x not 16-byte aligned: the x_group plan runs the slot kernel + placement
+    (same launch count) and gives the bit-identical result."""
+    import torch
+    n, m = 1 << 17, 2
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=71)
+    x_ref, plan = run(tds, a, b, c, d, params=_xg_params(np.float32, [4], 8))
+    ta, tb, tc, td = to_dev(a, b, c, d)
+    buf = torch.zeros(m * n + 1, dtype=torch.float32, device="cuda")
+    out = buf[1:].view(m, n)
+    x = tds.solve_batched(plan, ta, tb, tc, td, out=out)
+    torch.cuda.synchronize()
+    assert np.array_equal(x.cpu().numpy(), x_ref)
+
+
+def test_fused_placement_batch_isolation(tds):
+    """A poisoned neighbour system leaves the others bit-identical (x_group = 8)."""
+    n, m = 1 << 17, 4
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=72)
+    kw = _xg_params(np.float32, [4], 8)
+    x0, _ = run(tds, a, b, c, d, params=kw)
+    d2 = d.copy(); b2 = b.copy()
+    d2[2] *= 1e6; b2[2] += 5
+    x1, _ = run(tds, a, b2, c, d2, params=kw)
+    for s in (0, 1, 3):
+        assert np.array_equal(x0[s], x1[s])
+
+
+def test_fused_placement_back_to_back(tds):
+    """Fused and unfused plans back to back on one stream through one workspace."""
+    import torch
+    cases = [(1 << 20, 2, _xg_params(np.float32, [7], 8)), (1 << 17, 3, _xg_params(np.float32, [4], 4)),
+             (1 << 17, 3, _xg_params(np.float32, [4], 0)), (8192, 8, None)]
+    plans, data, refs, wbytes = [], [], [], 0
+    for i, (n, m, params) in enumerate(cases):
+        a, b, c, d = inputs.generate(n, m, np.float32, seed=80 + i)
+        plan = tds.Plan(n, m, "float32", device=0, mode="static")
+        if params:
+            plan.set_params(cluster=1, **params)
+        plans.append(plan)
+        data.append(to_dev(a, b, c, d))
+        refs.append((a, b, c, d))
+        wbytes = max(wbytes, plan.workspace_bytes)
+    ws = torch.empty(max(wbytes, 1), dtype=torch.uint8, device="cuda")
+    outs = [torch.empty_like(dv[3]) for dv in data]
+    for rep in range(3):
+        for plan, (ta, tb, tc, td), x in zip(plans, data, outs):
+            tds.solve_batched(plan, ta, tb, tc, td, out=x, workspace=ws)
+    torch.cuda.synchronize()
+    for (a, b, c, d), x in zip(refs, outs):
+        check(a, b, c, d, x.cpu().numpy(), np.float32)
