@@ -1,0 +1,9 @@
+for c in 2 4; do
+  timeout 300 python bench.py --config $c --steps 30 --warmup 5 --no-e2e --no-cpu-baseline --soak-s 0 --tune-cache gpurun_out/tune_ag.txt > gpurun_out/ag_cfg$c.json 2>/dev/null
+  python -c "
+import json; d=json.load(open('gpurun_out/ag_cfg$c.json')); print('cfg$c', d['ms_per_step'], '%.3e'%d['value'], d['config']['plan']['cluster'])"
+done
+timeout 900 python -m pytest tests -m gpu -x -q -p no:cacheprovider 2>&1 | tail -3
+timeout 300 compute-sanitizer --tool racecheck python scripts/sanitize.py 2>&1 | grep -E "BAD|SUMMARY"
+timeout 300 compute-sanitizer --tool synccheck python scripts/sanitize.py 2>&1 | grep -E "BAD|SUMMARY"
+timeout 300 compute-sanitizer --tool memcheck python scripts/sanitize.py 2>&1 | grep -E "BAD|SUMMARY"
