@@ -40,11 +40,12 @@ __device__ __forceinline__ void reduced_solve_pipe(T *z, int Z, int NT, int t, i
 // Warp-level on-chip solve of one subsystem held as R rows per thread (x
 // returned in rd).  c = log2(R) CR levels in registers, 5 CR levels across
 // the lanes of each warp (shuffles), then the one remaining row per warp is
-// solved by warp 0 with shuffle PCR, and everything is back-substituted.  The
+// solved with shuffle PCR, and everything is back-substituted.  The
 // only row of a warp that reaches into the next warp is lane 31's: its chains
 // are deferred until one barrier publishes the next warp's rows (lane 0's
 // row s-1 per register level, lane s-1's row per lane level; both depend on
-// nothing beyond their own warp).  5 barriers per subsystem in total.
+// nothing beyond their own warp).  Every warp then solves the one-row-per-warp
+// system itself (no barrier to distribute its x).
 template <typename T, int R, typename Hook>
 __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[R], T *scr, int lane, int warp,
                                                 int nwarps, Hook &&after_barrier) {
@@ -132,7 +133,11 @@ __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[
         top[64 + warp] = zd;
     }
     __syncthreads();
-    if (warp == 0) {  // one row per warp: pure PCR with shuffles (every row decouples, x = d)
+    // one row per warp: pure PCR with shuffles (every row decouples, x = d),
+    // solved redundantly by EVERY warp (identical arithmetic), so each warp
+    // takes its own x and the previous warp's by shuffle -- no third barrier
+    T xw, xprev;
+    {
         T a = lane < nwarps ? top[lane] : T(0), c = lane < nwarps ? top[32 + lane] : T(0),
           d = lane < nwarps ? top[64 + lane] : T(0);
         for (int s = 1; s < nwarps; s <<= 1) {
@@ -140,16 +145,20 @@ __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[
             const T xa = __shfl_down_sync(FULL, a, s), xc = __shfl_down_sync(FULL, c, s),
                     xd = __shfl_down_sync(FULL, d, s);
             const bool hl = lane >= s, hr = lane + s < nwarps;
-            if (lane < nwarps)
-                row_update(a, c, d, hl ? la : T(0), hl ? lc : T(0), hl ? ld : T(0), hr ? xa : T(0), hr ? xc : T(0),
-                           hr ? xd : T(0));
+            T na = a, nc = c, nd = d;
+            row_update(na, nc, nd, hl ? la : T(0), hl ? lc : T(0), hl ? ld : T(0), hr ? xa : T(0), hr ? xc : T(0),
+                       hr ? xd : T(0));
+            a = lane < nwarps ? na : a;
+            c = lane < nwarps ? nc : c;
+            d = lane < nwarps ? nd : d;
         }
-        if (lane < nwarps) xtop[lane] = d;
+        const T xme = __shfl_sync(FULL, d, warp);
+        const T xpw = __shfl_sync(FULL, d, warp > 0 ? warp - 1 : 0);
+        xw = lane == 31 ? xme : T(0);
+        xprev = warp > 0 ? xpw : T(0);  // row -1 of this warp: previous warp's lane 31
     }
-    __syncthreads();
+    (void)xtop;
     // back substitution across lanes, then in registers
-    T xw = lane == 31 ? xtop[warp] : T(0);
-    const T xprev = warp > 0 ? xtop[warp - 1] : T(0);  // row -1 of this warp: previous warp's lane 31
 #pragma unroll
     for (int l = 5; l >= 1; --l) {
         const int s = 1 << (l - 1);

@@ -1,0 +1,5 @@
+for c in 4 2 3 4 2 3; do
+timeout 300 python bench.py --config $c --steps 30 --warmup 5 --no-e2e --no-cpu-baseline --soak-s 0 --tune-cache gpurun_out/tune_rw.txt > gpurun_out/rw.json 2>/dev/null
+python -c "
+import json; d=json.load(open('gpurun_out/rw.json')); print('cfg$c', d['ms_per_step'], '%.3e'%d['value'], d['clocks']['sm_mhz'], d['clocks']['reasons'], [(k['kernel'], round(k['ms'],4)) for k in d['roofline']['per_kernel']])"
+done
