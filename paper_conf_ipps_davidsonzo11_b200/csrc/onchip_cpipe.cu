@@ -37,6 +37,66 @@ __device__ __forceinline__ void csync() {
     if constexpr (C > 1) cg::this_cluster().sync(); else __syncthreads();
 }
 
+// One warp solves a system of 32 * RZ normalised rows (lane l holds rows
+// l RZ .. l RZ + RZ - 1) by cyclic reduction: log2(RZ) levels in registers,
+// 5 across the lanes (shuffles), back substitution in reverse order; rows
+// outside the system are identity rows.  No barrier (the cluster's top rows,
+// C = 4 / 8, replace 6 / 7 shared-memory PCR levels with 14 barriers).
+template <typename T, int RZ>
+__device__ __forceinline__ void warp_cr_solve(T (&ra)[RZ], T (&rc)[RZ], T (&rd)[RZ], int lane) {
+    constexpr unsigned FULL = 0xffffffffu;
+    constexpr int CR = ilog2c(RZ);
+#pragma unroll
+    for (int l = 1; l <= CR; ++l) {
+        const int s = 1 << (l - 1);
+        const T na = __shfl_down_sync(FULL, ra[s - 1], 1), nc = __shfl_down_sync(FULL, rc[s - 1], 1),
+                nd = __shfl_down_sync(FULL, rd[s - 1], 1);
+        const bool hn = lane < 31;
+#pragma unroll
+        for (int v = (1 << l) - 1; v < RZ; v += (1 << l)) {
+            const bool last = v + s >= RZ;
+            row_update(ra[v], rc[v], rd[v], ra[v - s], rc[v - s], rd[v - s], last ? (hn ? na : T(0)) : ra[v + s],
+                       last ? (hn ? nc : T(0)) : rc[v + s], last ? (hn ? nd : T(0)) : rd[v + s]);
+        }
+    }
+    T za = ra[RZ - 1], zc = rc[RZ - 1], zd = rd[RZ - 1];
+#pragma unroll
+    for (int l = 1; l <= 5; ++l) {
+        const int s = 1 << (l - 1);
+        const T la = __shfl_up_sync(FULL, za, s), lc = __shfl_up_sync(FULL, zc, s), ld = __shfl_up_sync(FULL, zd, s);
+        const T xa = __shfl_down_sync(FULL, za, s), xc = __shfl_down_sync(FULL, zc, s),
+                xd = __shfl_down_sync(FULL, zd, s);
+        const bool hr = lane + s < 32;
+        T a = za, c = zc, d = zd;
+        row_update(a, c, d, la, lc, ld, hr ? xa : T(0), hr ? xc : T(0), hr ? xd : T(0));
+        const bool upd = (lane & ((1 << l) - 1)) == (1 << l) - 1;
+        za = upd ? a : za;
+        zc = upd ? c : zc;
+        zd = upd ? d : zd;
+    }
+    T xw = lane == 31 ? zd : T(0);  // the last row decouples: x = d
+#pragma unroll
+    for (int l = 5; l >= 1; --l) {
+        const int s = 1 << (l - 1);
+        const T xl = __shfl_up_sync(FULL, xw, s);
+        const T xr = __shfl_down_sync(FULL, xw, s);
+        const T xn = zd - za * (lane >= s ? xl : T(0)) - zc * (lane + s < 32 ? xr : T(0));
+        xw = (lane & ((1 << l) - 1)) == s - 1 ? xn : xw;
+    }
+    T xleft = __shfl_up_sync(FULL, xw, 1);
+    if (lane == 0) xleft = T(0);
+    rd[RZ - 1] = xw;
+#pragma unroll
+    for (int l = CR; l >= 1; --l) {
+        const int s = 1 << (l - 1);
+#pragma unroll
+        for (int v = s - 1; v < RZ - 1; v += 2 * s) {
+            const T xlv = (v >= s) ? rd[v - s] : xleft;
+            rd[v] = rd[v] - ra[v] * xlv - rc[v] * rd[v + s];
+        }
+    }
+}
+
 template <typename T>
 __device__ __forceinline__ T *peer(T *p, int rank) {  // DSMEM address of p in cluster CTA `rank`
     return cg::this_cluster().map_shared_rank(p, rank);
@@ -284,8 +344,27 @@ __global__ void __launch_bounds__(512, 1)
         if constexpr (C > 1) {
             if (C * nwarps > 32 || warp == 0) mbar_wait(&mb_top, uint32_t(it & 1));
         }
-        if (C * nwarps > 32) {
-            // CTA 0: PCR over the Z = C * nwarps top rows in shared memory (every row decouples, x = d)
+        if (C * nwarps > 32 && C * nwarps == ZMAX) {
+            // the Z = 64 / 128 top rows (C = 4 / 8, 16 warps): cyclic reduction in one warp (2 / 4 rows per lane)
+            constexpr int RZ = ZMAX / 32;
+            if (warp == 0) {
+                T za2[RZ], zc2[RZ], zd2[RZ];
+#pragma unroll
+                for (int v = 0; v < RZ; ++v) {
+                    za2[v] = top[lane * RZ + v];
+                    zc2[v] = top[ZMAX + lane * RZ + v];
+                    zd2[v] = top[2 * ZMAX + lane * RZ + v];
+                }
+                warp_cr_solve<T, RZ>(za2, zc2, zd2, lane);
+#pragma unroll
+                for (int v = 0; v < RZ; ++v) {  // this CTA's x of the top rows, and the previous CTA's last one
+                    const int z = lane * RZ + v, r = z / nwarps, w = z % nwarps;
+                    if (r == rank) xtop[w] = zd2[v];
+                    if (z == rank * nwarps - 1) xtop[32] = zd2[v];
+                }
+            }
+        } else if (C * nwarps > 32) {
+            // PCR over the Z = C * nwarps top rows in shared memory (every row decouples, x = d)
             const int Z = C * nwarps;
             T *za2 = top, *zc2 = top + ZMAX, *zd2 = top + 2 * ZMAX;
             for (int s = 1; s < Z; s <<= 1) {
