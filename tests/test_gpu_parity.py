@@ -457,6 +457,40 @@ def test_config4_sampled(tds):
     check(a[idx], b[idx], c[idx], d[idx], x[idx], np.float32)
 
 
+BENCH_SHAPES = [  # the tuned plans bench.py times (profiles/r01h_bench_*), pinned explicitly
+    (2, np.float32, dict(k_pass=[], cr_levels=4, thomas_chains=16, cluster=8, tl_levels=5)),
+    (3, np.float32, dict(k_pass=[7], cr_levels=4, thomas_chains=16, cluster=1, tl_levels=5, split_threads=512,
+                         split_tile_rows=8192)),
+    (3, np.float64, dict(k_pass=[8], cr_levels=3, thomas_chains=16, cluster=1, tl_levels=5, split_threads=512,
+                         split_tile_rows=4096)),
+    (4, np.float32, dict(k_pass=[], cr_levels=4, thomas_chains=32, cluster=2, tl_levels=5))]
+
+
+@pytest.mark.parametrize("how", ["pinned", "tuned"])
+@pytest.mark.parametrize("cfg,dtype,params", BENCH_SHAPES, ids=["cfg2", "cfg3f32", "cfg3f64", "cfg4"])
+def test_bench_launch_configuration_full_size(tds, tmp_path, how, cfg, dtype, params):
+    """BASELINE.json configs 2-4 at full size in the launch configuration
+    bench.py times: the plan the tuner picks on this device (as bench.py does)
+    and the tuned shape recorded in profiles/, against the oracle (config 4:
+    every system on the GPU, 64 sampled systems through the oracle)."""
+    import torch
+    n, m = {2: (65536, 256), 3: (1 << 20, 16), 4: (16384, 4096)}[cfg]
+    a, b, c, d = inputs.generate(n, m, dtype, seed=inputs.config_seed(cfg, dtype))
+    plan = tds.Plan(n, m, "float32" if dtype == np.float32 else "float64", device=0, mode="static")
+    if how == "tuned":
+        plan.tune(cache_path=str(tmp_path / "tune.txt"))
+    else:
+        plan.set_params(**params)
+    ta, tb, tc, td = to_dev(a, b, c, d)
+    x = tds.solve_batched(plan, ta, tb, tc, td)
+    torch.cuda.synchronize()
+    x = x.cpu().numpy()
+    if cfg == 4:
+        idx = np.sort(np.concatenate([[0, m - 1], np.random.default_rng(1).choice(m, 62, replace=False)]))
+        a, b, c, d, x = a[idx], b[idx], c[idx], d[idx], x[idx]
+    check(a, b, c, d, x, dtype)
+
+
 @pytest.mark.slow
 def test_config5_single_gpu_part(tds):
     """1 x 2^26 fp32 (the single-GPU half of config 5's schedule: 2 passes)."""
