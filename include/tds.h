@@ -221,6 +221,28 @@ tds_status tds_split_batched(const tds_plan_t plan, const void *a, const void *b
                              const void *d, void *a_out, void *c_out, void *d_out,
                              void *workspace, size_t workspace_bytes, void *cuda_stream);
 
+/* ---- batch-interleaved layout (ADI-style batches) ----- */
+
+/* Bytes of device workspace tds_solve_interleaved needs for `plan`: the
+ * plan's own workspace plus four system-major copies of the m x n arrays
+ * (each rounded up to 256 bytes).  The plan must be dense (batch_stride == n).
+ * Errors: INVALID_ARG (NULL), UNSUPPORTED (strided or split-only plan). */
+tds_status tds_interleaved_workspace_bytes(const tds_plan_t plan, size_t *bytes);
+
+/* Same solve as tds_solve_batched for arrays in the INTERLEAVED layout:
+ * element i of system s at ptr[i * m + s] (row-major n x m, the layout of
+ * ADI sweeps along the fast axis).  The arrays are transposed into the
+ * workspace by a shared-memory tile kernel (reads coalesced along systems,
+ * writes along rows), solved by the plan's kernels in place, and x is
+ * transposed back: 2 x 4 s extra HBM bytes per equation in, 2 s out.
+ * x: device, interleaved, may alias d exactly.  workspace: device, 256-byte
+ * aligned, >= tds_interleaved_workspace_bytes.  Same errors as
+ * tds_solve_batched (plus UNSUPPORTED for a strided plan); enqueued on
+ * cuda_stream, asynchronous. */
+tds_status tds_solve_interleaved(const tds_plan_t plan, const void *a, const void *b, const void *c,
+                                 const void *d, void *x, void *workspace, size_t workspace_bytes,
+                                 void *cuda_stream);
+
 /* ---- misc ---------------------------------------------------------------------- */
 
 const char *tds_status_string(tds_status status);

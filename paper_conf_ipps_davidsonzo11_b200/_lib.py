@@ -25,6 +25,7 @@ EXPORTED = (
     "tds_plan", "tds_plan_from_props", "tds_device_props_query", "tds_plan_info_get",
     "tds_plan_set_params", "tds_plan_permutation", "tds_plan_destroy", "tds_tune",
     "tds_plan_tune_trials", "tds_solve_batched", "tds_solve_stages", "tds_split_batched", "tds_status_string",
+    "tds_interleaved_workspace_bytes", "tds_solve_interleaved",
     "tds_last_error", "tds_version",
 )
 
@@ -87,6 +88,8 @@ def load() -> ctypes.CDLL:
         "tds_solve_batched": (I32, [P, VP, VP, VP, VP, VP, VP, SZ, VP]),
         "tds_solve_stages": (I32, [P, VP, VP, VP, VP, VP, VP, SZ, VP, ctypes.c_int32, ctypes.c_int32]),
         "tds_split_batched": (I32, [P, VP, VP, VP, VP, VP, VP, VP, VP, SZ, VP]),
+        "tds_interleaved_workspace_bytes": (I32, [P, ctypes.POINTER(ctypes.c_size_t)]),
+        "tds_solve_interleaved": (I32, [P, VP, VP, VP, VP, VP, VP, SZ, VP]),
         "tds_status_string": (ctypes.c_char_p, [I32]),
         "tds_last_error": (ctypes.c_char_p, []),
         "tds_version": (I32, []),

@@ -158,6 +158,13 @@ class Plan:
         L.check(self._lib.tds_plan_tune_trials(self._h, ctypes.byref(t)))
         return int(t.value)
 
+    @property
+    def interleaved_workspace_bytes(self) -> int:
+        """tds_interleaved_workspace_bytes (dense plans only)."""
+        v = ctypes.c_size_t()
+        L.check(self._lib.tds_interleaved_workspace_bytes(self._h, ctypes.byref(v)))
+        return int(v.value)
+
     def workspace(self):
         import torch
         nbytes = self.workspace_bytes
@@ -206,6 +213,27 @@ def solve_batched(plan: Plan, a, b, c, d, out=None, workspace=None, stream=None)
     wbytes = workspace.numel() * workspace.element_size() if workspace is not None else 0
     L.check(plan._lib.tds_solve_batched(plan.handle, a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
                                         out.data_ptr(), wptr, wbytes, _stream_ptr(stream, dev)))
+    return out
+
+
+def solve_interleaved(plan: Plan, a, b, c, d, out=None, workspace=None, stream=None):
+    """tds_solve_interleaved: the same solve for arrays in the batch-interleaved
+    layout (element i of system s at [i, s] of an (n, m) tensor).  Returns x, (n, m)."""
+    import torch
+    info, _, want, dev = plan._solve_info()
+    need = info.n * info.m
+    for name, t in (("a", a), ("b", b), ("c", c), ("d", d)):
+        _check_fast(t, need, want, name)
+    if out is None:
+        out = torch.empty_like(d)
+    else:
+        _check_fast(out, need, want, "out")
+    if workspace is None:
+        workspace = torch.empty(plan.interleaved_workspace_bytes, dtype=torch.uint8, device=f"cuda:{dev}")
+    wbytes = workspace.numel() * workspace.element_size()
+    L.check(plan._lib.tds_solve_interleaved(plan.handle, a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
+                                            out.data_ptr(), workspace.data_ptr(), wbytes,
+                                            _stream_ptr(stream, dev)))
     return out
 
 

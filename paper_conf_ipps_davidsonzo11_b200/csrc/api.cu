@@ -287,6 +287,39 @@ static tds_status split_chunks(const tds_plan_info &I, const T *a, const T *b, c
     return TDS_OK;
 }
 
+// Interleaved layout (tds_solve_interleaved): the plan's workspace, then the
+// four transposed (system-major) arrays, each rounded to 256 bytes; x is
+// solved in place over the transposed d.
+static size_t interleaved_array_bytes(const tds_plan_info &I) {
+    return size_t(round_up(I.m * I.n * dsize(I.dtype), 256));
+}
+static tds_status interleaved_plan_ok(const tds_plan_st *plan) {
+    if (!plan) return fail(TDS_ERR_INVALID_ARG, "plan is NULL");
+    if (plan->info.params.split_only) return fail(TDS_ERR_UNSUPPORTED, "split-only plan: use tds_split_batched");
+    if (plan->info.batch_stride != plan->info.n)
+        return fail(TDS_ERR_UNSUPPORTED, "interleaved layout needs a dense plan (batch_stride == n)");
+    return TDS_OK;
+}
+
+template <typename T>
+static tds_status solve_interleaved_impl(const tds_plan_info &I, const T *a, const T *b, const T *c, const T *d,
+                                         T *x, void *ws, cudaStream_t st) {
+    char *base = static_cast<char *>(ws) + round_up(int64_t(I.workspace_bytes), 256);
+    const size_t ab = interleaved_array_bytes(I);
+    T *sys[4];
+    for (int q = 0; q < 4; ++q) sys[q] = reinterpret_cast<T *>(base + q * ab);
+    const T *in[4] = {a, b, c, d};
+    cudaError_t e = launch_transpose<T>(in, sys, 4, I.n, I.m, st);  // n x m -> m x n
+    if (e != cudaSuccess) return cuda_fail(e, "interleave transpose launch");
+    tds_status s = solve_chunks<T>(I, sys[0], sys[1], sys[2], sys[3], sys[3], ws, st, 0, I.launches - 1);
+    if (s != TDS_OK) return s;
+    const T *xin[1] = {sys[3]};
+    T *xout[1] = {x};
+    e = launch_transpose<T>(xin, xout, 1, I.m, I.n, st);  // m x n -> n x m
+    if (e != cudaSuccess) return cuda_fail(e, "interleave transpose launch");
+    return TDS_OK;
+}
+
 static tds_status check_arrays(const tds_plan_info &I, std::initializer_list<const void *> ptrs) {
     const size_t es = size_t(dsize(I.dtype));
     for (const void *p : ptrs) {
@@ -379,6 +412,46 @@ tds_status tds_split_batched(const tds_plan_t plan, const void *a, const void *b
             : split_chunks<double>(I, (const double *)a, (const double *)b, (const double *)c,
                                    (const double *)d, (double *)a_out, (double *)c_out, (double *)d_out, workspace,
                                    st);
+    if (s == TDS_OK) clear_error();
+    return s;
+}
+
+tds_status tds_interleaved_workspace_bytes(const tds_plan_t plan, size_t *bytes) {
+    tds_status s = interleaved_plan_ok(plan);
+    if (s != TDS_OK) return s;
+    if (!bytes) return fail(TDS_ERR_INVALID_ARG, "bytes is NULL");
+    *bytes = size_t(round_up(int64_t(plan->info.workspace_bytes), 256)) + 4 * interleaved_array_bytes(plan->info);
+    clear_error();
+    return TDS_OK;
+}
+
+tds_status tds_solve_interleaved(const tds_plan_t plan, const void *a, const void *b, const void *c, const void *d,
+                                 void *x, void *workspace, size_t workspace_bytes, void *cuda_stream) {
+    tds_status s = interleaved_plan_ok(plan);
+    if (s != TDS_OK) return s;
+    const tds_plan_info &I = plan->info;
+    if ((s = check_arrays(I, {a, b, c, d, x})) != TDS_OK) return s;
+    const size_t bytes = size_t(I.m * I.n * dsize(I.dtype));
+    for (const void *p : {a, b, c})
+        if (overlaps(x, bytes, p, bytes)) return fail(TDS_ERR_INVALID_ARG, "x overlaps a, b or c");
+    if (x != d && overlaps(x, bytes, d, bytes))
+        return fail(TDS_ERR_INVALID_ARG, "x partially overlaps d (only x == d is allowed)");
+    size_t need = 0;
+    tds_interleaved_workspace_bytes(plan, &need);
+    if (!workspace) return fail(TDS_ERR_WORKSPACE, "workspace is NULL");
+    if (workspace_bytes < need)
+        return fail(TDS_ERR_WORKSPACE, "workspace " + std::to_string(workspace_bytes) + " < required " +
+                                           std::to_string(need));
+    if (reinterpret_cast<uintptr_t>(workspace) % 256) return fail(TDS_ERR_WORKSPACE, "workspace not 256-byte aligned");
+    for (const void *p : {a, b, c, d, (const void *)x})
+        if (overlaps(workspace, need, p, bytes)) return fail(TDS_ERR_INVALID_ARG, "workspace overlaps an array");
+    if ((s = check_device(plan)) != TDS_OK) return s;
+    cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
+    s = I.dtype == TDS_F32
+            ? solve_interleaved_impl<float>(I, (const float *)a, (const float *)b, (const float *)c,
+                                            (const float *)d, (float *)x, workspace, st)
+            : solve_interleaved_impl<double>(I, (const double *)a, (const double *)b, (const double *)c,
+                                             (const double *)d, (double *)x, workspace, st);
     if (s == TDS_OK) clear_error();
     return s;
 }

@@ -143,6 +143,11 @@ size_t onchip_pipe_smem_bytes(int32_t dtype, int32_t threads, int32_t R, int32_t
 // one CTA per subsystem whose threads hold 64 bytes of rows per array (fp32
 // c = 4, fp64 c = 3; up to 512 threads) or 32 bytes (fp32 c = 3, fp64 c = 2;
 // up to 1024 threads).
+// in: rows x cols row-major -> out: cols x rows, `narrays` (1 or 4) arrays (interleave.cu)
+template <typename T>
+cudaError_t launch_transpose(const T *const *in, T *const *out, int narrays, int64_t rows, int64_t cols,
+                             cudaStream_t st);
+
 template <typename T>
 cudaError_t launch_onchip_gpipe(const OnchipArgs<T> &A, int64_t nslots, int threads, int sm_count, cudaStream_t st);
 

@@ -182,3 +182,22 @@ def test_x_group_validation(tds):
     r = tds.Plan(1 << 20, 2, "float64", props=_props(rp.B200))
     r.set_params(k_pass=[8], cr_levels=3, thomas_chains=16, cluster=1, tl_levels=5, x_group=2)
     assert r.info["launches"] == 2
+
+
+def test_interleaved_workspace_and_errors(tds):
+    """tds_interleaved_workspace_bytes: plan workspace + four 256-byte-rounded
+    m x n copies; strided plans are refused; argument errors before launch."""
+    p = tds.Plan(1 << 20, 16, props=_props(rp.B200))
+    ws = p.info["workspace_bytes"]
+    r256 = lambda v: -(-v // 256) * 256
+    assert p.interleaved_workspace_bytes == r256(ws) + 4 * r256(16 * (1 << 20) * 4)
+    q = tds.Plan(1000, 3, props=_props(rp.B200), batch_stride=1024)
+    with pytest.raises(tds.TdsError) as e:
+        q.interleaved_workspace_bytes
+    assert e.value.name == "TDS_ERR_UNSUPPORTED"
+    lib = tds._lib.load()
+    h = p.handle
+    assert lib.tds_solve_interleaved(h, None, 8, 8, 8, 8, 256, 1 << 40, None) == 1    # NULL a
+    assert lib.tds_solve_interleaved(h, 8, 8, 8, 8, 8, None, 0, None) == 1            # x overlaps a
+    assert lib.tds_solve_interleaved(h, 1 << 20, 2 << 30, 3 << 30, 4 << 30, 5 << 30, None, 0, None) == 4  # no ws
+    assert lib.tds_interleaved_workspace_bytes(h, None) == 1
