@@ -55,6 +55,8 @@ def parse():
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--soak-s", type=float, default=1.5, help="untimed load before timing (clock sampling)")
+    ap.add_argument("--graph", action="store_true",
+                    help="each step replays a CUDA graph of one solve (launch-latency-bound configs)")
     return ap.parse_args()
 
 
@@ -303,6 +305,21 @@ def run_tds(args):
             step()
         torch.cuda.synchronize()
 
+    if args.graph:  # one solve captured once; a step is then one graph replay
+        gs = torch.cuda.Stream()
+        gs.wait_stream(torch.cuda.current_stream())
+        with torch.cuda.stream(gs):
+            step()
+        torch.cuda.current_stream().wait_stream(gs)
+        torch.cuda.synchronize()
+        graph = torch.cuda.CUDAGraph()
+        with torch.cuda.graph(graph):
+            tds.solve_batched(plan, ta, tb, tc, td, out=x, workspace=ws)
+        step = graph.replay
+        for _ in range(max(args.warmup, 3)):
+            step()
+        torch.cuda.synchronize()
+
     # ---- timed region: K steps back to back (value, ms_per_step)
     K = args.steps
     e_start, e_stop = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
@@ -444,6 +461,7 @@ def run_tds(args):
                                                                      "theta", "split_segments", "x_group",
                                                                      "onchip_threads", "workspace_bytes")},
                    "tune_trials": trials, "tune_s": round(tune_s, 2),
+                   "launch": "cuda_graph_replay" if args.graph else "eager",
                    "l2": f"no flush: per-step working set {(5 * eqs_per_step * s + info['workspace_bytes']) / 2**20:.0f} MiB > L2 126 MiB"
                    if 5 * eqs_per_step * s + info["workspace_bytes"] > L2_BYTES else
                    "working set fits L2: warm-L2 latency number",
