@@ -55,7 +55,7 @@ __device__ __forceinline__ void warp_cr_solve(T (&ra)[RZ], T (&rc)[RZ], T (&rd)[
 #pragma unroll
         for (int v = (1 << l) - 1; v < RZ; v += (1 << l)) {
             const bool last = v + s >= RZ;
-            row_update(ra[v], rc[v], rd[v], ra[v - s], rc[v - s], rd[v - s], last ? (hn ? na : T(0)) : ra[v + s],
+            row_update_early(ra[v], rc[v], rd[v], ra[v - s], rc[v - s], rd[v - s], last ? (hn ? na : T(0)) : ra[v + s],
                        last ? (hn ? nc : T(0)) : rc[v + s], last ? (hn ? nd : T(0)) : rd[v + s]);
         }
     }
@@ -68,7 +68,7 @@ __device__ __forceinline__ void warp_cr_solve(T (&ra)[RZ], T (&rc)[RZ], T (&rd)[
                 xd = __shfl_down_sync(FULL, zd, s);
         const bool hr = lane + s < 32;
         T a = za, c = zc, d = zd;
-        row_update(a, c, d, la, lc, ld, hr ? xa : T(0), hr ? xc : T(0), hr ? xd : T(0));
+        row_update_early(a, c, d, la, lc, ld, hr ? xa : T(0), hr ? xc : T(0), hr ? xd : T(0));
         const bool upd = (lane & ((1 << l) - 1)) == (1 << l) - 1;
         za = upd ? a : za;
         zc = upd ? c : zc;
@@ -252,7 +252,7 @@ __global__ void __launch_bounds__(512, 1)
             for (int v = (1 << l) - 1; v < R; v += (1 << l)) {
                 const bool last = v == R - 1;
                 T a = ra[v], c = rc[v], d = rd[v];
-                row_update(a, c, d, ra[v - s], rc[v - s], rd[v - s], last ? na : ra[(v + s) % R],
+                row_update_early(a, c, d, ra[v - s], rc[v - s], rd[v - s], last ? na : ra[(v + s) % R],
                            last ? nc : rc[(v + s) % R], last ? nd : rd[(v + s) % R]);
                 const bool keep = last && lane == 31;
                 ra[v] = keep ? ra[v] : a;
@@ -290,7 +290,7 @@ __global__ void __launch_bounds__(512, 1)
                 f[2] = zd;
             }
             T a = za, c = zc, d = zd;
-            row_update(a, c, d, la, lc, ld, xa, xc, xd);
+            row_update_early(a, c, d, la, lc, ld, xa, xc, xd);
             const bool upd = (lane & ((1 << l) - 1)) == (1 << l) - 1 && lane != 31;
             za = upd ? a : za;
             zc = upd ? c : zc;
@@ -313,7 +313,7 @@ __global__ void __launch_bounds__(512, 1)
             for (int l = 1; l <= CR; ++l) {
                 const int s = 1 << (l - 1);
                 const T *e = en + (l - 1) * 3;
-                row_update(ra[R - 1], rc[R - 1], rd[R - 1], ra[R - 1 - s], rc[R - 1 - s], rd[R - 1 - s],
+                row_update_early(ra[R - 1], rc[R - 1], rd[R - 1], ra[R - 1 - s], rc[R - 1 - s], rd[R - 1 - s],
                            h ? e[0] : T(0), h ? e[1] : T(0), h ? e[2] : T(0));
             }
             za = ra[R - 1];
@@ -323,7 +323,7 @@ __global__ void __launch_bounds__(512, 1)
             for (int l = 1; l <= 5; ++l) {
                 const T *f = lft + (warp * 5 + l - 1) * 3;
                 const T *w = wn + (l - 1) * 3;
-                row_update(za, zc, zd, f[0], f[1], f[2], h ? w[0] : T(0), h ? w[1] : T(0), h ? w[2] : T(0));
+                row_update_early(za, zc, zd, f[0], f[1], f[2], h ? w[0] : T(0), h ? w[1] : T(0), h ? w[2] : T(0));
             }
             const int z = rank * nwarps + warp;
             if constexpr (C > 1) {  // all-gather: to every CTA (itself included), counted on its mb_top
@@ -374,7 +374,7 @@ __global__ void __launch_bounds__(512, 1)
                     c = zc2[t];
                     d = zd2[t];
                     const bool hl = t >= s, hr = t + s < Z;
-                    row_update(a, c, d, hl ? za2[t - s] : T(0), hl ? zc2[t - s] : T(0), hl ? zd2[t - s] : T(0),
+                    row_update_early(a, c, d, hl ? za2[t - s] : T(0), hl ? zc2[t - s] : T(0), hl ? zd2[t - s] : T(0),
                                hr ? za2[t + s] : T(0), hr ? zc2[t + s] : T(0), hr ? zd2[t + s] : T(0));
                 }
                 __syncthreads();
@@ -399,7 +399,7 @@ __global__ void __launch_bounds__(512, 1)
                         xd = __shfl_down_sync(FULL, d, s);
                 const bool hl = lane >= s, hr = lane + s < Z;
                 T na = a, nc = c, nd = d;
-                row_update(na, nc, nd, hl ? la : T(0), hl ? lc : T(0), hl ? ld : T(0), hr ? xa : T(0),
+                row_update_early(na, nc, nd, hl ? la : T(0), hl ? lc : T(0), hl ? ld : T(0), hr ? xa : T(0),
                            hr ? xc : T(0), hr ? xd : T(0));
                 a = lane < Z ? na : a;
                 c = lane < Z ? nc : c;
