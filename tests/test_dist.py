@@ -129,3 +129,31 @@ def test_huge_system_single_gpu_kernels():
     torch.cuda.synchronize()
     xr = oracle.thomas(a, b, c, d)[0]
     assert np.abs(x.cpu().numpy() - xr).max() / np.abs(xr).max() <= 1e-4
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("n,m,params", [
+    (1 << 20, 8, dict(k_pass=[7], cr_levels=4, thomas_chains=16, cluster=1, tl_levels=5)),
+    (16384, 96, dict(k_pass=[], cr_levels=4, thomas_chains=32, cluster=2, tl_levels=5)),
+    (65536, 24, dict(k_pass=[], cr_levels=4, thomas_chains=16, cluster=8, tl_levels=5))],
+    ids=["cfg3-shape", "cfg4-shape", "cfg2-shape"])
+@pytest.mark.parametrize("world", [2, 3, 8])
+def test_batch_shards_bit_identical_gpu(n, m, params, world):
+    """SURVEY §8(c) "Sharding": x of every rank's shard (its own Plan(n, m_rank)
+    with the broadcast integer plan, inputs generated with global system
+    indices) is bit-identical to the same systems of the unsharded solve."""
+    import paper_conf_ipps_davidsonzo11_b200 as tds
+    from paper_conf_ipps_davidsonzo11_b200 import dist as tdist
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=11)
+    full = tds.Plan(n, m, "float32", device=0)
+    full.set_params(**params)
+    xall = tds.solve_batched(full, *[torch.from_numpy(v).cuda() for v in (a, b, c, d)]).cpu().numpy()
+    for r in range(world):
+        s0, s1 = tdist.shard_range(m, world, r)
+        if s1 <= s0:
+            continue
+        sh = inputs.generate(n, s1 - s0, np.float32, seed=11, first_system=s0)
+        plan = tds.Plan(n, s1 - s0, "float32", device=0)
+        plan.set_params_list(full.params_list())
+        x = tds.solve_batched(plan, *[torch.from_numpy(v).cuda() for v in sh]).cpu().numpy()
+        assert np.array_equal(x, xall[s0:s1])
