@@ -715,7 +715,10 @@ IL_CASES = [  # (dtype, n, m, params or None for the static plan)
     (np.float32, 1 << 17, 7, dict(k_pass=[4], cr_levels=4, thomas_chains=16, tl_levels=5)),
     (np.float32, 300001, 3, None),                                      # ragged, split passes
     (np.float64, 4096, 129, None), (np.float64, 1 << 16, 9, dict(k_pass=[4], cr_levels=3, thomas_chains=16,
-                                                                    tl_levels=5))]
+                                                                    tl_levels=5)),
+    # whole 16-byte rows and columns: the TMA transposer (ragged edge tiles)
+    (np.float32, 3000, 36, None), (np.float64, 4096, 130, None), (np.float64, 1000, 66, None),
+    (np.float32, 1 << 17, 8, dict(k_pass=[4], cr_levels=4, thomas_chains=16, tl_levels=5))]
 
 
 @pytest.mark.parametrize("dtype,n,m,params", IL_CASES)
