@@ -1,7 +1,6 @@
-for cd in "3 f32" "2 f32" "4 f32" "3 f64" "3 f32" "2 f32" "4 f32"; do
-set -- $cd
-timeout 300 python bench.py --config $1 --dtype $2 --steps 30 --warmup 5 --no-e2e --no-cpu-baseline --soak-s 0 --tune-cache gpurun_out/tune_ru.txt > gpurun_out/rw.json 2>/dev/null
+for e in 0 1 0 1; do
+TDS_ONCHIP_XEARLY=$e timeout 300 python bench.py --config 3 --steps 30 --warmup 5 --no-e2e --no-cpu-baseline --soak-s 0 --tune-cache gpurun_out/tune_xe.txt > gpurun_out/rw.json 2>/dev/null
 python -c "
-import json; d=json.load(open('gpurun_out/rw.json')); print('cfg$1 $2', round(d['ms_per_step'],4), '%.3e'%d['value'], d['config']['plan']['k_pass'], [(k['kernel'], round(k['ms'],4)) for k in d['roofline']['per_kernel']])"
+import json; d=json.load(open('gpurun_out/rw.json')); print('xearly=$e', round(d['ms_per_step'],4), '%.3e'%d['value'], [(k['kernel'], round(k['ms'],4)) for k in d['roofline']['per_kernel']])"
 done
-timeout 900 python -m pytest tests -m gpu -x -q -p no:cacheprovider 2>&1 | tail -3
+TDS_ONCHIP_XEARLY=1 timeout 900 python -m pytest tests/test_gpu_parity.py -m gpu -x -q -p no:cacheprovider -k "pipe or back_to_back or single_pass or unaligned or stride or bench_launch" 2>&1 | tail -2
