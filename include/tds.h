@@ -24,7 +24,8 @@
  * NUMERICS.  No pivoting (the paper's solvers do not pivot): the precondition
  * is a nonsingular, diagonally dominant (or SPD) system.  Breakdown is NOT
  * detected: a zero pivot yields inf/NaN in x.  fp32 uses the hardware
- * approximate reciprocal; fp64 uses IEEE division.
+ * approximate reciprocal (rcp.approx, <= 1 ulp); fp64 uses the hardware
+ * reciprocal seed refined by two Newton steps (~1 ulp) -- DESIGN.md R16.
  *
  * CONVENTIONS (every entry point):
  *  - Layout: element i of system s is at ptr[s * batch_stride + i]
