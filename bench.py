@@ -248,10 +248,19 @@ def run_tds(args):
     world, rank, local = dist_env()
     if world != args.gpus and world > 1:
         print(f"warning: WORLD_SIZE={world} != --gpus {args.gpus}", file=sys.stderr)
+    # TDS_BENCH_SAME_DEVICE=1 + TDS_BENCH_BACKEND=gloo: functional dry run of the
+    # N > 1 path with every rank on cuda:0 (timings meaningless; NCCL refuses
+    # two ranks on one device)
+    if os.environ.get("TDS_BENCH_SAME_DEVICE") == "1":
+        local = 0
     torch.cuda.set_device(local)
     dev = torch.device("cuda", local)
     if world > 1:
-        dist.init_process_group("nccl", device_id=dev)
+        backend = os.environ.get("TDS_BENCH_BACKEND", "nccl")
+        if backend == "nccl":
+            dist.init_process_group("nccl", device_id=dev)
+        else:
+            dist.init_process_group(backend)
 
     def barrier():
         if world > 1:
