@@ -782,3 +782,53 @@ def test_cuda_graph_capture_replay(tds, params):
         xe = tds.solve_batched(plan, *to_dev(a, b, c, d)).cpu().numpy()
         assert np.array_equal(xg, xe)
         check(a, b, c, d, xg, np.float32)
+
+
+# ------------------------------------------------ randomized plan fuzz (seeded)
+
+def _fuzz_cases(count=320, seed=2024):
+    rng = np.random.default_rng(seed)
+    out = []
+    for i in range(count):
+        dtype = np.float32 if rng.random() < 0.7 else np.float64
+        n = int(rng.choice([rng.integers(1, 5000), rng.integers(5000, 300000), 1 << int(rng.integers(10, 19))]))
+        m = int(rng.integers(1, 7))
+        k = int(rng.integers(0, 12))
+        passes = 0 if k == 0 else int(rng.integers(1, min(3, k) + 1))
+        kp = [] if k == 0 else [k // passes + (1 if j < k % passes else 0) for j in range(passes)]
+        c_lv = int(rng.integers(0, 5 if dtype == np.float32 else 4))
+        params = dict(k_pass=kp, cr_levels=c_lv, thomas_chains=int(2 ** rng.integers(0, 7)),
+                      cluster=int(rng.choice([1, 1, 1, 2, 4, 8])), tl_levels=int(rng.choice([0, 1, 3, 5])),
+                      x_group=int(rng.choice([0, 0, 0, 4, 8])), split_threads=int(rng.choice([256, 512])),
+                      chunk_systems=int(rng.choice([0, 0, 1, 2])))
+        out.append((i, dtype, n, m, params))
+    try:  # keep the plans the planner accepts for B200 (host-only check; all of them if libtds is not built)
+        import dataclasses
+        import paper_conf_ipps_davidsonzo11_b200 as tds_mod
+        from oracle import plan as rp
+        props = dataclasses.asdict(rp.B200)
+        keep = []
+        for case in out:
+            _, dt, n, m, params = case
+            pl = tds_mod.Plan(n, m, "float32" if dt == np.float32 else "float64", props=props)
+            try:
+                pl.set_params(**dict({"cluster": 1, "tl_levels": 0}, **params))
+                keep.append(case)
+            except tds_mod.TdsError:
+                pass
+        return keep
+    except (OSError, RuntimeError, ImportError):
+        return out
+
+
+@pytest.mark.parametrize("i,dtype,n,m,params", _fuzz_cases(), ids=lambda v: None)
+def test_plan_fuzz(tds, i, dtype, n, m, params):
+    """Seeded random plans (k, pass schedule, c, T, cluster, c2, x_group,
+    split CTA size, chunking) over random n, m: every plan the planner accepts
+    solves to the oracle's x within the tolerances."""
+    a, b, c, d = inputs.generate(n, m, dtype, seed=1000 + i)
+    try:
+        x, plan = run(tds, a, b, c, d, params=params)
+    except tds.TdsError as e:
+        pytest.skip(f"plan rejected: {e}")
+    check(a, b, c, d, x, dtype)
