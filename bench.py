@@ -139,14 +139,14 @@ def algorithmic_bytes(info: dict, s: int):
     for p in range(info["passes"]):
         out.append((7 if p == 0 else 6) * s * eqs)
     out.append((5 if info["passes"] == 0 else 4) * s * eqs)
-    if info["k"] > 0 and info["x_group"] == 0:
+    if info["k"] > 0 and info["x_group"] == 0 and info["strided"] == 0:
         out.append(2 * s * eqs)
     return out
 
 
 def stage_names(info):
     names = [f"split_pass_{p}(k_p={info['k_pass'][p]})" for p in range(info["passes"])] + ["onchip_cr_pcr_thomas"]
-    if info["k"] > 0 and info["x_group"] == 0:
+    if info["k"] > 0 and info["x_group"] == 0 and info["strided"] == 0:
         names.append("place_x")
     return names
 
@@ -297,7 +297,7 @@ def run_tds(args):
     info = plan.info
     ws = plan.workspace()
     NL = info["launches"]                            # kernel launches per step (all chunks)
-    S = info["passes"] + 1 + (1 if info["k"] > 0 and info["x_group"] == 0 else 0)  # kernels per chunk
+    S = info["passes"] + 1 + (1 if info["k"] > 0 and info["x_group"] == 0 and info["strided"] == 0 else 0)
     stream = torch.cuda.current_stream()
 
     def step():
@@ -467,7 +467,7 @@ def run_tds(args):
                                                                      "cr_levels", "thomas_chains",
                                                                      "cluster", "tl_levels", "chunk_systems",
                                                                      "chunks", "launches", "split_tile_rows", "split_threads",
-                                                                     "theta", "split_segments", "x_group",
+                                                                     "theta", "split_segments", "x_group", "strided",
                                                                      "onchip_threads", "workspace_bytes")},
                    "tune_trials": trials, "tune_s": round(tune_s, 2),
                    "launch": "cuda_graph_replay" if args.graph else "eager",

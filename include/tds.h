@@ -113,6 +113,13 @@ typedef struct {
                                         (n / 2^k = threads x 2^c), tl_levels = 5,
                                         2^c sizeof(T) = 64, G sizeof(T) >= 16, and
                                         2^k sizeof(T), batch_stride sizeof(T) multiples of 16 */
+    int32_t strided;                 /* 1: the paper's strided base-kernel variant:
+                                        the split leaves the 2^k subsystems interleaved in
+                                        place (rows in original order) and the on-chip kernel
+                                        gathers residue class r with stride 2^k and scatters x
+                                        in place (no de-interleave, no placement kernel); needs
+                                        one split pass with k_pass <= 4, cluster 1,
+                                        tl_levels 5, 2^c sizeof(T) = 64, x_group 0 */
 } tds_params;
 
 /* Everything a plan decided (read-only view). */

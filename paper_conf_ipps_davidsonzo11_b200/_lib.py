@@ -46,7 +46,7 @@ class Params(ctypes.Structure):
                 ("split_tile_rows", ctypes.c_int32),
                 ("split_threads", ctypes.c_int32), ("theta", ctypes.c_int32),
                 ("chunk_systems", ctypes.c_int32), ("split_only", ctypes.c_int32),
-                ("x_group", ctypes.c_int32)]
+                ("x_group", ctypes.c_int32), ("strided", ctypes.c_int32)]
 
 
 class PlanInfo(ctypes.Structure):

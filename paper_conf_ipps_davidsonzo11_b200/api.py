@@ -44,7 +44,7 @@ def params_to_dict(p: L.Params) -> dict:
             "cr_levels": p.cr_levels, "thomas_chains": p.thomas_chains, "cluster": p.cluster,
             "tl_levels": p.tl_levels, "chunk_systems": p.chunk_systems,
             "split_tile_rows": p.split_tile_rows, "split_threads": p.split_threads, "theta": p.theta,
-            "x_group": p.x_group}
+            "x_group": p.x_group, "strided": p.strided}
 
 
 class Plan:

@@ -77,7 +77,7 @@ static WsBufs<T> ws_bufs(const tds_plan_info &I, void *ws) {
 template <typename T>
 static tds_status run_split(const tds_plan_info &I, const T *a, const T *b, const T *c, const T *d,
                             const WsBufs<T> &w, cudaStream_t st, int *out_buf, int first = 0,
-                            int last = 1 << 30) {
+                            int last = 1 << 30, bool natural = false) {
     const tds_params &P = I.params;
     int kprev = 0;
     for (int p = 0; p < P.passes; ++p) {
@@ -118,6 +118,10 @@ static tds_status run_split(const tds_plan_info &I, const T *a, const T *b, cons
         const int64_t e = P.split_tile_rows + 2 * ((int64_t(1) << kp) - 1);
         A.ep = int32_t(e + (e >> std::max(kp, 5)) + 1);
         A.vec = raw ? vec_ok(I, {a, b, c, d}) : 1;
+        if (natural) {  // strided variant: one pass, rows kept in original order (per system stride)
+            A.natural = 1;
+            A.out_slot = round_up(I.n, 16 / int64_t(sizeof(T)));
+        }
         const int64_t grid = m_in * A.segs;
         if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "split grid exceeds 2^31-1 CTAs");
         cudaError_t err;
@@ -153,6 +157,8 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
     A.cluster = P.cluster;
     A.tl_levels = P.tl_levels;
     A.x_group = P.x_group;
+    // strided variant (the paper's in-place subsystems): needs the TMA split kernel (16-byte aligned input)
+    const bool strided_ok = P.strided && P.k > 0 && vec_ok(I, {a, b, c, d});
     int64_t grid;
     if (P.k == 0) {
         A.a = a;
@@ -165,7 +171,7 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
         A.vec = 1;
         WsBufs<T> w = ws_bufs<T>(I, ws);
         int ob = 0;
-        tds_status s = run_split<T>(I, a, b, c, d, w, st, &ob, first, last);
+        tds_status s = run_split<T>(I, a, b, c, d, w, st, &ob, first, last, strided_ok);
         if (s != TDS_OK) return s;
         A.a = w.a[ob];
         A.b = nullptr;
@@ -184,7 +190,12 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
     if (P.passes >= first && P.passes <= last) {
         if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "on-chip grid exceeds 2^31-1 CTAs");
         cudaError_t err;
-        if (P.k == 0 && onchip_cpipe_ok(I) && A.vec) {
+        if (strided_ok) {
+            // gather residue classes with stride 2^k from the in-place split output, x scattered in place
+            A.x = x;
+            err = launch_onchip_strided<T>(A, I.m << P.k, I.onchip_threads, round_up(I.n, 16 / int64_t(sizeof(T))),
+                                           st);
+        } else if (P.k == 0 && onchip_cpipe_ok(I) && A.vec) {
             // persistent, TMA-fed warp-form kernel on one CTA or a 2-CTA cluster per system
             err = launch_onchip_cpipe<T>(A, I.onchip_threads, sm_count_current(), st);
         } else if (P.x_group > 0 && uintptr_t(x) % 16 == 0) {
@@ -203,8 +214,10 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
     }
     // x_group plans place x inside the on-chip stage (a misaligned x falls back
     // to the slot kernel + placement, both counted as that one stage)
-    const bool place = P.x_group == 0 ? P.passes + 1 >= first && P.passes + 1 <= last
-                                      : uintptr_t(x) % 16 != 0 && P.passes >= first && P.passes <= last;
+    const bool fused = P.x_group > 0 || P.strided;
+    const bool fused_ok = P.strided ? strided_ok : uintptr_t(x) % 16 == 0;
+    const bool place = !fused ? P.passes + 1 >= first && P.passes + 1 <= last
+                              : !fused_ok && P.passes >= first && P.passes <= last;
     if (P.k > 0 && place) {
         cudaError_t err = launch_place_x<T>(A.xs, x, I.n, I.m, I.batch_stride, I.slot_rows, P.k,
                                             vec_ok(I, {(const void *)x}), A.geom, st);
@@ -258,7 +271,7 @@ static tds_status split_impl(const tds_plan_info &I, const T *a, const T *b, con
 template <typename T>
 static tds_status solve_chunks(const tds_plan_info &I, const T *a, const T *b, const T *c, const T *d, T *x,
                                void *ws, cudaStream_t st, int first, int last) {
-    const int S = I.params.passes + 1 + (I.params.k > 0 && I.params.x_group == 0 ? 1 : 0);
+    const int S = I.params.passes + 1 + (I.params.k > 0 && I.params.x_group == 0 && !I.params.strided ? 1 : 0);
     const int64_t mc = chunk_m(I.params, I.m);
     for (int64_t ch = 0; ch * mc < I.m; ++ch) {
         const int lf = std::max<int64_t>(first - ch * S, 0);

@@ -122,6 +122,7 @@ struct SplitArgs {
     int32_t ep;              // padded shared-memory length per array
     int32_t vec;             // input rows may be read with 16-byte vector loads
     PassGeom geom;           // passes applied to the input
+    int32_t natural;         // output rows in original order (strided variant; first pass, k_p <= 4)
 };
 
 template <typename T>
@@ -166,6 +167,10 @@ size_t onchip_pipe_smem_bytes(int32_t dtype, int32_t threads, int32_t R, int32_t
 template <typename T>
 cudaError_t launch_transpose(const T *const *in, T *const *out, int narrays, int64_t rows, int64_t cols,
                              cudaStream_t st);
+
+template <typename T>
+cudaError_t launch_onchip_strided(const OnchipArgs<T> &A, int64_t nslots, int threads, int64_t ws_stride,
+                                  cudaStream_t st);
 
 template <typename T>
 cudaError_t launch_onchip_gpipe(const OnchipArgs<T> &A, int64_t nslots, int threads, int sm_count, cudaStream_t st);

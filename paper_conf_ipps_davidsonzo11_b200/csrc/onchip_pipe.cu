@@ -639,6 +639,67 @@ __global__ void __launch_bounds__(512, 1)
     cg::this_cluster().sync();  // no CTA leaves while a peer may still push into it
 }
 
+// ---- the paper's strided base-kernel variant (plan strided = 1):
+// the split pass left the 2^K subsystems interleaved in place (row i of
+// system s at a'[s * stride + i]), so subsystem (s, r) is gathered with
+// stride 2^K straight into registers (scalar loads; a warp's loads touch 32
+// different sectors) and its x is scattered the same way into the caller's
+// array -- no de-interleave, no x slots, no placement kernel, no TMA (the
+// rows of one subsystem are not contiguous).  Same arithmetic as the warp
+// form of the pipe kernel (solve_item_warp), so x is bit-identical to the
+// de-interleaved path under the same plan.  Persistent, one subsystem per CTA
+// at a time.
+template <typename T, int R>
+__global__ void __launch_bounds__(512, 1)
+    onchip_strided_kernel(const OnchipArgs<T> A, int64_t nslots, int64_t ws_stride) {
+    extern __shared__ __align__(16) unsigned char smem_raw[];
+    T *scr = reinterpret_cast<T *>(smem_raw);
+    const int NT = blockDim.x, t = threadIdx.x, lane = t & 31, warp = t >> 5, nwarps = NT >> 5;
+    const int64_t KK = int64_t(1) << A.K;
+    pdl_wait();  // the split pass is complete before any global access
+    for (int64_t q = blockIdx.x; q < nslots; q += gridDim.x) {
+        const int64_t sys = q >> A.K, r = q & (KK - 1);
+        const int64_t L = r < A.n ? (A.n - r + KK - 1) >> A.K : 0;
+        if (L == 0) continue;  // CTA-uniform
+        const int64_t jt = int64_t(t) * R, g0 = sys * ws_stride + r;
+        T ra[R], rc[R], rd[R];
+#pragma unroll
+        for (int v = 0; v < R; ++v) {
+            const bool in = jt + v < L;  // rows past the subsystem: identity (0, 1, 0, 0)
+            const int64_t g = g0 + (jt + v) * KK;
+            ra[v] = in ? __ldcs(A.a + g) : T(0);
+            rc[v] = in ? __ldcs(A.c + g) : T(0);
+            rd[v] = in ? __ldcs(A.d + g) : T(0);
+        }
+        solve_item_warp<T, R>(ra, rc, rd, scr, lane, warp, nwarps, [] {});
+        T *x = A.x + sys * A.batch_stride + r;
+#pragma unroll
+        for (int v = 0; v < R; ++v)
+            if (jt + v < L) x[(jt + v) * KK] = rd[v];
+    }
+}
+
+template <typename T>
+cudaError_t launch_onchip_strided(const OnchipArgs<T> &A, int64_t nslots, int threads, int64_t ws_stride,
+                                  cudaStream_t st) {
+    constexpr int R = 64 / int(sizeof(T));
+    if (threads % 32 || threads > 512 || nslots > 0x7fffffffLL) return cudaErrorInvalidConfiguration;
+    const int nw = threads / 32;
+    const size_t smem = size_t(nw * (3 * ilog2c(R) + 30) + 128) * sizeof(T);
+    auto kern = onchip_strided_kernel<T, R>;
+    int occ = 1;
+    cudaError_t e = kernel_setup((const void *)kern, threads, smem, 1, &occ);
+    if (e != cudaSuccess) return e;
+    const int64_t grid = std::min<int64_t>(nslots, int64_t(std::max(occ, 1)) * sm_count_current());
+    e = launch_pdl(kern, dim3(unsigned(std::max<int64_t>(grid, 1))), dim3(threads), smem, st, 1, A, nslots,
+                   ws_stride);
+    if (e != cudaSuccess) return e;
+    return cudaGetLastError();
+}
+
+template cudaError_t launch_onchip_strided<float>(const OnchipArgs<float> &, int64_t, int, int64_t, cudaStream_t);
+template cudaError_t launch_onchip_strided<double>(const OnchipArgs<double> &, int64_t, int, int64_t, cudaStream_t);
+
 size_t onchip_gpipe_smem_bytes(int32_t dtype, int32_t threads) {
     const int64_t R = 64 / dsize(dtype), nw = threads / 32;
     return 1024 + size_t((6 * int64_t(threads) * R + nw * (3 * ilog2c(int(R)) + 30) + 128 + 8) * dsize(dtype));

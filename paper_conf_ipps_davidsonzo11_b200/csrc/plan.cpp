@@ -170,6 +170,13 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
         }
     }
     if (p.chunk_systems < 0) return fail(TDS_ERR_INVALID_ARG, "chunk_systems >= 0");
+    if (p.strided != 0) {  // the paper's strided base-kernel variant (onchip_strided.cu)
+        if (p.strided != 1) return fail(TDS_ERR_INVALID_ARG, "strided must be 0 or 1");
+        if (p.split_only || p.passes != 1 || p.k_pass[0] > 4 || p.x_group != 0)
+            return fail(TDS_ERR_UNSUPPORTED, "strided needs one split pass with k_pass <= 4 and x_group 0");
+        if (p.cluster != 1 || p.tl_levels != 5 || R * dsize(dtype) != 64)
+            return fail(TDS_ERR_UNSUPPORTED, "strided needs cluster 1, tl_levels 5, 64 bytes of rows per thread");
+    }
     if (p.x_group != 0) {  // fused x placement (onchip_pipe.cu, gpipe kernel)
         const int G = p.x_group, ds = dsize(dtype);
         if (G != 2 && G != 4 && G != 8) return fail(TDS_ERR_INVALID_ARG, "x_group must be 0, 2, 4 or 8");
@@ -192,7 +199,7 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
     info.subsys_per_cta = 1;
     const int64_t mc = chunk_m(p, m);  // systems per chunk
     info.chunks = (int32_t)cdiv(m, mc);
-    info.launches = info.chunks * (p.passes + 1 + (p.k > 0 && p.x_group == 0 ? 1 : 0));
+    info.launches = info.chunks * (p.passes + 1 + (p.k > 0 && p.x_group == 0 && p.strided == 0 ? 1 : 0));
     if (p.passes > 0) {
         int kk = 0;
         int64_t elems = 0;

@@ -261,6 +261,27 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
             if (t == 0) bulk_wait_read0();
             __syncthreads();
         }
+        if constexpr (KP <= 4) {
+            if (A.natural) {  // strided variant: rows stay in original order (no de-interleave)
+                if (lane >= 1 && lane <= 30 && i0 < L) {
+                    const int64_t o = sigma * A.out_slot + i0;
+                    if (i0 + R <= L) {
+                        store_run<T, R>(A.oa + o, ra);
+                        store_run<T, R>(A.oc + o, rc);
+                        store_run<T, R>(A.od + o, rd);
+                    } else {
+#pragma unroll
+                        for (int v = 0; v < R; ++v)
+                            if (i0 + v < L) {
+                                A.oa[o + v] = ra[v];
+                                A.oc[o + v] = rc[v];
+                                A.od[o + v] = rd[v];
+                            }
+                    }
+                }
+                continue;
+            }
+        }
         if constexpr (KP <= 4 && TSTORE) {
             constexpr int NR = 1 << KP, G = R >> KP;
             if (lane >= 1 && lane <= 30) {  // residue rr, positions 16(a-1)/2^KP + u

@@ -138,7 +138,7 @@ static void tune_onchip(TuneCtx &C, tds_params &best, double &t_best) {
     bool improved = true;
     while (improved && !out_of_time(C)) {
         improved = false;
-        tds_params cand[16];
+        tds_params cand[18];
         int nc = 0;
         // the warp-level form (CR across all 32 lanes, shuffles only) is a
         // different kernel path, not a neighbour of tl_levels = 4: try it directly
@@ -173,6 +173,12 @@ static void tune_onchip(TuneCtx &C, tds_params &best, double &t_best) {
                 if (best.x_group < 8) { cand[nc] = best; cand[nc++].x_group = best.x_group * 2; }
             }
         }
+        // the paper's strided base-kernel variant (one pass of <= 4 levels): on / off
+        if (best.k > 0 && best.passes == 1 && best.k_pass[0] <= 4 && best.cluster == 1 && best.tl_levels == 5 &&
+            best.x_group == 0 && (1 << best.cr_levels) * dsize(I.dtype) == 64) {
+            cand[nc] = best;
+            cand[nc++].strided = best.strided ? 0 : 1;
+        }
         for (int i = 0; i < nc; ++i) {
             clamp_onchip(I, cand[i]);
             if (std::memcmp(&cand[i], &best, sizeof(best)) == 0) continue;
@@ -206,6 +212,7 @@ static void fit_onchip(const tds_plan_info &I, const tds_device_props &props, td
     while (thr(p) > cap(p.cr_levels) && p.cluster < 16 && props.cc_major >= 9) p.cluster *= 2;
     p.tl_levels = ilog2i(p.cluster);
     p.x_group = 0;  // re-enabled by tune_onchip where the new subsystem size allows it
+    p.strided = 0;
     clamp_onchip(I, p);
 }
 
@@ -228,7 +235,7 @@ static std::string params_str(const tds_params &p) {
     for (int i = 0; i < TDS_MAX_PASSES; ++i) o << " " << p.k_pass[i];
     o << " " << p.cr_levels << " " << p.thomas_chains << " " << p.cluster << " " << p.tl_levels << " "
       << p.split_tile_rows << " " << p.split_threads << " " << p.theta << " " << p.chunk_systems << " "
-      << p.x_group;
+      << p.x_group << " " << p.strided;
     return o.str();
 }
 
@@ -248,6 +255,7 @@ static bool cache_lookup(const std::string &path, const std::string &key, tds_pa
             q.theta >> q.chunk_systems;
         if (is) {
             if (!(is >> q.x_group)) q.x_group = 0;  // lines written before x_group existed
+            if (!(is >> q.strided)) q.strided = 0;
             p = q;
             found = true;
         }

@@ -201,3 +201,17 @@ def test_interleaved_workspace_and_errors(tds):
     assert lib.tds_solve_interleaved(h, 8, 8, 8, 8, 8, None, 0, None) == 1            # x overlaps a
     assert lib.tds_solve_interleaved(h, 1 << 20, 2 << 30, 3 << 30, 4 << 30, 5 << 30, None, 0, None) == 4  # no ws
     assert lib.tds_interleaved_workspace_bytes(h, None) == 1
+
+
+def test_strided_variant_validation(tds):
+    """The paper's strided base-kernel variant (tds_params.strided): one split
+    pass of <= 4 levels, warp form, cluster 1; two launches (no placement)."""
+    p = tds.Plan(65536, 8, props=_props(rp.B200))
+    base = dict(k_pass=[3], cr_levels=4, thomas_chains=16, cluster=1, tl_levels=5)
+    p.set_params(**base, strided=1)
+    assert p.info["strided"] == 1 and p.info["launches"] == 2
+    for kw in [dict(strided=2), dict(strided=1, k_pass=[2, 1]), dict(strided=1, k_pass=[5]),
+               dict(strided=1, tl_levels=3), dict(strided=1, cr_levels=3), dict(strided=1, cluster=2),
+               dict(strided=1, x_group=8)]:
+        with pytest.raises(tds.TdsError):
+            p.set_params(**dict(base, **kw))

@@ -832,3 +832,55 @@ def test_plan_fuzz(tds, i, dtype, n, m, params):
     except tds.TdsError as e:
         pytest.skip(f"plan rejected: {e}")
     check(a, b, c, d, x, dtype)
+
+
+# ------------------------------------- the paper's strided base-kernel variant
+
+SV_CASES = [  # (dtype, n, m, k)
+    (np.float32, 65536, 5, 3), (np.float32, 16384, 7, 1), (np.float32, 32768, 3, 2), (np.float32, 100003, 3, 4),
+    (np.float32, 8191 * 4 + 3, 2, 2), (np.float64, 32768, 3, 3), (np.float64, 9001, 4, 2)]
+
+
+@pytest.mark.parametrize("dtype,n,m,k", SV_CASES)
+def test_strided_variant(tds, dtype, n, m, k):
+    """strided = 1 (subsystems left interleaved by the split, gathered with
+    stride 2^k on chip, x scattered in place): the oracle's x within the
+    tolerances and BIT-identical to the de-interleaved path of the same plan
+    (same split arithmetic, same on-chip solve)."""
+    c_lv = 4 if dtype == np.float32 else 3
+    kw = dict(k_pass=[k], cr_levels=c_lv, thomas_chains=1, tl_levels=5)
+    a, b, c, d = inputs.generate(n, m, dtype, seed=70 + k)
+    x1, plan = run(tds, a, b, c, d, params=dict(kw, strided=1))
+    assert plan.info["strided"] == 1 and plan.info["launches"] == 2
+    check(a, b, c, d, x1, dtype)
+    x0, _ = run(tds, a, b, c, d, params=dict(kw, strided=0))
+    assert np.array_equal(x1, x0)
+
+
+def test_strided_variant_unaligned_input_and_stride(tds):
+    """Unaligned input rows (no TMA split): the strided plan falls back to the
+    de-interleaved kernels, same x; a padded batch stride leaves the padding."""
+    import torch
+    n, m = 20000, 3
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=77)
+    kw = dict(k_pass=[2], cr_levels=4, thomas_chains=1, tl_levels=5, strided=1)
+    xr, _ = run(tds, a, b, c, d, params=kw)
+    plan = tds.Plan(n, m, "float32", device=0)
+    plan.set_params(cluster=1, **kw)
+    ta, tb, tc, td = (torch.zeros(m * n + 1, dtype=torch.float32, device="cuda")[1:].view(m, n) for _ in range(4))
+    for t_, v in zip((ta, tb, tc, td), (a, b, c, d)):
+        t_.copy_(torch.from_numpy(v))
+    x = tds.solve_batched(plan, ta, tb, tc, td)
+    torch.cuda.synchronize()
+    assert np.array_equal(x.cpu().numpy(), xr)
+    stride = n + 12
+    pad = lambda v: np.pad(v, ((0, 0), (0, stride - n)), constant_values=7.0)
+    A, B, C, D = (torch.from_numpy(pad(v).reshape(-1)).cuda() for v in (a, b, c, d))
+    plan2 = tds.Plan(n, m, "float32", device=0, batch_stride=stride)
+    plan2.set_params(cluster=1, **kw)
+    out = torch.full_like(D, 7.0)
+    tds.solve_batched(plan2, A, B, C, D, out=out)
+    torch.cuda.synchronize()
+    xs = out.cpu().numpy().reshape(m, stride)
+    assert np.all(xs[:, n:] == 7.0)
+    assert np.array_equal(xs[:, :n], xr)
