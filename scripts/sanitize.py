@@ -34,9 +34,21 @@ CASES = [  # (label, dtype, n, m, params or None for the static plan)
     ("f64 k8 + pipe", F64, 1 << 20, 1, dict(k_pass=[8], cr_levels=3, thomas_chains=16, tl_levels=5)),
     ("f64 k0 cpipe C=2", F64, 8192, 2, dict(k_pass=[], cr_levels=3, thomas_chains=16, cluster=2, tl_levels=5)),
     ("f64 x_group 2", F64, 1 << 16, 2, dict(k_pass=[4], cr_levels=3, thomas_chains=1, tl_levels=5, x_group=2)),
+    ("strided k3", F32, 65536, 2, dict(k_pass=[3], cr_levels=4, thomas_chains=1, tl_levels=5, strided=1)),
+    ("f64 strided k2", F64, 9001, 2, dict(k_pass=[2], cr_levels=3, thomas_chains=1, tl_levels=5, strided=1)),
 ]
 
 bad = 0
+# the interleaved layout (TMA transposer and the plain tile transposer)
+for label, dt, n, m in [("interleaved TMA transpose", F32, 3000, 36), ("interleaved tile transpose", F32, 1000, 33)]:
+    a, b, c, d = inputs.generate(n, m, dt, seed=6)
+    plan = tds.Plan(n, m, "float32", device=0, mode="static")
+    ti = [torch.from_numpy(np.ascontiguousarray(v.T)).cuda() for v in (a, b, c, d)]
+    x = tds.solve_interleaved(plan, *ti).cpu().numpy().T
+    err = oracle.rel_err(np.ascontiguousarray(x), oracle.thomas(a, b, c, d))
+    ok = err <= 1e-4
+    bad += not ok
+    print(f"{'ok ' if ok else 'BAD'} {label}: n={n} m={m} rel_err={err:.2e}", flush=True)
 for label, dt, n, m, params in CASES:
     a, b, c, d = inputs.generate(n, m, dt, seed=5)
     plan = tds.Plan(n, m, "float32" if dt == F32 else "float64", device=0, mode="static")
