@@ -1,0 +1,49 @@
+"""Long randomized plan fuzz (diagnostic; the test suite runs a seeded 320-draw
+subset): random n, m, dtype and plan parameters, every plan the planner
+accepts solved on the GPU and checked against the oracle.
+
+    python scripts/fuzz_long.py [draws] [seed]
+"""
+import sys
+
+import numpy as np
+import torch
+
+sys.path.insert(0, ".")
+import oracle  # noqa: E402
+import paper_conf_ipps_davidsonzo11_b200 as tds  # noqa: E402
+from paper_conf_ipps_davidsonzo11_b200 import inputs  # noqa: E402
+
+draws = int(sys.argv[1]) if len(sys.argv) > 1 else 2000
+rng = np.random.default_rng(int(sys.argv[2]) if len(sys.argv) > 2 else 7)
+ran = bad = 0
+for i in range(draws):
+    dtype = np.float32 if rng.random() < 0.7 else np.float64
+    n = int(rng.choice([rng.integers(1, 5000), rng.integers(5000, 400000), 1 << int(rng.integers(10, 20))]))
+    m = int(rng.integers(1, 9))
+    k = int(rng.integers(0, 13))
+    passes = 0 if k == 0 else int(rng.integers(1, min(3, k) + 1))
+    kp = [] if k == 0 else [k // passes + (1 if j < k % passes else 0) for j in range(passes)]
+    c_lv = int(rng.integers(0, 5 if dtype == np.float32 else 4))
+    params = dict(k_pass=kp, cr_levels=c_lv, thomas_chains=int(2 ** rng.integers(0, 7)),
+                  cluster=int(rng.choice([1, 1, 1, 2, 4, 8, 16])), tl_levels=int(rng.choice([0, 1, 2, 3, 5])),
+                  x_group=int(rng.choice([0, 0, 0, 2, 4, 8])), strided=int(rng.choice([0, 0, 1])),
+                  split_threads=int(rng.choice([128, 256, 512])), split_tile_rows=int(rng.choice([2048, 4096, 8192])),
+                  theta=int(rng.choice([1, 16, 148, 4736])), chunk_systems=int(rng.choice([0, 0, 1, 2, 3])))
+    plan = tds.Plan(n, m, "float32" if dtype == np.float32 else "float64", device=0)
+    try:
+        plan.set_params(**params)
+    except tds.TdsError:
+        continue
+    a, b, c, d = inputs.generate(n, m, dtype, seed=5000 + i)
+    x = tds.solve_batched(plan, *[torch.from_numpy(v).cuda() for v in (a, b, c, d)])
+    torch.cuda.synchronize()
+    x = x.cpu().numpy()
+    err = oracle.rel_err(x, oracle.thomas(a, b, c, d))
+    ok = np.all(np.isfinite(x)) and err <= (1e-4 if dtype == np.float32 else 1e-10)
+    ran += 1
+    if not ok:
+        bad += 1
+        print(f"BAD draw {i}: {dtype.__name__} n={n} m={m} {params} err={err:.3e}", flush=True)
+print(f"fuzz: {ran} plans run, {bad} bad", flush=True)
+sys.exit(1 if bad else 0)
