@@ -16,7 +16,7 @@ from paper_conf_ipps_davidsonzo11_b200 import inputs  # noqa: E402
 
 draws = int(sys.argv[1]) if len(sys.argv) > 1 else 2000
 rng = np.random.default_rng(int(sys.argv[2]) if len(sys.argv) > 2 else 7)
-ran = bad = 0
+ran = bad = inter = 0
 for i in range(draws):
     dtype = np.float32 if rng.random() < 0.7 else np.float64
     n = int(rng.choice([rng.integers(1, 5000), rng.integers(5000, 400000), 1 << int(rng.integers(10, 20))]))
@@ -41,9 +41,14 @@ for i in range(draws):
     x = x.cpu().numpy()
     err = oracle.rel_err(x, oracle.thomas(a, b, c, d))
     ok = np.all(np.isfinite(x)) and err <= (1e-4 if dtype == np.float32 else 1e-10)
+    if ok and plan.info["batch_stride"] == n and rng.random() < 0.3:  # the interleaved layout: bit-identical
+        xi = tds.solve_interleaved(plan, *[torch.from_numpy(np.ascontiguousarray(v.T)).cuda() for v in (a, b, c, d)])
+        torch.cuda.synchronize()
+        ok = bool(np.array_equal(xi.cpu().numpy().T, x))
+        inter += 1
     ran += 1
     if not ok:
         bad += 1
         print(f"BAD draw {i}: {dtype.__name__} n={n} m={m} {params} err={err:.3e}", flush=True)
-print(f"fuzz: {ran} plans run, {bad} bad", flush=True)
+print(f"fuzz: {ran} plans run ({inter} also through the interleaved layout), {bad} bad", flush=True)
 sys.exit(1 if bad else 0)
