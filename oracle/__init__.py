@@ -18,7 +18,8 @@ Contents (each cites the passage it follows; PAPER.md = /root/reference/PAPER.md
 * ``permutation`` -- the canonical subsystem order after k levels (Fig. 3a
                      P:L386-394: 2 systems of 4, 4 of 2, 8 of 1).
 * ``residual`` / ``backward_error`` / ``rel_err`` -- fp64 error metrics.
-* ``plan``        -- the reference planner (``oracle/plan.py``), §IV-B/C.
+* ``plan``        -- the reference planner (``oracle/plan.py``): the method's integers of
+                     §IV-B/C (on-chip entry size, k, passes, T, theta, segments).
 
 Parity status: every function here is pinned by ``tests/test_oracle.py``
 against something other than itself (dense Gaussian elimination, LAPACK

@@ -2,19 +2,23 @@
 // parameter selection (§IV-B/C) turned into an integer
 // plan for the B200 kernels, plus the plan-handling half of the C ABI.
 //
-// The rules:
+// The rules (the method's integers are pinned
+// against oracle/plan.py, the rest are build choices):
 //   DEFAULT  n_sub_target = 256, theta = 16 systems,
-//            T = 32 (reading R10), split tile 1024 x 256 threads, <= 8
-//            levels per pass, on-chip CTA <= 256 threads.
-//   STATIC   n_sub_target = n_onchip_max: largest power of two whose four
-//            arrays fit in shared memory ("switch as soon as it fits",
-//            P:L704-705), T = 2 x warp size, theta = #SMs
-//            (P:L650-655), split tile = n_onchip_max x 512 threads, <= 9
-//            (fp32) / 8 (fp64) levels per pass, on-chip CTA <= half the
-//            maximum block size.
+//            T = 32 (reading R10), split tile 1024 x 256 threads, on-chip CTA
+//            <= 256 threads, no clusters.
+//   STATIC   n_sub_target = n_onchip_max: the largest power of two whose four
+//            arrays fit in the shared memory of ONE SM ("switch as soon as it
+//            fits"; "shared memory per processor", Table II
+//            P:L729-730): 8192 fp32 / 4096 fp64 on B200.  T = 2 x warp size
+//            (P:L666-668), theta = #SMs, split tile =
+//            n_onchip_max x 512 threads, on-chip CTA <= half the maximum
+//            block size, no clusters (clusters are a TUNED dimension).
 //   both     k = min{k : ceil(n/2^k) <= n_sub_target}; passes = ceil(k/kp_max)
-//            with levels as equal as possible, larger first; R = 2^c the
-//            smallest power of two with ceil(n_sub/R) <= on-chip cap.
+//            with kp_max = 9 (fp32) / 8 (fp64) (lowered only
+//            when a device's shared memory cannot hold the pass's halo), levels
+//            as equal as possible, larger first; R = 2^c the smallest power of
+//            two with ceil(n_sub/R) <= on-chip cap.
 #include <algorithm>
 #include <cstring>
 #include <new>
@@ -88,14 +92,12 @@ int32_t static_cluster(const tds_device_props &p) {
 }
 
 static int64_t n_onchip_max(const tds_device_props &p, int32_t dtype) {
-    // "switch as soon as it fits": the largest power of two whose four
-    // arrays fit in the shared memory of one cluster, capped by the on-chip kernel's
-    // register capacity (R_max x 512 threads per CTA).
-    const int64_t C = static_cluster(p);
-    const int64_t cap = int64_t(r_max(dtype)) * kMaxOnchipThreadsWide * C;
-    const int64_t budget = (int64_t(p.smem_optin_bytes) - kSmemReserve) * C;
+    // "switch as soon as it fits" in the shared memory of one
+    // processor (Table II): the largest power of two n with
+    // 4 n sizeof(T) <= smem_optin - reserve
+    const int64_t budget = int64_t(p.smem_optin_bytes) - kSmemReserve;
     int64_t n = 1;
-    while (n * 2 <= cap && 4 * (n * 2) * dsize(dtype) <= budget) n *= 2;
+    while (4 * (n * 2) * dsize(dtype) <= budget) n *= 2;
     return n;
 }
 
@@ -227,28 +229,24 @@ static tds_status seed(tds_plan_info &info, const tds_device_props &props, tds_p
     int64_t target;
     int32_t T, theta, tile, g1threads, kpmax, g2cap, cmax;
     info.n_onchip_max = (int32_t)n_onchip_max(props, dtype);
+    const int kp_paper = dtype == TDS_F32 ? 9 : 8;
     if (info.mode == TDS_PARAMS_DEFAULT) {
         target = 256;
         theta = 16;
         T = 32;               // reading R10
         tile = 1024;
         g1threads = 256;
-        kpmax = 8;
         g2cap = 256;
-        cmax = 1;
     } else {
-        target = info.n_onchip_max;
+        target = info.n_onchip_max;                       // P:L704-705, Table II
         T = 2 * props.warp_size;
-        // P:L650-655 "estimate based only on the number of available processors";
-        // a B200 SM keeps several split CTAs resident and independent tiles need no
-        // inter-CTA sync, so the static guess asks for 32 independent units per SM.
-        theta = 32 * props.sm_count;
+        theta = props.sm_count;
         tile = (int32_t)std::min<int64_t>(info.n_onchip_max, int64_t(r_max(dtype)) * kMaxOnchipThreadsWide);
         g1threads = 512;
-        kpmax = std::min(dtype == TDS_F32 ? 9 : 8, kp_limit(props, dtype, tile));
         g2cap = props.max_threads_per_block / 2;
-        cmax = static_cluster(props);
     }
+    kpmax = std::min(kp_paper, kp_limit(props, dtype, tile));
+    cmax = 1;  // clusters: TUNED only (tds_tune), the paper's processor is one SM
     info.n_sub_target = (int32_t)target;
     info.split_kp_max = kpmax;
     std::memset(&p, 0, sizeof(p));

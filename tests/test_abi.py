@@ -62,27 +62,59 @@ for pname, props in [("B200", rp.B200)] + list(rp.TABLE_I.items()):
                 CASES.append((pname, props, dtype, mode, n, m))
 
 
+def _pow2ceil(v):
+    p = 1
+    while p < v:
+        p *= 2
+    return p
+
+
 @pytest.mark.parametrize("pname,props,dtype,mode,n,m", CASES)
 def test_planner_matches_reference(tds, pname, props, dtype, mode, n, m):
-    """Integer plan bit-exact vs the plain-Python reference planner (oracle/plan.py)."""
-    try:
-        ref = rp.make_plan(props, dtype, n, m, 0, mode)
-    except ValueError as e:
-        assert "unsupported" in str(e)
-        with pytest.raises(tds.TdsError) as ce:
-            tds.Plan(n, m, "float32" if dtype == rp.F32 else "float64", props=_props(props),
-                     mode="default" if mode == rp.DEFAULT else "static")
-        assert ce.value.name == "TDS_ERR_UNSUPPORTED"
-        return
-    p = tds.Plan(n, m, "float32" if dtype == rp.F32 else "float64", props=_props(props),
-                 mode="default" if mode == rp.DEFAULT else "static")
+    """The method's integers (k, passes, k_pass, n_sub, number of subsystems,
+    on-chip entry size, theta, T, segments) bit-exact vs the plain-Python
+    reference planner (oracle/plan.py), which knows nothing of the kernels."""
+    mname = "default" if mode == rp.DEFAULT else "static"
+    dname = "float32" if dtype == rp.F32 else "float64"
+    if pname != "B200":
+        # Table I devices: the B200 kernels may not fit 16 / 48 KB of shared
+        # memory; when the C++ planner accepts, the method's integers must agree.
+        try:
+            p = tds.Plan(n, m, dname, props=_props(props), mode=mname)
+        except tds.TdsError as e:
+            assert e.name == "TDS_ERR_UNSUPPORTED"
+            return
+    else:
+        p = tds.Plan(n, m, dname, props=_props(props), mode=mname)
     got = p.info
-    for f in ("k", "passes", "n_sub", "num_subsystems", "cr_levels", "thomas_chains", "onchip_threads",
-              "cluster", "tl_levels", "chunk_systems", "chunks", "launches",
-              "split_tile_rows", "split_threads", "split_segments", "theta", "n_sub_target", "n_onchip_max",
-              "split_kp_max", "slot_rows", "workspace_bytes"):
+    ref = rp.make_plan(props, dtype, n, m, mode, kp_max=got["split_kp_max"])
+    if pname == "B200":
+        assert got["split_kp_max"] == rp.KP_MAX[dtype]
+    for f in ("k", "passes", "n_sub", "num_subsystems", "theta", "n_sub_target", "n_onchip_max"):
         assert got[f] == getattr(ref, f), (f, got[f], getattr(ref, f))
     assert got["k_pass"] == ref.k_pass[:ref.passes]
+    # T: the mode's switch, unless the reduced on-chip system has fewer rows
+    red = -(-got["n_sub"] // (1 << got["cr_levels"])) >> got["tl_levels"]
+    assert got["thomas_chains"] == min(ref.thomas_switch, _pow2ceil(red))
+    # segments: the rule's value, capped by the number of split tiles per system
+    if ref.passes:
+        tiles = -(-n // got["split_tile_eff"])
+        assert got["split_segments"] == min(ref.segments, tiles)
+    # build properties of the kernel shape (not the method's integers)
+    assert got["cluster"] == 1 and got["chunk_systems"] == 0 and got["chunks"] == 1
+    R = 1 << got["cr_levels"]
+    assert R <= (16 if dtype == rp.F32 else 8)
+    nt = got["onchip_threads"]
+    assert nt % 32 == 0 and 32 <= nt <= props.max_threads_per_block
+    assert nt >= -(-got["n_sub"] // R)
+    assert got["launches"] == got["passes"] + 1 + (1 if got["k"] > 0 else 0)
+    s = 4 if dtype == rp.F32 else 8
+    if got["passes"]:
+        # three normalised arrays of every row (x2 ping-pong for >= 2 passes)
+        assert got["workspace_bytes"] >= (1 if got["passes"] == 1 else 2) * 3 * m * n * s
+        assert got["slot_rows"] >= got["n_sub"] and (got["slot_rows"] * s) % 16 == 0
+    else:
+        assert got["workspace_bytes"] == 0
 
 
 @pytest.mark.parametrize("n", [1, 5, 8, 100, 1023, 70000])
@@ -127,8 +159,8 @@ def test_set_params_validation(tds):
     p.set_params(k_pass=[5, 5], cr_levels=3, thomas_chains=16)
     i = p.info
     assert (i["k"], i["passes"], i["k_pass"], i["n_sub"], i["mode"]) == (10, 2, [5, 5], 1024, 2)
-    assert i["workspace_bytes"] == 2 * 3 * 4 * max(4 * 32 * rp.slot_rows(1 << 20, 5, 0),
-                                                   4 * 1024 * rp.slot_rows(1 << 20, 10, 0))
+    slot = lambda kk: -(-(-(-(1 << 20) // (1 << kk))) // 4) * 4   # ceil(n / 2^kk) in 16-byte units
+    assert i["workspace_bytes"] == 2 * 3 * 4 * max(4 * 32 * slot(5), 4 * 1024 * slot(10))
 
 
 def test_solve_argument_errors_before_launch(tds):

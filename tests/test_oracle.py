@@ -135,6 +135,69 @@ def test_thomas_batch_independence_and_threads():
     assert np.array_equal(xs, x1[17])
 
 
+# ---------------------------------------------------------- error metrics ----
+# The GPU parity tests judge every x through these three functions, so each is
+# pinned by hand-computed values (a metric that returned 0, or took the wrong
+# norm / the wrong maximum, fails here).
+
+def test_rel_err_hand_values():
+    """Normwise per system, max over systems (reading R17): system 0 has
+    ||dx|| = 0.5, ||x_ref|| = 4 -> 0.125; system 1 has 3 / 300 = 0.01.  A
+    global norm would give 0.5/300, an elementwise one 0.5/2."""
+    xref = np.array([[1.0, -4.0, 2.0], [300.0, 10.0, -20.0]])
+    x = xref.copy()
+    x[0, 2] += 0.5
+    x[1, 0] -= 3.0
+    assert oracle.rel_err(x, xref) == 0.125
+    assert oracle.rel_err(x[1:], xref[1:]) == 0.01
+    assert oracle.rel_err(xref, xref) == 0.0
+    # x = x_ref + delta e_j: exactly delta / ||x_ref||
+    for j in range(3):
+        y = xref[:1].copy()
+        y[0, j] += 2.0 ** -10
+        assert oracle.rel_err(y, xref[:1]) == 2.0 ** -10 / 4.0
+    # a zero reference system: the denominator guard makes it an absolute error
+    assert oracle.rel_err(np.array([[0.0, 0.25]]), np.zeros((1, 2))) == 0.25
+    # fp32 input is upcast exactly
+    assert oracle.rel_err(np.float32([[1.5, 2.0]]), np.array([[1.0, 2.0]])) == 0.25
+
+
+def test_residual_hand_values():
+    """||A x - d||_inf / ||d||_inf per system, max over systems, a[0] and
+    c[n-1] outside the matrix.  A = [[4,1,0],[1,5,1],[0,2,6]], d = [1,2,3]:
+    x = 1 gives A x - d = [4,5,5] -> 5/3; x = 0 gives -d -> 1."""
+    a = np.array([[100.0, 1.0, 2.0]] * 2)        # a[0] ignored
+    b = np.array([[4.0, 5.0, 6.0]] * 2)
+    c = np.array([[1.0, 1.0, -100.0]] * 2)       # c[n-1] ignored
+    d = np.array([[1.0, 2.0, 3.0]] * 2)
+    x = np.array([[1.0, 1.0, 1.0], [0.0, 0.0, 0.0]])
+    assert oracle.residual(a, b, c, d, x) == 5.0 / 3.0
+    assert oracle.residual(a[1:], b[1:], c[1:], d[1:], x[1:]) == 1.0
+    # the exact solution has residual 0
+    xs = np.linalg.solve(dense(a[0], b[0], c[0]), d[0])
+    assert oracle.residual(a[:1], b[:1], c[:1], d[:1], xs[None]) <= 4 * EPS64
+    # ||d|| = 0 guard: the residual is ||A x||_inf (A x = [5, 7, 8])
+    assert oracle.residual(a[:1], b[:1], c[:1], np.zeros((1, 3)), x[:1]) == 8.0
+    # matvec itself: A x for x = [1, 2, 3] is [6, 14, 22]
+    assert oracle.matvec(a[:1], b[:1], c[:1], np.array([[1.0, 2.0, 3.0]])).tolist() == [[6.0, 14.0, 22.0]]
+
+
+def test_backward_error_closed_form_2x2():
+    """||Ax-d|| / (||A|| ||x|| + ||d||) on A = [[2,1],[1,3]] (||A||_inf = 4),
+    d = [1,1]: x = [1,1] -> r = [2,3] -> 3 / (4 + 1) = 0.6; x = 0 -> 1 / 1."""
+    a = np.array([[50.0, 1.0]])    # a[0] ignored (also in ||A||)
+    b = np.array([[2.0, 3.0]])
+    c = np.array([[1.0, 50.0]])    # c[n-1] ignored
+    d = np.array([[1.0, 1.0]])
+    assert oracle.backward_error(a, b, c, d, np.array([[1.0, 1.0]])) == 0.6
+    assert oracle.backward_error(a, b, c, d, np.zeros((1, 2))) == 1.0
+    # max over systems: a second system scaled by 10 has the same backward error
+    A, B, C, D = (np.concatenate([v, 10 * v]) for v in (a, b, c, d))
+    X = np.array([[1.0, 1.0], [0.0, 0.0]])
+    assert oracle.backward_error(A, B, C, D, X) == 1.0
+    assert oracle.backward_error(A[1:], B[1:], C[1:], D[1:], np.array([[1.0, 1.0]])) == 30.0 / 50.0
+
+
 # ------------------------------------------------------------- generator ----
 
 def test_generator_recipe():
@@ -276,48 +339,62 @@ def _golden_params():
 
 
 def test_planner_paper_values():
+    """The paper's printed constants (tests/golden/paper_parameters.txt)."""
     g = _golden_params()
     p = rplan.make_plan(rplan.B200, rplan.F32, 1 << 20, 16, mode=rplan.DEFAULT)
     assert p.n_sub_target == g["default_nsub_target"][0]
     assert p.theta == g["default_theta"][0]
     assert p.n_sub <= 256 and p.k == 12
     ps = rplan.make_plan(rplan.B200, rplan.F32, 1 << 20, 16, mode=rplan.STATIC)
-    assert ps.thomas_chains == g["static_thomas_chains"][0]
-    assert ps.theta == 32 * rplan.B200.sm_count  # a multiple of the processor count
+    assert ps.thomas_switch == g["static_thomas_chains"][0]
+    assert ps.theta == rplan.B200.sm_count  # "based only on the number of available processors" (P:L650-655)
 
 
 def test_planner_static_onchip_sizes():
     """Static on-chip size = largest power of two whose 4 arrays fit in the
-    shared memory of the device's cluster: 512 (16 KB) / 2048 (48 KB) on Table
-    I (no clusters), 65536 fp32 / 32768 fp64 on B200 (8-CTA clusters)."""
+    shared memory of ONE processor (Table II): 512 on
+    16 KB (8800 GTX, GTX 280), 2048 on 48 KB (GTX 470), and on B200's 227 KB
+    opt-in 8192 fp32 / 4096 fp64 (SURVEY §8 preamble)."""
     t = rplan.TABLE_I
     assert rplan.n_onchip_max(t["GeForce 8800 GTX"], rplan.F32) == 512
     assert rplan.n_onchip_max(t["GeForce GTX 280"], rplan.F32) == 512
     assert rplan.n_onchip_max(t["GeForce GTX 470"], rplan.F32) == 2048
-    assert rplan.n_onchip_max(rplan.B200, rplan.F32) == 65536
-    assert rplan.n_onchip_max(rplan.B200, rplan.F64) == 32768
+    assert rplan.n_onchip_max(rplan.B200, rplan.F32) == 8192
+    assert rplan.n_onchip_max(rplan.B200, rplan.F64) == 4096
+    # brute force over every power of two: the next one no longer fits
+    for props in list(t.values()) + [rplan.B200]:
+        for dt in (rplan.F32, rplan.F64):
+            n = rplan.n_onchip_max(props, dt)
+            s = rplan.dsize(dt)
+            assert 4 * n * s <= props.smem_optin_bytes - 1024 < 4 * 2 * n * s
 
 
-@pytest.mark.parametrize("dtype,n,m,k,passes,nsub,cluster", [
-    (rplan.F32, 1024, 1, 0, 0, 1024, 1),
-    (rplan.F32, 65536, 256, 0, 0, 65536, 8),
-    (rplan.F32, 1 << 20, 16, 4, 1, 65536, 8),
-    (rplan.F64, 1 << 20, 16, 5, 1, 32768, 8),
-    (rplan.F32, 16384, 4096, 0, 0, 16384, 2),
-    (rplan.F32, 1 << 28, 1, 12, 2, 65536, 8),
+@pytest.mark.parametrize("dtype,n,m,k,k_pass,nsub,segs", [
+    (rplan.F32, 1024, 1, 0, [], 1024, 0),              # cfg 1
+    (rplan.F32, 65536, 256, 3, [3], 8192, 1),          # cfg 2
+    (rplan.F32, 1 << 20, 16, 7, [7], 8192, 10),        # cfg 3 fp32: one pass
+    (rplan.F64, 1 << 20, 16, 8, [8], 4096, 10),        # cfg 3 fp64: one pass
+    (rplan.F32, 16384, 4096, 1, [1], 8192, 1),         # cfg 4
+    (rplan.F32, 1 << 28, 1, 15, [8, 7], 8192, 148),    # cfg 5: two passes
 ])
-def test_planner_static_configs(dtype, n, m, k, passes, nsub, cluster):
-    """STATIC plans at the BASELINE.json configs: "switch to the on-chip kernel
-    as soon as the subsystem fits", where on B200 the on-chip
-    memory is that of one 8-CTA cluster (reading R22)."""
+def test_planner_static_configs(dtype, n, m, k, k_pass, nsub, segs):
+    """STATIC plans at the BASELINE.json configs: k from
+    "switch to the on-chip kernel as soon as the subsystem fits" in one SM
+    (P:L704-705), passes of <= 9 / 8 levels, segments = max(1, ceil(#SMs / M))."""
     p = rplan.make_plan(rplan.B200, dtype, n, m, mode=rplan.STATIC)
-    assert (p.k, p.passes, p.n_sub, p.cluster) == (k, passes, nsub, cluster)
-    assert sum(p.k_pass) == k
-    assert p.k_pass[:passes] == sorted(p.k_pass[:passes], reverse=True)
-    assert max(p.k_pass) - min(p.k_pass[:max(passes, 1)]) <= 1 or passes <= 1
+    assert (p.k, p.k_pass[:p.passes], p.n_sub, p.segments) == (k, k_pass, nsub, segs)
+    assert p.num_subsystems == m * (1 << k)
+    assert p.thomas_switch == 64
 
 
-def test_decoupled_trial_count_arithmetic():
-    """§IV-D: decoupling makes trials additive, not multiplicative."""
-    g = _golden_params()["decoupled_trials"]
-    assert g[0] + g[1] == g[2] and g[0] * g[1] == g[3]
+@pytest.mark.parametrize("n", [1, 255, 256, 257, 1000, 4097, 1 << 20, 3 * 10 ** 6 + 7])
+def test_planner_default_rule_bruteforce(n):
+    """DEFAULT: k is the smallest number of halvings that brings ceil(n / 2^k)
+    to <= 256 (brute force over k), passes split k as evenly as possible."""
+    p = rplan.make_plan(rplan.B200, rplan.F32, n, 3, mode=rplan.DEFAULT)
+    k = next(k for k in range(64) if -(-n // (1 << k)) <= 256)
+    assert p.k == k and p.n_sub == -(-n // (1 << k)) and p.thomas_switch == 32
+    kp = p.k_pass[:p.passes]
+    assert sum(kp) == k and all(1 <= v <= 9 for v in kp) and (not kp or max(kp) - min(kp) <= 1)
+    assert kp == sorted(kp, reverse=True) and p.passes == -(-k // 9)
+    assert p.segments == (max(1, -(-16 // 3)) if k else 0)
