@@ -9,6 +9,21 @@ namespace tds {
 
 constexpr int kMaxPasses = TDS_MAX_PASSES;
 
+// Mutation-test builds only (scripts/mutation_check.sh, -DTDS_MUTATE=k):
+// site k drops one long-range coupling term so the coupling tests
+// (tests/test_coupling.py) can be shown to fail.  Product builds: 0, every
+// site compiles away.
+//   1 warp-form top PCR (onchip_pipe solve_item_warp): warps >= 2 apart
+//   2 cpipe: the last warp's chain loses the next CTA's rows (DSMEM hand-off)
+//   3 cpipe: the cluster's all-gathered top system, strides >= 4
+//   4 pipe shared-memory form: reduced PCR, strides >= 4
+//   5 onchip (generic / cluster) leader PCR, strides >= 4
+//   6 onchip cluster: the deferred chain loses the next CTA's ghost rows
+#ifndef TDS_MUTATE
+#define TDS_MUTATE 0
+#endif
+#define TDS_MUT(k, cond) (TDS_MUTATE == (k) && (cond))
+
 // Reciprocal.  fp32: the SFU approximation (MUFU.RCP, <= 1 ulp) -- the
 // north_star's fp32 tolerance (1e-4 error, 1e-5 residual) leaves room for it
 // (reading R16).  fp64: the SFU seed (MUFU.RCP64H) refined by two

@@ -88,7 +88,7 @@ __device__ __forceinline__ void reduced_solve(T *z, int Z, int NT, int t, int lo
             const int i = t + q * NT;
             if (i < Z) {
                 T a = za[i], c = zc[i], d = zd[i];
-                const bool hl = i >= s, hr = i + s < Z;
+                const bool hl = i >= s, hr = i + s < Z && !TDS_MUT(5, s >= 4);
                 row_update(a, c, d, hl ? za[i - s] : T(0), hl ? zc[i - s] : T(0), hl ? zd[i - s] : T(0),
                            hr ? za[i + s] : T(0), hr ? zc[i + s] : T(0), hr ? zd[i + s] : T(0));
                 na[q] = a;
@@ -296,8 +296,10 @@ __global__ void __launch_bounds__(R * sizeof(T) >= 64 ? 512 : 1024) onchip_kerne
 #pragma unroll
             for (int l = 1; l <= CR; ++l) {
                 const int s = 1 << (l - 1);
+                const bool g = !TDS_MUT(6, crank + 1 < C);
                 row_update(ra[R - 1], rc[R - 1], rd[R - 1], ra[R - 1 - s], rc[R - 1 - s], rd[R - 1 - s],
-                           ghost[3 * (l - 1)], ghost[3 * (l - 1) + 1], ghost[3 * (l - 1) + 2]);
+                           g ? ghost[3 * (l - 1)] : T(0), g ? ghost[3 * (l - 1) + 1] : T(0),
+                           g ? ghost[3 * (l - 1) + 2] : T(0));
             }
             T a = ra[R - 1], c = rc[R - 1], d = rd[R - 1];
             for (int l = 1; l <= c2; ++l) {

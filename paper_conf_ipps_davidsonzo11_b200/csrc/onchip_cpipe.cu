@@ -66,7 +66,7 @@ __device__ __forceinline__ void warp_cr_solve(T (&ra)[RZ], T (&rc)[RZ], T (&rd)[
         const T la = __shfl_up_sync(FULL, za, s), lc = __shfl_up_sync(FULL, zc, s), ld = __shfl_up_sync(FULL, zd, s);
         const T xa = __shfl_down_sync(FULL, za, s), xc = __shfl_down_sync(FULL, zc, s),
                 xd = __shfl_down_sync(FULL, zd, s);
-        const bool hr = lane + s < 32;
+        const bool hr = lane + s < 32 && !TDS_MUT(3, s >= 4);
         T a = za, c = zc, d = zd;
         row_update_early(a, c, d, la, lc, ld, hr ? xa : T(0), hr ? xc : T(0), hr ? xd : T(0));
         const bool upd = (lane & ((1 << l) - 1)) == (1 << l) - 1;
@@ -300,7 +300,7 @@ __global__ void __launch_bounds__(512, 1)
         __syncthreads();  // (1) every warp's first rows are published (this CTA)
         if (lane == 31) {  // the deferred chains; the last warp uses the next CTA's pushed rows
             const bool last_warp = warp == nwarps - 1;
-            const bool h = !last_warp || rank + 1 < C;
+            const bool h = !last_warp || (rank + 1 < C && !TDS_MUT(2, true));
             const T *en = e_in + (warp + 1) * CR * 3, *wn = w_in + (warp + 1) * 15;
             if constexpr (C > 1) {
                 if (last_warp && rank + 1 < C) {
@@ -373,7 +373,7 @@ __global__ void __launch_bounds__(512, 1)
                     a = za2[t];
                     c = zc2[t];
                     d = zd2[t];
-                    const bool hl = t >= s, hr = t + s < Z;
+                    const bool hl = t >= s, hr = t + s < Z && !TDS_MUT(3, s >= 4);
                     row_update_early(a, c, d, hl ? za2[t - s] : T(0), hl ? zc2[t - s] : T(0), hl ? zd2[t - s] : T(0),
                                hr ? za2[t + s] : T(0), hr ? zc2[t + s] : T(0), hr ? zd2[t + s] : T(0));
                 }
@@ -397,7 +397,7 @@ __global__ void __launch_bounds__(512, 1)
                         ld = __shfl_up_sync(FULL, d, s);
                 const T xa = __shfl_down_sync(FULL, a, s), xc = __shfl_down_sync(FULL, c, s),
                         xd = __shfl_down_sync(FULL, d, s);
-                const bool hl = lane >= s, hr = lane + s < Z;
+                const bool hl = lane >= s, hr = lane + s < Z && !TDS_MUT(3, s >= 4);
                 T na = a, nc = c, nd = d;
                 row_update_early(na, nc, nd, hl ? la : T(0), hl ? lc : T(0), hl ? ld : T(0), hr ? xa : T(0),
                            hr ? xc : T(0), hr ? xd : T(0));

@@ -144,7 +144,7 @@ __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[
             const T la = __shfl_up_sync(FULL, a, s), lc = __shfl_up_sync(FULL, c, s), ld = __shfl_up_sync(FULL, d, s);
             const T xa = __shfl_down_sync(FULL, a, s), xc = __shfl_down_sync(FULL, c, s),
                     xd = __shfl_down_sync(FULL, d, s);
-            const bool hl = lane >= s, hr = lane + s < nwarps;
+            const bool hl = lane >= s, hr = lane + s < nwarps && !TDS_MUT(1, s >= 2);
             T na = a, nc = c, nd = d;
             row_update(na, nc, nd, hl ? la : T(0), hl ? lc : T(0), hl ? ld : T(0), hr ? xa : T(0), hr ? xc : T(0),
                        hr ? xd : T(0));
@@ -453,7 +453,7 @@ __device__ __forceinline__ void reduced_solve_pipe(T *z, int Z, int NT, int t, i
             const int i = t + q * NT;
             if (i < Z) {
                 T a = za[i], c = zc[i], d = zd[i];
-                const bool hl = i >= s, hr = i + s < Z;
+                const bool hl = i >= s, hr = i + s < Z && !TDS_MUT(4, s >= 4);
                 row_update(a, c, d, hl ? za[i - s] : T(0), hl ? zc[i - s] : T(0), hl ? zd[i - s] : T(0),
                            hr ? za[i + s] : T(0), hr ? zc[i + s] : T(0), hr ? zd[i + s] : T(0));
                 na[q] = a;
