@@ -141,7 +141,15 @@ typedef struct {
     int32_t launches;         /* kernel launches per solve (tds_solve_stages range)    */
     int64_t slot_rows;        /* workspace rows reserved per subsystem (final pass)    */
     size_t workspace_bytes;   /* bytes tds_solve_batched needs (0 when k == 0)         */
+    int32_t onchip_form;      /* stage 3->4 form the on-chip kernel runs (16-byte aligned
+                                 arrays): TDS_FORM_PCR_THOMAS = the paper's base kernel
+                                 (PCR until T chains, Thomas per chain, §III-A) after c / c2
+                                 CR levels; TDS_FORM_WARP_CR = CR in registers and across the
+                                 32 lanes, shuffle PCR / CR on the per-warp top rows (T
+                                 unused); -1 for a split-only plan                          */
 } tds_plan_info;
+
+enum { TDS_FORM_PCR_THOMAS = 0, TDS_FORM_WARP_CR = 1 };
 
 /* ---- planning (host only, no device work) -------------------------------- */
 
@@ -191,6 +199,18 @@ tds_status tds_tune(tds_plan_t plan, void *cuda_stream, const char *cache_path);
 
 /* Trials run by the most recent tds_tune on this plan (0 on a cache hit). */
 tds_status tds_plan_tune_trials(const tds_plan_t plan, int32_t *trials);
+
+/* TEST-ONLY: tds_tune's search (§IV-D: decoupled stages, hill climb from the
+ * plan's current parameters, 2 % ties, cache) with the trial cost supplied by
+ * the caller instead of timed device solves -- no device work, so a plan from
+ * tds_plan_from_props works.  cost (host callback): the "median time" of one
+ * solve with *params (called only for parameter sets the planner accepts;
+ * return >= 1e30 to refuse one, NaN to abort the search).  user is passed
+ * through.  cache_path as in tds_tune.  tds_plan_tune_trials reports the
+ * number of cost calls.  Errors: INVALID_ARG (NULL plan / cost), TUNE (the
+ * seed was refused or the search aborted). */
+tds_status tds_tune_search(tds_plan_t plan, double (*cost)(const tds_params *params, void *user), void *user,
+                           const char *cache_path);
 
 /* ---- solving ---------------------------------------------------------------- */
 
@@ -250,6 +270,21 @@ tds_status tds_interleaved_workspace_bytes(const tds_plan_t plan, size_t *bytes)
 tds_status tds_solve_interleaved(const tds_plan_t plan, const void *a, const void *b, const void *c,
                                  const void *d, void *x, void *workspace, size_t workspace_bytes,
                                  void *cuda_stream);
+
+/* ---- synthetic inputs ------------------------- */
+
+/* Fill a, b, c, d (device, dtype, m x batch_stride; padding untouched) with the
+ * seeded diagonally dominant systems of the input recipe, bit-identical to the
+ * host generator (inputs.py, family "dd" with margin mu; "weak" is mu < 1):
+ * h = splitmix64(seed ^ (array_id << 56) ^ ((first_system + s) * n + i)),
+ * a, c, d = exact dyadic 2u - 1 from the top 24 (fp32) / 53 (fp64) bits of h
+ * (array ids 0, 2, 3), a_0 = c_{n-1} = 0, b = (|a| + |c|) + mu rounded to
+ * nearest in the target precision.  first_system: global index of system 0
+ * (a rank of a sharded batch draws exactly the unsharded rows).  Enqueued on
+ * cuda_stream.  Errors: INVALID_ARG (dtype, n < 1, m < 1, stride < n, NULL or
+ * misaligned pointer), CUDA (launch). */
+tds_status tds_generate(tds_dtype dtype, int64_t n, int64_t m, int64_t batch_stride, uint64_t seed,
+                        int64_t first_system, double mu, void *a, void *b, void *c, void *d, void *cuda_stream);
 
 /* ---- misc ---------------------------------------------------------------------- */
 

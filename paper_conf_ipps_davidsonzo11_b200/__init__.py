@@ -7,6 +7,7 @@ error (there is no CPU fallback).
 """
 from . import inputs  # noqa: F401  (seeded generator; no solver arithmetic)
 from ._lib import TdsError  # noqa: F401
-from .api import Plan, device_props, solve_batched, solve_interleaved, split_batched, version  # noqa: F401
+from .api import Plan, device_props, generate, solve_batched, solve_interleaved, split_batched, version  # noqa: F401
 
-__all__ = ["Plan", "solve_batched", "solve_interleaved", "split_batched", "device_props", "version", "TdsError", "inputs"]
+__all__ = ["Plan", "solve_batched", "solve_interleaved", "split_batched", "generate", "device_props", "version",
+           "TdsError", "inputs"]

@@ -26,7 +26,7 @@ EXPORTED = (
     "tds_plan_set_params", "tds_plan_permutation", "tds_plan_destroy", "tds_tune",
     "tds_plan_tune_trials", "tds_solve_batched", "tds_solve_stages", "tds_split_batched", "tds_status_string",
     "tds_interleaved_workspace_bytes", "tds_solve_interleaved",
-    "tds_last_error", "tds_version",
+    "tds_last_error", "tds_version", "tds_tune_search", "tds_generate",
 )
 
 
@@ -58,8 +58,12 @@ class PlanInfo(ctypes.Structure):
                 ("onchip_threads", ctypes.c_int32), ("subsys_per_cta", ctypes.c_int32),
                 ("split_segments", ctypes.c_int32), ("split_tile_eff", ctypes.c_int32),
                 ("chunks", ctypes.c_int32), ("launches", ctypes.c_int32),
-                ("slot_rows", ctypes.c_int64), ("workspace_bytes", ctypes.c_size_t)]
+                ("slot_rows", ctypes.c_int64), ("workspace_bytes", ctypes.c_size_t),
+                ("onchip_form", ctypes.c_int32)]
 
+
+# tds_tune_search's cost callback: double (*)(const tds_params *, void *)
+COST_FN = ctypes.CFUNCTYPE(ctypes.c_double, ctypes.POINTER(Params), ctypes.c_void_p)
 
 _lib = None
 
@@ -90,6 +94,8 @@ def load() -> ctypes.CDLL:
         "tds_split_batched": (I32, [P, VP, VP, VP, VP, VP, VP, VP, VP, SZ, VP]),
         "tds_interleaved_workspace_bytes": (I32, [P, ctypes.POINTER(ctypes.c_size_t)]),
         "tds_solve_interleaved": (I32, [P, VP, VP, VP, VP, VP, VP, SZ, VP]),
+        "tds_tune_search": (I32, [P, COST_FN, VP, ctypes.c_char_p]),
+        "tds_generate": (I32, [I32, I64, I64, I64, ctypes.c_uint64, I64, ctypes.c_double, VP, VP, VP, VP, VP]),
         "tds_status_string": (ctypes.c_char_p, [I32]),
         "tds_last_error": (ctypes.c_char_p, []),
         "tds_version": (I32, []),

@@ -158,6 +158,20 @@ class Plan:
         L.check(self._lib.tds_plan_tune_trials(self._h, ctypes.byref(t)))
         return int(t.value)
 
+    def tune_search(self, cost, cache_path: Optional[str] = None) -> int:
+        """tds_tune_search (TEST-ONLY): the tuner's search with ``cost(params
+        dict) -> float`` in place of timed device solves.  Returns the number
+        of cost calls (0 on a cache hit)."""
+        def cb(p, _user):
+            return float(cost(params_to_dict(p.contents)))
+        fn = L.COST_FN(cb)
+        cp = cache_path.encode() if cache_path else None
+        self._cache = None
+        L.check(self._lib.tds_tune_search(self._h, fn, None, cp))
+        t = ctypes.c_int32()
+        L.check(self._lib.tds_plan_tune_trials(self._h, ctypes.byref(t)))
+        return int(t.value)
+
     @property
     def interleaved_workspace_bytes(self) -> int:
         """tds_interleaved_workspace_bytes (dense plans only)."""
@@ -266,6 +280,24 @@ def split_batched(plan: Plan, a, b, c, d, workspace=None, stream=None):
     L.check(plan._lib.tds_split_batched(plan.handle, _ptr(a), _ptr(b), _ptr(c), _ptr(d), _ptr(oa), _ptr(oc),
                                         _ptr(od), wptr, wbytes, _stream_ptr(stream)))
     return oa, oc, od
+
+
+def generate(n: int, m: int, dtype="float32", seed: int = 1, first_system: int = 0, mu: float = 1.0,
+             device: int = 0, batch_stride: int = 0, out=None, stream=None):
+    """tds_generate: the seeded synthetic systems (inputs.py's "dd" family)
+    drawn on the device.  Returns (a, b, c, d) as (m, batch_stride or n) CUDA
+    tensors (or fills ``out``)."""
+    import torch
+    code = _dtype_code(dtype)
+    stride = int(batch_stride) or int(n)
+    tdt = torch.float32 if code == L.TDS_F32 else torch.float64
+    if out is None:
+        out = tuple(torch.empty((int(m), stride), dtype=tdt, device=f"cuda:{device}") for _ in range(4))
+    for name, t in zip("abcd", out):
+        _check_fast(t, (int(m) - 1) * stride + int(n), tdt, name)
+    L.check(L.load().tds_generate(code, int(n), int(m), stride, int(seed) & 0xFFFFFFFFFFFFFFFF, int(first_system),
+                                  float(mu), *(t.data_ptr() for t in out), _stream_ptr(stream, int(out[0].device.index))))
+    return out
 
 
 def version() -> int:

@@ -226,6 +226,15 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
     return TDS_OK;
 }
 
+int32_t onchip_form_of(const tds_plan_info &I) {
+    const tds_params &P = I.params;
+    bool warp;
+    if (P.strided || P.x_group > 0) warp = true;  // onchip_strided / onchip_gpipe: solve_item_warp
+    else if (P.k == 0) warp = onchip_cpipe_ok(I);
+    else warp = onchip_pipe_ok(I) && P.tl_levels == 5;
+    return warp ? TDS_FORM_WARP_CR : TDS_FORM_PCR_THOMAS;
+}
+
 // Gather workspace slots into the canonical order (diagnostic path only).
 template <typename T>
 __global__ void gather_canonical_kernel(const T *sa, const T *sc, const T *sd, T *oa, T *oc, T *od, int64_t n,

@@ -3,6 +3,8 @@
 #include <cuda_runtime.h>
 #include <stdint.h>
 
+#include <algorithm>
+
 #include "tds_internal.h"
 
 namespace tds {
@@ -223,5 +225,10 @@ cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batc
 template <typename T>
 cudaError_t launch_onchip(const OnchipArgs<T> &A, int cr_levels, bool raw, int64_t grid, int threads,
                           size_t smem, cudaStream_t st);
+
+// G4 seeded input generator (gen.cu), bit-identical to inputs.py's "dd" family.
+template <typename T>
+cudaError_t launch_generate(T *a, T *b, T *c, T *d, int64_t n, int64_t m, int64_t stride, uint64_t seed,
+                            int64_t first_system, double mu, cudaStream_t st);
 
 }  // namespace tds

@@ -1,0 +1,99 @@
+// gen.cu -- G4: the seeded synthetic-input generator on the device
+// (SURVEY.md §8(d) "Concrete synthetic inputs"), bit-identical
+// to the host generator paper_conf_ipps_davidsonzo11_b200/inputs.py (family
+// "dd" / "weak"), so a bench rank or the tuner draws its batch in HBM instead
+// of generating gigabytes on the host and copying them over PCIe.
+//
+//   h = splitmix64(seed ^ (array_id << 56) ^ global_row),
+//   global_row = (first_system + s) * n + i;
+//   fp32: u = top 24 bits of h, value (u - 2^23) 2^-23 (exact, in [-1, 1));
+//   fp64: u = top 53 bits,      value (u - 2^52) 2^-52;
+//   a, c, d from array ids 0, 2, 3; a_0 = c_{n-1} = 0;
+//   b = (|a| + |c|) + mu, both additions rounded to nearest in the target
+//   precision (no FMA: __fadd_rn / __dadd_rn).
+// No solver arithmetic here.
+#include "common.cuh"
+#include "pipe.cuh"
+
+namespace tds {
+
+__device__ __forceinline__ uint64_t splitmix64_dev(uint64_t z) {
+    z += 0x9E3779B97F4A7C15ull;
+    z = (z ^ (z >> 30)) * 0xBF58476D1CE4E5B9ull;
+    z = (z ^ (z >> 27)) * 0x94D049BB133111EBull;
+    return z ^ (z >> 31);
+}
+
+__device__ __forceinline__ float upm1(uint64_t h, float) {
+    const int64_t u = int64_t(h >> 40);                      // 24 bits
+    return float(double(u - (int64_t(1) << 23)) * 0x1p-23);  // exact
+}
+__device__ __forceinline__ double upm1(uint64_t h, double) {
+    const int64_t u = int64_t(h >> 11);  // 53 bits
+    return double(u - (int64_t(1) << 52)) * 0x1p-52;
+}
+__device__ __forceinline__ float add_rn(float x, float y) { return __fadd_rn(x, y); }
+__device__ __forceinline__ double add_rn(double x, double y) { return __dadd_rn(x, y); }
+
+template <typename T>
+__global__ void __launch_bounds__(256) generate_kernel(T *a, T *b, T *c, T *d, int64_t n, int64_t m, int64_t stride,
+                                                       uint64_t seed, int64_t first_system, T mu) {
+    const uint64_t ka = seed ^ (uint64_t(0) << 56), kc = seed ^ (uint64_t(2) << 56), kd = seed ^ (uint64_t(3) << 56);
+    const int64_t total = n * m;
+    for (int64_t e = blockIdx.x * int64_t(blockDim.x) + threadIdx.x; e < total;
+         e += int64_t(gridDim.x) * blockDim.x) {
+        const int64_t s = e / n, i = e - s * n;
+        const uint64_t row = uint64_t((first_system + s) * n + i);
+        const T va = i > 0 ? upm1(splitmix64_dev(row ^ ka), T(0)) : T(0);
+        const T vc = i < n - 1 ? upm1(splitmix64_dev(row ^ kc), T(0)) : T(0);
+        const T vd = upm1(splitmix64_dev(row ^ kd), T(0));
+        const int64_t o = s * stride + i;
+        a[o] = va;
+        c[o] = vc;
+        d[o] = vd;
+        b[o] = add_rn(add_rn(fabs(va), fabs(vc)), mu);
+    }
+}
+
+template <typename T>
+cudaError_t launch_generate(T *a, T *b, T *c, T *d, int64_t n, int64_t m, int64_t stride, uint64_t seed,
+                            int64_t first_system, double mu, cudaStream_t st) {
+    const int64_t total = n * m;
+    const int64_t blocks = std::min<int64_t>(int64_t(sm_count_current()) * 16, cdiv(total, 256));
+    generate_kernel<T><<<unsigned(std::max<int64_t>(blocks, 1)), 256, 0, st>>>(a, b, c, d, n, m, stride, seed,
+                                                                                first_system, T(mu));
+    return cudaGetLastError();
+}
+
+template cudaError_t launch_generate<float>(float *, float *, float *, float *, int64_t, int64_t, int64_t, uint64_t,
+                                            int64_t, double, cudaStream_t);
+template cudaError_t launch_generate<double>(double *, double *, double *, double *, int64_t, int64_t, int64_t,
+                                             uint64_t, int64_t, double, cudaStream_t);
+
+}  // namespace tds
+
+using namespace tds;
+
+extern "C" tds_status tds_generate(tds_dtype dtype, int64_t n, int64_t m, int64_t batch_stride, uint64_t seed,
+                                   int64_t first_system, double mu, void *a, void *b, void *c, void *d,
+                                   void *cuda_stream) {
+    if (dtype != TDS_F32 && dtype != TDS_F64) return fail(TDS_ERR_INVALID_ARG, "dtype");
+    if (n < 1 || m < 1 || first_system < 0) return fail(TDS_ERR_INVALID_ARG, "n, m >= 1 and first_system >= 0");
+    if (batch_stride == 0) batch_stride = n;
+    if (batch_stride < n) return fail(TDS_ERR_INVALID_ARG, "batch_stride < n");
+    const size_t es = size_t(dsize(dtype));
+    for (const void *p : {a, b, c, d}) {
+        if (!p) return fail(TDS_ERR_INVALID_ARG, "NULL array pointer");
+        if (reinterpret_cast<uintptr_t>(p) % es) return fail(TDS_ERR_INVALID_ARG, "array not aligned to sizeof(T)");
+    }
+    cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
+    const cudaError_t e =
+        dtype == TDS_F32
+            ? launch_generate<float>((float *)a, (float *)b, (float *)c, (float *)d, n, m, batch_stride, seed,
+                                     first_system, mu, st)
+            : launch_generate<double>((double *)a, (double *)b, (double *)c, (double *)d, n, m, batch_stride, seed,
+                                      first_system, mu, st);
+    if (e != cudaSuccess) return fail(TDS_ERR_CUDA, std::string("generate launch: ") + cudaGetErrorString(e));
+    clear_error();
+    return TDS_OK;
+}

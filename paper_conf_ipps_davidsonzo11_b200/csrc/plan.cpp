@@ -220,6 +220,7 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
         info.split_segments = 0;
         info.split_tile_eff = 0;
     }
+    info.onchip_form = p.split_only ? -1 : onchip_form_of(info);
     return TDS_OK;
 }
 

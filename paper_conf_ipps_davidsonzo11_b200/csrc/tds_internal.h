@@ -42,5 +42,7 @@ int32_t split_tile_eff(const tds_params &p, int pass);
 int64_t chunk_m(const tds_params &p, int64_t m);
 int32_t static_cluster(const tds_device_props &p);
 tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_params &p);
+// The on-chip form the dispatch selects (api.cu solve_impl) for 16-byte aligned arrays.
+int32_t onchip_form_of(const tds_plan_info &I);
 
 }  // namespace tds
