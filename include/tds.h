@@ -249,6 +249,48 @@ tds_status tds_split_batched(const tds_plan_t plan, const void *a, const void *b
                              const void *d, void *a_out, void *c_out, void *d_out,
                              void *workspace, size_t workspace_bytes, void *cuda_stream);
 
+/* Same solve for NORMALISED systems (b = 1, the form every split pass leaves,
+ * SURVEY.md §8(c)): a, c, d only, no b array is read.  a[0] and c[n-1] of
+ * each system multiply identity rows and are ignored (they must be finite).
+ * The plan needs k >= 1 and strided == 0 (the k = 0 on-chip kernels read b);
+ * else UNSUPPORTED.  Otherwise as tds_solve_batched.  Used by the one-huge-
+ * system path (dist.py solve_huge: the all-to-all delivers normalised residue
+ * systems, so no b' = 1 array is materialised). */
+tds_status tds_solve_normalized(const tds_plan_t plan, const void *a, const void *c, const void *d, void *x,
+                                void *workspace, size_t workspace_bytes, void *cuda_stream);
+
+/* Where the split passes leave the split system inside the workspace (host
+ * only).  Three arrays a', c', d' of NORMALISED rows (b' = 1) start at element
+ * offsets a_offset, c_offset, d_offset (elements of the plan's dtype from the
+ * workspace base); slot (s << k) + r (r < 2^k, s < m) holds residue class r of
+ * system s -- original rows r + 2^k j, j = 0 .. ceil((n - r) / 2^k) - 1 --
+ * contiguously from element slot * slot_rows (Fig. 3a; canonical
+ * order, R23).  UNSUPPORTED for k = 0, strided or chunked plans. */
+typedef struct {
+    int64_t a_offset, c_offset, d_offset;
+    int64_t slot_rows;   /* elements between consecutive slots (>= ceil(n / 2^k)) */
+    int64_t num_slots;   /* m * 2^k */
+} tds_slots_layout;
+tds_status tds_plan_slots_layout(const tds_plan_t plan, tds_slots_layout *out);
+
+/* Run only the plan's split passes (PAPER.md stages 1-2), leaving the split
+ * system in the workspace as tds_plan_slots_layout describes -- the zero-copy
+ * source of the one-huge-system all-to-all (each residue class's rows of a
+ * block are one contiguous run).  Split-only plans are accepted.  Same array,
+ * workspace and device rules as tds_solve_batched; enqueued on cuda_stream. */
+tds_status tds_split_slots(const tds_plan_t plan, const void *a, const void *b, const void *c, const void *d,
+                           void *workspace, size_t workspace_bytes, void *cuda_stream);
+
+/* The residue-class -> original-order transpose of Fig. 3a:
+ * x[s * batch_stride + r + 2^k j] = xs[((s << k) + r) * slot_rows + j] for
+ * every system s < m, residue r < 2^k and row r + 2^k j < n.  xs, x: device,
+ * dtype, must not overlap; xs is left intact.  The x placement kernel of the
+ * solve (TMA transposer); also the unpacking of the one-huge-system x
+ * return.  Errors: INVALID_ARG (k < 1, slot_rows < ceil(n/2^k), NULL,
+ * misaligned, overlap), CUDA.  Enqueued on cuda_stream. */
+tds_status tds_unpack_residues(tds_dtype dtype, int64_t n, int64_t m, int32_t k, int64_t slot_rows, const void *xs,
+                               void *x, int64_t batch_stride, void *cuda_stream);
+
 /* ---- batch-interleaved layout (ADI-style batches) ----- */
 
 /* Bytes of device workspace tds_solve_interleaved needs for `plan`: the
@@ -285,6 +327,14 @@ tds_status tds_solve_interleaved(const tds_plan_t plan, const void *a, const voi
  * misaligned pointer), CUDA (launch). */
 tds_status tds_generate(tds_dtype dtype, int64_t n, int64_t m, int64_t batch_stride, uint64_t seed,
                         int64_t first_system, double mu, void *a, void *b, void *c, void *d, void *cuda_stream);
+
+/* Rows [row0, row0 + count) of ONE system of n rows drawn by the same recipe
+ * (global_row = row; a_0 = c_{n-1} = 0), rows outside [0, n) as identity rows
+ * (a, b, c, d) = (0, 1, 0, 0): the halo-padded row block a rank of the
+ * one-huge-system path owns.  a, b, c, d: device, count elements each.
+ * Errors as tds_generate. */
+tds_status tds_generate_rows(tds_dtype dtype, int64_t n, int64_t row0, int64_t count, uint64_t seed, double mu,
+                             void *a, void *b, void *c, void *d, void *cuda_stream);
 
 /* ---- misc ---------------------------------------------------------------------- */
 

@@ -26,7 +26,8 @@ EXPORTED = (
     "tds_plan_set_params", "tds_plan_permutation", "tds_plan_destroy", "tds_tune",
     "tds_plan_tune_trials", "tds_solve_batched", "tds_solve_stages", "tds_split_batched", "tds_status_string",
     "tds_interleaved_workspace_bytes", "tds_solve_interleaved",
-    "tds_last_error", "tds_version", "tds_tune_search", "tds_generate",
+    "tds_last_error", "tds_version", "tds_tune_search", "tds_generate", "tds_generate_rows",
+    "tds_solve_normalized", "tds_plan_slots_layout", "tds_split_slots", "tds_unpack_residues",
 )
 
 
@@ -60,6 +61,11 @@ class PlanInfo(ctypes.Structure):
                 ("chunks", ctypes.c_int32), ("launches", ctypes.c_int32),
                 ("slot_rows", ctypes.c_int64), ("workspace_bytes", ctypes.c_size_t),
                 ("onchip_form", ctypes.c_int32)]
+
+
+class SlotsLayout(ctypes.Structure):
+    _fields_ = [("a_offset", ctypes.c_int64), ("c_offset", ctypes.c_int64), ("d_offset", ctypes.c_int64),
+                ("slot_rows", ctypes.c_int64), ("num_slots", ctypes.c_int64)]
 
 
 # tds_tune_search's cost callback: double (*)(const tds_params *, void *)
@@ -96,6 +102,11 @@ def load() -> ctypes.CDLL:
         "tds_solve_interleaved": (I32, [P, VP, VP, VP, VP, VP, VP, SZ, VP]),
         "tds_tune_search": (I32, [P, COST_FN, VP, ctypes.c_char_p]),
         "tds_generate": (I32, [I32, I64, I64, I64, ctypes.c_uint64, I64, ctypes.c_double, VP, VP, VP, VP, VP]),
+        "tds_generate_rows": (I32, [I32, I64, I64, I64, ctypes.c_uint64, ctypes.c_double, VP, VP, VP, VP, VP]),
+        "tds_solve_normalized": (I32, [P, VP, VP, VP, VP, VP, SZ, VP]),
+        "tds_plan_slots_layout": (I32, [P, ctypes.POINTER(SlotsLayout)]),
+        "tds_split_slots": (I32, [P, VP, VP, VP, VP, VP, SZ, VP]),
+        "tds_unpack_residues": (I32, [I32, I64, I64, I32, I64, VP, VP, I64, VP]),
         "tds_status_string": (ctypes.c_char_p, [I32]),
         "tds_last_error": (ctypes.c_char_p, []),
         "tds_version": (I32, []),

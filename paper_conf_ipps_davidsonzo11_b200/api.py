@@ -179,6 +179,13 @@ class Plan:
         L.check(self._lib.tds_interleaved_workspace_bytes(self._h, ctypes.byref(v)))
         return int(v.value)
 
+    def slots_layout(self) -> dict:
+        """tds_plan_slots_layout: where tds_split_slots leaves the split system
+        in the workspace (element offsets of a', c', d', slot_rows, num_slots)."""
+        lay = L.SlotsLayout()
+        L.check(self._lib.tds_plan_slots_layout(self._h, ctypes.byref(lay)))
+        return {f: int(getattr(lay, f)) for f, _ in L.SlotsLayout._fields_}
+
     def workspace(self):
         import torch
         nbytes = self.workspace_bytes
@@ -227,6 +234,78 @@ def solve_batched(plan: Plan, a, b, c, d, out=None, workspace=None, stream=None)
     wbytes = workspace.numel() * workspace.element_size() if workspace is not None else 0
     L.check(plan._lib.tds_solve_batched(plan.handle, a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
                                         out.data_ptr(), wptr, wbytes, _stream_ptr(stream, dev)))
+    return out
+
+
+def solve_normalized(plan: Plan, a, c, d, out=None, workspace=None, stream=None):
+    """tds_solve_normalized: the same solve for normalised systems (b = 1; no
+    b array).  The plan needs k >= 1.  Returns x."""
+    import torch
+    info, need, want, dev = plan._solve_info()
+    for name, t in (("a", a), ("c", c), ("d", d)):
+        _check_fast(t, need, want, name)
+    if out is None:
+        out = torch.empty_like(d)
+    else:
+        _check_fast(out, need, want, "out")
+    if workspace is None and info.workspace_bytes > 0:
+        workspace = plan.workspace()
+    wptr = workspace.data_ptr() if workspace is not None else None
+    wbytes = workspace.numel() * workspace.element_size() if workspace is not None else 0
+    L.check(plan._lib.tds_solve_normalized(plan.handle, a.data_ptr(), c.data_ptr(), d.data_ptr(), out.data_ptr(),
+                                           wptr, wbytes, _stream_ptr(stream, dev)))
+    return out
+
+
+def split_slots(plan: Plan, a, b, c, d, workspace, stream=None):
+    """tds_split_slots: run the split passes only; returns (a', c', d') as
+    (num_slots, slot_rows) views into ``workspace`` (slot (s << k) + r = residue
+    r of system s, normalised rows, Fig. 3a order)."""
+    info, need, want, dev = plan._solve_info()
+    for name, t in (("a", a), ("b", b), ("c", c), ("d", d)):
+        _check_fast(t, need, want, name)
+    lay = plan.slots_layout()
+    wbytes = workspace.numel() * workspace.element_size()
+    L.check(plan._lib.tds_split_slots(plan.handle, a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
+                                      workspace.data_ptr(), wbytes, _stream_ptr(stream, dev)))
+    return slot_views(plan, workspace, lay)
+
+
+def slot_views(plan: Plan, workspace, lay: Optional[dict] = None):
+    """(a', c', d') views of the split slots inside ``workspace`` (no device work)."""
+    info, _, want, _ = plan._solve_info()
+    lay = lay or plan.slots_layout()
+    typed = workspace.view(want)
+    size = lay["num_slots"] * lay["slot_rows"]
+    return tuple(typed[lay[k]:lay[k] + size].view(lay["num_slots"], lay["slot_rows"])
+                 for k in ("a_offset", "c_offset", "d_offset"))
+
+
+def unpack_residues(xs, x, n: int, m: int, k: int, slot_rows: int, batch_stride: int = 0, stream=None):
+    """tds_unpack_residues: x[s*stride + r + 2^k j] = xs[((s << k) + r) * slot_rows + j]."""
+    want = xs.dtype
+    _check_fast(xs, (m << k) * slot_rows, want, "xs")
+    stride = int(batch_stride) or int(n)
+    _check_fast(x, (m - 1) * stride + n, want, "x")
+    L.check(L.load().tds_unpack_residues(_dtype_code(want), int(n), int(m), int(k), int(slot_rows), xs.data_ptr(),
+                                         x.data_ptr(), stride, _stream_ptr(stream, int(x.device.index))))
+    return x
+
+
+def generate_rows(n: int, row0: int, count: int, dtype="float32", seed: int = 1, mu: float = 1.0, device: int = 0,
+                  out=None, stream=None):
+    """tds_generate_rows: rows [row0, row0 + count) of one seeded system of n
+    rows (identity rows outside [0, n)).  Returns (a, b, c, d), each (count,)."""
+    import torch
+    code = _dtype_code(dtype)
+    tdt = torch.float32 if code == L.TDS_F32 else torch.float64
+    if out is None:
+        out = tuple(torch.empty(int(count), dtype=tdt, device=f"cuda:{device}") for _ in range(4))
+    for name, t in zip("abcd", out):
+        _check_fast(t, int(count), tdt, name)
+    L.check(L.load().tds_generate_rows(code, int(n), int(row0), int(count), int(seed) & 0xFFFFFFFFFFFFFFFF,
+                                       float(mu), *(t.data_ptr() for t in out),
+                                       _stream_ptr(stream, int(out[0].device.index))))
     return out
 
 

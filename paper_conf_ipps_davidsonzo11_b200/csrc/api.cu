@@ -87,8 +87,8 @@ static tds_status run_split(const tds_plan_info &I, const T *a, const T *b, cons
             continue;
         }
         SplitArgs<T> A{};
-        const bool raw = (p == 0);
-        if (raw) {
+        const bool raw = (p == 0 && b != nullptr);  // b == nullptr: normalised input (b = 1, tds_solve_normalized)
+        if (p == 0) {
             A.a = a;
             A.b = b;
             A.c = c;
@@ -117,7 +117,7 @@ static tds_status run_split(const tds_plan_info &I, const T *a, const T *b, cons
         A.segs = split_segments(m_in, cdiv(len_in, split_tile_eff(P, p)), P.theta);
         const int64_t e = P.split_tile_rows + 2 * ((int64_t(1) << kp) - 1);
         A.ep = int32_t(e + (e >> std::max(kp, 5)) + 1);
-        A.vec = raw ? vec_ok(I, {a, b, c, d}) : 1;
+        A.vec = p == 0 ? (raw ? vec_ok(I, {a, b, c, d}) : vec_ok(I, {a, c, d})) : 1;
         if (natural) {  // strided variant: one pass, rows kept in original order (per system stride)
             A.natural = 1;
             A.out_slot = round_up(I.n, 16 / int64_t(sizeof(T)));
@@ -241,7 +241,7 @@ __global__ void gather_canonical_kernel(const T *sa, const T *sc, const T *sd, T
                                         int32_t K, int64_t slot, PassGeom geom) {
     const int64_t sigma = blockIdx.x;
     const int64_t sys = sigma >> K;
-    const int64_t r = slot_residue(sigma & ((int64_t(1) << K) - 1), geom.npass, geom.kpass);
+    const int64_t r = sigma & ((int64_t(1) << K) - 1);
     if (r >= n) return;
     const int64_t L = (n - r + (int64_t(1) << K) - 1) >> K;
     const int64_t q = n >> K, rem = n & ((int64_t(1) << K) - 1);
@@ -436,6 +436,117 @@ tds_status tds_split_batched(const tds_plan_t plan, const void *a, const void *b
                                    st);
     if (s == TDS_OK) clear_error();
     return s;
+}
+
+static tds_status check_solve_args(const tds_plan_info &I, const void *a, const void *b, const void *c,
+                                   const void *d, void *x, void *workspace, size_t workspace_bytes) {
+    tds_status s = b ? check_arrays(I, {a, b, c, d, x}) : check_arrays(I, {a, c, d, x});
+    if (s != TDS_OK) return s;
+    const size_t bytes = size_t(((I.m - 1) * I.batch_stride + I.n) * dsize(I.dtype));
+    for (const void *p : {a, b, c})
+        if (p && overlaps(x, bytes, p, bytes)) return fail(TDS_ERR_INVALID_ARG, "x overlaps a, b or c");
+    if (x != d && overlaps(x, bytes, d, bytes))
+        return fail(TDS_ERR_INVALID_ARG, "x partially overlaps d (only x == d is allowed)");
+    if ((s = check_workspace(I, workspace, workspace_bytes)) != TDS_OK) return s;
+    if (workspace && I.workspace_bytes)
+        for (const void *p : {a, b, c, d, (const void *)x})
+            if (p && overlaps(workspace, I.workspace_bytes, p, bytes))
+                return fail(TDS_ERR_INVALID_ARG, "workspace overlaps an array");
+    return TDS_OK;
+}
+
+tds_status tds_solve_normalized(const tds_plan_t plan, const void *a, const void *c, const void *d, void *x,
+                                void *workspace, size_t workspace_bytes, void *cuda_stream) {
+    if (!plan) return fail(TDS_ERR_INVALID_ARG, "plan is NULL");
+    const tds_plan_info &I = plan->info;
+    if (I.params.split_only) return fail(TDS_ERR_UNSUPPORTED, "split-only plan");
+    if (I.params.k < 1 || I.params.strided)
+        return fail(TDS_ERR_UNSUPPORTED, "normalised input needs a plan with k >= 1 split levels and strided = 0");
+    tds_status s = check_solve_args(I, a, nullptr, c, d, x, workspace, workspace_bytes);
+    if (s != TDS_OK) return s;
+    if ((s = check_device(plan)) != TDS_OK) return s;
+    cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
+    s = I.dtype == TDS_F32
+            ? solve_chunks<float>(I, (const float *)a, nullptr, (const float *)c, (const float *)d, (float *)x,
+                                  workspace, st, 0, I.launches - 1)
+            : solve_chunks<double>(I, (const double *)a, nullptr, (const double *)c, (const double *)d, (double *)x,
+                                   workspace, st, 0, I.launches - 1);
+    if (s == TDS_OK) clear_error();
+    return s;
+}
+
+tds_status tds_plan_slots_layout(const tds_plan_t plan, tds_slots_layout *out) {
+    if (!plan || !out) return fail(TDS_ERR_INVALID_ARG, "NULL argument");
+    const tds_plan_info &I = plan->info;
+    if (I.params.k < 1 || I.params.strided) return fail(TDS_ERR_UNSUPPORTED, "slots need k >= 1 and strided = 0");
+    if (I.chunks != 1) return fail(TDS_ERR_UNSUPPORTED, "slots of a chunked plan are reused per chunk");
+    const int nbuf = I.params.passes >= 2 ? 2 : 1;
+    const int64_t E = int64_t(I.workspace_bytes / (size_t(nbuf) * 3 * size_t(dsize(I.dtype))));
+    const int ob = (I.params.passes - 1) & 1;
+    out->a_offset = (3 * ob + 0) * E;
+    out->c_offset = (3 * ob + 1) * E;
+    out->d_offset = (3 * ob + 2) * E;
+    out->slot_rows = I.slot_rows;
+    out->num_slots = I.m << I.params.k;
+    return TDS_OK;
+}
+
+tds_status tds_split_slots(const tds_plan_t plan, const void *a, const void *b, const void *c, const void *d,
+                           void *workspace, size_t workspace_bytes, void *cuda_stream) {
+    tds_slots_layout L;
+    tds_status s = tds_plan_slots_layout(plan, &L);
+    if (s != TDS_OK) return s;
+    const tds_plan_info &I = plan->info;
+    if ((s = check_arrays(I, {a, b, c, d})) != TDS_OK) return s;
+    if ((s = check_workspace(I, workspace, workspace_bytes)) != TDS_OK) return s;
+    const size_t bytes = size_t(((I.m - 1) * I.batch_stride + I.n) * dsize(I.dtype));
+    for (const void *p : {a, b, c, d})
+        if (overlaps(workspace, I.workspace_bytes, p, bytes)) return fail(TDS_ERR_INVALID_ARG, "workspace overlaps an array");
+    if ((s = check_device(plan)) != TDS_OK) return s;
+    cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
+    int ob = 0;
+    if (I.dtype == TDS_F32) {
+        WsBufs<float> w = ws_bufs<float>(I, workspace);
+        s = run_split<float>(I, (const float *)a, (const float *)b, (const float *)c, (const float *)d, w, st, &ob);
+    } else {
+        WsBufs<double> w = ws_bufs<double>(I, workspace);
+        s = run_split<double>(I, (const double *)a, (const double *)b, (const double *)c, (const double *)d, w, st,
+                              &ob);
+    }
+    if (s == TDS_OK) clear_error();
+    return s;
+}
+
+tds_status tds_unpack_residues(tds_dtype dtype, int64_t n, int64_t m, int32_t k, int64_t slot_rows, const void *xs,
+                               void *x, int64_t batch_stride, void *cuda_stream) {
+    if (dtype != TDS_F32 && dtype != TDS_F64) return fail(TDS_ERR_INVALID_ARG, "dtype");
+    if (n < 1 || m < 1 || k < 1 || k > 30) return fail(TDS_ERR_INVALID_ARG, "n, m >= 1 and 1 <= k <= 30");
+    if (batch_stride == 0) batch_stride = n;
+    if (batch_stride < n) return fail(TDS_ERR_INVALID_ARG, "batch_stride < n");
+    const int64_t es = dsize(dtype);
+    if (slot_rows < cdiv(n, int64_t(1) << k)) return fail(TDS_ERR_INVALID_ARG, "slot_rows < ceil(n / 2^k)");
+    if (!xs || !x || reinterpret_cast<uintptr_t>(xs) % es || reinterpret_cast<uintptr_t>(x) % es)
+        return fail(TDS_ERR_INVALID_ARG, "NULL or misaligned array");
+    const size_t xb = size_t(((m - 1) * batch_stride + n) * es), sb = size_t((m << k) * slot_rows * es);
+    if (overlaps(xs, sb, x, xb)) return fail(TDS_ERR_INVALID_ARG, "x overlaps xs");
+    PassGeom g{};
+    g.npass = 1;
+    g.kpass[0] = k;
+    cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
+    tds_plan_info I{};
+    I.dtype = dtype;
+    I.batch_stride = batch_stride;
+    const int vec = vec_ok(I, {x});
+    // place_x's TMA transposer needs whole 16-byte slot rows
+    const int64_t vslot = (slot_rows * es) % 16 == 0 && reinterpret_cast<uintptr_t>(xs) % 16 == 0 ? vec : 0;
+    const cudaError_t e = dtype == TDS_F32
+                              ? launch_place_x<float>((const float *)xs, (float *)x, n, m, batch_stride, slot_rows, k,
+                                                      int(vslot), g, st, false)
+                              : launch_place_x<double>((const double *)xs, (double *)x, n, m, batch_stride, slot_rows,
+                                                       k, int(vslot), g, st, false);
+    if (e != cudaSuccess) return cuda_fail(e, "unpack launch");
+    clear_error();
+    return TDS_OK;
 }
 
 tds_status tds_interleaved_workspace_bytes(const tds_plan_t plan, size_t *bytes) {

@@ -103,10 +103,6 @@ __device__ __forceinline__ void row_update2(float2 &a, float2 &c, float2 &d, flo
 // levels, slot (s << K) + r holds the residue-r subsystem of system s.  Each
 // pass writes the new residue digit rho of input slot sigma (levels kprev
 // before it, kp in it) to residue r + (rho << kprev).
-__device__ __forceinline__ int64_t slot_residue(int64_t rho, int /*npass*/, const int32_t * /*kpass*/) {
-    return rho;
-}
-
 __device__ __forceinline__ int64_t out_slot_index(int64_t sigma, int kprev, int kp, int64_t rho) {
     const int64_t sys = sigma >> kprev, r = sigma & ((int64_t(1) << kprev) - 1);
     return (sys << (kprev + kp)) + r + (rho << kprev);
@@ -221,7 +217,7 @@ inline bool onchip_cpipe_ok(const tds_plan_info &I) {
 
 template <typename T>
 cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batch_stride, int64_t slot, int K,
-                           int vec, const PassGeom &geom, cudaStream_t st);
+                           int vec, const PassGeom &geom, cudaStream_t st, bool xs_scratch = true);
 template <typename T>
 cudaError_t launch_onchip(const OnchipArgs<T> &A, int cr_levels, bool raw, int64_t grid, int threads,
                           size_t smem, cudaStream_t st);

@@ -55,6 +55,32 @@ __global__ void __launch_bounds__(256) generate_kernel(T *a, T *b, T *c, T *d, i
     }
 }
 
+// Rows [row0, row0 + count) of ONE system of n rows (global_row = row); rows
+// outside [0, n) are identity rows (0, 1, 0, 0) -- a rank's halo-padded block
+// of a system split over several GPUs (dist.py solve_huge).
+template <typename T>
+__global__ void __launch_bounds__(256) generate_rows_kernel(T *a, T *b, T *c, T *d, int64_t n, int64_t row0,
+                                                            int64_t count, uint64_t seed, T mu) {
+    const uint64_t ka = seed ^ (uint64_t(0) << 56), kc = seed ^ (uint64_t(2) << 56), kd = seed ^ (uint64_t(3) << 56);
+    for (int64_t e = blockIdx.x * int64_t(blockDim.x) + threadIdx.x; e < count; e += int64_t(gridDim.x) * blockDim.x) {
+        const int64_t i = row0 + e;
+        if (i < 0 || i >= n) {
+            a[e] = T(0);
+            b[e] = T(1);
+            c[e] = T(0);
+            d[e] = T(0);
+            continue;
+        }
+        const uint64_t row = uint64_t(i);
+        const T va = i > 0 ? upm1(splitmix64_dev(row ^ ka), T(0)) : T(0);
+        const T vc = i < n - 1 ? upm1(splitmix64_dev(row ^ kc), T(0)) : T(0);
+        a[e] = va;
+        c[e] = vc;
+        d[e] = upm1(splitmix64_dev(row ^ kd), T(0));
+        b[e] = add_rn(add_rn(fabs(va), fabs(vc)), mu);
+    }
+}
+
 template <typename T>
 cudaError_t launch_generate(T *a, T *b, T *c, T *d, int64_t n, int64_t m, int64_t stride, uint64_t seed,
                             int64_t first_system, double mu, cudaStream_t st) {
@@ -73,6 +99,29 @@ template cudaError_t launch_generate<double>(double *, double *, double *, doubl
 }  // namespace tds
 
 using namespace tds;
+
+extern "C" tds_status tds_generate_rows(tds_dtype dtype, int64_t n, int64_t row0, int64_t count, uint64_t seed,
+                                        double mu, void *a, void *b, void *c, void *d, void *cuda_stream) {
+    if (dtype != TDS_F32 && dtype != TDS_F64) return fail(TDS_ERR_INVALID_ARG, "dtype");
+    if (n < 1 || count < 1) return fail(TDS_ERR_INVALID_ARG, "n, count >= 1");
+    const size_t es = size_t(dsize(dtype));
+    for (const void *p : {a, b, c, d}) {
+        if (!p) return fail(TDS_ERR_INVALID_ARG, "NULL array pointer");
+        if (reinterpret_cast<uintptr_t>(p) % es) return fail(TDS_ERR_INVALID_ARG, "array not aligned to sizeof(T)");
+    }
+    cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
+    const int64_t blocks = std::max<int64_t>(1, std::min<int64_t>(int64_t(sm_count_current()) * 16, cdiv(count, 256)));
+    if (dtype == TDS_F32)
+        generate_rows_kernel<float><<<unsigned(blocks), 256, 0, st>>>((float *)a, (float *)b, (float *)c, (float *)d, n,
+                                                                      row0, count, seed, float(mu));
+    else
+        generate_rows_kernel<double><<<unsigned(blocks), 256, 0, st>>>((double *)a, (double *)b, (double *)c,
+                                                                       (double *)d, n, row0, count, seed, mu);
+    const cudaError_t e = cudaGetLastError();
+    if (e != cudaSuccess) return fail(TDS_ERR_CUDA, std::string("generate launch: ") + cudaGetErrorString(e));
+    clear_error();
+    return TDS_OK;
+}
 
 extern "C" tds_status tds_generate(tds_dtype dtype, int64_t n, int64_t m, int64_t batch_stride, uint64_t seed,
                                    int64_t first_system, double mu, void *a, void *b, void *c, void *d,

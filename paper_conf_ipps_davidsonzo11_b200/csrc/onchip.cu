@@ -164,7 +164,7 @@ __global__ void __launch_bounds__(R * sizeof(T) >= 64 ? 512 : 1024) onchip_kerne
         in_base = sys * A.batch_stride;
     } else {
         sys = sigma >> A.K;
-        r = slot_residue(sigma & ((int64_t(1) << A.K) - 1), A.geom.npass, A.geom.kpass);
+        r = sigma & ((int64_t(1) << A.K) - 1);
         if (r >= A.n) return;  // empty slot (2^K > n): uniform across the cluster
         L = (A.n - r + (int64_t(1) << A.K) - 1) >> A.K;
         in_base = sigma * A.slot;

@@ -202,7 +202,7 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
     const int64_t KK = int64_t(1) << A.K;
 
     auto slot_len = [&](int64_t sigma) -> int64_t {
-        const int64_t r = slot_residue(sigma & (KK - 1), A.geom.npass, A.geom.kpass);
+        const int64_t r = sigma & (KK - 1);
         return r < A.n ? (A.n - r + KK - 1) >> A.K : 0;
     };
     const int64_t tma_rows = int64_t(tma_lines) * ELINE;  // rows of every slot in whole TMA lines

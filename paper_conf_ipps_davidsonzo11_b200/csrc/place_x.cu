@@ -278,7 +278,7 @@ __global__ void __launch_bounds__(kTpThreads) place_x_tma_kernel(const PlaceArgs
 
 template <typename T>
 cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batch_stride, int64_t slot, int K,
-                           int vec, const PassGeom &geom, cudaStream_t st) {
+                           int vec, const PassGeom &geom, cudaStream_t st, bool xs_scratch) {
     PlaceArgs<T> A{};
     A.xs = xs;
     A.x = x;
@@ -314,7 +314,7 @@ cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batc
             const int64_t grid =
                 std::max<int64_t>(1, std::min<int64_t>(ntiles, int64_t(std::max(occ, 1)) * sm_count_current()));
             // x slots are scratch whose last reader is this kernel: drop their lines from L2 once loaded
-            const int32_t disc = (slot * int64_t(sizeof(T))) % 128 == 0 && uintptr_t(xs) % 128 == 0;
+            const int32_t disc = xs_scratch && (slot * int64_t(sizeof(T))) % 128 == 0 && uintptr_t(xs) % 128 == 0;
             e = launch_pdl(kern, dim3(unsigned(grid)), dim3(kTpThreads), smem, st, 1, A, tm, ntiles, jtiles, lfull, m,
                            disc);
             if (e != cudaSuccess) return e;
@@ -342,8 +342,8 @@ cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batc
 }
 
 template cudaError_t launch_place_x<float>(const float *, float *, int64_t, int64_t, int64_t, int64_t, int, int,
-                                           const PassGeom &, cudaStream_t);
+                                           const PassGeom &, cudaStream_t, bool);
 template cudaError_t launch_place_x<double>(const double *, double *, int64_t, int64_t, int64_t, int64_t, int, int,
-                                            const PassGeom &, cudaStream_t);
+                                            const PassGeom &, cudaStream_t, bool);
 
 }  // namespace tds

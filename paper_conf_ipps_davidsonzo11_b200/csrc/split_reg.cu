@@ -39,7 +39,7 @@ __global__ void __launch_bounds__(kRegSplitThreads, 2) split_reg_kernel(const Sp
         L = A.n;
     } else {
         const int64_t rho = sigma & ((int64_t(1) << kprev) - 1);
-        const int64_t r = slot_residue(rho, A.geom.npass, A.geom.kpass);
+        const int64_t r = rho;
         L = r < A.n ? (A.n - r + (int64_t(1) << kprev) - 1) >> kprev : 0;
     }
     const int64_t in_base = sigma * A.in_stride;

@@ -6,30 +6,48 @@ Two decompositions:
   P:L503-505): each rank solves a contiguous block of systems with the same
   integer plan; no data-path collective (``shard_range``, ``broadcast_plan``).
 
-* **One huge system** split by contiguous row blocks (``solve_huge``).  Rank g
-  owns rows [g*B, (g+1)*B).  After k_d PCR levels every residue class mod
-  2^k_d is an independent tridiagonal system (Fig. 3a), but each
-  class still spans every rank's rows, so a halo exchange alone cannot
-  decouple the ranks (SURVEY.md §0 point 2).  The steps:
+* **One huge system** split by contiguous row blocks (``HugeRank`` /
+  ``solve_huge``) -- the paper's Stage 1, several processors cooperating on one
+  system, lifted to several GPUs.  Rank g owns rows [g B, (g+1) B)
+  inside a halo-padded block ``ext`` of E = B + 2H rows (global rows
+  g B - H .. g B + B + H; identity rows (0, 1, 0, 0) outside [0, n)).  After
+  k_d PCR levels every residue class mod 2^k_d is an independent system
+  (Fig. 3a), but each class still spans every rank's rows, so a
+  halo exchange alone cannot decouple the ranks (SURVEY.md §0 point 2):
 
-  1. halo exchange: H = 2^k_d boundary rows of a, b, c, d with rank g-1 and
-     g+1 (point-to-point; ranks 0 and G-1 pad with identity rows);
-  2. local split: k_d fused PCR levels over the extended block of B + 2H rows
-     (``tds_split_batched`` on a split-only plan); rows [H, H+B) are exact;
-  3. all-to-all: residue classes [h*q, (h+1)*q) (q = 2^k_d / G) go to rank h,
-     each rank contributing its B / 2^k_d rows of every class;
-  4. local solve of the q owned classes (normalised, b' = 1), each a system of
-     n / 2^k_d rows (``tds_solve_batched``: more split passes + on-chip);
-  5. all-to-all of x back and placement into the local rows.
+  1. halo exchange: H rows of a, b, c, d with ranks g-1 and g+1, received
+     straight into ext's padding (point-to-point, no copy);
+  2. local split: k_d fused PCR levels over ext (``tds_split_slots``): the
+     split system stays in the workspace, residue r of the block in slot r,
+     rows [H, H + B) of ext exact (H >= 2^k_d - 1);
+  3. all-to-all: residue classes [h q, (h+1) q) (q = 2^k_d / G) go to rank h.
+     Every (array, residue) run of the block is ONE contiguous slot segment, so
+     the sends read the split's slots in place and the receives land in place
+     in the destination's residue systems -- no pack / unpack copies (only the
+     rank's own 1/G share is copied locally);
+  4. local solve of the q owned residue systems (normalised, b' = 1:
+     ``tds_solve_normalized``, no b array), in ``chunks`` groups of residues:
+     group c is solved while group c+1 is still arriving (SURVEY §7 H6);
+  5. x return: the solve's x runs go back to their owners (again contiguous
+     segments on both sides), then ONE residue->row transpose
+     (``tds_unpack_residues``, the placement kernel) writes x in row order.
 
-The local compute is injectable (``split_fn``, ``solve_fn``) so the index
-arithmetic and the collectives can be exercised on CPU with gloo against the
-oracle; the defaults run libtds on the rank's GPU.
+  With G = 1 there is nothing to exchange: the residue systems are read in
+  place from the split's slots (a slot view with batch_stride = slot_rows).
+
+The communication is a generator protocol: ``huge_steps`` yields at every
+exchange, so the same code runs over torch.distributed point-to-point ops
+(``P2PTransport``: NCCL on GPUs, gloo on CPU) or over the G ranks of a
+single-GPU loopback world (``solve_huge_loopback``: every rank's buffers and
+kernels on one device, messages as device copies) -- the full multi-rank data
+path exercised with the real kernels on one GPU.  The local compute is a
+backend object (``CudaBackend`` runs libtds; the gloo tests plug in the CPU
+oracle).
 """
 from __future__ import annotations
 
 import math
-from typing import Callable, Optional, Sequence, Tuple
+from typing import List, Optional, Sequence, Tuple
 
 import torch
 import torch.distributed as dist
@@ -66,109 +84,302 @@ def solve_sharded(a, b, c, d, mode: str = "static", plan: Optional[api.Plan] = N
 
 # ------------------------------------------------------------------ one huge system
 
-def _gpu_split(a, b, c, d, kd: int):
-    """k_d PCR levels over (1, E) arrays on the GPU; canonical order, b' = 1."""
-    E = d.shape[-1]
-    plan = api.Plan(E, 1, str(d.dtype).replace("torch.", ""), device=d.device.index or 0, mode="static")
-    plan.set_params(k_pass=_schedule(kd), split_only=1, cluster=1, tl_levels=0)
-    return api.split_batched(plan, a.reshape(1, E), b.reshape(1, E), c.reshape(1, E), d.reshape(1, E))
-
-
-def _gpu_solve(a, b, c, d):
-    m, n = d.shape
-    plan = api.Plan(n, m, str(d.dtype).replace("torch.", ""), device=d.device.index or 0, mode="static")
-    return api.solve_batched(plan, a.contiguous(), b.contiguous(), c.contiguous(), d.contiguous())
-
-
-def _schedule(k: int, kpmax: int = 4) -> list:
-    P = -(-k // kpmax)
-    return [k // P + (1 if i < k % P else 0) for i in range(P)]
-
-
 def huge_kd(world: int, kd: Optional[int] = None) -> int:
     """Levels split before the exchange: at least log2(world) so every rank owns a class."""
     base = max(1, int(math.ceil(math.log2(world)))) if world > 1 else 1
     return max(base, kd or 0)
 
 
-def solve_huge(a_loc, b_loc, c_loc, d_loc, n: int, group=None, kd: Optional[int] = None,
-               split_fn: Callable = _gpu_split, solve_fn: Callable = _gpu_solve):
-    """Solve one system of n rows whose row block [g*B, (g+1)*B) lives on rank g.
+def huge_halo(kd: int, itemsize: int) -> int:
+    """Halo rows per side: >= 2^k_d - 1 (exactness of k_d fused levels), a
+    multiple of 2^k_d (residues of ext rows = residues of global rows) and of
+    16 bytes per residue (the G = 1 slot views stay 16-byte aligned)."""
+    return (1 << kd) * max(1, 16 // itemsize)
 
-    a_loc .. d_loc: 1-D tensors of B = n / G rows (the rank's block; a_0 and
-    c_{n-1} of the global system are ignored).  Returns x for the local rows.
-    Requirements: G a power of two, B a multiple of 2^k_d.
-    """
+
+def _schedule(k: int, kpmax: int = 8) -> list:
+    P = -(-k // kpmax)
+    return [k // P + (1 if i < k % P else 0) for i in range(P)]
+
+
+class CudaBackend:
+    """libtds on this rank's GPU: split to slots, normalised solves, x unpack."""
+
+    def __init__(self, dtype: torch.dtype, device, mode: str = "static"):
+        self.dtype, self.device, self.mode = dtype, torch.device(device), mode
+        self.name = str(dtype).replace("torch.", "")
+
+    def empty(self, *shape):
+        return torch.empty(*shape, dtype=self.dtype, device=self.device)
+
+    def make_split(self, E: int, kd: int):
+        plan = api.Plan(E, 1, self.name, device=self.device.index or 0, mode="static")
+        plan.set_params(k_pass=_schedule(kd), split_only=1, cluster=1, tl_levels=0)
+        ws = plan.workspace()
+        return plan, ws, api.slot_views(plan, ws)
+
+    def split(self, state, ext):
+        plan, ws, _ = state
+        api.split_slots(plan, ext[0], ext[1], ext[2], ext[3], ws)
+
+    def make_solve(self, NL: int, m: int, stride: int):
+        plan = api.Plan(NL, m, self.name, device=self.device.index or 0, mode="static", batch_stride=stride)
+        return plan, plan.workspace()
+
+    def solve(self, state, a, c, d, x):
+        plan, ws = state
+        api.solve_normalized(plan, a, c, d, out=x, workspace=ws)
+
+    def unpack(self, xs, out, B: int, kd: int, slot_rows: int):
+        api.unpack_residues(xs, out, B, 1, kd, slot_rows)
+
+
+class HugeRank:
+    """One rank's buffers, plans and message lists for ``huge_steps`` (all
+    allocated once; a solve only enqueues kernels and exchanges)."""
+
+    def __init__(self, n: int, G: int, g: int, backend, kd: Optional[int] = None, chunks: int = 1):
+        itemsize = torch.empty((), dtype=backend.dtype).element_size()
+        self.n, self.G, self.g, self.be = n, G, g, backend
+        self.kd = kd = huge_kd(G, kd)
+        self.NR = NR = 1 << kd
+        self.B = B = n // G
+        if G & (G - 1) or B * G != n or B % NR or NR % G:
+            raise ValueError(f"solve_huge: need G a power of two, n = G B, B % 2^kd == 0, 2^kd % G == 0 "
+                             f"(G={G}, n={n}, kd={kd})")
+        self.q = q = NR // G                     # residue classes (local systems) per rank
+        if q % chunks:
+            raise ValueError(f"chunks ({chunks}) must divide the {q} residue systems per rank")
+        self.chunks = chunks
+        self.H = H = huge_halo(kd, itemsize)
+        self.E = E = B + 2 * H
+        self.Bj = Bj = B // NR                   # rows of one residue class inside the block
+        self.NL = NL = n // NR                   # rows of one residue system
+        self.off = H // NR                       # first valid position of each slot
+        self.ext = backend.empty(4, E)           # a, b, c, d of global rows gB - H .. gB + B + H
+        self.ext.zero_()
+        self.ext[1].fill_(1)                     # identity rows until the halo arrives (stay at the ends)
+        self.split_state = backend.make_split(E, kd)
+        self.slots = self.split_state[2]         # (a', c', d') as (NR, stride) views
+        self.stride = self.slots[0].shape[1]
+        qc = q // chunks
+        if G == 1:
+            # the residue systems are read in place from the slots (batch_stride = slot stride)
+            flat = [v.reshape(-1) for v in self.slots]
+            self.sys = None
+            span = (qc - 1) * self.stride + NL
+            self.chunk_in = [tuple(f[self.off + c * qc * self.stride:][:span] for f in flat) for c in range(chunks)]
+            self.solve_states = [backend.make_solve(NL, qc, self.stride) for _ in range(chunks)]
+        else:
+            self.sys = [backend.empty(q, NL) for _ in range(3)]
+            self.chunk_in = [tuple(v[c * qc:(c + 1) * qc] for v in self.sys) for c in range(chunks)]
+            self.solve_states = [backend.make_solve(NL, qc, NL) for _ in range(chunks)]
+        self.xs = backend.empty(q, NL)            # x of the local residue systems
+        self.chunk_x = [self.xs[c * qc:(c + 1) * qc] for c in range(chunks)]
+        self.xrecv = self.xs if G == 1 else backend.empty(NR, Bj)
+
+    @property
+    def local(self):
+        """(a, b, c, d) views of the rank's own rows (fill them before solving)."""
+        return tuple(self.ext[t, self.H:self.H + self.B] for t in range(4))
+
+    # -------- message lists: (peer, tensor) in the order both sides post them
+    def halo_messages(self):
+        H, B, E, g = self.H, self.B, self.E, self.g
+        sends, recvs = [], []
+        if g > 0:
+            sends += [(g - 1, self.ext[t, H:2 * H]) for t in range(4)]
+            recvs += [(g - 1, self.ext[t, 0:H]) for t in range(4)]
+        if g < self.G - 1:
+            sends += [(g + 1, self.ext[t, B:B + H]) for t in range(4)]
+            recvs += [(g + 1, self.ext[t, B + H:E]) for t in range(4)]
+        return sends, recvs
+
+    def _chunk(self, c):
+        qc = self.q // self.chunks
+        return range(c * qc, (c + 1) * qc)
+
+    def a2a_messages(self, c):
+        sends, recvs, local = [], [], []
+        o, Bj, q, g = self.off, self.Bj, self.q, self.g
+        for h in range(self.G):
+            for t in range(3):
+                for rl in self._chunk(c):
+                    seg_out = self.slots[t][h * q + rl, o:o + Bj]        # my rows of residue h q + rl
+                    seg_in = self.sys[t][rl, h * Bj:(h + 1) * Bj]        # rank h's rows of my residue rl
+                    if h == g:
+                        local.append((seg_out, seg_in))
+                    else:
+                        sends.append((h, seg_out))
+                        recvs.append((h, seg_in))
+        return sends, recvs, local
+
+    def xret_messages(self, c):
+        sends, recvs, local = [], [], []
+        Bj, q, g = self.Bj, self.q, self.g
+        for h in range(self.G):
+            for rl in self._chunk(c):
+                seg_out = self.xs[rl, h * Bj:(h + 1) * Bj]               # x of my residue rl, rank h's rows
+                seg_in = self.xrecv[h * q + rl]                           # x of residue h q + rl, my rows
+                if h == g:
+                    local.append((seg_out, seg_in))
+                else:
+                    sends.append((h, seg_out))
+                    recvs.append((h, seg_in))
+        return sends, recvs, local
+
+    # -------- compute
+    def split(self):
+        self.be.split(self.split_state, self.ext)
+
+    def solve(self, c):
+        a, cc, d = self.chunk_in[c]
+        self.be.solve(self.solve_states[c], a, cc, d, self.chunk_x[c])
+
+    def unpack(self, out):
+        self.be.unpack(self.xrecv, out, self.B, self.kd, self.xrecv.shape[1] if self.G > 1 else self.NL)
+
+
+def huge_steps(R: HugeRank, out, mark=None):
+    """One solve of rank R's part; a generator that yields ("post", sends,
+    recvs) and ("wait", handle) at every exchange (the driver performs them).
+    ``mark(phase)`` (optional) is called at the phase boundaries "halo",
+    "split", "exchange_solve", "unpack", "end" (per-phase event timing)."""
+    mark = mark or (lambda phase: None)
+    mark("halo")
+    if R.G > 1:
+        h = yield ("post",) + R.halo_messages()
+        yield ("wait", h)
+    mark("split")
+    R.split()
+    mark("exchange_solve")
+    if R.G > 1:
+        a2a = []
+        for c in range(R.chunks):
+            sends, recvs, local = R.a2a_messages(c)
+            a2a.append((yield ("post", sends, recvs)))
+            for src, dst in local:
+                dst.copy_(src)
+        xret = []
+        for c in range(R.chunks):
+            yield ("wait", a2a[c])
+            R.solve(c)
+            sends, recvs, local = R.xret_messages(c)
+            xret.append((yield ("post", sends, recvs)))
+            for src, dst in local:
+                dst.copy_(src)
+        for c in range(R.chunks):
+            yield ("wait", xret[c])
+    else:
+        for c in range(R.chunks):
+            R.solve(c)
+    mark("unpack")
+    R.unpack(out)
+    mark("end")
+    return out
+
+
+class P2PTransport:
+    """torch.distributed point-to-point (batch_isend_irecv): NCCL on GPUs (the
+    ops run on NCCL's stream, ordered after the current stream's kernels and
+    waited on by it), gloo on CPU."""
+
+    def __init__(self, group=None):
+        self.group = group
+
+    def post(self, sends, recvs):
+        ops = [dist.P2POp(dist.isend, t, peer, self.group) for peer, t in sends]
+        ops += [dist.P2POp(dist.irecv, t, peer, self.group) for peer, t in recvs]
+        return dist.batch_isend_irecv(ops) if ops else []
+
+    @staticmethod
+    def wait(works):
+        for w in works:
+            w.wait()
+
+
+def run_steps(gen, transport: P2PTransport):
+    """Drive one rank's ``huge_steps`` generator over a real transport."""
+    try:
+        msg = next(gen)
+        while True:
+            if msg[0] == "post":
+                msg = gen.send(transport.post(msg[1], msg[2]))
+            else:
+                transport.wait(msg[1])
+                msg = gen.send(None)
+    except StopIteration as e:
+        return e.value
+
+
+def solve_huge_loopback(ranks: Sequence[HugeRank], outs: Sequence):
+    """Run G ranks' ``huge_steps`` in ONE process (one device): a message from
+    rank g to rank h is a copy from g's send tensor to h's receive tensor,
+    matched in posting order per (g, h) pair exactly as NCCL matches them."""
+    G = len(ranks)
+    gens = [huge_steps(R, o) for R, o in zip(ranks, outs)]
+    pending = {}                                   # (src, dst) -> [sends], [recvs]
+    state, done = [None] * G, [False] * G
+    for g, gen in enumerate(gens):
+        try:
+            state[g] = next(gen)
+        except StopIteration:                      # G = 1: nothing to exchange
+            done[g] = True
+    while not all(done):
+        progressed = False
+        for g in range(G):
+            while not done[g] and state[g][0] == "post":
+                _, sends, recvs = state[g]
+                for peer, t in sends:
+                    pending.setdefault((g, peer), ([], []))[0].append(t)
+                for peer, t in recvs:
+                    pending.setdefault((peer, g), ([], []))[1].append(t)
+                try:
+                    state[g] = gens[g].send(None)
+                except StopIteration:
+                    done[g] = True
+                progressed = True
+        # every rank is waiting (or done): deliver every matched message
+        for key, (sends, recvs) in pending.items():
+            k = min(len(sends), len(recvs))
+            for src, dst in zip(sends[:k], recvs[:k]):
+                assert src.numel() == dst.numel(), key
+                dst.copy_(src)
+            del sends[:k], recvs[:k]
+        for g in range(G):
+            if not done[g] and state[g][0] == "wait":
+                try:
+                    state[g] = gens[g].send(None)
+                except StopIteration:
+                    done[g] = True
+                progressed = True
+        if not progressed:
+            raise RuntimeError("loopback deadlock")
+    return outs
+
+
+def solve_huge(a_loc, b_loc, c_loc, d_loc, n: int, group=None, kd: Optional[int] = None, backend=None,
+               chunks: int = 1, rank_state: Optional[HugeRank] = None):
+    """Solve one system of n rows whose row block [g B, (g+1) B) lives on rank
+    g (1-D tensors of B rows; a_0 and c_{n-1} of the global system are
+    ignored).  Returns x for the local rows.  ``rank_state`` reuses the
+    buffers and plans of an earlier call (allocate once with ``HugeRank``)."""
     G = dist.get_world_size(group) if dist.is_initialized() else 1
     g = dist.get_rank(group) if dist.is_initialized() else 0
-    kd = huge_kd(G, kd)
-    NR = 1 << kd
-    B = d_loc.shape[-1]
-    if G & (G - 1) or B * G != n or B % NR:
-        raise ValueError(f"solve_huge: need G a power of two, n = G*B, B % 2^kd == 0 (G={G}, n={n}, kd={kd})")
-    H = NR                      # halo rows per side (>= 2^kd - 1, aligned to the residue period)
-    dev, dt = d_loc.device, d_loc.dtype
-    loc = torch.stack([a_loc, b_loc, c_loc, d_loc])  # (4, B)
-    if g == 0:
-        loc[0, 0] = 0
-    if g == G - 1:
-        loc[2, B - 1] = 0
-
-    # 1. halo exchange with g-1 / g+1
-    ident = torch.zeros(4, H, dtype=dt, device=dev)
-    ident[1] = 1
-    left, right = ident.clone(), ident.clone()
-    if G > 1:
-        ops = []
-        if g > 0:
-            ops.append(dist.P2POp(dist.isend, loc[:, :H].contiguous(), g - 1, group))
-            ops.append(dist.P2POp(dist.irecv, left, g - 1, group))
-        if g < G - 1:
-            ops.append(dist.P2POp(dist.isend, loc[:, B - H:].contiguous(), g + 1, group))
-            ops.append(dist.P2POp(dist.irecv, right, g + 1, group))
-        for r in dist.batch_isend_irecv(ops):
-            r.wait()
-    ext = torch.cat([left, loc, right], dim=1)  # (4, E), E = B + 2H; ext row e = global row g*B - H + e
-
-    # 2. local split (k_d levels); canonical order: residue r, position j (ext row r + NR*j)
-    sa, sc, sd = split_fn(ext[0], ext[1], ext[2], ext[3], kd)
-    E = B + 2 * H
-    per = E // NR                                # rows per residue in the extended block
-    Bj = B // NR                                 # valid rows per residue (positions 1 .. Bj)
-    split = torch.stack([sa.reshape(NR, per), sc.reshape(NR, per), sd.reshape(NR, per)])  # (3, NR, per)
-    valid = split[:, :, H // NR: H // NR + Bj]   # (3, NR, Bj)
-
-    # 3. all-to-all: residues [h*q, (h+1)*q) -> rank h
-    q = NR // G
-    send = valid.reshape(3, G, q, Bj).permute(1, 0, 2, 3).contiguous()  # (G, 3, q, Bj)
-    recv = torch.empty_like(send)
-    if G > 1:
-        dist.all_to_all_single(recv, send, group=group)
-    else:
-        recv.copy_(send)
-    # recv[src]: rows j-block src of my q residues -> (3, q, G*Bj) systems
-    sys = recv.permute(1, 2, 0, 3).reshape(3, q, G * Bj)
-
-    # 4. local solve of the owned residue systems (normalised: b' = 1)
-    ones = torch.ones_like(sys[0])
-    xs = solve_fn(sys[0].contiguous(), ones, sys[1].contiguous(), sys[2].contiguous())  # (q, n/NR)
-
-    # 5. x back: rank h returns j-block g of its residues to rank g
-    xsend = xs.reshape(q, G, Bj).permute(1, 0, 2).contiguous()  # (G, q, Bj)
-    xrecv = torch.empty_like(xsend)
-    if G > 1:
-        dist.all_to_all_single(xrecv, xsend, group=group)
-    else:
-        xrecv.copy_(xsend)
-    # xrecv[h][rl][jj] = x of global row (h*q + rl) + NR*(g*Bj + jj) = local row (h*q+rl) + NR*jj
-    x_loc = xrecv.reshape(NR, Bj).t().contiguous().reshape(B)
-    return x_loc
+    if backend is None:
+        backend = CudaBackend(d_loc.dtype, d_loc.device)
+    R = rank_state or HugeRank(n, G, g, backend, kd=kd, chunks=chunks)
+    for dst, src in zip(R.local, (a_loc, b_loc, c_loc, d_loc)):
+        dst.copy_(src)
+    out = backend.empty(R.B)
+    return run_steps(huge_steps(R, out), P2PTransport(group))
 
 
 def huge_bytes(n: int, world: int, s: int = 4, kd: Optional[int] = None) -> dict:
-    """Bytes each rank moves over the interconnect in solve_huge."""
+    """Bytes each rank moves over the interconnect in solve_huge (NVLink)."""
     kd = huge_kd(world, kd)
     B = n // world
-    return {"halo": 2 * 4 * (1 << kd) * s if world > 1 else 0,
+    H = huge_halo(kd, s)
+    return {"halo": 2 * 4 * H * s if world > 1 else 0,
             "all_to_all_split": 3 * B * s * (world - 1) // world,
             "all_to_all_x": B * s * (world - 1) // world}

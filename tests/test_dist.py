@@ -25,19 +25,47 @@ def _free_port():
     return p
 
 
-def cpu_split(a, b, c, d, kd):
-    """Oracle k_d PCR levels, normalised (b' = 1), canonical residue order."""
-    A, B, C, D = (v.detach().double().numpy()[None] for v in (a, b, c, d))
-    sa, sb, sc, sd = oracle.pcr_split(A, B, C, D, kd)
-    perm = oracle.permutation(A.shape[1], kd)
-    return tuple(torch.from_numpy(np.ascontiguousarray(v[0, perm] / sb[0, perm])) for v in (sa, sc, sd))
+class OracleBackend:
+    """solve_huge's local compute on the CPU oracle (test infrastructure): the
+    split by oracle.pcr_split (normalised, canonical residue slots), the
+    residue systems by fp64 Thomas, the unpack by a transpose."""
+
+    def __init__(self, dtype=torch.float64):
+        self.dtype = dtype
+
+    def empty(self, *shape):
+        return torch.empty(*shape, dtype=self.dtype)
+
+    def make_split(self, E, kd):
+        NR = 1 << kd
+        assert E % NR == 0
+        buf = torch.empty(3, NR, E // NR, dtype=self.dtype)
+        return kd, buf, (buf[0], buf[1], buf[2])
+
+    def split(self, state, ext):
+        kd, buf, _ = state
+        E = ext.shape[1]
+        A, B, C, D = (ext[t].double().numpy()[None] for t in range(4))
+        sa, sb, sc, sd = oracle.pcr_split(A, B, C, D, kd)
+        perm = oracle.permutation(E, kd)
+        for t, v in enumerate((sa, sc, sd)):
+            buf[t] = torch.from_numpy((v[0, perm] / sb[0, perm]).reshape(buf.shape[1], buf.shape[2]))
+
+    def make_solve(self, NL, m, stride):
+        return NL, m, stride
+
+    def solve(self, state, a, c, d, x):
+        NL, m, stride = state
+        view = (lambda t: torch.as_strided(t, (m, NL), (stride, 1))) if a.dim() == 1 else (lambda t: t)
+        A, C, D = (view(t).double().numpy() for t in (a, c, d))
+        x.copy_(torch.from_numpy(oracle.thomas(A, np.ones_like(A), C, D)))
+
+    def unpack(self, xs, out, B, kd, slot_rows):
+        NR = 1 << kd
+        out.copy_(xs[:, :B // NR].t().reshape(B))
 
 
-def cpu_solve(a, b, c, d):
-    return torch.from_numpy(oracle.thomas(a.numpy(), b.numpy(), c.numpy(), d.numpy()))
-
-
-def _huge_worker(rank, world, port, n, kd, q):
+def _huge_worker(rank, world, port, n, kd, chunks, q):
     os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
     dist.init_process_group("gloo", rank=rank, world_size=world)
     try:
@@ -46,31 +74,69 @@ def _huge_worker(rank, world, port, n, kd, q):
         B = n // world
         sl = slice(rank * B, (rank + 1) * B)
         loc = [torch.from_numpy(np.ascontiguousarray(v[0, sl])) for v in (a, b, c, d)]
-        x = tdist.solve_huge(*loc, n=n, kd=kd, split_fn=cpu_split, solve_fn=cpu_solve)
+        x = tdist.solve_huge(*loc, n=n, kd=kd, backend=OracleBackend(), chunks=chunks)
         xr = oracle.thomas(a, b, c, d)[0, sl]
         err = float(np.abs(x.numpy() - xr).max() / np.abs(xr).max())
-        q.put((rank, err))
+        q.put((rank, err, x.numpy().tobytes()))
     finally:
         dist.destroy_process_group()
 
 
-@pytest.mark.parametrize("world,n,kd", [(2, 4096, 1), (2, 4096, 3), (4, 8192, 2), (4, 8192, 4)])
-def test_huge_system_gloo(world, n, kd):
-    """One system split by row blocks over `world` gloo ranks: halo exchange,
-    k_d local PCR levels, all-to-all of residue classes, local solves, x back.
-    Must equal the single-process oracle solution."""
+@pytest.mark.parametrize("world,n,kd,chunks", [(2, 4096, 1, 1), (2, 4096, 3, 2), (4, 8192, 2, 1), (4, 8192, 4, 4)])
+def test_huge_system_gloo(world, n, kd, chunks):
+    """One system split by row blocks over `world` gloo ranks (point-to-point
+    ops, the NCCL pattern): halo exchange into the padding, k_d PCR levels,
+    all-to-all of residue slot segments (chunked), residue solves, x back,
+    unpack.  Must equal the single-process oracle solution, and bit-equal the
+    same solve in a one-process loopback world."""
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _free_port()
-    procs = [ctx.Process(target=_huge_worker, args=(r, world, port, n, kd, q)) for r in range(world)]
+    procs = [ctx.Process(target=_huge_worker, args=(r, world, port, n, kd, chunks, q)) for r in range(world)]
     for p in procs:
         p.start()
-    res = dict(q.get(timeout=120) for _ in range(world))
+    res = {r: (e, xb) for r, e, xb in (q.get(timeout=120) for _ in range(world))}
     for p in procs:
         p.join(60)
         assert p.exitcode == 0
     assert sorted(res) == list(range(world))
-    assert max(res.values()) <= 1e-11, res
+    assert max(e for e, _ in res.values()) <= 1e-11, res
+    xs = _loopback_cpu(n, world, kd, chunks)
+    for r in range(world):
+        assert xs[r].numpy().tobytes() == res[r][1]
+
+
+def _loopback_cpu(n, G, kd, chunks, seed=31):
+    from paper_conf_ipps_davidsonzo11_b200 import dist as tdist
+    a, b, c, d = inputs.generate(n, 1, np.float64, seed=seed, mu=0.3)
+    be = OracleBackend()
+    ranks = [tdist.HugeRank(n, G, g, be, kd=kd, chunks=chunks) for g in range(G)]
+    B = n // G
+    for g, R in enumerate(ranks):
+        for dst, v in zip(R.local, (a, b, c, d)):
+            dst.copy_(torch.from_numpy(v[0, g * B:(g + 1) * B]))
+    outs = [be.empty(B) for _ in range(G)]
+    return tdist.solve_huge_loopback(ranks, outs)
+
+
+@pytest.mark.parametrize("kd,chunks", [(3, 1), (3, 2), (4, 1)])
+def test_huge_loopback_cpu_bit_identical_over_G(kd, chunks):
+    """The loopback world (G ranks in one process): x is the oracle's, and
+    bit-identical for G = 1, 2, 4, 8 (every row's split coefficients come from
+    the same operands whatever the block boundaries; the residue systems are
+    the same)."""
+    n = 4096
+    a, b, c, d = inputs.generate(n, 1, np.float64, seed=31, mu=0.3)
+    xr = oracle.thomas(a, b, c, d)[0]
+    ref = None
+    for G in (1, 2, 4, 8):
+        if (1 << kd) % G or (1 << kd) // G % chunks:
+            continue
+        x = torch.cat(_loopback_cpu(n, G, kd, chunks)).numpy()
+        assert np.abs(x - xr).max() <= 1e-11 * np.abs(xr).max()
+        if ref is None:
+            ref = x
+        assert np.array_equal(x, ref), G
 
 
 def _shard_worker(rank, world, port, q):
@@ -113,14 +179,20 @@ def test_batch_sharding_gloo():
 
 
 def test_huge_bytes_accounting():
+    """NVLink bytes per rank: config 5 at 8 GPUs moves 3 split
+    arrays x 7/8 of its 2^25 rows (~ 352 MB) out and in, and 7/8 of its x
+    (~ 117 MB) back."""
     from paper_conf_ipps_davidsonzo11_b200 import dist as tdist
-    b = tdist.huge_bytes(1 << 28, 8)
+    b = tdist.huge_bytes(1 << 28, 8, kd=8)
     assert b["all_to_all_split"] == 3 * (1 << 25) * 4 * 7 // 8
+    assert b["all_to_all_x"] == (1 << 25) * 4 * 7 // 8
+    assert b["halo"] == 2 * 4 * 1024 * 4
 
 
 @pytest.mark.gpu
 def test_huge_system_single_gpu_kernels():
-    """The huge-system path (G = 1) with the libtds split-only plan and solve."""
+    """The huge-system path (G = 1, torch.distributed not initialised) with
+    the libtds kernels: split to slots, residue systems read in place."""
     from paper_conf_ipps_davidsonzo11_b200 import dist as tdist
     n = 1 << 20
     a, b, c, d = inputs.generate(n, 1, np.float32, seed=5)
@@ -129,6 +201,120 @@ def test_huge_system_single_gpu_kernels():
     torch.cuda.synchronize()
     xr = oracle.thomas(a, b, c, d)[0]
     assert np.abs(x.cpu().numpy() - xr).max() / np.abs(xr).max() <= 1e-4
+
+
+def _loopback_gpu(n, G, kd, chunks, dtype, seed=5):
+    from paper_conf_ipps_davidsonzo11_b200 import dist as tdist
+    tdt = torch.float32 if dtype == np.float32 else torch.float64
+    be = tdist.CudaBackend(tdt, "cuda:0")
+    ranks = [tdist.HugeRank(n, G, g, be, kd=kd, chunks=chunks) for g in range(G)]
+    B = n // G
+    import paper_conf_ipps_davidsonzo11_b200 as tds
+    for g, R in enumerate(ranks):  # each rank draws its own rows (device generator, global row index)
+        tds.api.generate_rows(n, g * B, B, "float32" if dtype == np.float32 else "float64", seed=seed, out=R.local)
+    outs = [be.empty(B) for _ in range(G)]
+    tdist.solve_huge_loopback(ranks, outs)
+    torch.cuda.synchronize()
+    return torch.cat(outs).cpu().numpy()
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("kd,chunks", [(3, 1), (5, 4), (8, 8)])
+def test_huge_loopback_gpu(dtype, kd, chunks):
+    """The whole multi-rank huge-system data path on ONE GPU (G = 1, 2, 4, 8
+    ranks in a loopback world, libtds kernels, messages as device copies):
+    the oracle's x within the tolerance and bit-identical for every G."""
+    n = 1 << 20
+    a, b, c, d = inputs.generate(n, 1, dtype, seed=5)
+    xr = oracle.thomas(a, b, c, d)[0]
+    ref = None
+    for G in (1, 2, 4, 8):
+        if (1 << kd) % G or (1 << kd) // G % chunks:
+            continue
+        x = _loopback_gpu(n, G, kd, chunks, dtype)
+        err = np.abs(x - xr).max() / np.abs(xr).max()
+        assert err <= (1e-4 if dtype == np.float32 else 1e-10), (G, err)
+        if ref is None:
+            ref = x
+        assert np.array_equal(x, ref), G
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("n,kp", [(4096 + 256, [3]), (1 << 20, [8]), (100000, [5]), (1 << 18, [4, 4])])
+def test_split_slots_pack_bit_exact(dtype, n, kp):
+    """G3 pack: tds_split_slots leaves residue r of system s in slot (s << k) + r
+    -- the same numbers, bit for bit, as the canonical diagnostic split
+    (tds_split_batched) in the torch reference layout."""
+    import paper_conf_ipps_davidsonzo11_b200 as tds
+    name = "float32" if dtype == np.float32 else "float64"
+    m = 2
+    dv = [torch.from_numpy(v).cuda() for v in inputs.generate(n, m, dtype, seed=3)]
+    plan = tds.Plan(n, m, name, device=0)
+    plan.set_params(k_pass=kp, split_only=1, cluster=1, tl_levels=0)
+    ref = tds.split_batched(plan, *dv)
+    ws = plan.workspace()
+    views = tds.api.split_slots(plan, *dv, workspace=ws)
+    torch.cuda.synchronize()
+    k = sum(kp)
+    NR = 1 << k
+    lay = plan.slots_layout()
+    assert lay["num_slots"] == m * NR and lay["slot_rows"] >= -(-n // NR)
+    for v, r_ in zip(views, ref):
+        off = 0
+        for r in range(NR):
+            L = -(-(n - r) // NR)
+            for s in range(m):
+                assert torch.equal(v[s * NR + r, :L], r_[s, off:off + L])
+            off += L
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("n,m,k,slot", [(1 << 16, 3, 5, 2048), (1 << 16, 1, 8, 256), (5000, 2, 2, 1260),
+                                        (4096, 2, 6, 96)])
+def test_unpack_residues_bit_exact(dtype, n, m, k, slot):
+    """G3 unpack: tds_unpack_residues is the residue -> row transpose of the
+    torch reference: x[s, r + 2^k j] = xs[(s << k) + r, j]; xs left intact."""
+    import paper_conf_ipps_davidsonzo11_b200 as tds
+    tdt = torch.float32 if dtype == np.float32 else torch.float64
+    NR = 1 << k
+    xs = torch.randn(m * NR, slot, dtype=tdt, device="cuda")
+    keep = xs.clone()
+    x = torch.full((m, n), 7.0, dtype=tdt, device="cuda")
+    tds.api.unpack_residues(xs, x, n, m, k, slot)
+    torch.cuda.synchronize()
+    ref = torch.empty(m, n, dtype=tdt, device="cuda")
+    for r in range(NR):
+        L = -(-(n - r) // NR)
+        ref[:, r::NR] = xs.view(m, NR, slot)[:, r, :L]
+    assert torch.equal(x, ref) and torch.equal(xs, keep)
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("n,m,params", [(1 << 20, 4, dict(k_pass=[7], cr_levels=4, thomas_chains=1, tl_levels=5)),
+                                        (100000, 3, dict(k_pass=[5], cr_levels=3, thomas_chains=32, tl_levels=0)),
+                                        (1 << 18, 2, dict(k_pass=[3, 3], cr_levels=4, thomas_chains=1, tl_levels=5))])
+def test_solve_normalized_equals_b_one(dtype, n, m, params):
+    """tds_solve_normalized (no b array) is bit-identical to tds_solve_batched
+    with a materialised b = 1 (normalising by rcp(1) = 1 is exact)."""
+    import paper_conf_ipps_davidsonzo11_b200 as tds
+    name = "float32" if dtype == np.float32 else "float64"
+    if dtype == np.float64:
+        params = dict(params, cr_levels=3)
+    a, b, c, d = inputs.generate(n, m, dtype, seed=8)
+    an, cn, dn = (v / b for v in (a, c, d))
+    ta, tc, td = (torch.from_numpy(np.ascontiguousarray(v)).cuda() for v in (an, cn, dn))
+    plan = tds.Plan(n, m, name, device=0)
+    plan.set_params(cluster=1, **params)
+    x1 = tds.api.solve_normalized(plan, ta, tc, td)
+    x2 = tds.solve_batched(plan, ta, torch.ones_like(ta), tc, td)
+    torch.cuda.synchronize()
+    assert torch.equal(x1, x2)
+    xr = oracle.thomas(an, np.ones_like(an), cn, dn)
+    assert oracle.rel_err(x1.cpu().numpy(), xr) <= (1e-4 if dtype == np.float32 else 1e-10)
 
 
 @pytest.mark.gpu
