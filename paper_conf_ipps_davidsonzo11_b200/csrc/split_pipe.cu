@@ -39,6 +39,12 @@ __constant__ int tds_split_ablation;
 #define TDS_ABL(bit) false
 #endif
 
+// Experiment switch (-DTDS_SPLIT_STG=1): the tile's outputs leave by vector
+// STG from registers instead of shared-memory staging + TMA tensor stores.
+#ifndef TDS_SPLIT_STG
+#define TDS_SPLIT_STG 0
+#endif
+
 template <int KP, int NT_>
 struct SplitShape {
     static constexpr int R = kRegSplitRows;
@@ -55,7 +61,7 @@ struct SplitShape {
     // B blocks stored; with 512 threads rounded so a residue's positions per tile
     // (NB * 256 / 2^KP) stay a 16-byte multiple (TMA store rows)
     static constexpr int NBQ = (KP >= 8 ? 4 : KP == 7 ? 2 : 1);
-    static constexpr int NB = NT == 512 ? NBMAX - NBMAX % NBQ : NBMAX;
+    static constexpr int NB = (NT == 512 && !TDS_SPLIT_STG) ? NBMAX - NBMAX % NBQ : NBMAX;
     static constexpr int TV = KP > 4 ? NB * 16 * R : AV * R;              // output rows per tile
     static constexpr int HEAD = R + LEFT * R;                             // window rows before the tile
     static_assert(TV % (1 << KP) == 0, "tile must hold whole residue periods");
@@ -77,7 +83,7 @@ struct SplitShape {
     static constexpr int NBOX = PT / BOXP;
     static_assert(PT % BOXP == 0, "whole boxes");
     template <typename T>
-    __host__ __device__ static constexpr bool tstore() { return (PT * int(sizeof(T))) % 16 == 0; }
+    __host__ __device__ static constexpr bool tstore() { return !TDS_SPLIT_STG && (PT * int(sizeof(T))) % 16 == 0; }
     template <typename T>
     __host__ __device__ static constexpr int tbuf_elems() {
         const int tr = KP > 4 ? (sizeof(T) == 4 ? 3 : 1) * AV * 16 : 0;

@@ -209,12 +209,15 @@ static tds_params search(Search &S, const tds_params &seed, double &t_best) {
     // reverse.  For each k both pass schedules are tried -- register split
     // passes (k_p <= 4), the persistent TMA split kernel's limit (k_p <= 8)
     // and the seed's k_p limit -- with the smallest cluster that holds the
-    // subsystem; the walk tolerates two non-improving steps (splitting and
-    // on-chip costs trade off unevenly).
+    // subsystem; the walk up tolerates two non-improving steps (splitting and
+    // on-chip costs trade off unevenly), the walk down goes on while the
+    // subsystems fit on chip (k = 0, no split pass at all, is a regime of its
+    // own: a local minimum the climb must not miss -- config 4 from its static
+    // seed k = 1).
     for (int dir : {+1, -1}) {
         tds_params walk = best;
         int misses = 0;
-        while (misses < 3 && !out_of_time(S)) {
+        while ((dir < 0 || misses < 3) && !out_of_time(S)) {
             tds_params base = walk;
             base.k += dir;
             if (base.k < 0 || base.k > 30 || (int64_t(1) << base.k) > 2 * I.n) break;

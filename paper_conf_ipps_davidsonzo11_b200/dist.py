@@ -124,6 +124,16 @@ class CudaBackend:
 
     def make_solve(self, NL: int, m: int, stride: int):
         plan = api.Plan(NL, m, self.name, device=self.device.index or 0, mode="static", batch_stride=stride)
+        if plan.info["k"] == 0:
+            # normalised input needs >= 1 split level (the k = 0 kernels read b): one level, the
+            # static on-chip shape for the halved subsystems
+            T0 = plan.info["thomas_chains"]
+            for T in [T0] + [t for t in (32, 16, 8, 4, 2, 1) if t < T0]:
+                try:
+                    plan.set_params(k_pass=[1], cluster=1, tl_levels=0, thomas_chains=T)
+                    break
+                except api.L.TdsError:
+                    continue
         return plan, plan.workspace()
 
     def solve(self, state, a, c, d, x):
@@ -174,7 +184,8 @@ class HugeRank:
             self.sys = [backend.empty(q, NL) for _ in range(3)]
             self.chunk_in = [tuple(v[c * qc:(c + 1) * qc] for v in self.sys) for c in range(chunks)]
             self.solve_states = [backend.make_solve(NL, qc, NL) for _ in range(chunks)]
-        self.xs = backend.empty(q, NL)            # x of the local residue systems
+        # x of the local residue systems (G = 1: with the slots' stride, unpacked in place)
+        self.xs = backend.empty(q, self.stride if G == 1 else NL)
         self.chunk_x = [self.xs[c * qc:(c + 1) * qc] for c in range(chunks)]
         self.xrecv = self.xs if G == 1 else backend.empty(NR, Bj)
 
@@ -237,7 +248,7 @@ class HugeRank:
         self.be.solve(self.solve_states[c], a, cc, d, self.chunk_x[c])
 
     def unpack(self, out):
-        self.be.unpack(self.xrecv, out, self.B, self.kd, self.xrecv.shape[1] if self.G > 1 else self.NL)
+        self.be.unpack(self.xrecv, out, self.B, self.kd, self.xrecv.shape[1])
 
 
 def huge_steps(R: HugeRank, out, mark=None):
