@@ -229,8 +229,9 @@ tds_status tds_solve_batched(const tds_plan_t plan, const void *a, const void *b
 /* Run only launches first_stage..last_stage (inclusive) of the kernel sequence
  * tds_solve_batched enqueues.  The sequence is, for each chunk of
  * chunk_systems systems in order: split passes 0..passes-1 (PAPER.md stages
- * 1-2), the on-chip kernel (stages 3-4) and, when k > 0 and x_group == 0, the x placement;
- * launch index = chunk * S + stage with S = passes + 1 + (k > 0 && x_group == 0), and
+ * 1-2), the on-chip kernel (stages 3-4) and, when k > 0, x_group == 0 and strided == 0, the x
+ * placement; launch index = chunk * S + stage with
+ * S = passes + 1 + (k > 0 && x_group == 0 && strided == 0), and
  * info.launches = chunks * S.  Calling every launch in order on one stream is
  * identical to tds_solve_batched (used to time each kernel with events between
  * them); each launch consumes what the previous one left in the workspace, so a
@@ -296,7 +297,7 @@ tds_status tds_unpack_residues(tds_dtype dtype, int64_t n, int64_t m, int32_t k,
 /* Bytes of device workspace tds_solve_interleaved needs for `plan`: the
  * plan's own workspace plus four system-major copies of the m x n arrays
  * (each rounded up to 256 bytes).  The plan must be dense (batch_stride == n).
- * Errors: INVALID_ARG (NULL), UNSUPPORTED (strided or split-only plan). */
+ * Errors: INVALID_ARG (NULL), UNSUPPORTED (padded -- batch_stride != n -- or split-only plan). */
 tds_status tds_interleaved_workspace_bytes(const tds_plan_t plan, size_t *bytes);
 
 /* Same solve as tds_solve_batched for arrays in the INTERLEAVED layout:
@@ -307,7 +308,7 @@ tds_status tds_interleaved_workspace_bytes(const tds_plan_t plan, size_t *bytes)
  * transposed back: 2 x 4 s extra HBM bytes per equation in, 2 s out.
  * x: device, interleaved, may alias d exactly.  workspace: device, 256-byte
  * aligned, >= tds_interleaved_workspace_bytes.  Same errors as
- * tds_solve_batched (plus UNSUPPORTED for a strided plan); enqueued on
+ * tds_solve_batched (plus UNSUPPORTED for a padded plan, batch_stride != n); enqueued on
  * cuda_stream, asynchronous. */
 tds_status tds_solve_interleaved(const tds_plan_t plan, const void *a, const void *b, const void *c,
                                  const void *d, void *x, void *workspace, size_t workspace_bytes,

@@ -202,13 +202,17 @@ def _check_tensor(t, plan_info, name):
     import torch
     want = torch.float32 if plan_info.dtype == L.TDS_F32 else torch.float64
     need = (plan_info.m - 1) * plan_info.batch_stride + plan_info.n
-    _check_fast(t, need, want, name)
+    _check_fast(t, need, want, name, int(plan_info.device))
 
 
-def _check_fast(t, need, want, name):
-    """Argument checks of the Python face (the C ABI re-checks pointers / sizes)."""
+def _check_fast(t, need, want, name, dev=None):
+    """Argument checks of the Python face (the C ABI re-checks pointers / sizes);
+    ``dev``: the plan's device -- a tensor on another GPU is refused here (the
+    kernels would fault on it)."""
     if getattr(t, "is_cuda", False) is not True:
         raise TypeError(f"{name} must be a CUDA tensor")
+    if dev is not None and t.device.index != dev:
+        raise ValueError(f"{name} is on cuda:{t.device.index}, the plan on cuda:{dev}")
     if t.dtype != want:
         raise TypeError(f"{name} has dtype {t.dtype}, plan expects {want}")
     if t.numel() < need or not t.is_contiguous():
@@ -220,14 +224,14 @@ def solve_batched(plan: Plan, a, b, c, d, out=None, workspace=None, stream=None)
     tensors laid out as the plan says (m x batch_stride).  Returns x."""
     import torch
     info, need, want, dev = plan._solve_info()
-    _check_fast(a, need, want, "a")
-    _check_fast(b, need, want, "b")
-    _check_fast(c, need, want, "c")
-    _check_fast(d, need, want, "d")
+    _check_fast(a, need, want, "a", dev)
+    _check_fast(b, need, want, "b", dev)
+    _check_fast(c, need, want, "c", dev)
+    _check_fast(d, need, want, "d", dev)
     if out is None:
         out = torch.empty_like(d)
     else:
-        _check_fast(out, need, want, "out")
+        _check_fast(out, need, want, "out", dev)
     if workspace is None and info.workspace_bytes > 0:
         workspace = plan.workspace()
     wptr = workspace.data_ptr() if workspace is not None else None
@@ -243,11 +247,11 @@ def solve_normalized(plan: Plan, a, c, d, out=None, workspace=None, stream=None)
     import torch
     info, need, want, dev = plan._solve_info()
     for name, t in (("a", a), ("c", c), ("d", d)):
-        _check_fast(t, need, want, name)
+        _check_fast(t, need, want, name, dev)
     if out is None:
         out = torch.empty_like(d)
     else:
-        _check_fast(out, need, want, "out")
+        _check_fast(out, need, want, "out", dev)
     if workspace is None and info.workspace_bytes > 0:
         workspace = plan.workspace()
     wptr = workspace.data_ptr() if workspace is not None else None
@@ -263,7 +267,7 @@ def split_slots(plan: Plan, a, b, c, d, workspace, stream=None):
     r of system s, normalised rows, Fig. 3a order)."""
     info, need, want, dev = plan._solve_info()
     for name, t in (("a", a), ("b", b), ("c", c), ("d", d)):
-        _check_fast(t, need, want, name)
+        _check_fast(t, need, want, name, dev)
     lay = plan.slots_layout()
     wbytes = workspace.numel() * workspace.element_size()
     L.check(plan._lib.tds_split_slots(plan.handle, a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
@@ -316,11 +320,11 @@ def solve_interleaved(plan: Plan, a, b, c, d, out=None, workspace=None, stream=N
     info, _, want, dev = plan._solve_info()
     need = info.n * info.m
     for name, t in (("a", a), ("b", b), ("c", c), ("d", d)):
-        _check_fast(t, need, want, name)
+        _check_fast(t, need, want, name, dev)
     if out is None:
         out = torch.empty_like(d)
     else:
-        _check_fast(out, need, want, "out")
+        _check_fast(out, need, want, "out", dev)
     if workspace is None:
         workspace = torch.empty(plan.interleaved_workspace_bytes, dtype=torch.uint8, device=f"cuda:{dev}")
     wbytes = workspace.numel() * workspace.element_size()

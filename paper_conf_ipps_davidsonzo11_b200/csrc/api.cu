@@ -274,7 +274,7 @@ static tds_status split_impl(const tds_plan_info &I, const T *a, const T *b, con
 }
 
 // Run launches [first, last] of the chunked sequence: for each chunk of
-// chunk_systems systems, S = passes + 1 + (k > 0 && x_group == 0) kernels.  Chunks reuse one
+// chunk_systems systems, S = passes + 1 + (k > 0 && x_group == 0 && strided == 0) kernels.  Chunks reuse one
 // workspace, so a chunk's split output is still in L2 when its on-chip kernel
 // and x placement read it.
 template <typename T>
@@ -342,6 +342,24 @@ static tds_status solve_interleaved_impl(const tds_plan_info &I, const T *a, con
     return TDS_OK;
 }
 
+// Launch geometry of every kernel of a solve, checked before the first launch
+// (so an UNSUPPORTED never leaves earlier launches of the same call enqueued).
+static tds_status check_geometry(const tds_plan_info &I) {
+    const tds_params &P = I.params;
+    const int64_t mc = chunk_m(P, I.m);  // the largest chunk
+    int kprev = 0;
+    for (int p = 0; p < P.passes; ++p) {
+        const int64_t m_in = mc << kprev;
+        const int64_t len_in = cdiv(I.n, int64_t(1) << kprev);
+        const int64_t segs = split_segments(m_in, cdiv(len_in, split_tile_eff(P, p)), P.theta);
+        if (m_in * segs > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "split grid exceeds 2^31-1 CTAs");
+        kprev += P.k_pass[p];
+    }
+    const int64_t grid = P.k == 0 ? mc * P.cluster : (mc << P.k) * P.cluster;
+    if (!P.split_only && grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "on-chip grid exceeds 2^31-1 CTAs");
+    return TDS_OK;
+}
+
 static tds_status check_arrays(const tds_plan_info &I, std::initializer_list<const void *> ptrs) {
     const size_t es = size_t(dsize(I.dtype));
     for (const void *p : ptrs) {
@@ -406,6 +424,7 @@ tds_status tds_solve_stages(const tds_plan_t plan, const void *a, const void *b,
         for (const void *p : {a, b, c, d, (const void *)x})
             if (overlaps(workspace, I.workspace_bytes, p, bytes))
                 return fail(TDS_ERR_INVALID_ARG, "workspace overlaps an array");
+    if ((s = check_geometry(I)) != TDS_OK) return s;
     if ((s = check_device(plan)) != TDS_OK) return s;
     cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
     s = I.dtype == TDS_F32
@@ -464,6 +483,7 @@ tds_status tds_solve_normalized(const tds_plan_t plan, const void *a, const void
         return fail(TDS_ERR_UNSUPPORTED, "normalised input needs a plan with k >= 1 split levels and strided = 0");
     tds_status s = check_solve_args(I, a, nullptr, c, d, x, workspace, workspace_bytes);
     if (s != TDS_OK) return s;
+    if ((s = check_geometry(I)) != TDS_OK) return s;
     if ((s = check_device(plan)) != TDS_OK) return s;
     cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
     s = I.dtype == TDS_F32
@@ -502,6 +522,7 @@ tds_status tds_split_slots(const tds_plan_t plan, const void *a, const void *b, 
     const size_t bytes = size_t(((I.m - 1) * I.batch_stride + I.n) * dsize(I.dtype));
     for (const void *p : {a, b, c, d})
         if (overlaps(workspace, I.workspace_bytes, p, bytes)) return fail(TDS_ERR_INVALID_ARG, "workspace overlaps an array");
+    if ((s = check_geometry(I)) != TDS_OK) return s;
     if ((s = check_device(plan)) != TDS_OK) return s;
     cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
     int ob = 0;
@@ -578,6 +599,7 @@ tds_status tds_solve_interleaved(const tds_plan_t plan, const void *a, const voi
     if (reinterpret_cast<uintptr_t>(workspace) % 256) return fail(TDS_ERR_WORKSPACE, "workspace not 256-byte aligned");
     for (const void *p : {a, b, c, d, (const void *)x})
         if (overlaps(workspace, need, p, bytes)) return fail(TDS_ERR_INVALID_ARG, "workspace overlaps an array");
+    if ((s = check_geometry(I)) != TDS_OK) return s;
     if ((s = check_device(plan)) != TDS_OK) return s;
     cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
     s = I.dtype == TDS_F32
