@@ -19,6 +19,13 @@ for k in split_pipe onchip place_x; do
       python bench.py --config 3 --tune-cache $cache --steps 2 --warmup 1 --soak-s 0 --no-e2e --no-cpu-baseline > /dev/null 2>&1
   echo "prof $k rc=$?"
 done
+# the fp64 split (the kernel furthest below its roofline) and the k = 0 cluster kernel of config 4
+timeout 900 ncu --set full --clock-control none --import-source on -k regex:split_pipe -s 2 -c 1 -o gpurun_out/prof_split_pipe_f64_$tag \
+    python bench.py --config 3 --dtype f64 --tune-cache $cache --steps 2 --warmup 1 --soak-s 0 --no-e2e --no-cpu-baseline > /dev/null 2>&1
+echo "prof split f64 rc=$?"
+timeout 900 ncu --set full --clock-control none --import-source on -k regex:onchip_cpipe -s 2 -c 1 -o gpurun_out/prof_cpipe_cfg4_$tag \
+    python bench.py --config 4 --tune-cache $cache --steps 2 --warmup 1 --soak-s 0 --no-e2e --no-cpu-baseline > /dev/null 2>&1
+echo "prof cpipe rc=$?"
 cp gpurun_out/${tag}_launches_cfg3_f32.csv gpurun_out/launches_$tag.csv
 cp gpurun_out/${tag}_bench_cfg3_f32.json gpurun_out/bench_$tag.json
 ls gpurun_out | head -80

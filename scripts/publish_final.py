@@ -89,8 +89,11 @@ def main():
           f"Command: `bash scripts/gpu_final.sh {tag}` (bench tunes and caches the plan; ncu runs read the cache). "
           "Captures: `ncu --set full --clock-control none --import-source on -k regex:<kernel> -s 2 -c 1` "
           "(cold L2, serialised).", "", "```"]
-    for k in ("split_pipe", "onchip", "place_x"):
+    for k in ("split_pipe", "onchip", "place_x", "split_pipe_f64", "cpipe_cfg4"):
         rep = os.path.join(G, f"prof_{k}_{tag}.ncu-rep")
+        if k in ("split_pipe_f64", "cpipe_cfg4"):
+            md.append("")
+            md.append(f"# {'config 3 fp64' if k == 'split_pipe_f64' else 'config 4 fp32'}")
         if os.path.exists(rep):
             md.append(subprocess.run([sys.executable, os.path.join(ROOT, "scripts", "ncu_summary.py"), rep],
                                      capture_output=True, text=True).stdout.rstrip())
