@@ -21,7 +21,7 @@ CFGS = ["cfg3_f32", "cfg3_f64", "cfg2_f32", "cfg4_f32", "cfg1_f32", "cfg5_f32"]
 
 
 def stage_of(kernel: str):
-    k = kernel.split("(")[0].split("<")[0].replace("void ", "").strip()
+    k = kernel.split("(")[0].split("<")[0].replace("void ", "").replace("tds::", "").strip()
     if k.startswith("split_"):
         return "split_pass"
     if k.startswith("onchip"):
