@@ -579,6 +579,18 @@ def run_huge(args):
     chunks = args.huge_chunks if world > 1 else 1
     be = tdist.CudaBackend(tdt, dev)
     R = tdist.HugeRank(n, world, rank, be, kd=kd, chunks=chunks)
+    trials = 0
+    if args.mode == "tuned":
+        # the residue solves' plan: tuned on rank 0, broadcast (identical kernels on every rank)
+        if rank == 0:
+            cache = args.tune_cache or tempfile.mktemp(suffix=".tds_tune")
+            R.tune_residues(cache_path=cache)
+            if not args.tune_cache and os.path.exists(cache):
+                os.unlink(cache)
+        if world > 1:
+            vec = torch.tensor(R.residue_params(), dtype=torch.int64, device=dev)
+            hz.dist.broadcast(vec, 0)
+            R.set_residue_params(vec.tolist())
     tds.api.generate_rows(n, rank * R.B, R.B, name, seed=seed, out=R.local, device=hz.local)
     x = be.empty(R.B)
     transport = tdist.P2PTransport()
@@ -685,7 +697,7 @@ def run_huge(args):
                 "on the device by tds_generate_rows)",
         "config": {"workload": f"config5: 1 x {n} {args.dtype} split by rows over {world} GPU(s)", "n": n, "m": 1,
                    "rows_per_rank": B, "k_d": kd, "halo_rows": R.H, "chunks": R.chunks,
-                   "residue_systems_per_rank": R.q, "residue_plan": _plan_summary(info),
+                   "residue_systems_per_rank": R.q, "mode": args.mode, "residue_plan": _plan_summary(info),
                    "launch": "eager (NCCL point-to-point between the kernels)",
                    "l2": "no flush: per-step working set > 10 GiB > L2 126 MiB",
                    "parallelism": f"one system over {world} rank(s): halo exchange + all-to-all of residue classes "

@@ -239,6 +239,34 @@ class HugeRank:
                     recvs.append((h, seg_in))
         return sends, recvs, local
 
+    # -------- residue-solve plan (all chunks share one shape)
+    def residue_params(self) -> list:
+        return self.solve_states[0][0].params_list()
+
+    def set_residue_params(self, vals) -> None:
+        """Apply one integer plan to every chunk's residue solve (e.g. tuned on
+        rank 0 and broadcast); a plan with k = 0 (normalised input needs a
+        split level) is refused by tds_solve_normalized, so it is not applied."""
+        new = []
+        for plan, _ in self.solve_states:
+            old = plan.params_list()
+            plan.set_params_list(vals)
+            if plan.info["k"] == 0:
+                plan.set_params_list(old)
+            new.append((plan, plan.workspace()))
+        self.solve_states = new
+
+    def tune_residues(self, cache_path=None) -> list:
+        """tds_tune on the residue-solve shape (this rank's device); applied to
+        every chunk.  Returns the integer plan (to broadcast)."""
+        plan = self.solve_states[0][0]
+        before = plan.params_list()
+        plan.tune(cache_path=cache_path)
+        vals = plan.params_list()
+        plan.set_params_list(before)
+        self.set_residue_params(vals)
+        return self.residue_params()
+
     # -------- compute
     def split(self):
         self.be.split(self.split_state, self.ext)

@@ -343,3 +343,24 @@ def test_batch_shards_bit_identical_gpu(n, m, params, world):
         plan.set_params_list(full.params_list())
         x = tds.solve_batched(plan, *[torch.from_numpy(v).cuda() for v in sh]).cpu().numpy()
         assert np.array_equal(x, xall[s0:s1])
+
+
+@pytest.mark.gpu
+def test_huge_tuned_residue_plan(tmp_path):
+    """The residue solves with a tds_tune'd plan (bench.py --config 5 tunes
+    it on rank 0 and broadcasts it): same x as the static plan within the
+    tolerance, and every chunk runs the same integer plan."""
+    from paper_conf_ipps_davidsonzo11_b200 import dist as tdist
+    import paper_conf_ipps_davidsonzo11_b200 as tds
+    n, kd = 1 << 20, 5
+    be = tdist.CudaBackend(torch.float32, "cuda:0")
+    R = tdist.HugeRank(n, 1, 0, be, kd=kd, chunks=2)
+    vals = R.tune_residues(cache_path=str(tmp_path / "t.txt"))
+    assert all(p.params_list() == vals for p, _ in R.solve_states)
+    tds.api.generate_rows(n, 0, n, "float32", seed=5, out=R.local)
+    out = be.empty(n)
+    tdist.solve_huge_loopback([R], [out])
+    torch.cuda.synchronize()
+    a, b, c, d = inputs.generate(n, 1, np.float32, seed=5)
+    xr = oracle.thomas(a, b, c, d)[0]
+    assert np.abs(out.cpu().numpy() - xr).max() / np.abs(xr).max() <= 1e-4
