@@ -364,3 +364,40 @@ def test_huge_tuned_residue_plan(tmp_path):
     a, b, c, d = inputs.generate(n, 1, np.float32, seed=5)
     xr = oracle.thomas(a, b, c, d)[0]
     assert np.abs(out.cpu().numpy() - xr).max() / np.abs(xr).max() <= 1e-4
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("family,kw", [("poisson", {}), ("const", {"param": 1e-6})])
+@pytest.mark.parametrize("kd,chunks", [(3, 1), (5, 2)])
+def test_huge_loopback_gpu_coupling(family, kw, kd, chunks):
+    """The multi-rank huge-system path on long-range-coupled fp64 systems
+    (every row couples to rows on every other rank): the halo exchange, the
+    residue all-to-all and the x return must carry the coupling.  Oracle
+    within 10 kappa eps_64, bit-identical over G = 1, 2, 4, 8."""
+    import math
+    from paper_conf_ipps_davidsonzo11_b200 import dist as tdist
+    n = 1 << 18
+    a, b, c, d = inputs.generate(n, 1, np.float64, seed=7, family=family, **kw)
+    xr = oracle.thomas(a, b, c, d)[0]
+    delta = kw.get("param", 0.0)
+    cs = math.cos(math.pi / (n + 1))
+    kappa = (2 + delta + 2 * cs) / (2 + delta - 2 * cs)
+    be = tdist.CudaBackend(torch.float64, "cuda:0")
+    ref = None
+    for G in (1, 2, 4, 8):
+        if (1 << kd) % G or (1 << kd) // G % chunks:
+            continue
+        B = n // G
+        ranks = [tdist.HugeRank(n, G, g, be, kd=kd, chunks=chunks) for g in range(G)]
+        for g, R in enumerate(ranks):
+            for dst, v in zip(R.local, (a, b, c, d)):
+                dst.copy_(torch.from_numpy(v[0, g * B:(g + 1) * B]))
+        outs = [be.empty(B) for _ in range(G)]
+        tdist.solve_huge_loopback(ranks, outs)
+        torch.cuda.synchronize()
+        x = torch.cat(outs).cpu().numpy()
+        err = np.abs(x - xr).max() / np.abs(xr).max()
+        assert err <= 10 * kappa * 2.22e-16, (G, err)
+        if ref is None:
+            ref = x
+        assert np.array_equal(x, ref), G
