@@ -2,7 +2,7 @@
 tuned plan).  Diagnostic only."""
 import json, os, sys, time
 import torch
-sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.dirname(os.path.abspath(__file__)))))
 import paper_conf_ipps_davidsonzo11_b200 as tds  # noqa: E402
 from paper_conf_ipps_davidsonzo11_b200 import api  # noqa: E402
 n, m = 1 << 20, 16

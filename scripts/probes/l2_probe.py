@@ -7,7 +7,7 @@ import sys
 
 import torch
 
-sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.dirname(os.path.abspath(__file__)))))
 import paper_conf_ipps_davidsonzo11_b200 as tds  # noqa: E402
 from paper_conf_ipps_davidsonzo11_b200 import api  # noqa: E402
 

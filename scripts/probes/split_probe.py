@@ -1,13 +1,13 @@
 """Probe: split-stage time of config 3 (16 x 2^20 fp32) for split kernel
 variants (threads per CTA, k_p).  Diagnostic only.
-    python scripts/split_probe.py [--only THREADS KP]   (one variant, e.g. under ncu)"""
+    python scripts/probes/split_probe.py [--only THREADS KP]   (one variant, e.g. under ncu)"""
 import json
 import os
 import sys
 
 import torch
 
-sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.dirname(os.path.abspath(__file__)))))
 import paper_conf_ipps_davidsonzo11_b200 as tds  # noqa: E402
 from paper_conf_ipps_davidsonzo11_b200 import api  # noqa: E402
 
