@@ -67,6 +67,9 @@ def parse():
     ap.add_argument("--scaling", default="strong", choices=["strong", "weak"],
                     help="strong: the config's M systems in total, sharded over the ranks (default); "
                          "weak: M systems per rank")
+    ap.add_argument("--systems", type=int, default=0,
+                    help="override the config's number of systems M (probe: one rank's share of a strong-scaled "
+                         "batch, e.g. --systems 2 = config 3 at 8 GPUs)")
     ap.add_argument("--huge-kd", type=int, default=8, help="config 5: levels split before the exchange")
     ap.add_argument("--huge-chunks", type=int, default=4, help="config 5: residue groups overlapped with the "
                                                              "all-to-all (N > 1)")
@@ -365,6 +368,7 @@ def run_tds(args):
     hz = Harness(args)
     world, rank, dev = hz.world, hz.rank, hz.dev
     n, M = CONFIGS[args.config]
+    M = args.systems or M
     dt = np.float32 if args.dtype == "f32" else np.float64
     name = "float32" if dt == np.float32 else "float64"
     tdt = torch.float32 if dt == np.float32 else torch.float64
