@@ -61,4 +61,31 @@ for label, dt, n, m, params in CASES:
     ok = err <= (1e-4 if dt == F32 else 1e-10)
     bad += not ok
     print(f"{'ok ' if ok else 'BAD'} {label}: n={n} m={m} rel_err={err:.2e}", flush=True)
+# round 2: device generator, the one-huge-system path in a loopback world (split to
+# slots, normalised residue solves, exchange copies, x unpack), normalised solve
+from paper_conf_ipps_davidsonzo11_b200 import dist as tdist  # noqa: E402
+for label, dt, n, G, kd, chunks in [("huge loopback G=4 kd=3", F32, 1 << 16, 4, 3, 1),
+                                    ("huge loopback G=2 kd=4 chunks=2", F64, 1 << 15, 2, 4, 2),
+                                    ("huge G=1 kd=5", F32, 1 << 16, 1, 5, 1)]:
+    tdt = torch.float32 if dt == F32 else torch.float64
+    name = "float32" if dt == F32 else "float64"
+    be = tdist.CudaBackend(tdt, "cuda:0")
+    ranks = [tdist.HugeRank(n, G, g, be, kd=kd, chunks=chunks) for g in range(G)]
+    B = n // G
+    for g, R in enumerate(ranks):
+        tds.api.generate_rows(n, g * B, B, name, seed=5, out=R.local)
+    outs = [be.empty(B) for _ in range(G)]
+    tdist.solve_huge_loopback(ranks, outs)
+    torch.cuda.synchronize()
+    a, b, c, d = inputs.generate(n, 1, dt, seed=5)
+    err = oracle.rel_err(torch.cat(outs).cpu().numpy()[None], oracle.thomas(a, b, c, d))
+    ok = err <= (1e-4 if dt == F32 else 1e-10)
+    bad += not ok
+    print(f"{'ok ' if ok else 'BAD'} {label}: n={n} rel_err={err:.2e}", flush=True)
+gen = tds.generate(3000, 5, "float64", seed=9, first_system=2)
+torch.cuda.synchronize()
+ref = inputs.generate(3000, 5, F64, seed=9, first_system=2)
+ok = all(np.array_equal(r, g.cpu().numpy()) for r, g in zip(ref, gen))
+bad += not ok
+print(f"{'ok ' if ok else 'BAD'} tds_generate f64 bit-identical", flush=True)
 sys.exit(1 if bad else 0)
