@@ -16,7 +16,7 @@ from paper_conf_ipps_davidsonzo11_b200 import inputs  # noqa: E402
 
 draws = int(sys.argv[1]) if len(sys.argv) > 1 else 2000
 rng = np.random.default_rng(int(sys.argv[2]) if len(sys.argv) > 2 else 7)
-ran = bad = inter = 0
+ran = bad = inter = coupled = 0
 for i in range(draws):
     dtype = np.float32 if rng.random() < 0.7 else np.float64
     n = int(rng.choice([rng.integers(1, 5000), rng.integers(5000, 400000), 1 << int(rng.integers(10, 20))]))
@@ -35,12 +35,25 @@ for i in range(draws):
         plan.set_params(**params)
     except tds.TdsError:
         continue
-    a, b, c, d = inputs.generate(n, m, dtype, seed=5000 + i)
+    # fp64 draws: half of them on long-range-coupled families (Poisson, tridiag(-1, 2 + 1e-6, -1)) with
+    # 10 kappa eps tolerances -- random plans must carry the coupling, not only the dd-random data
+    fam = "dd"
+    if dtype == np.float64 and rng.random() < 0.5:
+        fam = "poisson" if rng.random() < 0.5 else "const"
+    kw = {"param": 1e-6} if fam == "const" else {}
+    a, b, c, d = inputs.generate(n, m, dtype, seed=5000 + i, family=fam, **kw)
     x = tds.solve_batched(plan, *[torch.from_numpy(v).cuda() for v in (a, b, c, d)])
     torch.cuda.synchronize()
     x = x.cpu().numpy()
     err = oracle.rel_err(x, oracle.thomas(a, b, c, d))
-    ok = np.all(np.isfinite(x)) and err <= (1e-4 if dtype == np.float32 else 1e-10)
+    if fam == "dd":
+        tol = 1e-4 if dtype == np.float32 else 1e-10
+    else:
+        delta = kw.get("param", 0.0)
+        cs = np.cos(np.pi / (n + 1))
+        tol = 10 * (2 + delta + 2 * cs) / max(2 + delta - 2 * cs, 1e-300) * 2.22e-16
+        coupled += 1
+    ok = np.all(np.isfinite(x)) and err <= tol
     if ok and plan.info["batch_stride"] == n and rng.random() < 0.3:  # the interleaved layout: bit-identical
         xi = tds.solve_interleaved(plan, *[torch.from_numpy(np.ascontiguousarray(v.T)).cuda() for v in (a, b, c, d)])
         torch.cuda.synchronize()
@@ -49,6 +62,7 @@ for i in range(draws):
     ran += 1
     if not ok:
         bad += 1
-        print(f"BAD draw {i}: {dtype.__name__} n={n} m={m} {params} err={err:.3e}", flush=True)
-print(f"fuzz: {ran} plans run ({inter} also through the interleaved layout), {bad} bad", flush=True)
+        print(f"BAD draw {i}: {dtype.__name__} {fam} n={n} m={m} {params} err={err:.3e}", flush=True)
+print(f"fuzz: {ran} plans run ({inter} also through the interleaved layout, {coupled} on coupled fp64 "
+      f"families), {bad} bad", flush=True)
 sys.exit(1 if bad else 0)

@@ -5,3 +5,4 @@ for tool in memcheck racecheck synccheck; do
   timeout 1500 compute-sanitizer --tool $tool --print-limit 20 python scripts/sanitize.py > $O/san_$tool.txt 2>&1
   echo "== $tool rc=$?"; grep -E "SUMMARY|BAD" $O/san_$tool.txt | head -20; grep -c "^ok" $O/san_$tool.txt
 done
+timeout 2400 python scripts/fuzz_long.py 3000 11 > $O/fuzz.txt 2>&1; echo "fuzz rc=$?"; tail -5 $O/fuzz.txt
