@@ -402,9 +402,11 @@ static bool ensure_ws(TuneCtx &C, size_t need) {
     return true;
 }
 
-// Median time (ms) of the full solve with parameters p (already validated);
-// kRejected if the solve refuses to launch; NaN on a device fault (sticky:
-// the search stops).
+// Median time (ms) of the full solve with parameters p (already validated),
+// measured as bench.py runs it: `inner` solves back to back between two
+// events (inner chosen so one sample spans >= ~0.4 ms; small problems would
+// otherwise time the host launch gaps, not the kernels); kRejected if the
+// solve refuses to launch; NaN on a device fault (sticky: the search stops).
 static double trial(TuneCtx &C, const tds_params &p) {
     tds_plan_st tmp = *C.plan;
     if (derive(tmp.info, tmp.props, p) != TDS_OK) return kRejected;
@@ -413,14 +415,17 @@ static double trial(TuneCtx &C, const tds_params &p) {
     if (cudaEventCreate(&e0) != cudaSuccess || cudaEventCreate(&e1) != cudaSuccess) return NAN;
     std::vector<float> ms;
     bool launched = true, fault = false;
+    int inner = 1;
     for (int r = 0; r < C.reps + 2 && launched && !fault; ++r) {
         cudaEventRecord(e0, C.st);
-        launched = tds_solve_batched(&tmp, C.a, C.b, C.c, C.d, C.x, C.ws, C.ws_bytes, C.st) == TDS_OK;
+        for (int i = 0; i < inner && launched; ++i)
+            launched = tds_solve_batched(&tmp, C.a, C.b, C.c, C.d, C.x, C.ws, C.ws_bytes, C.st) == TDS_OK;
         cudaEventRecord(e1, C.st);
         if (cudaEventSynchronize(e1) != cudaSuccess) fault = true;
         float t = 0;
         cudaEventElapsedTime(&t, e0, e1);
-        if (r >= 2) ms.push_back(t);
+        if (r == 0 && inner == 1 && t > 0) inner = std::max(1, std::min(64, int(0.4f / t + 0.999f)));
+        if (r >= 2) ms.push_back(t / float(inner));
     }
     cudaEventDestroy(e0);
     cudaEventDestroy(e1);
