@@ -637,6 +637,30 @@ def run_huge(args):
     names = ["split_to_slots(k_d=%d)" % kd, "residue_solves(k=%d, %d passes)" % (local_k, info["passes"]),
              "unpack_residues"]
     abytes = [ab_split, ab_solve, ab_unpack]
+    timing_note = ("CUDA events between the phases of K extra steps on rank 0 (phase 2 includes the all-to-all "
+                   f"and x return when N > 1; halo exchange {ph_all[0]:.4f} ms apart)")
+    n_launch = 1 + R.chunks * info["launches"] + 1
+    if R.full is not None:
+        # G = 1: the split and the residue solves are ONE plan; time its kernels like the batch arm
+        fplan, fws = R.full
+        finfo = fplan.info
+        NLf = finfo["launches"]
+        fa = [R.ext[t, R.H:R.H + n] for t in range(4)]
+        evk = [[torch.cuda.Event(enable_timing=True) for _ in range(NLf + 1)] for _ in range(K)]
+        torch.cuda.synchronize()
+        for i in range(K):
+            for st in range(NLf):
+                evk[i][st].record()
+                tds.api.solve_stages(fplan, *fa, x, fws, st, st)
+            evk[i][NLf].record()
+        torch.cuda.synchronize()
+        ph = [sum(evk[i][st].elapsed_time(evk[i][st + 1]) for i in range(K)) / K for st in range(NLf)]
+        names = stage_names(finfo)
+        abytes = algorithmic_bytes(dict(finfo, m=1), s)
+        timing_note = ("N = 1: split and residue solves run as ONE plan (passes [k_d] + the residue plan's, x "
+                       "placed in row order); CUDA events between its kernels, K extra steps")
+        n_launch = NLf
+        info = finfo
     dom = int(np.argmax(ph))
     achieved = abytes[dom] / (ph[dom] / 1e3) / 1e9
     roofline = {
@@ -646,8 +670,7 @@ def run_huge(args):
         "share_of_step": ph[dom] / sum(ph),
         "per_kernel": [{"kernel": nm, "ms": t, "algorithmic_bytes": a_, "gbs": a_ / (t / 1e3) / 1e9}
                        for nm, t, a_ in zip(names, ph, abytes)],
-        "kernel_timing": "CUDA events between the phases of K extra steps on rank 0 (phase 2 includes the "
-                         f"all-to-all and x return when N > 1; halo exchange {ph_all[0]:.4f} ms apart)",
+        "kernel_timing": timing_note,
         "step": {"algorithmic_bytes": sum(abytes), "bytes_per_eq": sum(abytes) / B,
                  "gbs": sum(abytes) / (total_ms / K / 1e3) / 1e9,
                  "frac": sum(abytes) / (total_ms / K / 1e3) / 1e9 / hbm_peak},
@@ -705,7 +728,8 @@ def run_huge(args):
                 "on the device by tds_generate_rows)",
         "config": {"workload": f"config5: 1 x {n} {args.dtype} split by rows over {world} GPU(s)", "n": n, "m": 1,
                    "rows_per_rank": B, "k_d": kd, "halo_rows": R.H, "chunks": R.chunks,
-                   "residue_systems_per_rank": R.q, "mode": args.mode, "residue_plan": _plan_summary(info),
+                   "residue_systems_per_rank": R.q, "mode": args.mode, "plan": _plan_summary(info),
+                   "fused_single_gpu_plan": R.full is not None,
                    "launch": "eager (NCCL point-to-point between the kernels)",
                    "l2": "no flush: per-step working set > 10 GiB > L2 126 MiB",
                    "parallelism": f"one system over {world} rank(s): halo exchange + all-to-all of residue classes "
@@ -714,7 +738,7 @@ def run_huge(args):
         "roofline": roofline,
         "cpu_baseline": cpu,
         "e2e": e2e,
-        "gpu_launches": K * (1 + R.chunks * info["launches"] + 1),
+        "gpu_launches": K * n_launch,
         "clocks": clocks,
     }
     print(json.dumps(line), flush=True)

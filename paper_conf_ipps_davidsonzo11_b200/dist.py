@@ -143,6 +143,25 @@ class CudaBackend:
     def unpack(self, xs, out, B: int, kd: int, slot_rows: int):
         api.unpack_residues(xs, out, B, 1, kd, slot_rows)
 
+    def make_full(self, n: int, kd: int, res_plan):
+        """G = 1: the k_d-level split and the residue solves as ONE plan --
+        passes [k_d] + the residue plan's, the residue plan's on-chip shape --
+        so x is placed straight into row order (no x slots round trip, no
+        unpack).  Same per-row arithmetic as the split + residue solves."""
+        p = res_plan.info
+        plan = api.Plan(n, 1, self.name, device=self.device.index or 0, mode="static")
+        keys = ("cr_levels", "thomas_chains", "cluster", "tl_levels", "split_tile_rows", "split_threads", "theta")
+        kw = {k: p[k] for k in keys}
+        try:
+            plan.set_params(k_pass=_schedule(kd) + p["k_pass"], x_group=p["x_group"], **kw)
+        except api.L.TdsError:
+            plan.set_params(k_pass=_schedule(kd) + p["k_pass"], x_group=0, **kw)
+        return plan, plan.workspace()
+
+    def solve_full(self, state, ext, H: int, n: int, out):
+        plan, ws = state
+        api.solve_batched(plan, *(ext[t, H:H + n] for t in range(4)), out=out, workspace=ws)
+
 
 class HugeRank:
     """One rank's buffers, plans and message lists for ``huge_steps`` (all
@@ -188,6 +207,9 @@ class HugeRank:
         self.xs = backend.empty(q, self.stride if G == 1 else NL)
         self.chunk_x = [self.xs[c * qc:(c + 1) * qc] for c in range(chunks)]
         self.xrecv = self.xs if G == 1 else backend.empty(NR, Bj)
+        # G = 1 with a backend that can fuse: split + residue solves as one plan
+        self.full = backend.make_full(n, kd, self.solve_states[0][0]) if G == 1 and hasattr(backend, "make_full") \
+            else None
 
     @property
     def local(self):
@@ -255,6 +277,8 @@ class HugeRank:
                 plan.set_params_list(old)
             new.append((plan, plan.workspace()))
         self.solve_states = new
+        if self.full is not None:
+            self.full = self.be.make_full(self.n, self.kd, self.solve_states[0][0])
 
     def tune_residues(self, cache_path=None) -> list:
         """tds_tune on the residue-solve shape (this rank's device); applied to
@@ -290,6 +314,12 @@ def huge_steps(R: HugeRank, out, mark=None):
         h = yield ("post",) + R.halo_messages()
         yield ("wait", h)
     mark("split")
+    if R.full is not None:  # G = 1, fused: one plan, x straight into row order
+        R.be.solve_full(R.full, R.ext, R.H, R.n, out)
+        mark("exchange_solve")
+        mark("unpack")
+        mark("end")
+        return out
     R.split()
     mark("exchange_solve")
     if R.G > 1:
