@@ -44,6 +44,14 @@ __constant__ int tds_split_ablation;
 #ifndef TDS_SPLIT_STG
 #define TDS_SPLIT_STG 0
 #endif
+// NB is rounded so a residue's positions per tile are whole 16-byte TMA store
+// rows for every CTA size (256-thread k_p = 8: 13 -> 12 B-blocks, so fp64 and
+// 256-thread fp32 tiles leave by TMA tensor stores instead of per-residue
+// scalar STG with 64-bit address arithmetic: config 3 fp64 split 0.285 ->
+// 0.269 ms, gpurun_out/r02i).  -DTDS_SPLIT_NBQ_ALL=0 restores the old rule.
+#ifndef TDS_SPLIT_NBQ_ALL
+#define TDS_SPLIT_NBQ_ALL 1
+#endif
 
 template <int KP, int NT_>
 struct SplitShape {
@@ -61,7 +69,7 @@ struct SplitShape {
     // B blocks stored; with 512 threads rounded so a residue's positions per tile
     // (NB * 256 / 2^KP) stay a 16-byte multiple (TMA store rows)
     static constexpr int NBQ = (KP >= 8 ? 4 : KP == 7 ? 2 : 1);
-    static constexpr int NB = (NT == 512 && !TDS_SPLIT_STG) ? NBMAX - NBMAX % NBQ : NBMAX;
+    static constexpr int NB = ((NT == 512 || TDS_SPLIT_NBQ_ALL) && !TDS_SPLIT_STG) ? NBMAX - NBMAX % NBQ : NBMAX;
     static constexpr int TV = KP > 4 ? NB * 16 * R : AV * R;              // output rows per tile
     static constexpr int HEAD = R + LEFT * R;                             // window rows before the tile
     static_assert(TV % (1 << KP) == 0, "tile must hold whole residue periods");
