@@ -52,6 +52,14 @@ __constant__ int tds_split_ablation;
 #ifndef TDS_SPLIT_NBQ_ALL
 #define TDS_SPLIT_NBQ_ALL 1
 #endif
+// fp64 class transpose in ONE round for the three arrays (class-major
+// [3][16][AV] buffer, XOR-swizzled 16-byte chunks, 92 KB) instead of three
+// rounds through one buffer (6 barriers per tile): 252 -> 212 registers,
+// config 3 fp64 split 0.277 -> 0.268 ms (gpurun_out/r02j).
+// -DTDS_SPLIT_TRC64=0 restores the three-round transpose.
+#ifndef TDS_SPLIT_TRC64
+#define TDS_SPLIT_TRC64 1
+#endif
 
 template <int KP, int NT_>
 struct SplitShape {
@@ -94,7 +102,7 @@ struct SplitShape {
     __host__ __device__ static constexpr bool tstore() { return !TDS_SPLIT_STG && (PT * int(sizeof(T))) % 16 == 0; }
     template <typename T>
     __host__ __device__ static constexpr int tbuf_elems() {
-        const int tr = KP > 4 ? (sizeof(T) == 4 ? 3 : 1) * AV * 16 : 0;
+        const int tr = KP > 4 ? ((sizeof(T) == 4 || TDS_SPLIT_TRC64) ? 3 : 1) * AV * 16 : 0;
         const int so = tstore<T>() ? 3 * TV : 0;
         return tr > so ? tr : so;
     }
@@ -114,7 +122,7 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
     static_assert(ROWS % ELINE == 0, "window of whole lines");
     constexpr int STG = S::template stage_elems<T>();          // elements per array stage (1024-byte multiple)
     constexpr int NA = RAW ? 4 : 3;                            // arrays streamed
-    constexpr int NTR = KP > 4 ? (sizeof(T) == 4 ? 3 : 1) : 0;  // arrays per transpose round
+    constexpr int NTR = KP > 4 ? ((sizeof(T) == 4 || TDS_SPLIT_TRC64) ? 3 : 1) : 0;  // arrays per transpose round
     extern __shared__ __align__(1024) unsigned char smem_raw[];
     T *stage = reinterpret_cast<T *>(smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u));  // 1024-aligned
     T *tbuf = stage + NA * STG;  // [NTR][AV * 16] transpose buffer / [3][TV] output staging
@@ -356,7 +364,7 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
             const int rho = t / CH, b = t % CH;
             const int mb = LEFT - 16 + 16 * b;  // member of u = 0
             const bool wr = lane >= 1 && lane <= 30;
-            if constexpr (NTR == 3) {  // fp32, one round: 3 class-major buffers [rho][m]
+            if constexpr (NTR == 3 && sizeof(T) == 4) {  // fp32, one round: 3 class-major buffers [rho][m]
                 if (wr) {
                     const int pm = trc_phys(ablk - 1);
                     trc_write<T, R, AV>(ra, tbuf + pm);
@@ -369,6 +377,19 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
                 trc_read<R>(ra, tbuf + rho * AV, ch);
                 trc_read<R>(rc, tbuf + AV * 16 + rho * AV, ch);
                 trc_read<R>(rd, tbuf + 2 * AV * 16 + rho * AV, ch);
+            } else if constexpr (NTR == 3) {  // fp64, one round (TDS_SPLIT_TRC64)
+                if (wr) {
+                    const int pm = trc_phys64(ablk - 1);
+                    trc_write<T, R, AV>(ra, tbuf + pm);
+                    trc_write<T, R, AV>(rc, tbuf + AV * 16 + pm);
+                    trc_write<T, R, AV>(rd, tbuf + 2 * AV * 16 + pm);
+                }
+                __syncthreads();
+                int ch[R / 2];
+                trc_read_chunks64<R, AV>(mb, ch);
+                trc_read64<R>(ra, tbuf + rho * AV, ch);
+                trc_read64<R>(rc, tbuf + AV * 16 + rho * AV, ch);
+                trc_read64<R>(rd, tbuf + 2 * AV * 16 + rho * AV, ch);
             } else {
                 int ad[R];
                 tr_read_addrs<R, AV, (LEFT - 16) & 15>(mb, rho, ad);  // three rounds through one buffer

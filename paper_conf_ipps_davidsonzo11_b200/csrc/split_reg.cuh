@@ -226,6 +226,39 @@ __device__ __forceinline__ void trc_read(float (&x)[R], const float *row, const 
     }
 }
 
+// fp64 class-major buffer [rho][m] (row stride AV doubles): member m at
+// 2 * (c ^ ((c >> 3) & 7)) + (m & 1), c = m >> 1 (16-byte chunks of two
+// members XOR-swizzled by the 128-byte block).  Layout-A writes are 16 scalar
+// stores of consecutive m across the warp; layout-B reads are 8 LDS.128 of two
+// consecutive members each, lanes 16 members apart: the 8 lanes of a
+// quarter-warp hit 8 different bank groups.
+__device__ __forceinline__ int trc_phys64(int m) {
+    const int c = m >> 1;
+    return ((c ^ ((c >> 3) & 7)) << 1) | (m & 1);
+}
+
+template <int R, int AV>
+__device__ __forceinline__ void trc_read_chunks64(int mb, int (&ch)[R / 2]) {
+#pragma unroll
+    for (int q = 0; q < R / 2; ++q) {
+        int c = mb / 2 + q;  // chunks outside [0, AV/2): a neighbouring lane's chunk (broadcast)
+        c = c < 0 ? c + 8 : c;
+        c = c > AV / 2 - 1 ? c - 8 : c;
+        c = c > AV / 2 - 1 ? c - 8 : c;
+        ch[q] = (c ^ ((c >> 3) & 7)) << 1;
+    }
+}
+
+template <int R>
+__device__ __forceinline__ void trc_read64(double (&x)[R], const double *row, const int (&ch)[R / 2]) {
+#pragma unroll
+    for (int q = 0; q < R / 2; ++q) {
+        const double2 f = *reinterpret_cast<const double2 *>(row + ch[q]);
+        x[2 * q] = f.x;
+        x[2 * q + 1] = f.y;
+    }
+}
+
 template <typename T, int R>
 __device__ __forceinline__ void tr_read(T (&x)[R], const T *buf, const int (&ad)[R]) {
 #pragma unroll
