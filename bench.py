@@ -376,14 +376,15 @@ def run_tds(args):
     seed = inputs.config_seed(args.config, dt)
     # strong scaling: the config's M systems in total, shard_range blocks per rank;
     # weak: M systems per rank (global indices rank * M ...)
+    if args.scaling == "strong" and M < world:  # fewer systems than ranks: nothing to shard
+        print(f"warning: {M} systems cannot feed {world} ranks under strong scaling; running weak", file=sys.stderr)
+        args.scaling = "weak"
     if args.scaling == "strong":
         s0, s1 = tdist.shard_range(M, world, rank)
     else:
         s0, s1 = rank * M, (rank + 1) * M
     m = s1 - s0
     m_total = M if args.scaling == "strong" else M * world
-    if m < 1:
-        raise SystemExit(f"strong scaling: {M} systems cannot feed {world} ranks")
     # inputs drawn on the device (G4 generator, bit-identical to inputs.py)
     ta, tb, tc, td = tds.generate(n, m, name, seed=seed, first_system=s0, device=hz.local)
     x = torch.empty_like(td)
