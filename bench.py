@@ -376,7 +376,7 @@ def run_tds(args):
     seed = inputs.config_seed(args.config, dt)
     # strong scaling: the config's M systems in total, shard_range blocks per rank;
     # weak: M systems per rank (global indices rank * M ...)
-    if args.scaling == "strong" and M < world:  # fewer systems than ranks: nothing to shard
+    if args.scaling == "strong" and M - (world - 1) * (-(-M // world)) < 1:  # some rank would get no system
         print(f"warning: {M} systems cannot feed {world} ranks under strong scaling; running weak", file=sys.stderr)
         args.scaling = "weak"
     if args.scaling == "strong":
