@@ -51,3 +51,19 @@ def test_tds_arm_config5_huge_system():
     assert d["scaling"] == "strong" and d["config"]["m"] == 1 and d["config"]["fused_single_gpu_plan"] is True
     assert d["config"]["interior_residual"] <= 1e-5
     assert d["roofline"]["nvlink_bytes_per_rank"]["all_to_all_split"] == 0
+
+
+def test_algorithmic_bytes_accounting():
+    """split pass 1 7 s/eq, later passes 6 s, on-chip 4 s (5 s
+    at k = 0), placement 2 s (k > 0, no x_group / strided)."""
+    sys.path.insert(0, ROOT)
+    import bench
+    info = dict(n=1 << 20, m=16, passes=1, k=7, k_pass=[7], x_group=0, strided=0)
+    eqs = 16 << 20
+    assert bench.algorithmic_bytes(info, 4) == [28 * eqs, 16 * eqs, 8 * eqs]  # 52 B/eq (SURVEY §8(d))
+    assert bench.stage_names(info) == ["split_pass_0(k_p=7)", "onchip_cr_pcr_thomas", "place_x"]
+    two = dict(info, passes=2, k=15, k_pass=[8, 7], m=1, n=1 << 28)
+    assert sum(bench.algorithmic_bytes(two, 4)) == 76 * (1 << 28)  # config 5: 28 + 24 + 16 + 8 B/eq
+    k0 = dict(info, passes=0, k=0, k_pass=[])
+    assert bench.algorithmic_bytes(k0, 4) == [20 * eqs]
+    assert bench.algorithmic_bytes(dict(info, x_group=8), 8) == [56 * eqs, 32 * eqs]
