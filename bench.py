@@ -202,7 +202,7 @@ def cpu_oracle_time(a, b, c, d, repeats=3, budget_s=25.0):
     # bounded sample: as many whole systems as fit ~2^25 rows (all of them for configs 1-3)
     ms = max(1, min(m, (1 << 25) // n))
     a64, b64, c64, d64 = (np.ascontiguousarray(v[:ms], dtype=np.float64) for v in (a, b, c, d))  # upcast: untimed
-    threads = min(oracle.num_threads(), ms)
+    threads = min(host_cores(), ms)  # the box's cores (torchrun sets OMP_NUM_THREADS=1)
     times, x = [], None
     t_start = time.perf_counter()
     for _ in range(repeats):
@@ -234,7 +234,7 @@ def run_reference(args):
         ns, ms = n, max(1, min(m, (1 << 25) // n))
     a, b, c, d = inputs.generate(ns, ms, dt, seed=inputs.config_seed(args.config, dt))
     a64, b64, c64, d64 = (np.ascontiguousarray(v, dtype=np.float64) for v in (a, b, c, d))
-    threads = min(oracle.num_threads(), ms)
+    threads = min(host_cores(), ms)  # the box's cores (torchrun sets OMP_NUM_THREADS=1)
     for _ in range(args.warmup):
         oracle.thomas(a64, b64, c64, d64, threads=threads)
     t0 = time.perf_counter()
