@@ -401,3 +401,31 @@ def test_huge_loopback_gpu_coupling(family, kw, kd, chunks):
         if ref is None:
             ref = x
         assert np.array_equal(x, ref), G
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("stride_pad,kp", [(3, [2]), (3, [6]), (16, [7]), (5, [4, 3])])
+def test_solve_normalized_padded_strides(stride_pad, kp):
+    """tds_solve_normalized with a padded (and for odd pads, non-16-byte)
+    batch stride: the register / shared-memory split kernels read the
+    normalised caller arrays; equal to the materialised-b = 1 solve and the
+    oracle; the padding is untouched."""
+    import paper_conf_ipps_davidsonzo11_b200 as tds
+    n, m = 50000, 3
+    stride = n + stride_pad
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=12)
+    an, cn, dn = (v / b for v in (a, c, d))
+    pad = lambda v: np.pad(v, ((0, 0), (0, stride_pad)), constant_values=7.0).reshape(-1)
+    ta, tc, td = (torch.from_numpy(pad(v)).cuda() for v in (an, cn, dn))
+    plan = tds.Plan(n, m, "float32", device=0, batch_stride=stride)
+    R = 16 if -(-n // (1 << sum(kp))) > 4096 else 8
+    plan.set_params(k_pass=kp, cluster=1, cr_levels=R.bit_length() - 1, thomas_chains=1, tl_levels=5)
+    out = torch.full_like(td, 7.0)
+    tds.api.solve_normalized(plan, ta, tc, td, out=out)
+    x2 = tds.solve_batched(plan, ta, torch.ones_like(ta), tc, td)
+    torch.cuda.synchronize()
+    xs = out.cpu().numpy().reshape(m, stride)
+    assert np.all(xs[:, n:] == 7.0)
+    assert np.array_equal(xs[:, :n], x2.cpu().numpy().reshape(m, stride)[:, :n])
+    xr = oracle.thomas(an, np.ones_like(an), cn, dn)
+    assert oracle.rel_err(xs[:, :n], xr) <= 1e-4
