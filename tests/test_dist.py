@@ -404,7 +404,7 @@ def test_huge_loopback_gpu_coupling(family, kw, kd, chunks):
 
 
 @pytest.mark.gpu
-@pytest.mark.parametrize("stride_pad,kp", [(3, [2]), (3, [6]), (16, [7]), (5, [4, 3])])
+@pytest.mark.parametrize("stride_pad,kp", [(3, [3]), (3, [6]), (16, [7]), (5, [4, 3])])
 def test_solve_normalized_padded_strides(stride_pad, kp):
     """tds_solve_normalized with a padded (and for odd pads, non-16-byte)
     batch stride: the register / shared-memory split kernels read the
