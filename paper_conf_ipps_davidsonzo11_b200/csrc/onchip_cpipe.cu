@@ -165,6 +165,7 @@ __global__ void __launch_bounds__(512, 1)
     for (int64_t it = 0;; ++it) {
         const int64_t sys = cid + it * ncl;
         if (sys >= A.m_systems) break;
+        pdl_trigger_if_last(sys + ncl >= A.m_systems);
         T *top = top_base + int(it & 1) * 3 * ZMAX;
         mbar_wait(&full_bar, uint32_t(it & 1));
         const int64_t i0 = row0 + int64_t(t) * R;  // first row of this thread

@@ -260,6 +260,7 @@ __global__ void __launch_bounds__(R * sizeof(T) == 32 ? 1024 : 512, 1)
     for (int64_t it = 0;; ++it) {
         const int64_t q = int64_t(blockIdx.x) + it * gridDim.x;
         if (q >= nslots) break;
+        pdl_trigger_if_last(q + gridDim.x >= nslots);
         const int64_t sigma = nslots - 1 - q;
         const int s = int(it & 1);
         const int64_t L = slot_len(sigma);

@@ -18,6 +18,15 @@ namespace tds {
 // on the stream drains; every thread waits here for that kernel's completion
 // and memory before its first global-memory access.  A no-op for a normal launch.
 __device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
+// Experiment switch (-DTDS_PDL_TRIGGER=1): a CTA that starts its LAST work item
+// lets the next kernel on the stream launch (its CTAs take the SMs this grid's
+// finished CTAs free; they still wait in pdl_wait for this grid's completion).
+#ifndef TDS_PDL_TRIGGER
+#define TDS_PDL_TRIGGER 0
+#endif
+__device__ __forceinline__ void pdl_trigger_if_last(bool last) {
+    if (TDS_PDL_TRIGGER && last) asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
+}
 
 // Host: per-launch setup that does not change between solves -- the dynamic
 // shared-memory opt-in, the non-portable cluster opt-in and the occupancy

@@ -220,6 +220,7 @@ __global__ void __launch_bounds__(kTpThreads) place_x_tma_kernel(const PlaceArgs
     for (int64_t it = 0;; ++it) {
         const int64_t w = int64_t(blockIdx.x) + it * gridDim.x;
         if (w >= ntiles) break;
+        pdl_trigger_if_last(w + gridDim.x >= ntiles);
         const int s = int(it & 1);
         mbar_wait(&full[s], uint32_t((it >> 1) & 1));
         if (l2_discard && t < NBX * E) {  // the x-slot lines of this tile are dead once in shared memory

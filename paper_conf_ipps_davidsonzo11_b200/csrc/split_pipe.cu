@@ -205,6 +205,7 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
     for (int64_t it = 0;; ++it) {
         const int64_t w = int64_t(blockIdx.x) + it * gridDim.x;
         if (w >= nitems) break;
+        pdl_trigger_if_last(w + gridDim.x >= nitems);
         int64_t sigma, t0, L, g0, gt;
         item_rows(w, sigma, t0, L, g0, gt);
         if (!TDS_ABL(2)) mbar_wait(&bar, uint32_t(it & 1));
