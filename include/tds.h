@@ -193,7 +193,13 @@ tds_status tds_plan_destroy(tds_plan_t plan);
  * Allocates and frees its own device buffers; synchronises `cuda_stream`.
  * cache_path (host string, may be NULL => $TDS_TUNE_CACHE or no cache): a
  * text file of saved results keyed by device, dtype, n and m ("save those
- * results for future runs"); a hit skips the search.
+ * results for future runs"); a hit skips the search.  A trial
+ * is the median over several samples of back-to-back solves (>= ~0.4 ms per
+ * sample); the Thomas switch T is not searched in the warp form (no T).  A
+ * trial that faults the device (sticky CUDA error) aborts the search with
+ * TUNE; the chosen parameters must reproduce the seed plan's x on the trial
+ * systems (relative 2e-4 fp32 / 1e-9 fp64) before they and the cache line
+ * are committed -- on any error the plan is unchanged.
  * Errors: INVALID_ARG, DEVICE_MISMATCH, NO_MEMORY, CUDA, TUNE. */
 tds_status tds_tune(tds_plan_t plan, void *cuda_stream, const char *cache_path);
 
