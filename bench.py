@@ -71,6 +71,9 @@ def parse():
                     help="override the config's number of systems M (probe: one rank's share of a strong-scaled "
                          "batch, e.g. --systems 2 = config 3 at 8 GPUs)")
     ap.add_argument("--huge-kd", type=int, default=8, help="config 5: levels split before the exchange")
+    ap.add_argument("--huge-transport", default="peer", choices=["peer", "p2p"],
+                    help="config 5, N > 1: peer = the split writes residue classes into the owners' symmetric "
+                         "memory (fused all-to-all); p2p = NCCL point-to-point of the slot segments")
     ap.add_argument("--huge-chunks", type=int, default=4, help="config 5: residue groups overlapped with the "
                                                              "all-to-all (N > 1)")
     return ap.parse_args()
@@ -587,7 +590,30 @@ def run_huge(args):
     kd = max(args.huge_kd, int(math.log2(world)) if world > 1 else 0)
     chunks = args.huge_chunks if world > 1 else 1
     be = tdist.CudaBackend(tdt, dev)
-    R = tdist.HugeRank(n, world, rank, be, kd=kd, chunks=chunks)
+    transport = tdist.P2PTransport()
+    transport_kind = "p2p"
+    R = None
+    if world > 1 and args.huge_transport == "peer":
+        # the residue buffers in torch symmetric memory: every rank's split writes each residue
+        # class straight into its owner over NVLink (tds_split_scatter), then a device barrier
+        try:
+            import torch.distributed._symmetric_memory as symm_mem
+            grp = hz.dist.group.WORLD
+            try:
+                symm_mem.enable_symm_mem_for_group(grp.group_name)
+            except Exception:
+                pass
+            R = tdist.HugeRank(n, world, rank, be, kd=kd, chunks=chunks,
+                               sys_alloc=lambda shape: symm_mem.empty(*shape, dtype=tdt, device=dev))
+            handle = symm_mem.rendezvous(R.sys_buf, grp)
+            R.set_peers([int(p_) for p_ in handle.buffer_ptrs])
+            transport = tdist.P2PTransport(symm=handle)
+            transport_kind = "peer (split + all-to-all fused: tds_split_scatter into symmetric memory)"
+        except Exception as e:  # no symmetric memory here: the point-to-point all-to-all
+            print(f"warning: peer mode unavailable ({e}); point-to-point all-to-all", file=sys.stderr)
+            R = None
+    if R is None:
+        R = tdist.HugeRank(n, world, rank, be, kd=kd, chunks=chunks)
     trials = 0
     if args.mode == "tuned":
         # the residue solves' plan: tuned on rank 0, broadcast (identical kernels on every rank)
@@ -602,7 +628,6 @@ def run_huge(args):
             R.set_residue_params(vec.tolist())
     tds.api.generate_rows(n, rank * R.B, R.B, name, seed=seed, out=R.local, device=hz.local)
     x = be.empty(R.B)
-    transport = tdist.P2PTransport()
 
     def solve():
         tdist.run_steps(tdist.huge_steps(R, x), transport)
@@ -731,7 +756,7 @@ def run_huge(args):
                    "rows_per_rank": B, "k_d": kd, "halo_rows": R.H, "chunks": R.chunks,
                    "residue_systems_per_rank": R.q, "mode": args.mode, "plan": _plan_summary(info),
                    "fused_single_gpu_plan": R.full is not None,
-                   "launch": "eager (NCCL point-to-point between the kernels)",
+                   "launch": "eager (NCCL point-to-point between the kernels)", "transport": transport_kind,
                    "l2": "no flush: per-step working set > 10 GiB > L2 126 MiB",
                    "parallelism": f"one system over {world} rank(s): halo exchange + all-to-all of residue classes "
                                   "(dist.solve_huge)",

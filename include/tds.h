@@ -288,6 +288,32 @@ tds_status tds_plan_slots_layout(const tds_plan_t plan, tds_slots_layout *out);
 tds_status tds_split_slots(const tds_plan_t plan, const void *a, const void *b, const void *c, const void *d,
                            void *workspace, size_t workspace_bytes, void *cuda_stream);
 
+/* The split pass with the all-to-all of the one-huge-system path FUSED into
+ * its output (the paper's Stage 1, over several GPUs): the plan's
+ * ONE split pass (m = 1 system, k <= 8 levels, 16-byte aligned a, b, c, d)
+ * writes residue class r = h q + rl (q = residues_per_group) straight into
+ * destination h's arrays: normalised a', c', d' of position first_pos + j of
+ * residue r go to dst[t][h][rl * dst_stride + j] for j in [0, num_pos) -- each
+ * tile's outputs leave by TMA tensor stores, so on a multi-GPU node the
+ * transfer to peer memory (dst pointers mapped from other GPUs, e.g. torch
+ * symmetric memory over NVLink) overlaps the split tile by tile; positions
+ * outside the window (the halo) are not written.  No workspace.  The caller
+ * orders the destinations' readers after this call (a barrier across the
+ * ranks).  Errors: INVALID_ARG (NULL, groups not in [1, 8], groups * q != 2^k,
+ * window outside floor(n / 2^k), dst_stride < num_pos or not a 16-byte
+ * multiple, NULL / misaligned / overlapping dst), UNSUPPORTED (m != 1, not
+ * one pass of <= 8 levels, misaligned inputs), CUDA. */
+typedef struct {
+    int32_t groups;             /* destinations (GPUs), <= 8                         */
+    int32_t residues_per_group; /* q: residues [h q, (h+1) q) go to destination h    */
+    int64_t first_pos;          /* first slot position stored of every residue       */
+    int64_t num_pos;            /* positions stored per residue                      */
+    int64_t dst_stride;         /* elements between consecutive residues at a dst    */
+    void *dst[3][8];            /* [a', c', d'][destination]: device (or peer) bases */
+} tds_scatter;
+tds_status tds_split_scatter(const tds_plan_t plan, const void *a, const void *b, const void *c, const void *d,
+                             const tds_scatter *spec, void *cuda_stream);
+
 /* The residue-class -> original-order transpose of Fig. 3a:
  * x[s * batch_stride + r + 2^k j] = xs[((s << k) + r) * slot_rows + j] for
  * every system s < m, residue r < 2^k and row r + 2^k j < n.  xs, x: device,

@@ -28,6 +28,7 @@ EXPORTED = (
     "tds_interleaved_workspace_bytes", "tds_solve_interleaved",
     "tds_last_error", "tds_version", "tds_tune_search", "tds_generate", "tds_generate_rows",
     "tds_solve_normalized", "tds_plan_slots_layout", "tds_split_slots", "tds_unpack_residues",
+    "tds_split_scatter",
 )
 
 
@@ -66,6 +67,12 @@ class PlanInfo(ctypes.Structure):
 class SlotsLayout(ctypes.Structure):
     _fields_ = [("a_offset", ctypes.c_int64), ("c_offset", ctypes.c_int64), ("d_offset", ctypes.c_int64),
                 ("slot_rows", ctypes.c_int64), ("num_slots", ctypes.c_int64)]
+
+
+class Scatter(ctypes.Structure):
+    _fields_ = [("groups", ctypes.c_int32), ("residues_per_group", ctypes.c_int32),
+                ("first_pos", ctypes.c_int64), ("num_pos", ctypes.c_int64), ("dst_stride", ctypes.c_int64),
+                ("dst", (ctypes.c_void_p * 8) * 3)]
 
 
 # tds_tune_search's cost callback: double (*)(const tds_params *, void *)
@@ -107,6 +114,7 @@ def load() -> ctypes.CDLL:
         "tds_plan_slots_layout": (I32, [P, ctypes.POINTER(SlotsLayout)]),
         "tds_split_slots": (I32, [P, VP, VP, VP, VP, VP, SZ, VP]),
         "tds_unpack_residues": (I32, [I32, I64, I64, I32, I64, VP, VP, I64, VP]),
+        "tds_split_scatter": (I32, [P, VP, VP, VP, VP, ctypes.POINTER(Scatter), VP]),
         "tds_status_string": (ctypes.c_char_p, [I32]),
         "tds_last_error": (ctypes.c_char_p, []),
         "tds_version": (I32, []),

@@ -275,6 +275,29 @@ def split_slots(plan: Plan, a, b, c, d, workspace, stream=None):
     return slot_views(plan, workspace, lay)
 
 
+def split_scatter(plan: Plan, a, b, c, d, dst, residues_per_group: int, first_pos: int, num_pos: int,
+                  dst_stride: int, stream=None):
+    """tds_split_scatter: the plan's one split pass with the all-to-all fused
+    into its stores -- residue h q + rl of position first_pos + j goes to
+    dst[t][h] + (rl * dst_stride + j) elements (t = a', c', d').  ``dst``: 3
+    lists of device addresses (ints; peer-mapped addresses allowed) or
+    tensors, one per destination."""
+    info, need, want, dev = plan._solve_info()
+    for name, t in (("a", a), ("b", b), ("c", c), ("d", d)):
+        _check_fast(t, need, want, name, dev)
+    spec = L.Scatter()
+    groups = len(dst[0])
+    spec.groups, spec.residues_per_group = groups, int(residues_per_group)
+    spec.first_pos, spec.num_pos, spec.dst_stride = int(first_pos), int(num_pos), int(dst_stride)
+    for t in range(3):
+        if len(dst[t]) != groups:
+            raise ValueError("dst: the same number of destinations for a', c', d'")
+        for h, p in enumerate(dst[t]):
+            spec.dst[t][h] = p if isinstance(p, int) else p.data_ptr()
+    L.check(plan._lib.tds_split_scatter(plan.handle, a.data_ptr(), b.data_ptr(), c.data_ptr(), d.data_ptr(),
+                                        ctypes.byref(spec), _stream_ptr(stream, dev)))
+
+
 def slot_views(plan: Plan, workspace, lay: Optional[dict] = None):
     """(a', c', d') views of the split slots inside ``workspace`` (no device work)."""
     info, _, want, _ = plan._solve_info()

@@ -77,7 +77,7 @@ static WsBufs<T> ws_bufs(const tds_plan_info &I, void *ws) {
 template <typename T>
 static tds_status run_split(const tds_plan_info &I, const T *a, const T *b, const T *c, const T *d,
                             const WsBufs<T> &w, cudaStream_t st, int *out_buf, int first = 0,
-                            int last = 1 << 30, bool natural = false) {
+                            int last = 1 << 30, bool natural = false, const ScatterHost *sc = nullptr) {
     const tds_params &P = I.params;
     int kprev = 0;
     for (int p = 0; p < P.passes; ++p) {
@@ -125,9 +125,11 @@ static tds_status run_split(const tds_plan_info &I, const T *a, const T *b, cons
         const int64_t grid = m_in * A.segs;
         if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "split grid exceeds 2^31-1 CTAs");
         cudaError_t err;
+        if (sc && !(kp <= kPipeSplitMaxKp && A.vec))
+            return fail(TDS_ERR_UNSUPPORTED, "a scatter needs the TMA split kernel (k <= 8, 16-byte aligned rows)");
         if (kp <= kPipeSplitMaxKp && A.vec) {
             // persistent, TMA-prefetched register kernel (16-byte aligned rows)
-            err = launch_split_pipe<T>(A, raw, m_in, len_in, I.params.split_threads, st);
+            err = launch_split_pipe<T>(A, raw, m_in, len_in, I.params.split_threads, st, sc);
         } else if (kp <= kRegSplitMaxKp) {
             err = launch_split_reg<T>(A, raw, grid, st);
         } else {
@@ -533,6 +535,57 @@ tds_status tds_split_slots(const tds_plan_t plan, const void *a, const void *b, 
         WsBufs<double> w = ws_bufs<double>(I, workspace);
         s = run_split<double>(I, (const double *)a, (const double *)b, (const double *)c, (const double *)d, w, st,
                               &ob);
+    }
+    if (s == TDS_OK) clear_error();
+    return s;
+}
+
+tds_status tds_split_scatter(const tds_plan_t plan, const void *a, const void *b, const void *c, const void *d,
+                             const tds_scatter *spec, void *cuda_stream) {
+    if (!plan || !spec) return fail(TDS_ERR_INVALID_ARG, "NULL argument");
+    const tds_plan_info &I = plan->info;
+    const tds_params &P = I.params;
+    if (P.passes != 1 || P.k_pass[0] > kPipeSplitMaxKp || I.m != 1 || P.strided || I.chunks != 1)
+        return fail(TDS_ERR_UNSUPPORTED, "a scatter needs one system (m = 1) split in ONE pass of <= 8 levels");
+    const int64_t NR = int64_t(1) << P.k;
+    if (spec->groups < 1 || spec->groups > 8 || int64_t(spec->residues_per_group) * spec->groups != NR)
+        return fail(TDS_ERR_INVALID_ARG, "groups in [1, 8] and groups * residues_per_group == 2^k");
+    const int64_t es = dsize(I.dtype);
+    if (spec->first_pos < 0 || spec->num_pos < 1 || spec->first_pos + spec->num_pos > I.n / NR ||
+        spec->dst_stride < spec->num_pos || (spec->dst_stride * es) % 16)
+        return fail(TDS_ERR_INVALID_ARG, "positions [first_pos, first_pos + num_pos) within floor(n / 2^k); "
+                                         "dst_stride >= num_pos, a 16-byte multiple");
+    tds_status s = check_arrays(I, {a, b, c, d});
+    if (s != TDS_OK) return s;
+    if (!vec_ok(I, {a, b, c, d})) return fail(TDS_ERR_UNSUPPORTED, "a scatter needs 16-byte aligned a, b, c, d");
+    ScatterHost sc{};
+    sc.groups = spec->groups;
+    sc.q = spec->residues_per_group;
+    sc.first_pos = spec->first_pos;
+    sc.num_pos = spec->num_pos;
+    sc.dst_stride = spec->dst_stride;
+    const size_t bytes = size_t(((I.m - 1) * I.batch_stride + I.n) * es);
+    const size_t dbytes = size_t((int64_t(sc.q - 1) * spec->dst_stride + spec->num_pos) * es);
+    for (int t = 0; t < 3; ++t)
+        for (int h = 0; h < sc.groups; ++h) {
+            const void *p = spec->dst[t][h];
+            if (!p || reinterpret_cast<uintptr_t>(p) % 16) return fail(TDS_ERR_INVALID_ARG, "NULL or misaligned dst");
+            for (const void *q : {a, b, c, d})
+                if (overlaps(p, dbytes, q, bytes)) return fail(TDS_ERR_INVALID_ARG, "dst overlaps an input");
+            sc.dst[t][h] = spec->dst[t][h];
+        }
+    if ((s = check_geometry(I)) != TDS_OK) return s;
+    if ((s = check_device(plan)) != TDS_OK) return s;
+    cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
+    int ob = 0;
+    if (I.dtype == TDS_F32) {
+        WsBufs<float> w{};
+        s = run_split<float>(I, (const float *)a, (const float *)b, (const float *)c, (const float *)d, w, st, &ob, 0,
+                             1 << 30, false, &sc);
+    } else {
+        WsBufs<double> w{};
+        s = run_split<double>(I, (const double *)a, (const double *)b, (const double *)c, (const double *)d, w, st,
+                              &ob, 0, 1 << 30, false, &sc);
     }
     if (s == TDS_OK) clear_error();
     return s;

@@ -136,6 +136,19 @@ struct SplitArgs {
     int32_t vec;             // input rows may be read with 16-byte vector loads
     PassGeom geom;           // passes applied to the input
     int32_t natural;         // output rows in original order (strided variant; first pass, k_p <= 4)
+    // fused split + all-to-all (tds_split_scatter): > 0 destinations; residues
+    // [h q, (h+1) q) of the tile go to destination h, positions shifted by -sc_first
+    int32_t sc_groups, sc_q;
+    int64_t sc_first;
+};
+
+// Host description of a scatter (tds_split_scatter): per destination h and
+// array t a base pointer; the destination is a [q][dst_stride] block of which
+// positions [0, num_pos) of every residue row are written.
+struct ScatterHost {
+    int32_t groups, q;
+    int64_t first_pos, num_pos, dst_stride;
+    void *dst[3][8];
 };
 
 template <typename T>
@@ -166,7 +179,7 @@ template <typename T>
 cudaError_t launch_split_reg(const SplitArgs<T> &A, bool raw, int64_t grid, cudaStream_t st);
 template <typename T>
 cudaError_t launch_split_pipe(const SplitArgs<T> &A, bool raw, int64_t m_in, int64_t max_len, int threads,
-                              cudaStream_t st);
+                              cudaStream_t st, const ScatterHost *sc = nullptr);
 template <typename T>
 cudaError_t launch_onchip_pipe(const OnchipArgs<T> &A, int64_t nslots, int threads, int cr_levels, int sm_count,
                                size_t smem, cudaStream_t st);

@@ -166,6 +166,10 @@ __device__ __forceinline__ void bulk_g2s(void *dst, const void *src, uint32_t by
 struct TmapSet {
     CUtensorMap m[4];
 };
+// the scatter views of a fused split + all-to-all: [array][destination], <= 8 destinations
+struct TmapSet24 {
+    CUtensorMap m[24];
+};
 
 __device__ __forceinline__ void tma_load_lines(void *dst, const CUtensorMap *map, int line, int slot, uint64_t *bar) {
     asm volatile(

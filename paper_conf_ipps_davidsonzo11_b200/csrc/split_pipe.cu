@@ -115,7 +115,7 @@ struct SplitShape {
 template <typename T, int KP, bool RAW, int NT>
 __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
     split_pipe_kernel(const SplitArgs<T> A, int64_t tps, int64_t nitems, const __grid_constant__ TmapSet tm,
-                      int32_t tma_lines, const __grid_constant__ TmapSet tmo) {
+                      int32_t tma_lines, const __grid_constant__ TmapSet tmo, const __grid_constant__ TmapSet24 tms) {
     using S = SplitShape<KP, NT>;
     constexpr int R = S::R, AV = S::AV, TV = S::TV, HEAD = S::HEAD, ROWS = S::ROWS, CH = S::CH;
     constexpr int TOFF = S::template toff<T>(), BL = S::template box_lines<T>(), ELINE = 128 / int(sizeof(T));
@@ -180,7 +180,18 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
     auto tma_store_tile = [&](int64_t sigma, int64_t t0, int kp_prev) {
         fence_proxy_async_smem();  // generic-proxy smem writes -> visible to the TMA
         __syncthreads();
-        if (t == 0 && !TDS_ABL(4)) {
+        if (t == 0 && !TDS_ABL(4) && A.sc_groups > 0) {
+            // fused all-to-all: residues [h q, (h+1) q) of the tile go straight to destination
+            // h's residue systems ({position, residue} view, positions shifted by -sc_first;
+            // the TMA unit drops the halo positions outside [0, num_pos))
+            const int j0 = int((t0 >> KP) - A.sc_first);
+            for (int q = 0; q < 3; ++q)
+                for (int bx = 0; bx < NBOX; ++bx)
+                    for (int h = 0; h < A.sc_groups; ++h)
+                        tma_store_box3(&tms.m[q * A.sc_groups + h],
+                                       tbuf + q * TV + bx * NRES * BOXP + h * A.sc_q * BOXP, j0 + bx * BOXP, 0, 0);
+            bulk_commit();
+        } else if (t == 0 && !TDS_ABL(4)) {
             const int j0 = int(t0 >> KP), r = int(sigma & ((int64_t(1) << kp_prev) - 1)), sys = int(sigma >> kp_prev);
 #pragma unroll
             for (int q = 0; q < 3; ++q)
@@ -473,7 +484,8 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
 }
 
 template <typename T, int KP, bool RAW, int NT>
-static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_len, cudaStream_t st) {
+static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_len, cudaStream_t st,
+                             const ScatterHost *sc) {
     using S = SplitShape<KP, NT>;
     auto kern = split_pipe_kernel<T, KP, RAW, NT>;
     const size_t smem = S::template smem_bytes<T>(RAW);
@@ -502,7 +514,30 @@ static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_le
                 return cudaErrorInvalidValue;
     }
     TmapSet tmo{};
-    if constexpr (S::template tstore<T>()) {  // output view {position, r, rho, system}
+    TmapSet24 tms{};
+    SplitArgs<T> B = A;
+    B.sc_groups = 0;
+    if (sc) {  // fused split + all-to-all: one {position, residue} view per destination and array
+        if constexpr (!S::template tstore<T>() || !RAW) {
+            return cudaErrorNotSupported;
+        } else {
+            if (sc->groups < 1 || sc->groups > 8 || sc->q * sc->groups != (1 << KP) || m_in != 1)
+                return cudaErrorInvalidValue;
+            for (int q = 0; q < 3; ++q)
+                for (int h = 0; h < sc->groups; ++h) {
+                    const uint64_t dims[3] = {uint64_t(sc->num_pos), uint64_t(sc->q), 1};
+                    const uint64_t strides[2] = {uint64_t(sc->dst_stride) * sizeof(T),
+                                                 uint64_t(sc->dst_stride) * sizeof(T) * uint64_t(sc->q)};
+                    const uint32_t box[3] = {uint32_t(S::BOXP), uint32_t(sc->q), 1};
+                    if (!encode_box3_tmap_plain(&tms.m[q * sc->groups + h], sc->dst[q][h], int(sizeof(T)), dims,
+                                                strides, box))
+                        return cudaErrorInvalidValue;
+                }
+            B.sc_groups = sc->groups;
+            B.sc_q = sc->q;
+            B.sc_first = sc->first_pos;
+        }
+    } else if constexpr (S::template tstore<T>()) {  // output view {position, r, rho, system}
         T *outs[3] = {A.oa, A.oc, A.od};
         const int64_t msys = m_in >> kprev;
         for (int q = 0; q < 3; ++q)
@@ -518,24 +553,25 @@ static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_le
         cudaMemcpyToSymbolAsync(tds_split_ablation, &v, sizeof(int), 0, cudaMemcpyHostToDevice, st);
     }
 #endif
-    cudaError_t le = launch_pdl(kern, dim3(unsigned(grid)), dim3(S::NT), smem, st, 1, A, tps, nitems, tm,
-                                int32_t(tma_lines), tmo);
+    cudaError_t le = launch_pdl(kern, dim3(unsigned(grid)), dim3(S::NT), smem, st, 1, B, tps, nitems, tm,
+                                int32_t(tma_lines), tmo, tms);
     if (le != cudaSuccess) return le;
     return cudaGetLastError();
 }
 
 template <typename T>
 cudaError_t launch_split_pipe(const SplitArgs<T> &A, bool raw, int64_t m_in, int64_t max_len, int threads,
-                              cudaStream_t st) {
+                              cudaStream_t st, const ScatterHost *sc) {
     // fp32: 512 threads (1 CTA/SM, 7.7K-row windows, less halo) when split_threads >= 512; fp64 always 256
     constexpr int NTW = sizeof(T) == 4 ? 512 : 256;
     const bool wide = threads >= 512;
 #define TDS_SP(KPV)                                                                                       \
     case KPV:                                                                                             \
         if (wide)                                                                                         \
-            return raw ? launch_sp<T, KPV, true, NTW>(A, m_in, max_len, st)                               \
-                       : launch_sp<T, KPV, false, NTW>(A, m_in, max_len, st);                             \
-        return raw ? launch_sp<T, KPV, true, 256>(A, m_in, max_len, st) : launch_sp<T, KPV, false, 256>(A, m_in, max_len, st)
+            return raw ? launch_sp<T, KPV, true, NTW>(A, m_in, max_len, st, sc)                           \
+                       : launch_sp<T, KPV, false, NTW>(A, m_in, max_len, st, sc);                         \
+        return raw ? launch_sp<T, KPV, true, 256>(A, m_in, max_len, st, sc)                                \
+                   : launch_sp<T, KPV, false, 256>(A, m_in, max_len, st, sc)
     switch (A.kp) {
         TDS_SP(1);
         TDS_SP(2);
@@ -550,7 +586,9 @@ cudaError_t launch_split_pipe(const SplitArgs<T> &A, bool raw, int64_t m_in, int
 #undef TDS_SP
 }
 
-template cudaError_t launch_split_pipe<float>(const SplitArgs<float> &, bool, int64_t, int64_t, int, cudaStream_t);
-template cudaError_t launch_split_pipe<double>(const SplitArgs<double> &, bool, int64_t, int64_t, int, cudaStream_t);
+template cudaError_t launch_split_pipe<float>(const SplitArgs<float> &, bool, int64_t, int64_t, int, cudaStream_t,
+                                              const ScatterHost *);
+template cudaError_t launch_split_pipe<double>(const SplitArgs<double> &, bool, int64_t, int64_t, int, cudaStream_t,
+                                               const ScatterHost *);
 
 }  // namespace tds

@@ -47,7 +47,7 @@ oracle).
 from __future__ import annotations
 
 import math
-from typing import List, Optional, Sequence, Tuple
+from typing import Callable, List, Optional, Sequence, Tuple
 
 import torch
 import torch.distributed as dist
@@ -122,6 +122,11 @@ class CudaBackend:
         plan, ws, _ = state
         api.split_slots(plan, ext[0], ext[1], ext[2], ext[3], ws)
 
+    def split_scatter(self, state, ext, dst, q: int, first_pos: int, num_pos: int, dst_stride: int):
+        """The split with the all-to-all fused into its TMA stores (tds_split_scatter)."""
+        plan = state[0]
+        api.split_scatter(plan, ext[0], ext[1], ext[2], ext[3], dst, q, first_pos, num_pos, dst_stride)
+
     def make_solve(self, NL: int, m: int, stride: int):
         plan = api.Plan(NL, m, self.name, device=self.device.index or 0, mode="static", batch_stride=stride)
         if plan.info["k"] == 0:
@@ -167,9 +172,14 @@ class HugeRank:
     """One rank's buffers, plans and message lists for ``huge_steps`` (all
     allocated once; a solve only enqueues kernels and exchanges)."""
 
-    def __init__(self, n: int, G: int, g: int, backend, kd: Optional[int] = None, chunks: int = 1):
+    def __init__(self, n: int, G: int, g: int, backend, kd: Optional[int] = None, chunks: int = 1,
+                 sys_alloc: Optional[Callable] = None):
+        """``sys_alloc(shape)``: allocator of the residue-system buffer (3, q, NL)
+        -- e.g. torch symmetric memory, so peers can write into it (peer mode,
+        ``set_peers``); default: the backend's allocator."""
         itemsize = torch.empty((), dtype=backend.dtype).element_size()
         self.n, self.G, self.g, self.be = n, G, g, backend
+        self.peer_dst = None                     # peer mode: tds_scatter destinations (set_peers)
         self.kd = kd = huge_kd(G, kd)
         self.NR = NR = 1 << kd
         self.B = B = n // G
@@ -200,7 +210,8 @@ class HugeRank:
             self.chunk_in = [tuple(f[self.off + c * qc * self.stride:][:span] for f in flat) for c in range(chunks)]
             self.solve_states = [backend.make_solve(NL, qc, self.stride) for _ in range(chunks)]
         else:
-            self.sys = [backend.empty(q, NL) for _ in range(3)]
+            self.sys_buf = sys_alloc((3, q, NL)) if sys_alloc else backend.empty(3, q, NL)
+            self.sys = [self.sys_buf[t] for t in range(3)]
             self.chunk_in = [tuple(v[c * qc:(c + 1) * qc] for v in self.sys) for c in range(chunks)]
             self.solve_states = [backend.make_solve(NL, qc, NL) for _ in range(chunks)]
         # x of the local residue systems (G = 1: with the slots' stride, unpacked in place)
@@ -210,6 +221,15 @@ class HugeRank:
         # G = 1 with a backend that can fuse: split + residue solves as one plan
         self.full = backend.make_full(n, kd, self.solve_states[0][0]) if G == 1 and hasattr(backend, "make_full") \
             else None
+
+    def set_peers(self, sys_ptrs: Sequence[int]) -> None:
+        """Peer mode: ``sys_ptrs[h]`` = device address (peer-mapped for h != g)
+        of rank h's residue-system buffer (3, q, NL).  The split then writes
+        every residue class straight into its owner (tds_split_scatter): the
+        all-to-all of the split data is fused into the split's TMA stores."""
+        s = self.ext.element_size()
+        q, NL, Bj, g = self.q, self.NL, self.Bj, self.g
+        self.peer_dst = [[int(sys_ptrs[h]) + (t * q * NL + g * Bj) * s for h in range(self.G)] for t in range(3)]
 
     @property
     def local(self):
@@ -314,6 +334,24 @@ def huge_steps(R: HugeRank, out, mark=None):
         h = yield ("post",) + R.halo_messages()
         yield ("wait", h)
     mark("split")
+    if R.peer_dst is not None and R.G > 1:  # peer mode: split + all-to-all in one kernel, then a barrier
+        R.be.split_scatter(R.split_state, R.ext, R.peer_dst, R.q, R.off, R.Bj, R.NL)
+        mark("exchange_solve")
+        yield ("barrier",)                  # every rank's split has written into every owner
+        for c in range(R.chunks):
+            R.solve(c)
+        xret = []
+        for c in range(R.chunks):
+            sends, recvs, local = R.xret_messages(c)
+            xret.append((yield ("post", sends, recvs)))
+            for src, dst in local:
+                dst.copy_(src)
+        for c in range(R.chunks):
+            yield ("wait", xret[c])
+        mark("unpack")
+        R.unpack(out)
+        mark("end")
+        return out
     if R.full is not None:  # G = 1, fused: one plan, x straight into row order
         R.be.solve_full(R.full, R.ext, R.H, R.n, out)
         mark("exchange_solve")
@@ -353,8 +391,17 @@ class P2PTransport:
     ops run on NCCL's stream, ordered after the current stream's kernels and
     waited on by it), gloo on CPU."""
 
-    def __init__(self, group=None):
-        self.group = group
+    def __init__(self, group=None, symm=None):
+        """``symm``: a torch symmetric-memory handle of the peer-mode residue
+        buffers -- its device-side barrier orders the peers' fused split
+        stores before the residue solves (else a process-group barrier)."""
+        self.group, self.symm = group, symm
+
+    def barrier(self):
+        if self.symm is not None:
+            self.symm.barrier()
+        else:
+            dist.barrier(group=self.group)
 
     def post(self, sends, recvs):
         ops = [dist.P2POp(dist.isend, t, peer, self.group) for peer, t in sends]
@@ -374,6 +421,9 @@ def run_steps(gen, transport: P2PTransport):
         while True:
             if msg[0] == "post":
                 msg = gen.send(transport.post(msg[1], msg[2]))
+            elif msg[0] == "barrier":
+                transport.barrier()
+                msg = gen.send(None)
             else:
                 transport.wait(msg[1])
                 msg = gen.send(None)
@@ -422,6 +472,15 @@ def solve_huge_loopback(ranks: Sequence[HugeRank], outs: Sequence):
                 except StopIteration:
                     done[g] = True
                 progressed = True
+        # a barrier releases only when every live rank has reached it
+        live = [g for g in range(G) if not done[g]]
+        if live and all(state[g][0] == "barrier" for g in live):
+            for g in live:
+                try:
+                    state[g] = gens[g].send(None)
+                except StopIteration:
+                    done[g] = True
+            progressed = True
         if not progressed:
             raise RuntimeError("loopback deadlock")
     return outs

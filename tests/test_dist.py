@@ -2,6 +2,7 @@
 world_size 2 and 4): the huge-system halo / all-to-all index arithmetic with
 oracle-backed local compute, batch sharding and plan broadcast.  A 1-GPU test
 runs the same huge-system path with the libtds kernels."""
+import ctypes
 import dataclasses
 import os
 import socket
@@ -429,3 +430,118 @@ def test_solve_normalized_padded_strides(stride_pad, kp):
     assert np.array_equal(xs[:, :n], x2.cpu().numpy().reshape(m, stride)[:, :n])
     xr = oracle.thomas(an, np.ones_like(an), cn, dn)
     assert oracle.rel_err(xs[:, :n], xr) <= 1e-4
+
+
+# ------------------------------------------- peer mode: the all-to-all fused into the split
+
+def _peer_ranks(n, G, kd, chunks, dtype, seed=5, family="dd", kw=None):
+    from paper_conf_ipps_davidsonzo11_b200 import dist as tdist
+    import paper_conf_ipps_davidsonzo11_b200 as tds
+    tdt = torch.float32 if dtype == np.float32 else torch.float64
+    be = tdist.CudaBackend(tdt, "cuda:0")
+    ranks = [tdist.HugeRank(n, G, g, be, kd=kd, chunks=chunks) for g in range(G)]
+    for R in ranks:  # every rank writes straight into its peers' residue buffers (one device here)
+        R.set_peers([P.sys_buf.data_ptr() for P in ranks])
+    B = n // G
+    if family == "dd":
+        for g, R in enumerate(ranks):
+            tds.api.generate_rows(n, g * B, B, "float32" if dtype == np.float32 else "float64", seed=seed,
+                                  out=R.local)
+    else:
+        a, b, c, d = inputs.generate(n, 1, dtype, seed=seed, family=family, **(kw or {}))
+        for g, R in enumerate(ranks):
+            for dst, v in zip(R.local, (a, b, c, d)):
+                dst.copy_(torch.from_numpy(v[0, g * B:(g + 1) * B]))
+    outs = [be.empty(B) for _ in range(G)]
+    tdist.solve_huge_loopback(ranks, outs)
+    torch.cuda.synchronize()
+    return torch.cat(outs).cpu().numpy()
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("G,kd,chunks", [(2, 3, 1), (4, 5, 2), (8, 8, 4)])
+def test_huge_peer_mode_loopback(dtype, G, kd, chunks):
+    """Peer mode (tds_split_scatter: every rank's split writes each residue
+    class straight into its owner's buffer, then a barrier): bit-identical to
+    the point-to-point all-to-all and to G = 1, and the oracle's x."""
+    n = 1 << 20
+    x = _peer_ranks(n, G, kd, chunks, dtype)
+    assert np.array_equal(x, _loopback_gpu(n, G, kd, chunks, dtype))
+    assert np.array_equal(x, _loopback_gpu(n, 1, kd, 1, dtype))
+    a, b, c, d = inputs.generate(n, 1, dtype, seed=5)
+    xr = oracle.thomas(a, b, c, d)[0]
+    assert np.abs(x - xr).max() / np.abs(xr).max() <= (1e-4 if dtype == np.float32 else 1e-10)
+
+
+@pytest.mark.gpu
+def test_huge_peer_mode_coupling():
+    """Peer mode on the Poisson matrix (every row couples across ranks)."""
+    import math
+    n, G, kd = 1 << 18, 4, 5
+    x = _peer_ranks(n, G, kd, 1, np.float64, seed=7, family="poisson")
+    a, b, c, d = inputs.generate(n, 1, np.float64, seed=7, family="poisson")
+    xr = oracle.thomas(a, b, c, d)[0]
+    cs = math.cos(math.pi / (n + 1))
+    kappa = (2 + 2 * cs) / (2 - 2 * cs)
+    assert np.abs(x - xr).max() / np.abs(xr).max() <= 10 * kappa * 2.22e-16
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("E,kd,G,off,num", [(4096 + 256, 3, 2, 4, 500), ((1 << 18) + 4096, 8, 8, 8, 1024),
+                                            (65536, 5, 4, 2, 2046)])
+def test_split_scatter_bit_exact(dtype, E, kd, G, off, num):
+    """tds_split_scatter writes residue h q + rl, positions [off, off + num),
+    to dst[t][h] + rl * stride: the same bits as the canonical split slots;
+    everything else in the destinations untouched (the halo positions are
+    clipped by the TMA stores)."""
+    import paper_conf_ipps_davidsonzo11_b200 as tds
+    name = "float32" if dtype == np.float32 else "float64"
+    tdt = torch.float32 if dtype == np.float32 else torch.float64
+    dv = [torch.from_numpy(v).cuda() for v in inputs.generate(E, 1, dtype, seed=4)]
+    plan = tds.Plan(E, 1, name, device=0)
+    plan.set_params(k_pass=[kd], split_only=1, cluster=1, tl_levels=0)
+    views = tds.api.split_slots(plan, *dv, workspace=plan.workspace())
+    NR, q = 1 << kd, (1 << kd) // G
+    stride = -(-(num + 3) // 4) * 4
+    dst = [[torch.full((q, stride), 7.0, dtype=tdt, device="cuda") for _ in range(G)] for _ in range(3)]
+    tds.api.split_scatter(plan, *dv, dst, q, off, num, stride)
+    torch.cuda.synchronize()
+    for t in range(3):
+        for h in range(G):
+            got = dst[t][h]
+            assert torch.equal(got[:, :num], views[t][h * q:(h + 1) * q, off:off + num])
+            assert bool((got[:, num:] == 7.0).all())
+
+
+def test_split_scatter_argument_errors():
+    """Rejected before anything is enqueued (plan from fake B200 properties)."""
+    import paper_conf_ipps_davidsonzo11_b200 as tds
+    from paper_conf_ipps_davidsonzo11_b200 import _lib as L
+    lib = L.load()
+    p = tds.Plan(4096, 1, "float32", props=dataclasses.asdict(rp.B200))
+    p.set_params(k_pass=[3], split_only=1, cluster=1, tl_levels=0)
+    spec = L.Scatter()
+    spec.groups, spec.residues_per_group, spec.first_pos, spec.num_pos, spec.dst_stride = 2, 4, 0, 100, 128
+    for t in range(3):
+        for h in range(2):
+            spec.dst[t][h] = (1 << 40) + (t * 2 + h) * (1 << 20)
+    A = 1 << 36
+    call = lambda: lib.tds_split_scatter(p.handle, A, A + (1 << 24), A + (2 << 24), A + (3 << 24),
+                                         ctypes.byref(spec), None)
+    assert call() in (5, 7)                      # valid: fails only at the device check (no GPU / no device)
+    spec.residues_per_group = 3
+    assert call() == 1                           # groups * q != 2^k
+    spec.residues_per_group = 4
+    spec.dst_stride = 50
+    assert call() == 1                           # dst_stride < num_pos
+    spec.dst_stride = 128
+    spec.num_pos = 1000
+    assert call() == 1                           # window past floor(n / 2^k) = 512
+    spec.num_pos = 100
+    spec.dst[1][1] = (1 << 40) + 8
+    assert call() == 1                           # misaligned dst
+    q2 = tds.Plan(4096, 2, "float32", props=dataclasses.asdict(rp.B200))
+    q2.set_params(k_pass=[3], split_only=1, cluster=1, tl_levels=0)
+    assert lib.tds_split_scatter(q2.handle, A, A, A, A, ctypes.byref(spec), None) == 2  # m != 1
