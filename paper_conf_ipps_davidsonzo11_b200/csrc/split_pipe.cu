@@ -184,12 +184,18 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
             // fused all-to-all: residues [h q, (h+1) q) of the tile go straight to destination
             // h's residue systems ({position, residue} view, positions shifted by -sc_first;
             // the TMA unit drops the halo positions outside [0, num_pos))
+            // (every tensor-map address a compile-time offset into the __grid_constant__
+            // parameter: a runtime index would make the compiler copy the maps to local memory)
             const int j0 = int((t0 >> KP) - A.sc_first);
+#pragma unroll
             for (int q = 0; q < 3; ++q)
+#pragma unroll
                 for (int bx = 0; bx < NBOX; ++bx)
-                    for (int h = 0; h < A.sc_groups; ++h)
-                        tma_store_box3(&tms.m[q * A.sc_groups + h],
-                                       tbuf + q * TV + bx * NRES * BOXP + h * A.sc_q * BOXP, j0 + bx * BOXP, 0, 0);
+#pragma unroll
+                    for (int h = 0; h < 8; ++h)
+                        if (h < A.sc_groups)
+                            tma_store_box3(&tms.m[q * 8 + h], tbuf + q * TV + bx * NRES * BOXP + h * A.sc_q * BOXP,
+                                           j0 + bx * BOXP, 0, 0);
             bulk_commit();
         } else if (t == 0 && !TDS_ABL(4)) {
             const int j0 = int(t0 >> KP), r = int(sigma & ((int64_t(1) << kp_prev) - 1)), sys = int(sigma >> kp_prev);
@@ -529,8 +535,8 @@ static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_le
                     const uint64_t strides[2] = {uint64_t(sc->dst_stride) * sizeof(T),
                                                  uint64_t(sc->dst_stride) * sizeof(T) * uint64_t(sc->q)};
                     const uint32_t box[3] = {uint32_t(S::BOXP), uint32_t(sc->q), 1};
-                    if (!encode_box3_tmap_plain(&tms.m[q * sc->groups + h], sc->dst[q][h], int(sizeof(T)), dims,
-                                                strides, box))
+                    if (!encode_box3_tmap_plain(&tms.m[q * 8 + h], sc->dst[q][h], int(sizeof(T)), dims, strides,
+                                                box))
                         return cudaErrorInvalidValue;
                 }
             B.sc_groups = sc->groups;
