@@ -115,7 +115,7 @@ struct SplitShape {
 template <typename T, int KP, bool RAW, int NT>
 __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
     split_pipe_kernel(const SplitArgs<T> A, int64_t tps, int64_t nitems, const __grid_constant__ TmapSet tm,
-                      int32_t tma_lines, const __grid_constant__ TmapSet tmo, const __grid_constant__ TmapSet24 tms) {
+                      int32_t tma_lines, const __grid_constant__ TmapSet tmo, const CUtensorMap *__restrict__ tms) {
     using S = SplitShape<KP, NT>;
     constexpr int R = S::R, AV = S::AV, TV = S::TV, HEAD = S::HEAD, ROWS = S::ROWS, CH = S::CH;
     constexpr int TOFF = S::template toff<T>(), BL = S::template box_lines<T>(), ELINE = 128 / int(sizeof(T));
@@ -184,8 +184,8 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
             // fused all-to-all: residues [h q, (h+1) q) of the tile go straight to destination
             // h's residue systems ({position, residue} view, positions shifted by -sc_first;
             // the TMA unit drops the halo positions outside [0, num_pos))
-            // (every tensor-map address a compile-time offset into the __grid_constant__
-            // parameter: a runtime index would make the compiler copy the maps to local memory)
+            // (the [array][destination] maps live in global memory: tds_split_scatter
+            // copies them there on the stream before the launch)
             const int j0 = int((t0 >> KP) - A.sc_first);
 #pragma unroll
             for (int q = 0; q < 3; ++q)
@@ -194,7 +194,7 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
 #pragma unroll
                     for (int h = 0; h < 8; ++h)
                         if (h < A.sc_groups)
-                            tma_store_box3(&tms.m[q * 8 + h], tbuf + q * TV + bx * NRES * BOXP + h * A.sc_q * BOXP,
+                            tma_store_box3(tms + q * 8 + h, tbuf + q * TV + bx * NRES * BOXP + h * A.sc_q * BOXP,
                                            j0 + bx * BOXP, 0, 0);
             bulk_commit();
         } else if (t == 0 && !TDS_ABL(4)) {
@@ -559,8 +559,19 @@ static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_le
         cudaMemcpyToSymbolAsync(tds_split_ablation, &v, sizeof(int), 0, cudaMemcpyHostToDevice, st);
     }
 #endif
+    // scatter maps: to global memory, stream-ordered (allocated and freed around the launch)
+    CUtensorMap *dmaps = nullptr;
+    if (B.sc_groups > 0) {
+        cudaError_t e2 = cudaMallocAsync(reinterpret_cast<void **>(&dmaps), sizeof(tms), st);
+        if (e2 == cudaSuccess) e2 = cudaMemcpyAsync(dmaps, &tms, sizeof(tms), cudaMemcpyHostToDevice, st);
+        if (e2 != cudaSuccess) return e2;
+    }
     cudaError_t le = launch_pdl(kern, dim3(unsigned(grid)), dim3(S::NT), smem, st, 1, B, tps, nitems, tm,
-                                int32_t(tma_lines), tmo, tms);
+                                int32_t(tma_lines), tmo, (const CUtensorMap *)dmaps);
+    if (dmaps) {
+        const cudaError_t e3 = cudaFreeAsync(dmaps, st);
+        if (le == cudaSuccess) le = e3;
+    }
     if (le != cudaSuccess) return le;
     return cudaGetLastError();
 }
