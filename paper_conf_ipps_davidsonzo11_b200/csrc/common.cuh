@@ -139,7 +139,8 @@ struct SplitArgs {
     // fused split + all-to-all (tds_split_scatter): > 0 destinations; residues
     // [h q, (h+1) q) of the tile go to destination h, positions shifted by -sc_first
     int32_t sc_groups, sc_q;
-    int64_t sc_first;
+    int64_t sc_first, sc_num, sc_stride;
+    T *sc_dst[3][8];  // the destinations again, for the boxes a TMA store cannot take (see split_pipe.cu)
 };
 
 // Host description of a scatter (tds_split_scatter): per destination h and

@@ -180,22 +180,36 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
     auto tma_store_tile = [&](int64_t sigma, int64_t t0, int kp_prev) {
         fence_proxy_async_smem();  // generic-proxy smem writes -> visible to the TMA
         __syncthreads();
+        // fused all-to-all: residues [h q, (h+1) q) of the tile go straight to destination
+        // h's residue systems ({position, residue} view, positions shifted by -sc_first;
+        // the TMA unit drops the positions past the window).  A TMA tensor STORE with a
+        // negative start coordinate is an illegal instruction on sm_100a (measured:
+        // scripts/probes/tma_store_probe.cu), so the boxes that start before the window --
+        // the first tile's, holding the left halo -- leave by plain stores of the window
+        // part (CTA-uniform branch; one tile of each system).
+        const int64_t jw = (t0 >> KP) - A.sc_first;  // window position of the tile's first position
+        if (A.sc_groups > 0 && jw < 0) {
+            for (int bx = 0; bx < NBOX && jw + int64_t(bx) * BOXP < 0; ++bx)
+                for (int e = t; e < 3 * NRES * BOXP; e += S::NT) {
+                    const int q = e / (NRES * BOXP), rr = (e / BOXP) % NRES, p = e % BOXP;
+                    const int64_t j = jw + int64_t(bx) * BOXP + p;
+                    if (j < 0 || j >= A.sc_num) continue;
+                    const int h = rr / A.sc_q, rl = rr % A.sc_q;
+                    A.sc_dst[q][h][int64_t(rl) * A.sc_stride + j] = tbuf[q * TV + bx * NRES * BOXP + rr * BOXP + p];
+                }
+        }
         if (t == 0 && !TDS_ABL(4) && A.sc_groups > 0) {
-            // fused all-to-all: residues [h q, (h+1) q) of the tile go straight to destination
-            // h's residue systems ({position, residue} view, positions shifted by -sc_first;
-            // the TMA unit drops the halo positions outside [0, num_pos))
             // (the [array][destination] maps live in global memory: tds_split_scatter
             // copies them there on the stream before the launch)
-            const int j0 = int((t0 >> KP) - A.sc_first);
 #pragma unroll
             for (int q = 0; q < 3; ++q)
 #pragma unroll
                 for (int bx = 0; bx < NBOX; ++bx)
 #pragma unroll
                     for (int h = 0; h < 8; ++h)
-                        if (h < A.sc_groups)
+                        if (h < A.sc_groups && jw + int64_t(bx) * BOXP >= 0)
                             tma_store_box3(tms + q * 8 + h, tbuf + q * TV + bx * NRES * BOXP + h * A.sc_q * BOXP,
-                                           j0 + bx * BOXP, 0, 0);
+                                           int(jw + int64_t(bx) * BOXP), 0, 0);
             bulk_commit();
         } else if (t == 0 && !TDS_ABL(4)) {
             const int j0 = int(t0 >> KP), r = int(sigma & ((int64_t(1) << kp_prev) - 1)), sys = int(sigma >> kp_prev);
@@ -542,6 +556,10 @@ static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_le
             B.sc_groups = sc->groups;
             B.sc_q = sc->q;
             B.sc_first = sc->first_pos;
+            B.sc_num = sc->num_pos;
+            B.sc_stride = sc->dst_stride;
+            for (int q = 0; q < 3; ++q)
+                for (int h = 0; h < sc->groups; ++h) B.sc_dst[q][h] = static_cast<T *>(sc->dst[q][h]);
         }
     } else if constexpr (S::template tstore<T>()) {  // output view {position, r, rho, system}
         T *outs[3] = {A.oa, A.oc, A.od};
