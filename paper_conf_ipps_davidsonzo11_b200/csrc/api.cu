@@ -551,10 +551,12 @@ tds_status tds_split_scatter(const tds_plan_t plan, const void *a, const void *b
     if (spec->groups < 1 || spec->groups > 8 || int64_t(spec->residues_per_group) * spec->groups != NR)
         return fail(TDS_ERR_INVALID_ARG, "groups in [1, 8] and groups * residues_per_group == 2^k");
     const int64_t es = dsize(I.dtype);
+    // (TMA tensor stores need 16-byte aligned box starts: the tiles' store coordinates
+    // are whole 16-byte runs after the shift by first_pos only if first_pos is)
     if (spec->first_pos < 0 || spec->num_pos < 1 || spec->first_pos + spec->num_pos > I.n / NR ||
-        spec->dst_stride < spec->num_pos || (spec->dst_stride * es) % 16)
+        spec->dst_stride < spec->num_pos || (spec->dst_stride * es) % 16 || (spec->first_pos * es) % 16)
         return fail(TDS_ERR_INVALID_ARG, "positions [first_pos, first_pos + num_pos) within floor(n / 2^k); "
-                                         "dst_stride >= num_pos, a 16-byte multiple");
+                                         "first_pos and dst_stride (>= num_pos) in 16-byte units");
     tds_status s = check_arrays(I, {a, b, c, d});
     if (s != TDS_OK) return s;
     if (!vec_ok(I, {a, b, c, d})) return fail(TDS_ERR_UNSUPPORTED, "a scatter needs 16-byte aligned a, b, c, d");

@@ -112,7 +112,7 @@ struct SplitShape {
     }
 };
 
-template <typename T, int KP, bool RAW, int NT>
+template <typename T, int KP, bool RAW, int NT, bool SC>
 __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
     split_pipe_kernel(const SplitArgs<T> A, int64_t tps, int64_t nitems, const __grid_constant__ TmapSet tm,
                       int32_t tma_lines, const __grid_constant__ TmapSet tmo, const CUtensorMap *__restrict__ tms) {
@@ -187,8 +187,8 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
         // scripts/probes/tma_store_probe.cu), so the boxes that start before the window --
         // the first tile's, holding the left halo -- leave by plain stores of the window
         // part (CTA-uniform branch; one tile of each system).
-        const int64_t jw = (t0 >> KP) - A.sc_first;  // window position of the tile's first position
-        if (A.sc_groups > 0 && jw < 0) {
+        const int64_t jw = SC ? (t0 >> KP) - A.sc_first : 0;  // window position of the tile's first position
+        if (SC && jw < 0) {
             for (int bx = 0; bx < NBOX && jw + int64_t(bx) * BOXP < 0; ++bx)
                 for (int e = t; e < 3 * NRES * BOXP; e += S::NT) {
                     const int q = e / (NRES * BOXP), rr = (e / BOXP) % NRES, p = e % BOXP;
@@ -198,7 +198,7 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
                     A.sc_dst[q][h][int64_t(rl) * A.sc_stride + j] = tbuf[q * TV + bx * NRES * BOXP + rr * BOXP + p];
                 }
         }
-        if (t == 0 && !TDS_ABL(4) && A.sc_groups > 0) {
+        if (SC && t == 0 && !TDS_ABL(4)) {
             // (the [array][destination] maps live in global memory: tds_split_scatter
             // copies them there on the stream before the launch)
 #pragma unroll
@@ -507,7 +507,9 @@ template <typename T, int KP, bool RAW, int NT>
 static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_len, cudaStream_t st,
                              const ScatterHost *sc) {
     using S = SplitShape<KP, NT>;
-    auto kern = split_pipe_kernel<T, KP, RAW, NT>;
+    // the fused split + all-to-all is its own instantiation (first pass only): the product
+    // kernels keep their code and registers
+    auto kern = (RAW && sc) ? split_pipe_kernel<T, KP, RAW, NT, RAW> : split_pipe_kernel<T, KP, RAW, NT, false>;
     const size_t smem = S::template smem_bytes<T>(RAW);
     int occ = 1;
     cudaError_t e = kernel_setup((const void *)kern, S::NT, smem, 1, &occ);
