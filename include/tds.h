@@ -299,12 +299,13 @@ tds_status tds_split_slots(const tds_plan_t plan, const void *a, const void *b, 
  * symmetric memory over NVLink) overlaps the split tile by tile; positions
  * outside the window (the halo) are not written.  No workspace.  The caller
  * orders the destinations' readers after this call (a barrier across the
- * ranks).  first_pos and dst_stride must be 16-byte multiples (TMA tensor
- * stores start on 16-byte boundaries; a store box starting before the window
+ * ranks).  first_pos, num_pos and dst_stride must be 16-byte multiples (TMA
+ * tensor stores start -- and clip at the window's end -- on 16-byte
+ * boundaries, measured on sm_100a; a store box starting before the window
  * -- the left halo -- leaves by plain stores: on sm_100a a TMA store with a
  * negative start coordinate is an illegal instruction).  Errors: INVALID_ARG
  * (NULL, groups not in [1, 8], groups * q != 2^k, window outside
- * floor(n / 2^k), dst_stride < num_pos, first_pos / dst_stride not 16-byte
+ * floor(n / 2^k), dst_stride < num_pos, first_pos / num_pos / dst_stride not 16-byte
  * multiples, NULL / misaligned / overlapping dst), UNSUPPORTED (m != 1, not
  * one pass of <= 8 levels, misaligned inputs), CUDA. */
 typedef struct {

@@ -554,9 +554,10 @@ tds_status tds_split_scatter(const tds_plan_t plan, const void *a, const void *b
     // (TMA tensor stores need 16-byte aligned box starts: the tiles' store coordinates
     // are whole 16-byte runs after the shift by first_pos only if first_pos is)
     if (spec->first_pos < 0 || spec->num_pos < 1 || spec->first_pos + spec->num_pos > I.n / NR ||
-        spec->dst_stride < spec->num_pos || (spec->dst_stride * es) % 16 || (spec->first_pos * es) % 16)
+        spec->dst_stride < spec->num_pos || (spec->dst_stride * es) % 16 || (spec->first_pos * es) % 16 ||
+        (spec->num_pos * es) % 16)
         return fail(TDS_ERR_INVALID_ARG, "positions [first_pos, first_pos + num_pos) within floor(n / 2^k); "
-                                         "first_pos and dst_stride (>= num_pos) in 16-byte units");
+                                         "first_pos, num_pos and dst_stride (>= num_pos) in 16-byte units");
     tds_status s = check_arrays(I, {a, b, c, d});
     if (s != TDS_OK) return s;
     if (!vec_ok(I, {a, b, c, d})) return fail(TDS_ERR_UNSUPPORTED, "a scatter needs 16-byte aligned a, b, c, d");

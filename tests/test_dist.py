@@ -490,7 +490,7 @@ def test_huge_peer_mode_coupling():
 @pytest.mark.gpu
 @pytest.mark.parametrize("dtype", [np.float32, np.float64])
 @pytest.mark.parametrize("E,kd,G,off,num", [(4096 + 256, 3, 2, 4, 500), ((1 << 18) + 4096, 8, 8, 8, 1024),
-                                            (65536, 5, 4, 4, 2042)])
+                                            (65536, 5, 4, 4, 2040)])
 def test_split_scatter_bit_exact(dtype, E, kd, G, off, num):
     """tds_split_scatter writes residue h q + rl, positions [off, off + num),
     to dst[t][h] + rl * stride: the same bits as the canonical split slots;
@@ -543,6 +543,9 @@ def test_split_scatter_argument_errors():
     spec.first_pos = 2
     assert call() == 1                           # first_pos not a 16-byte multiple (fp32: 4 elements)
     spec.first_pos = 0
+    spec.num_pos = 98
+    assert call() == 1                           # num_pos not a 16-byte multiple
+    spec.num_pos = 100
     spec.dst[1][1] = (1 << 40) + 8
     assert call() == 1                           # misaligned dst
     q2 = tds.Plan(4096, 2, "float32", props=dataclasses.asdict(rp.B200))
