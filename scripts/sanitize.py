@@ -66,11 +66,16 @@ for label, dt, n, m, params in CASES:
 from paper_conf_ipps_davidsonzo11_b200 import dist as tdist  # noqa: E402
 for label, dt, n, G, kd, chunks in [("huge loopback G=4 kd=3", F32, 1 << 16, 4, 3, 1),
                                     ("huge loopback G=2 kd=4 chunks=2", F64, 1 << 15, 2, 4, 2),
-                                    ("huge G=1 kd=5", F32, 1 << 16, 1, 5, 1)]:
+                                    ("huge G=1 kd=5", F32, 1 << 16, 1, 5, 1),
+                                    ("huge loopback peer G=4 kd=3", F32, 1 << 16, 4, 3, 1),
+                                    ("huge loopback peer G=2 kd=4", F64, 1 << 15, 2, 4, 1)]:
     tdt = torch.float32 if dt == F32 else torch.float64
     name = "float32" if dt == F32 else "float64"
     be = tdist.CudaBackend(tdt, "cuda:0")
     ranks = [tdist.HugeRank(n, G, g, be, kd=kd, chunks=chunks) for g in range(G)]
+    if "peer" in label:  # the split writes the residue classes straight into the owners (tds_split_scatter)
+        for R in ranks:
+            R.set_peers([P.sys_buf.data_ptr() for P in ranks])
     B = n // G
     for g, R in enumerate(ranks):
         tds.api.generate_rows(n, g * B, B, name, seed=5, out=R.local)
