@@ -319,6 +319,26 @@ typedef struct {
 tds_status tds_split_scatter(const tds_plan_t plan, const void *a, const void *b, const void *c, const void *d,
                              const tds_scatter *spec, void *cuda_stream);
 
+/* tds_solve_normalized with the x placement FUSED with the return of x to its
+ * owners (the one-huge-system path's second all-to-all): rows
+ * [h rows_per_group, (h+1) rows_per_group) of system s of x go to dst[h] +
+ * s * dst_system_stride -- the placement kernel's TMA tensor stores write them
+ * straight into (peer) memory.  Needs k >= 5, the TMA placement (n and
+ * rows_per_group multiples of 2^k, rows_per_group / 2^k a multiple of
+ * 4 * 128 / sizeof(T)), groups * rows_per_group == n, no chunking, strided 0,
+ * x_group 0.  No x array; d is not written.  The caller orders the owners'
+ * readers after the call (a barrier).  Errors: as tds_solve_normalized, plus
+ * INVALID_ARG for the shape rules and NULL / misaligned / overlapping dst. */
+typedef struct {
+    int32_t groups;              /* destinations (GPUs), <= 8                 */
+    int64_t rows_per_group;      /* rows of every system each destination owns */
+    int64_t dst_system_stride;   /* elements between systems at a destination  */
+    void *dst[8];                /* device (or peer) bases                     */
+} tds_xscatter;
+tds_status tds_solve_normalized_xscatter(const tds_plan_t plan, const void *a, const void *c, const void *d,
+                                         const tds_xscatter *spec, void *workspace, size_t workspace_bytes,
+                                         void *cuda_stream);
+
 /* The residue-class -> original-order transpose of Fig. 3a:
  * x[s * batch_stride + r + 2^k j] = xs[((s << k) + r) * slot_rows + j] for
  * every system s < m, residue r < 2^k and row r + 2^k j < n.  xs, x: device,

@@ -28,7 +28,7 @@ EXPORTED = (
     "tds_interleaved_workspace_bytes", "tds_solve_interleaved",
     "tds_last_error", "tds_version", "tds_tune_search", "tds_generate", "tds_generate_rows",
     "tds_solve_normalized", "tds_plan_slots_layout", "tds_split_slots", "tds_unpack_residues",
-    "tds_split_scatter",
+    "tds_split_scatter", "tds_solve_normalized_xscatter",
 )
 
 
@@ -75,6 +75,11 @@ class Scatter(ctypes.Structure):
                 ("dst", (ctypes.c_void_p * 8) * 3)]
 
 
+class XScatter(ctypes.Structure):
+    _fields_ = [("groups", ctypes.c_int32), ("rows_per_group", ctypes.c_int64),
+                ("dst_system_stride", ctypes.c_int64), ("dst", ctypes.c_void_p * 8)]
+
+
 # tds_tune_search's cost callback: double (*)(const tds_params *, void *)
 COST_FN = ctypes.CFUNCTYPE(ctypes.c_double, ctypes.POINTER(Params), ctypes.c_void_p)
 
@@ -115,6 +120,7 @@ def load() -> ctypes.CDLL:
         "tds_split_slots": (I32, [P, VP, VP, VP, VP, VP, SZ, VP]),
         "tds_unpack_residues": (I32, [I32, I64, I64, I32, I64, VP, VP, I64, VP]),
         "tds_split_scatter": (I32, [P, VP, VP, VP, VP, ctypes.POINTER(Scatter), VP]),
+        "tds_solve_normalized_xscatter": (I32, [P, VP, VP, VP, ctypes.POINTER(XScatter), VP, SZ, VP]),
         "tds_status_string": (ctypes.c_char_p, [I32]),
         "tds_last_error": (ctypes.c_char_p, []),
         "tds_version": (I32, []),

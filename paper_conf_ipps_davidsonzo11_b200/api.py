@@ -298,6 +298,27 @@ def split_scatter(plan: Plan, a, b, c, d, dst, residues_per_group: int, first_po
                                         ctypes.byref(spec), _stream_ptr(stream, dev)))
 
 
+def solve_normalized_xscatter(plan: Plan, a, c, d, dst, rows_per_group: int, dst_system_stride: int,
+                              workspace=None, stream=None):
+    """tds_solve_normalized_xscatter: the normalised solve whose x placement
+    writes rows [h rows_per_group, (h+1) rows_per_group) of every system
+    straight to dst[h] + s * dst_system_stride (device / peer addresses or
+    tensors)."""
+    info, need, want, dev = plan._solve_info()
+    for name, t in (("a", a), ("c", c), ("d", d)):
+        _check_fast(t, need, want, name, dev)
+    if workspace is None and info.workspace_bytes > 0:
+        workspace = plan.workspace()
+    spec = L.XScatter()
+    spec.groups, spec.rows_per_group, spec.dst_system_stride = len(dst), int(rows_per_group), int(dst_system_stride)
+    for h, p in enumerate(dst):
+        spec.dst[h] = p if isinstance(p, int) else p.data_ptr()
+    wptr = workspace.data_ptr() if workspace is not None else None
+    wbytes = workspace.numel() * workspace.element_size() if workspace is not None else 0
+    L.check(plan._lib.tds_solve_normalized_xscatter(plan.handle, a.data_ptr(), c.data_ptr(), d.data_ptr(),
+                                                    ctypes.byref(spec), wptr, wbytes, _stream_ptr(stream, dev)))
+
+
 def slot_views(plan: Plan, workspace, lay: Optional[dict] = None):
     """(a', c', d') views of the split slots inside ``workspace`` (no device work)."""
     info, _, want, _ = plan._solve_info()

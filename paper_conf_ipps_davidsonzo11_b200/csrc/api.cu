@@ -145,7 +145,8 @@ static tds_status run_split(const tds_plan_info &I, const T *a, const T *b, cons
 
 template <typename T>
 static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, const T *c, const T *d, T *x,
-                             void *ws, cudaStream_t st, int first = 0, int last = 1 << 30) {
+                             void *ws, cudaStream_t st, int first = 0, int last = 1 << 30,
+                             const XScatterHost *xsc = nullptr) {
     const tds_params &P = I.params;
     OnchipArgs<T> A{};
     A.x = x;
@@ -222,7 +223,7 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
                               : !fused_ok && P.passes >= first && P.passes <= last;
     if (P.k > 0 && place) {
         cudaError_t err = launch_place_x<T>(A.xs, x, I.n, I.m, I.batch_stride, I.slot_rows, P.k,
-                                            vec_ok(I, {(const void *)x}), A.geom, st);
+                                            xsc ? 1 : vec_ok(I, {(const void *)x}), A.geom, st, true, xsc);
         if (err != cudaSuccess) return cuda_fail(err, "place_x launch");
     }
     return TDS_OK;
@@ -493,6 +494,53 @@ tds_status tds_solve_normalized(const tds_plan_t plan, const void *a, const void
                                   workspace, st, 0, I.launches - 1)
             : solve_chunks<double>(I, (const double *)a, nullptr, (const double *)c, (const double *)d, (double *)x,
                                    workspace, st, 0, I.launches - 1);
+    if (s == TDS_OK) clear_error();
+    return s;
+}
+
+tds_status tds_solve_normalized_xscatter(const tds_plan_t plan, const void *a, const void *c, const void *d,
+                                         const tds_xscatter *spec, void *workspace, size_t workspace_bytes,
+                                         void *cuda_stream) {
+    if (!plan || !spec) return fail(TDS_ERR_INVALID_ARG, "NULL argument");
+    const tds_plan_info &I = plan->info;
+    const tds_params &P = I.params;
+    if (P.split_only || P.k < 5 || P.strided || P.x_group || I.chunks != 1)
+        return fail(TDS_ERR_UNSUPPORTED, "an x scatter needs k >= 5, no chunking, strided 0, x_group 0 (the TMA "
+                                         "placement)");
+    const int64_t es = dsize(I.dtype);
+    const int64_t KK = int64_t(1) << P.k, E = 128 / es;
+    const int64_t jb = spec->rows_per_group / KK;
+    if (spec->groups < 1 || spec->groups > 8 || spec->rows_per_group * spec->groups != I.n || I.n % KK ||
+        spec->rows_per_group % KK || jb % (4 * E) || spec->dst_system_stride < spec->rows_per_group ||
+        (spec->dst_system_stride * es) % 16)
+        return fail(TDS_ERR_INVALID_ARG, "groups in [1, 8] with groups * rows_per_group == n; rows_per_group a "
+                                         "multiple of 2^k * 4 * 128 bytes / sizeof(T); dst_system_stride >= "
+                                         "rows_per_group in 16-byte units");
+    tds_status s = check_solve_args(I, a, nullptr, c, d, const_cast<void *>(d), workspace, workspace_bytes);
+    if (s != TDS_OK) return s;
+    XScatterHost xsc{};
+    xsc.groups = spec->groups;
+    xsc.rows_per_group = spec->rows_per_group;
+    xsc.dst_system_stride = spec->dst_system_stride;
+    const size_t in_bytes = size_t(((I.m - 1) * I.batch_stride + I.n) * es);
+    const size_t dbytes = size_t(((I.m - 1) * spec->dst_system_stride + spec->rows_per_group) * es);
+    for (int h = 0; h < spec->groups; ++h) {
+        const void *p = spec->dst[h];
+        if (!p || reinterpret_cast<uintptr_t>(p) % 16) return fail(TDS_ERR_INVALID_ARG, "NULL or misaligned dst");
+        for (const void *q : {a, c, d})
+            if (overlaps(p, dbytes, q, in_bytes)) return fail(TDS_ERR_INVALID_ARG, "dst overlaps an input");
+        if (workspace && overlaps(p, dbytes, workspace, I.workspace_bytes))
+            return fail(TDS_ERR_INVALID_ARG, "dst overlaps the workspace");
+        xsc.dst[h] = spec->dst[h];
+    }
+    if ((s = check_geometry(I)) != TDS_OK) return s;
+    if ((s = check_device(plan)) != TDS_OK) return s;
+    cudaStream_t st = static_cast<cudaStream_t>(cuda_stream);
+    s = I.dtype == TDS_F32
+            ? solve_impl<float>(I, (const float *)a, nullptr, (const float *)c, (const float *)d, nullptr, workspace,
+                                st, 0, 1 << 30, &xsc)
+            : solve_impl<double>(I, (const double *)a, nullptr, (const double *)c, (const double *)d, nullptr,
+                                 workspace, st, 0, 1 << 30, &xsc);
     if (s == TDS_OK) clear_error();
     return s;
 }

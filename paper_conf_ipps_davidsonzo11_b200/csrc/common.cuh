@@ -229,9 +229,19 @@ inline bool onchip_cpipe_ok(const tds_plan_info &I) {
     return onchip_cpipe_smem_bytes(I.dtype, I.onchip_threads, C) + kSmemReserve + 16 <= size_t(232448);
 }
 
+// Host description of an x scatter (tds_solve_normalized_xscatter): rows
+// [h rows_per_group, (h+1) rows_per_group) of system s go to
+// dst[h] + s * dst_system_stride (+ row - h rows_per_group).
+struct XScatterHost {
+    int32_t groups;
+    int64_t rows_per_group, dst_system_stride;
+    void *dst[8];
+};
+
 template <typename T>
 cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batch_stride, int64_t slot, int K,
-                           int vec, const PassGeom &geom, cudaStream_t st, bool xs_scratch = true);
+                           int vec, const PassGeom &geom, cudaStream_t st, bool xs_scratch = true,
+                           const XScatterHost *xsc = nullptr);
 template <typename T>
 cudaError_t launch_onchip(const OnchipArgs<T> &A, int cr_levels, bool raw, int64_t grid, int threads,
                           size_t smem, cudaStream_t st);

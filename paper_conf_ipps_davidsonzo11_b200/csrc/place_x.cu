@@ -175,10 +175,11 @@ __global__ void __launch_bounds__(kPlaceThreads) place_x_tile_kernel(const Place
 // with plain loads and stores.
 constexpr int kTpBoxes = 4, kTpThreads = 256;
 
-template <typename T>
+template <typename T, bool XS>
 __global__ void __launch_bounds__(kTpThreads) place_x_tma_kernel(const PlaceArgs<T> A, const __grid_constant__ TmapSet tm,
                                                                 int64_t ntiles, int64_t jtiles, int64_t lfull,
-                                                                int64_t msys, int32_t l2_discard) {
+                                                                int64_t msys, int32_t l2_discard,
+                                                                const CUtensorMap *__restrict__ xmaps, int64_t jb) {
     constexpr int E = 128 / int(sizeof(T)), CH = 16 / int(sizeof(T)), NBX = kTpBoxes;
     constexpr int BOX = E * E;  // elements per box
     extern __shared__ __align__(1024) unsigned char smem_raw[];
@@ -261,8 +262,15 @@ __global__ void __launch_bounds__(kTpThreads) place_x_tma_kernel(const PlaceArgs
             int64_t sys, rt, jt;
             coords(w, sys, rt, jt);
 #pragma unroll
-            for (int bx = 0; bx < NBX; ++bx)
-                tma_store_box3(&tm.m[1], sout + bx * BOX, int(rt * E), int((jt * NBX + bx) * E), int(sys));
+            for (int bx = 0; bx < NBX; ++bx) {
+                const int64_t J = (jt * NBX + bx) * E;
+                if constexpr (XS) {  // x scatter: the box's rows belong to destination J / jb (boxes never straddle)
+                    const int64_t h = J / jb;
+                    if (J < lfull) tma_store_box3(xmaps + h, sout + bx * BOX, int(rt * E), int(J - h * jb), int(sys));
+                } else {
+                    tma_store_box3(&tm.m[1], sout + bx * BOX, int(rt * E), int(J), int(sys));
+                }
+            }
             bulk_commit();
             issue(w + 2 * int64_t(gridDim.x), s);  // stage s is free: every thread passed the barrier
         }
@@ -279,7 +287,7 @@ __global__ void __launch_bounds__(kTpThreads) place_x_tma_kernel(const PlaceArgs
 
 template <typename T>
 cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batch_stride, int64_t slot, int K,
-                           int vec, const PassGeom &geom, cudaStream_t st, bool xs_scratch) {
+                           int vec, const PassGeom &geom, cudaStream_t st, bool xs_scratch, const XScatterHost *xsc) {
     PlaceArgs<T> A{};
     A.xs = xs;
     A.x = x;
@@ -291,6 +299,45 @@ cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batc
     A.geom = geom;
     constexpr int E = 128 / int(sizeof(T));
     const int64_t lfull = n >> K;  // whole j rows of 2^K residues
+    if (xsc) {  // x scatter: only the TMA transposer, whole j rows, boxes inside one destination
+        const int64_t jb = xsc->rows_per_group >> K;
+        if (!((int64_t(1) << K) >= E && (lfull << K) == n && xsc->rows_per_group % (int64_t(1) << K) == 0 &&
+              jb % (kTpBoxes * E) == 0 && jb * xsc->groups == lfull && (m << K) < (int64_t(1) << 31)))
+            return cudaErrorNotSupported;
+        TmapSet tm{};
+        TmapSet24 xm{};
+        const uint64_t din[3] = {uint64_t(slot), uint64_t(m << K), 1};
+        const uint64_t sin_[2] = {uint64_t(slot) * sizeof(T), uint64_t(slot) * sizeof(T) * uint64_t(m << K)};
+        const uint32_t bin[3] = {uint32_t(E), uint32_t(E), 1};
+        if (!encode_box3_tmap(&tm.m[0], xs, int(sizeof(T)), din, sin_, bin)) return cudaErrorInvalidValue;
+        for (int h = 0; h < xsc->groups; ++h) {  // destination h: {2^K residues, jb j, m systems}
+            const uint64_t dout[3] = {uint64_t(1) << K, uint64_t(jb), uint64_t(m)};
+            const uint64_t sout_[2] = {(uint64_t(1) << K) * sizeof(T), uint64_t(xsc->dst_system_stride) * sizeof(T)};
+            const uint32_t bout[3] = {uint32_t(E), uint32_t(E), 1};
+            if (!encode_box3_tmap(&xm.m[h], xsc->dst[h], int(sizeof(T)), dout, sout_, bout)) return cudaErrorInvalidValue;
+        }
+        const int64_t rtiles = (int64_t(1) << K) / E;
+        const int64_t jtiles = lfull / (kTpBoxes * E);
+        const int64_t ntiles = m * rtiles * jtiles;
+        const size_t smem = 1024 + size_t(3 * kTpBoxes * E * E) * sizeof(T);
+        auto kern = place_x_tma_kernel<T, true>;
+        int occ = 1;
+        cudaError_t e = kernel_setup((const void *)kern, kTpThreads, smem, 1, &occ);
+        if (e != cudaSuccess) return e;
+        CUtensorMap *dmaps = nullptr;  // the destination maps in global memory, stream-ordered
+        e = cudaMallocAsync(reinterpret_cast<void **>(&dmaps), sizeof(xm), st);
+        if (e == cudaSuccess) e = cudaMemcpyAsync(dmaps, &xm, sizeof(xm), cudaMemcpyHostToDevice, st);
+        if (e != cudaSuccess) return e;
+        const int64_t grid =
+            std::max<int64_t>(1, std::min<int64_t>(ntiles, int64_t(std::max(occ, 1)) * sm_count_current()));
+        const int32_t disc = xs_scratch && (slot * int64_t(sizeof(T))) % 128 == 0 && uintptr_t(xs) % 128 == 0;
+        e = launch_pdl(kern, dim3(unsigned(grid)), dim3(kTpThreads), smem, st, 1, A, tm, ntiles, jtiles, lfull, m, disc,
+                       (const CUtensorMap *)dmaps, jb);
+        const cudaError_t e3 = cudaFreeAsync(dmaps, st);
+        if (e != cudaSuccess) return e;
+        if (e3 != cudaSuccess) return e3;
+        return cudaGetLastError();
+    }
     if ((int64_t(1) << K) >= E && vec && lfull > 0 && n > 0 && m > 0) {
         const int64_t rtiles = (int64_t(1) << K) / E;
         const int64_t jtiles = (lfull + kTpBoxes * E - 1) / (kTpBoxes * E);
@@ -308,7 +355,7 @@ cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batc
             encode_box3_tmap(&tm.m[0], xs, int(sizeof(T)), din, sin_, bin) &&
             encode_box3_tmap(&tm.m[1], x, int(sizeof(T)), dout, sout_, bout)) {
             const size_t smem = 1024 + size_t(3 * kTpBoxes * E * E) * sizeof(T);
-            auto kern = place_x_tma_kernel<T>;
+            auto kern = place_x_tma_kernel<T, false>;
             int occ = 1;
             cudaError_t e = kernel_setup((const void *)kern, kTpThreads, smem, 1, &occ);
             if (e != cudaSuccess) return e;
@@ -317,7 +364,7 @@ cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batc
             // x slots are scratch whose last reader is this kernel: drop their lines from L2 once loaded
             const int32_t disc = xs_scratch && (slot * int64_t(sizeof(T))) % 128 == 0 && uintptr_t(xs) % 128 == 0;
             e = launch_pdl(kern, dim3(unsigned(grid)), dim3(kTpThreads), smem, st, 1, A, tm, ntiles, jtiles, lfull, m,
-                           disc);
+                           disc, (const CUtensorMap *)nullptr, int64_t(0));
             if (e != cudaSuccess) return e;
             return cudaGetLastError();
         }
@@ -343,8 +390,8 @@ cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batc
 }
 
 template cudaError_t launch_place_x<float>(const float *, float *, int64_t, int64_t, int64_t, int64_t, int, int,
-                                           const PassGeom &, cudaStream_t, bool);
+                                           const PassGeom &, cudaStream_t, bool, const XScatterHost *);
 template cudaError_t launch_place_x<double>(const double *, double *, int64_t, int64_t, int64_t, int64_t, int, int,
-                                            const PassGeom &, cudaStream_t, bool);
+                                            const PassGeom &, cudaStream_t, bool, const XScatterHost *);
 
 }  // namespace tds

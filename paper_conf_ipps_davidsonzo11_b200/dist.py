@@ -127,6 +127,18 @@ class CudaBackend:
         plan = state[0]
         api.split_scatter(plan, ext[0], ext[1], ext[2], ext[3], dst, q, first_pos, num_pos, dst_stride)
 
+    def x_fusable(self, state, Bj: int) -> bool:
+        """Whether the residue solve can place x straight into the owners
+        (tds_solve_normalized_xscatter's shape rules)."""
+        info = state[0].info
+        k, E = info["k"], 128 // torch.empty((), dtype=self.dtype).element_size()
+        return (k >= 5 and info["chunks"] == 1 and info["x_group"] == 0 and info["strided"] == 0 and
+                info["n"] % (1 << k) == 0 and Bj % (1 << k) == 0 and (Bj >> k) % (4 * E) == 0)
+
+    def solve_xscatter(self, state, a, c, d, dst, Bj: int):
+        plan, ws = state
+        api.solve_normalized_xscatter(plan, a, c, d, dst, Bj, Bj, workspace=ws)
+
     def make_solve(self, NL: int, m: int, stride: int):
         plan = api.Plan(NL, m, self.name, device=self.device.index or 0, mode="static", batch_stride=stride)
         if plan.info["k"] == 0:
@@ -180,6 +192,7 @@ class HugeRank:
         itemsize = torch.empty((), dtype=backend.dtype).element_size()
         self.n, self.G, self.g, self.be = n, G, g, backend
         self.peer_dst = None                     # peer mode: tds_scatter destinations (set_peers)
+        self.x_fused = False                     # peer mode: x placed straight into its owners
         self.kd = kd = huge_kd(G, kd)
         self.NR = NR = 1 << kd
         self.B = B = n // G
@@ -210,14 +223,17 @@ class HugeRank:
             self.chunk_in = [tuple(f[self.off + c * qc * self.stride:][:span] for f in flat) for c in range(chunks)]
             self.solve_states = [backend.make_solve(NL, qc, self.stride) for _ in range(chunks)]
         else:
-            self.sys_buf = sys_alloc((3, q, NL)) if sys_alloc else backend.empty(3, q, NL)
-            self.sys = [self.sys_buf[t] for t in range(3)]
+            # one buffer: the residue systems (3, q, NL) and the returned x (NR, Bj) -- in peer
+            # mode both are written by the peers' kernels (symmetric memory on a multi-GPU node)
+            nsys = 3 * q * NL
+            self.sys_buf = sys_alloc((nsys + NR * Bj,)) if sys_alloc else backend.empty(nsys + NR * Bj)
+            self.sys = [self.sys_buf[t * q * NL:(t + 1) * q * NL].view(q, NL) for t in range(3)]
             self.chunk_in = [tuple(v[c * qc:(c + 1) * qc] for v in self.sys) for c in range(chunks)]
             self.solve_states = [backend.make_solve(NL, qc, NL) for _ in range(chunks)]
         # x of the local residue systems (G = 1: with the slots' stride, unpacked in place)
         self.xs = backend.empty(q, self.stride if G == 1 else NL)
         self.chunk_x = [self.xs[c * qc:(c + 1) * qc] for c in range(chunks)]
-        self.xrecv = self.xs if G == 1 else backend.empty(NR, Bj)
+        self.xrecv = self.xs if G == 1 else self.sys_buf[3 * q * NL:].view(NR, Bj)
         # G = 1 with a backend that can fuse: split + residue solves as one plan
         self.full = backend.make_full(n, kd, self.solve_states[0][0]) if G == 1 and hasattr(backend, "make_full") \
             else None
@@ -230,6 +246,12 @@ class HugeRank:
         s = self.ext.element_size()
         q, NL, Bj, g = self.q, self.NL, self.Bj, self.g
         self.peer_dst = [[int(sys_ptrs[h]) + (t * q * NL + g * Bj) * s for h in range(self.G)] for t in range(3)]
+        # x: chunk c's systems [c qc, (c+1) qc) -> rows g q + c qc ... of every owner's returned-x block
+        qc = q // self.chunks
+        self.peer_xdst = [[int(sys_ptrs[h]) + (3 * q * NL + (g * q + c * qc) * Bj) * s for h in range(self.G)]
+                          for c in range(self.chunks)]
+        self.x_fused = all(self.be.x_fusable(st_, Bj) for st_ in self.solve_states) if hasattr(self.be, "x_fusable") \
+            else False
 
     @property
     def local(self):
@@ -299,6 +321,8 @@ class HugeRank:
         self.solve_states = new
         if self.full is not None:
             self.full = self.be.make_full(self.n, self.kd, self.solve_states[0][0])
+        if self.peer_dst is not None and hasattr(self.be, "x_fusable"):
+            self.x_fused = all(self.be.x_fusable(st_, self.Bj) for st_ in self.solve_states)
 
     def tune_residues(self, cache_path=None) -> list:
         """tds_tune on the residue-solve shape (this rank's device); applied to
@@ -338,6 +362,15 @@ def huge_steps(R: HugeRank, out, mark=None):
         R.be.split_scatter(R.split_state, R.ext, R.peer_dst, R.q, R.off, R.Bj, R.NL)
         mark("exchange_solve")
         yield ("barrier",)                  # every rank's split has written into every owner
+        if R.x_fused:  # the placement writes x straight into its owners' blocks, then a barrier
+            for c in range(R.chunks):
+                a, cc, d = R.chunk_in[c]
+                R.be.solve_xscatter(R.solve_states[c], a, cc, d, R.peer_xdst[c], R.Bj)
+            yield ("barrier",)
+            mark("unpack")
+            R.unpack(out)
+            mark("end")
+            return out
         for c in range(R.chunks):
             R.solve(c)
         xret = []

@@ -551,3 +551,50 @@ def test_split_scatter_argument_errors():
     q2 = tds.Plan(4096, 2, "float32", props=dataclasses.asdict(rp.B200))
     q2.set_params(k_pass=[3], split_only=1, cluster=1, tl_levels=0)
     assert lib.tds_split_scatter(q2.handle, A, A, A, A, ctypes.byref(spec), None) == 2  # m != 1
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+@pytest.mark.parametrize("G,kd", [(2, 3), (4, 4)])
+def test_huge_peer_mode_x_fused(dtype, G, kd):
+    """Peer mode with BOTH exchanges fused: the split's stores scatter the
+    residue classes, the residue solves' placement writes x straight into its
+    owners (tds_solve_normalized_xscatter).  Bit-identical to the
+    point-to-point path, the oracle's x."""
+    from paper_conf_ipps_davidsonzo11_b200 import dist as tdist
+    n = 1 << 24
+    tdt = torch.float32 if dtype == np.float32 else torch.float64
+    be = tdist.CudaBackend(tdt, "cuda:0")
+    probe = tdist.HugeRank(n, G, 0, be, kd=kd)
+    probe.set_peers([probe.sys_buf.data_ptr()] * G)
+    assert probe.x_fused, (probe.solve_states[0][0].info["k"], probe.Bj)
+    del probe
+    x = _peer_ranks(n, G, kd, 1, dtype)
+    assert np.array_equal(x, _loopback_gpu(n, G, kd, 1, dtype))
+    a, b, c, d = inputs.generate(n, 1, dtype, seed=5)
+    xr = oracle.thomas(a, b, c, d)[0]
+    assert np.abs(x - xr).max() / np.abs(xr).max() <= (1e-4 if dtype == np.float32 else 1e-10)
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("dtype", [np.float32, np.float64])
+def test_solve_normalized_xscatter_bit_exact(dtype):
+    """x rows [h R, (h+1) R) of system s land at dst[h] + s * stride, the same
+    bits as tds_solve_normalized; nothing else written."""
+    import paper_conf_ipps_davidsonzo11_b200 as tds
+    n, m, G = 1 << 20, 3, 4
+    R = n // G
+    tdt = torch.float32 if dtype == np.float32 else torch.float64
+    a, b, c, d = inputs.generate(n, m, dtype, seed=21)
+    an, cn, dn = (torch.from_numpy(np.ascontiguousarray(v / b)).cuda() for v in (a, c, d))
+    plan = tds.Plan(n, m, "float32" if dtype == np.float32 else "float64", device=0)
+    plan.set_params(k_pass=[7] if dtype == np.float32 else [8], cluster=1,
+                    cr_levels=4 if dtype == np.float32 else 3, thomas_chains=1, tl_levels=5)
+    xref = tds.api.solve_normalized(plan, an, cn, dn)
+    stride = R + 64
+    dst = [torch.full((m, stride), 7.0, dtype=tdt, device="cuda") for _ in range(G)]
+    tds.api.solve_normalized_xscatter(plan, an, cn, dn, dst, R, stride)
+    torch.cuda.synchronize()
+    for h in range(G):
+        assert torch.equal(dst[h][:, :R], xref[:, h * R:(h + 1) * R])
+        assert bool((dst[h][:, R:] == 7.0).all())
