@@ -68,7 +68,8 @@ for label, dt, n, G, kd, chunks in [("huge loopback G=4 kd=3", F32, 1 << 16, 4, 
                                     ("huge loopback G=2 kd=4 chunks=2", F64, 1 << 15, 2, 4, 2),
                                     ("huge G=1 kd=5", F32, 1 << 16, 1, 5, 1),
                                     ("huge loopback peer G=4 kd=3", F32, 1 << 16, 4, 3, 1),
-                                    ("huge loopback peer G=2 kd=4", F64, 1 << 15, 2, 4, 1)]:
+                                    ("huge loopback peer G=2 kd=4", F64, 1 << 15, 2, 4, 1),
+                                    ("huge loopback peer x-fused G=2 kd=3", F32, 1 << 23, 2, 3, 1)]:
     tdt = torch.float32 if dt == F32 else torch.float64
     name = "float32" if dt == F32 else "float64"
     be = tdist.CudaBackend(tdt, "cuda:0")
