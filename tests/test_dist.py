@@ -598,3 +598,36 @@ def test_solve_normalized_xscatter_bit_exact(dtype):
     for h in range(G):
         assert torch.equal(dst[h][:, :R], xref[:, h * R:(h + 1) * R])
         assert bool((dst[h][:, R:] == 7.0).all())
+
+
+def test_solve_xscatter_argument_errors():
+    """tds_solve_normalized_xscatter's shape rules, before anything is enqueued."""
+    import paper_conf_ipps_davidsonzo11_b200 as tds
+    from paper_conf_ipps_davidsonzo11_b200 import _lib as L
+    lib = L.load()
+    p = tds.Plan(1 << 20, 2, "float32", props=dataclasses.asdict(rp.B200))
+    p.set_params(k_pass=[7], cluster=1, cr_levels=4, thomas_chains=1, tl_levels=5)
+    spec = L.XScatter()
+    spec.groups, spec.rows_per_group, spec.dst_system_stride = 4, 1 << 18, 1 << 18
+    for h in range(4):
+        spec.dst[h] = (1 << 40) + h * (1 << 24)
+    A, W = 1 << 36, 1 << 38
+    ws = p.workspace_bytes
+    call = lambda plan=p: lib.tds_solve_normalized_xscatter(plan.handle, A, A + (1 << 26), A + (2 << 26),
+                                                            ctypes.byref(spec), W, ws, None)
+    assert call() in (5, 7)                     # valid: fails only at the device check
+    spec.rows_per_group = 1 << 17
+    assert call() == 1                          # groups * rows_per_group != n
+    spec.rows_per_group, spec.groups = 1 << 19, 2
+    spec.dst_system_stride = (1 << 19) - 4
+    assert call() == 1                          # stride < rows_per_group
+    spec.dst_system_stride = 1 << 19
+    assert call() in (5, 7)
+    spec.dst[1] = (1 << 40) + 8
+    assert call() == 1                          # misaligned destination
+    spec.dst[1] = (1 << 40) + (1 << 24)
+    q = tds.Plan(65536, 2, "float32", props=dataclasses.asdict(rp.B200))
+    q.set_params(k_pass=[3], cluster=1, cr_levels=4, thomas_chains=1, tl_levels=5)
+    spec.groups, spec.rows_per_group, spec.dst_system_stride = 2, 32768, 32768
+    assert lib.tds_solve_normalized_xscatter(q.handle, A, A + (1 << 26), A + (2 << 26), ctypes.byref(spec), W,
+                                             q.workspace_bytes, None) == 2  # k < 5: no TMA placement
