@@ -119,7 +119,19 @@ typedef struct {
                                         gathers residue class r with stride 2^k and scatters x
                                         in place (no de-interleave, no placement kernel); needs
                                         one split pass with k_pass <= 4, cluster 1,
-                                        tl_levels 5, 2^c sizeof(T) = 64, x_group 0 */
+                                        tl_levels 5, 2^c sizeof(T) = 64, x_group 0.
+                                        2: the paper's second variant, coalesced loads with a
+                                        global-memory fallback: the same in-place
+                                        split output; one CTA solves G = 32 / sizeof(T)
+                                        consecutive residues (every access a whole 32-byte
+                                        sector), holds as many of their rows as fit in shared
+                                        memory and keeps the rest in the workspace, runs
+                                        log2(thomas_chains) PCR levels and Thomas per chain,
+                                        x stored in place; needs one split pass with
+                                        log2(G) <= k_pass <= 4, cr_levels 0, tl_levels 0,
+                                        cluster 1, x_group 0, G x thomas_chains <= 1024,
+                                        batch_stride x sizeof(T) a multiple of 16;
+                                        any subsystem length (no on-chip size limit) */
 } tds_params;
 
 /* Everything a plan decided (read-only view). */

@@ -57,7 +57,7 @@ struct WsBufs {
 template <typename T>
 static WsBufs<T> ws_bufs(const tds_plan_info &I, void *ws) {
     WsBufs<T> w{};
-    const int nbuf = I.params.passes >= 2 ? 2 : 1;
+    const int nbuf = I.params.passes >= 2 || I.params.strided == 2 ? 2 : 1;
     const int64_t E = int64_t(I.workspace_bytes / (size_t(nbuf) * 3 * sizeof(T)));
     T *base = static_cast<T *>(ws);
     for (int i = 0; i < nbuf; ++i) {
@@ -71,6 +71,14 @@ static WsBufs<T> ws_bufs(const tds_plan_info &I, void *ws) {
         w.d[1] = w.d[0];
     }
     return w;
+}
+
+// Per-system stride of the in-place (natural order) split output of the
+// strided variants: whole 32-byte sectors, so a coalesced group of
+// 32 / sizeof(T) residues is one aligned sector (onchip_coalesced.cu).
+template <typename T>
+static int64_t natural_stride(int64_t n) {
+    return round_up(n, 32 / int64_t(sizeof(T)));
 }
 
 // Launch the P split passes; returns the index of the buffer holding the result.
@@ -120,7 +128,7 @@ static tds_status run_split(const tds_plan_info &I, const T *a, const T *b, cons
         A.vec = p == 0 ? (raw ? vec_ok(I, {a, b, c, d}) : vec_ok(I, {a, c, d})) : 1;
         if (natural) {  // strided variant: one pass, rows kept in original order (per system stride)
             A.natural = 1;
-            A.out_slot = round_up(I.n, 16 / int64_t(sizeof(T)));
+            A.out_slot = natural_stride<T>(I.n);
         }
         const int64_t grid = m_in * A.segs;
         if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "split grid exceeds 2^31-1 CTAs");
@@ -162,6 +170,8 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
     A.x_group = P.x_group;
     // strided variant (the paper's in-place subsystems): needs the TMA split kernel (16-byte aligned input)
     const bool strided_ok = P.strided && P.k > 0 && vec_ok(I, {a, b, c, d});
+    if (P.strided == 2 && !strided_ok)  // no de-interleaved fallback: the plan's CTA size is the coalesced kernel's
+        return fail(TDS_ERR_UNSUPPORTED, "strided 2 needs 16-byte aligned a, b, c, d and batch_stride");
     int64_t grid;
     if (P.k == 0) {
         A.a = a;
@@ -193,11 +203,17 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
     if (P.passes >= first && P.passes <= last) {
         if (grid > 0x7fffffffLL) return fail(TDS_ERR_UNSUPPORTED, "on-chip grid exceeds 2^31-1 CTAs");
         cudaError_t err;
-        if (strided_ok) {
+        if (strided_ok && P.strided == 2) {
+            // coalesced 32-byte sectors of G adjacent residues, rows beyond shared memory in the workspace
+            WsBufs<T> w = ws_bufs<T>(I, ws);
+            int l2t = 0;
+            while ((1 << l2t) < P.thomas_chains) ++l2t;
+            err = launch_onchip_coalesced<T>(w.a, w.c, w.d, x, I.n, I.m, I.batch_stride,
+                                             natural_stride<T>(I.n), P.k, l2t, int64_t(smem_optin_current()) - kSmemReserve, st);
+        } else if (strided_ok) {
             // gather residue classes with stride 2^k from the in-place split output, x scattered in place
             A.x = x;
-            err = launch_onchip_strided<T>(A, I.m << P.k, I.onchip_threads, round_up(I.n, 16 / int64_t(sizeof(T))),
-                                           st);
+            err = launch_onchip_strided<T>(A, I.m << P.k, I.onchip_threads, natural_stride<T>(I.n), st);
         } else if (P.k == 0 && onchip_cpipe_ok(I) && A.vec) {
             // persistent, TMA-fed warp-form kernel on one CTA or a 2-CTA cluster per system
             err = launch_onchip_cpipe<T>(A, I.onchip_threads, sm_count_current(), st);
@@ -232,7 +248,8 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
 int32_t onchip_form_of(const tds_plan_info &I) {
     const tds_params &P = I.params;
     bool warp;
-    if (P.strided || P.x_group > 0) warp = true;  // onchip_strided / onchip_gpipe: solve_item_warp
+    if (P.strided == 2) warp = false;  // onchip_coalesced: PCR levels + Thomas per chain
+    else if (P.strided || P.x_group > 0) warp = true;  // onchip_strided / onchip_gpipe: solve_item_warp
     else if (P.k == 0) warp = onchip_cpipe_ok(I);
     else warp = onchip_pipe_ok(I) && P.tl_levels == 5;
     return warp ? TDS_FORM_WARP_CR : TDS_FORM_PCR_THOMAS;
@@ -550,7 +567,7 @@ tds_status tds_plan_slots_layout(const tds_plan_t plan, tds_slots_layout *out) {
     const tds_plan_info &I = plan->info;
     if (I.params.k < 1 || I.params.strided) return fail(TDS_ERR_UNSUPPORTED, "slots need k >= 1 and strided = 0");
     if (I.chunks != 1) return fail(TDS_ERR_UNSUPPORTED, "slots of a chunked plan are reused per chunk");
-    const int nbuf = I.params.passes >= 2 ? 2 : 1;
+    const int nbuf = I.params.passes >= 2 || I.params.strided == 2 ? 2 : 1;
     const int64_t E = int64_t(I.workspace_bytes / (size_t(nbuf) * 3 * size_t(dsize(I.dtype))));
     const int ob = (I.params.passes - 1) & 1;
     out->a_offset = (3 * ob + 0) * E;

@@ -21,6 +21,7 @@ constexpr int kMaxPasses = TDS_MAX_PASSES;
 //   4 pipe shared-memory form: reduced PCR, strides >= 4
 //   5 onchip (generic / cluster) leader PCR, strides >= 4
 //   6 onchip cluster: the deferred chain loses the next CTA's ghost rows
+//   7 onchip_coalesced: PCR levels, strides >= 4
 #ifndef TDS_MUTATE
 #define TDS_MUTATE 0
 #endif
@@ -198,6 +199,11 @@ cudaError_t launch_transpose(const T *const *in, T *const *out, int narrays, int
 template <typename T>
 cudaError_t launch_onchip_strided(const OnchipArgs<T> &A, int64_t nslots, int threads, int64_t ws_stride,
                                   cudaStream_t st);
+
+template <typename T>
+cudaError_t launch_onchip_coalesced(T *const wa[2], T *const wc[2], T *const wd[2], T *x, int64_t n, int64_t m,
+                                    int64_t batch_stride, int64_t ws_stride, int K, int log2T, int64_t smem_budget,
+                                    cudaStream_t st);
 
 template <typename T>
 cudaError_t launch_onchip_gpipe(const OnchipArgs<T> &A, int64_t nslots, int threads, int sm_count, cudaStream_t st);

@@ -93,6 +93,19 @@ inline int sm_count_current() {
     return sms[dev];
 }
 
+// Host: opt-in shared memory per CTA of the current device (cached).
+inline int smem_optin_current() {
+    static int v[64] = {0};
+    int dev = 0;
+    if (cudaGetDevice(&dev) != cudaSuccess || dev < 0 || dev >= 64) return 232448;
+    if (v[dev] == 0) {
+        int x = 0;
+        cudaDeviceGetAttribute(&x, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev);
+        v[dev] = x > 0 ? x : 232448;
+    }
+    return v[dev];
+}
+
 // Host: launch with programmatic stream serialisation (plus an optional cluster).
 template <typename... KArgs, typename... Args>
 inline cudaError_t launch_pdl(void (*kern)(KArgs...), dim3 grid, dim3 block, size_t smem, cudaStream_t st,

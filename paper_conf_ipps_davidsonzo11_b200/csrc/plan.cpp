@@ -139,8 +139,11 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
     if (p.split_only && p.k == 0) return fail(TDS_ERR_INVALID_ARG, "a split-only plan needs k >= 1");
     const int64_t n_sub = cdiv(n, int64_t(1) << std::min(p.k, 62));
     const int64_t nred = cdiv(n_sub, int64_t(R) * p.cluster);
-    const int64_t threads = p.split_only ? 32 : std::max<int64_t>(32, round_up(nred, 32));
-    if (!p.split_only) {  // the on-chip stage must fit (a split-only plan never launches it)
+    const bool coalesced = p.strided == 2;  // global fallback: no on-chip size limit
+    const int64_t threads = p.split_only ? 32
+                            : coalesced  ? coalesced_threads(dtype, n_sub, p.thomas_chains)
+                                         : std::max<int64_t>(32, round_up(nred, 32));
+    if (!p.split_only && !coalesced) {  // the on-chip stage must fit (a split-only plan never launches it)
         if (threads > onchip_max_threads(R, dsize(dtype)))
             return fail(TDS_ERR_UNSUPPORTED, "subsystem too large for the on-chip kernel (n_sub / (2^c cluster) > "
                                              "1024, or > 512 when 2^c * sizeof(T) >= 64)");
@@ -172,12 +175,27 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
         }
     }
     if (p.chunk_systems < 0) return fail(TDS_ERR_INVALID_ARG, "chunk_systems >= 0");
-    if (p.strided != 0) {  // the paper's strided base-kernel variant (onchip_strided.cu)
-        if (p.strided != 1) return fail(TDS_ERR_INVALID_ARG, "strided must be 0 or 1");
+    if (p.strided == 1) {  // the paper's strided base-kernel variant (onchip_pipe.cu, strided kernel)
         if (p.split_only || p.passes != 1 || p.k_pass[0] > 4 || p.x_group != 0)
             return fail(TDS_ERR_UNSUPPORTED, "strided needs one split pass with k_pass <= 4 and x_group 0");
         if (p.cluster != 1 || p.tl_levels != 5 || R * dsize(dtype) != 64)
             return fail(TDS_ERR_UNSUPPORTED, "strided needs cluster 1, tl_levels 5, 64 bytes of rows per thread");
+    } else if (coalesced) {  // the paper's coalesced variant with global fallback (onchip_coalesced.cu)
+        const int G = 32 / dsize(dtype);
+        if (p.split_only || p.passes != 1 || p.k_pass[0] > 4 || (1 << p.k) < G || p.x_group != 0)
+            return fail(TDS_ERR_UNSUPPORTED, "strided 2 needs one split pass with log2(32 / sizeof(T)) <= k_pass "
+                                             "<= 4 and x_group 0");
+        if (p.cluster != 1 || p.cr_levels != 0 || p.tl_levels != 0)
+            return fail(TDS_ERR_UNSUPPORTED, "strided 2 needs cluster 1, cr_levels 0, tl_levels 0");
+        if (n_sub >= (int64_t(1) << 31))
+            return fail(TDS_ERR_UNSUPPORTED, "strided 2 needs n / 2^k < 2^31");
+        if ((info.batch_stride * dsize(dtype)) % 16)
+            return fail(TDS_ERR_UNSUPPORTED, "strided 2 needs batch_stride x sizeof(T) a multiple of 16 (it reads "
+                                             "the TMA split's in-place output)");
+        if (int64_t(G) * p.thomas_chains > 1024)
+            return fail(TDS_ERR_INVALID_ARG, "strided 2 needs (32 / sizeof(T)) x thomas_chains <= 1024");
+    } else if (p.strided != 0) {
+        return fail(TDS_ERR_INVALID_ARG, "strided must be 0, 1 or 2");
     }
     if (p.x_group != 0) {  // fused x placement (onchip_pipe.cu, gpipe kernel)
         const int G = p.x_group, ds = dsize(dtype);
@@ -211,7 +229,8 @@ tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_
         }
         const int64_t E = round_up(elems, 64);
         info.slot_rows = slot_rows(n, p.k, dtype);
-        info.workspace_bytes = size_t((p.passes == 1 ? 1 : 2) * 3 * E * dsize(dtype));
+        // two buffers for multi-pass plans and for the coalesced variant's global-fallback ping-pong
+        info.workspace_bytes = size_t((p.passes == 1 && !coalesced ? 1 : 2) * 3 * E * dsize(dtype));
         info.split_tile_eff = split_tile_eff(p, 0);
         info.split_segments = split_segments(mc, cdiv(n, info.split_tile_eff), p.theta);
     } else {

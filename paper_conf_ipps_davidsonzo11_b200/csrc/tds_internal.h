@@ -44,5 +44,9 @@ int32_t static_cluster(const tds_device_props &p);
 tds_status derive(tds_plan_info &info, const tds_device_props &props, const tds_params &p);
 // The on-chip form the dispatch selects (api.cu solve_impl) for 16-byte aligned arrays.
 int32_t onchip_form_of(const tds_plan_info &I);
+// The coalesced base-kernel variant (strided = 2, onchip_coalesced.cu): rows per
+// subsystem held in shared memory, and the CTA size.
+int32_t coalesced_rows_in_smem(int32_t dtype, int64_t L, int64_t smem_budget);
+int32_t coalesced_threads(int32_t dtype, int64_t L, int32_t thomas_chains);
 
 }  // namespace tds

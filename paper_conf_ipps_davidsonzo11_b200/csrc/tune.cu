@@ -103,13 +103,15 @@ static void clamp_onchip(const tds_plan_st *plan, tds_params &p) {
     if (warp_form(plan, p)) p.thomas_chains = 1;
 }
 
-// Stage 3->4: hill climb over (form, c, T, c2, cluster, x placement) for the current k.
+static void fit_onchip(const tds_plan_st *plan, tds_params &p);
+
+// Stage 3->4: hill climb over (form, c, T, c2, cluster, x placement, load variant) for the current k.
 static void tune_onchip(Search &S, tds_params &best, double &t_best) {
     const tds_plan_info &I = S.plan->info;
     bool improved = true;
     while (improved && !out_of_time(S)) {
         improved = false;
-        tds_params cand[18];
+        tds_params cand[20];
         int nc = 0;
         // the warp-level form (CR across all 32 lanes, shuffles only) is a
         // different kernel path, not a neighbour of tl_levels = 4: try it directly
@@ -156,6 +158,23 @@ static void tune_onchip(Search &S, tds_params &best, double &t_best) {
             best.x_group == 0 && (1 << best.cr_levels) * dsize(I.dtype) == 64) {
             cand[nc] = best;
             cand[nc++].strided = best.strided ? 0 : 1;
+        }
+        // the paper's coalesced base-kernel variant with global fallback (strided = 2):
+        // on from any form of a one-pass plan of log2(G) <= k <= 4 levels (the paper's
+        // T = 64 to start), off back to the fitted default form
+        if (best.k > 0 && best.passes == 1 && best.k_pass[0] <= 4 && (1 << best.k) >= 32 / dsize(I.dtype) &&
+            best.x_group == 0) {
+            cand[nc] = best;
+            if (best.strided == 2) {
+                fit_onchip(S.plan, cand[nc]);
+            } else {
+                cand[nc].strided = 2;
+                cand[nc].cr_levels = 0;
+                cand[nc].tl_levels = 0;
+                cand[nc].cluster = 1;
+                cand[nc].thomas_chains = std::min(64, 1024 / (32 / dsize(I.dtype)));
+            }
+            ++nc;
         }
         for (int i = 0; i < nc; ++i) {
             clamp_onchip(S.plan, cand[i]);

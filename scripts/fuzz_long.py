@@ -16,7 +16,7 @@ from paper_conf_ipps_davidsonzo11_b200 import inputs  # noqa: E402
 
 draws = int(sys.argv[1]) if len(sys.argv) > 1 else 2000
 rng = np.random.default_rng(int(sys.argv[2]) if len(sys.argv) > 2 else 7)
-ran = bad = inter = coupled = 0
+ran = bad = inter = coupled = cv = 0
 for i in range(draws):
     dtype = np.float32 if rng.random() < 0.7 else np.float64
     n = int(rng.choice([rng.integers(1, 5000), rng.integers(5000, 400000), 1 << int(rng.integers(10, 20))]))
@@ -27,9 +27,11 @@ for i in range(draws):
     c_lv = int(rng.integers(0, 5 if dtype == np.float32 else 4))
     params = dict(k_pass=kp, cr_levels=c_lv, thomas_chains=int(2 ** rng.integers(0, 7)),
                   cluster=int(rng.choice([1, 1, 1, 2, 4, 8, 16])), tl_levels=int(rng.choice([0, 1, 2, 3, 5])),
-                  x_group=int(rng.choice([0, 0, 0, 2, 4, 8])), strided=int(rng.choice([0, 0, 1])),
+                  x_group=int(rng.choice([0, 0, 0, 2, 4, 8])), strided=int(rng.choice([0, 0, 1, 2])),
                   split_threads=int(rng.choice([128, 256, 512])), split_tile_rows=int(rng.choice([2048, 4096, 8192])),
                   theta=int(rng.choice([1, 16, 148, 4736])), chunk_systems=int(rng.choice([0, 0, 1, 2, 3])))
+    if params["strided"] == 2:  # the coalesced variant: PCR-Thomas without register / thread CR levels
+        params.update(cr_levels=0, tl_levels=0)
     plan = tds.Plan(n, m, "float32" if dtype == np.float32 else "float64", device=0)
     try:
         plan.set_params(**params)
@@ -60,9 +62,10 @@ for i in range(draws):
         ok = bool(np.array_equal(xi.cpu().numpy().T, x))
         inter += 1
     ran += 1
+    cv += plan.info["strided"] == 2
     if not ok:
         bad += 1
         print(f"BAD draw {i}: {dtype.__name__} {fam} n={n} m={m} {params} err={err:.3e}", flush=True)
 print(f"fuzz: {ran} plans run ({inter} also through the interleaved layout, {coupled} on coupled fp64 "
-      f"families), {bad} bad", flush=True)
+      f"families, {cv} coalesced-variant plans), {bad} bad", flush=True)
 sys.exit(1 if bad else 0)

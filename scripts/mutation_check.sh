@@ -2,11 +2,11 @@
 # Mutation check of the coupling tests ("a debug build that
 # zeroes the top-row coupling makes the new tests fail").
 #
-#   scripts/mutation_check.sh build      # here (CPU): libtds_mut{1..6}.so under build/mut/
+#   scripts/mutation_check.sh build      # here (CPU): libtds_mut{1..7}.so under build/mut/
 #   scripts/mutation_check.sh run OUT    # on the GPU box: run tests/test_coupling.py against each
 #
 # Each mutant is the product library with ONE long-range coupling term
-# dropped (csrc/common.cuh TDS_MUTATE sites 1-6); only the three on-chip
+# dropped (csrc/common.cuh TDS_MUTATE sites 1-7); only the four on-chip
 # translation units are recompiled, the rest are the product objects.
 set -u
 ROOT=$(cd "$(dirname "$0")/.." && pwd)
@@ -15,7 +15,7 @@ MUT=$ROOT/build/mut
 NVCC=${NVCC:-/usr/local/cuda/bin/nvcc}
 ARCH="-gencode arch=compute_100a,code=sm_100a"
 FLAGS="-O3 -std=c++17 -lineinfo $ARCH -Xcompiler -fPIC"
-SITES="1 2 3 4 5 6"
+SITES="${SITES:-1 2 3 4 5 6 7}"
 case "${1:-}" in
 build)
     make -C "$CSRC" -j8 >/dev/null || exit 1
@@ -25,7 +25,7 @@ build)
         for f in "$ROOT"/build/csrc/*.o; do
             b=$(basename "$f" .o)
             case $b in
-            onchip|onchip_pipe|onchip_cpipe)
+            onchip|onchip_pipe|onchip_cpipe|onchip_coalesced)
                 $NVCC $FLAGS -DTDS_MUTATE=$k -c "$CSRC/$b.cu" -o "$MUT/o$k/$b.o" &
                 objs="$objs $MUT/o$k/$b.o" ;;
             *) objs="$objs $f" ;;

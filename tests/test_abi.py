@@ -242,8 +242,37 @@ def test_strided_variant_validation(tds):
     base = dict(k_pass=[3], cr_levels=4, thomas_chains=16, cluster=1, tl_levels=5)
     p.set_params(**base, strided=1)
     assert p.info["strided"] == 1 and p.info["launches"] == 2
-    for kw in [dict(strided=2), dict(strided=1, k_pass=[2, 1]), dict(strided=1, k_pass=[5]),
+    for kw in [dict(strided=2), dict(strided=3), dict(strided=1, k_pass=[2, 1]), dict(strided=1, k_pass=[5]),
                dict(strided=1, tl_levels=3), dict(strided=1, cr_levels=3), dict(strided=1, cluster=2),
                dict(strided=1, x_group=8)]:
+        with pytest.raises(tds.TdsError):
+            p.set_params(**dict(base, **kw))
+
+
+def test_coalesced_variant_validation(tds):
+    """The paper's second base-kernel variant (tds_params.strided = 2,
+    P:L286-292): one split pass of log2(32 / sizeof(T)) <= k <= 4 levels,
+    cr_levels = tl_levels = 0, cluster 1; two launches (x stored in place),
+    two workspace buffers (the global-fallback ping-pong), the PCR-Thomas
+    form, and no on-chip size limit (rows beyond shared memory stay global)."""
+    base = dict(k_pass=[3], cr_levels=0, thomas_chains=64, cluster=1, tl_levels=0, strided=2)
+    p = tds.Plan(65536, 8, props=_props(rp.B200))
+    p.set_params(**base)
+    one = tds.Plan(65536, 8, props=_props(rp.B200))
+    one.set_params(k_pass=[3], cr_levels=4, thomas_chains=1, cluster=1, tl_levels=5)
+    assert p.info["strided"] == 2 and p.info["launches"] == 2
+    assert p.info["workspace_bytes"] == 2 * one.info["workspace_bytes"]
+    assert p.info["onchip_form"] == 0  # TDS_FORM_PCR_THOMAS
+    assert p.info["onchip_threads"] == 512  # 8 residues x T = 64 chains
+    big = tds.Plan(1 << 20, 16, props=_props(rp.B200))  # 65536-row subsystems: beyond any on-chip kernel
+    big.set_params(**dict(base, k_pass=[4], thomas_chains=128))
+    assert big.info["onchip_threads"] == 1024 and big.info["n_sub"] == 65536
+    with pytest.raises(tds.TdsError):
+        big.set_params(**dict(base, k_pass=[4], strided=0, cr_levels=4, tl_levels=5))
+    d = tds.Plan(9001, 4, "float64", props=_props(rp.B200), batch_stride=9002)
+    d.set_params(**dict(base, k_pass=[2], thomas_chains=256))  # fp64: G = 4, 4 x 256 threads
+    assert d.info["onchip_threads"] == 1024
+    for kw in [dict(k_pass=[2]), dict(k_pass=[5]), dict(k_pass=[2, 1]), dict(cr_levels=1), dict(tl_levels=1),
+               dict(cluster=2), dict(x_group=8), dict(thomas_chains=256), dict(split_only=1)]:
         with pytest.raises(tds.TdsError):
             p.set_params(**dict(base, **kw))

@@ -25,7 +25,8 @@ Each FORM names the kernel the C++ dispatch (csrc/api.cu solve_impl) selects
 for its plan: k = 0 warp form -> onchip_cpipe (cluster 1/2/4/8), cluster 16 ->
 onchip (generic, leader PCR-Thomas), k > 0 with 64 bytes of rows per thread ->
 onchip_pipe (tl_levels 5: warp form, else shared-memory PCR-Thomas), x_group
--> onchip_gpipe, strided -> onchip_strided, k > 0 with cluster > 1 -> onchip.
+-> onchip_gpipe, strided 1 -> onchip_strided, strided 2 -> onchip_coalesced,
+k > 0 with cluster > 1 -> onchip.
 Shapes are the BASELINE configs' (2^20 split by 2^8, 16384 on a cluster, 65536
 on 16 CTAs) with enough systems that the persistent kernels loop.
 """
@@ -60,6 +61,10 @@ FORMS = [
     ("xgroup8", F64, 1 << 20, 2, dict(k_pass=[8], cr_levels=3, cluster=1, x_group=8, **_W), "batched"),
     ("strided_k4", F64, 65536, 3, dict(k_pass=[4], cr_levels=3, cluster=1, strided=1, **_W), "batched"),
     ("interleaved_c4", F64, 16384, 40, dict(k_pass=[], cr_levels=3, cluster=4, **_W), "interleaved"),
+    ("coalesced_k4", F64, 65536, 3, dict(k_pass=[4], cr_levels=0, thomas_chains=64, tl_levels=0, cluster=1,
+                                         strided=2), "batched"),                   # 4096 rows: global fallback
+    ("coalesced_k2_T8", F64, 4096, 8, dict(k_pass=[2], cr_levels=0, thomas_chains=8, tl_levels=0, cluster=1,
+                                           strided=2), "batched"),                 # 1024 rows on chip
 ]
 
 FAMILIES = [("poisson", {}), ("const", {"param": 1e-6}), ("weak", {"param": 0.01}), ("adi", {"param": 100.0})]
@@ -77,6 +82,8 @@ FORMS32 = [
     ("xgroup8", F32, 16384, 40, dict(k_pass=[3], cr_levels=4, cluster=1, x_group=8, **_W), "batched"),
     ("strided_k1", F32, 16384, 40, dict(k_pass=[1], cr_levels=4, cluster=1, strided=1, **_W), "batched"),
     ("interleaved_c2", F32, 16384, 64, dict(k_pass=[], cr_levels=4, cluster=2, **_W), "interleaved"),
+    ("coalesced_k3", F32, 16384, 40, dict(k_pass=[3], cr_levels=0, thomas_chains=16, tl_levels=0, cluster=1,
+                                          strided=2), "batched"),                  # 2048 rows: global fallback
 ]
 
 

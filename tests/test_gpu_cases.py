@@ -57,6 +57,14 @@ def _cases():
     return out
 
 
+CV = [(dt, n, m, tgp._cv_params(k, T), tgp.cv_stride(dt, n)) for dt, n, m, k, T in tgp.CV_CASES]
+
+
+@pytest.mark.parametrize("dtype,n,m,params,stride", CV)
+def test_coalesced_case_is_accepted(tds, dtype, n, m, params, stride):
+    assert _accepts(tds, dtype, n, m, params, stride)["strided"] == 2
+
+
 CASES = _cases()
 
 

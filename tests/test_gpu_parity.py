@@ -871,6 +871,96 @@ def test_plan_fuzz(tds, i, dtype, n, m, params):
     check(a, b, c, d, x, dtype)
 
 
+# ------------------------------------- the paper's coalesced base-kernel variant (strided = 2)
+
+CV_CASES = [  # (dtype, n, m, k, T): J = 1205 rows per subsystem fit in shared memory, the rest is global
+    (np.float32, 16384, 7, 4, 16),        # L = 1024: every row on chip, no fallback
+    (np.float32, 65536, 5, 3, 64),        # L = 8192: 85 % of the rows through the global fallback
+    (np.float32, 100003, 3, 4, 64),       # ragged: residues of 6251 and 6250 rows in one group
+    (np.float32, 8191 * 4 + 3, 2, 3, 1),  # T = 1: Thomas on whole subsystems, ragged
+    (np.float32, 1 << 20, 2, 4, 128),     # L = 65536 (config-3 systems, one pass of 4 levels)
+    (np.float32, 4096, 3, 4, 128),        # T = 128 of L = 256: chains of 2 rows
+    (np.float32, 27, 3, 4, 2),            # n < 2^k: residues 27.. of the last group are empty
+    (np.float32, 1205 * 8 + 8, 2, 3, 8),  # L = J + 1: exactly one global row per subsystem
+    (np.float64, 32768, 3, 2, 64),        # fp64 group of 4 residues, L = 8192
+    (np.float64, 9001, 4, 3, 256),        # fp64 ragged, T = 256 (1024 threads)
+    (np.float64, 2411 * 4, 2, 2, 32)]     # fp64 L = 2411: J + 1206 global rows
+
+
+def _cv_params(k, T):
+    return dict(k_pass=[k], cr_levels=0, thomas_chains=T, cluster=1, tl_levels=0, strided=2)
+
+
+def cv_stride(dtype, n):
+    """The variant reads the TMA split's in-place output: systems start on 16 bytes."""
+    e = 16 // np.dtype(dtype).itemsize
+    return -(-n // e) * e
+
+
+@pytest.mark.parametrize("dtype,n,m,k,T", CV_CASES)
+def test_coalesced_variant(tds, dtype, n, m, k, T):
+    """strided = 2: groups of 32 / sizeof(T) adjacent residues
+    read as whole sectors, rows beyond shared memory read and written in the
+    workspace (global fallback), PCR-Thomas, x stored in place: the oracle's
+    x within the tolerances, two launches (ragged n on a 16-byte batch stride)."""
+    import torch
+    a, b, c, d = inputs.generate(n, m, dtype, seed=170 + k)
+    stride = cv_stride(dtype, n)
+    pad = lambda v: np.pad(v, ((0, 0), (0, stride - n)), constant_values=3.0)
+    A, B, C, D = (torch.from_numpy(pad(v).reshape(-1)).cuda() for v in (a, b, c, d))
+    plan = tds.Plan(n, m, "float32" if dtype == np.float32 else "float64", device=0, batch_stride=stride)
+    plan.set_params(**_cv_params(k, T))
+    assert plan.info["strided"] == 2 and plan.info["launches"] == 2
+    out = torch.full_like(D, 5.0)
+    tds.solve_batched(plan, A, B, C, D, out=out)
+    torch.cuda.synchronize()
+    xs = out.cpu().numpy().reshape(m, stride)
+    assert np.all(xs[:, n:] == 5.0)
+    check(a, b, c, d, np.ascontiguousarray(xs[:, :n]), dtype)
+
+
+def test_coalesced_variant_stride_and_alignment(tds):
+    """A padded batch stride leaves the padding; unaligned input rows are
+    refused (UNSUPPORTED: the variant reads the TMA split's in-place output),
+    and so is a batch stride that is not a 16-byte multiple (planner)."""
+    import torch
+    n, m, stride = 20000, 3, 20012
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=178)
+    pad = lambda v: np.pad(v, ((0, 0), (0, stride - n)), constant_values=7.0)
+    A, B, C, D = (torch.from_numpy(pad(v).reshape(-1)).cuda() for v in (a, b, c, d))
+    plan = tds.Plan(n, m, "float32", device=0, batch_stride=stride)
+    plan.set_params(**_cv_params(3, 32))
+    out = torch.full_like(D, 7.0)
+    tds.solve_batched(plan, A, B, C, D, out=out)
+    torch.cuda.synchronize()
+    xs = out.cpu().numpy().reshape(m, stride)
+    assert np.all(xs[:, n:] == 7.0)
+    check(a, b, c, d, xs[:, :n], np.float32)
+    plan2 = tds.Plan(n, m, "float32", device=0)
+    plan2.set_params(**_cv_params(3, 32))
+    ta, tb, tc, td = (torch.zeros(m * n + 1, dtype=torch.float32, device="cuda")[1:].view(m, n) for _ in range(4))
+    with pytest.raises(tds.TdsError) as e:
+        tds.solve_batched(plan2, ta, tb, tc, td)
+    assert e.value.name == "TDS_ERR_UNSUPPORTED"
+    plan3 = tds.Plan(20001, m, "float32", device=0)
+    with pytest.raises(tds.TdsError) as e:
+        plan3.set_params(**_cv_params(3, 32))
+    assert e.value.name == "TDS_ERR_UNSUPPORTED"
+
+
+def test_coalesced_variant_interleaved_layout(tds):
+    """The variant under the batch-interleaved entry point (tds_solve_interleaved)."""
+    import torch
+    n, m = 4096, 64
+    a, b, c, d = inputs.generate(n, m, np.float32, seed=179)
+    plan = tds.Plan(n, m, "float32", device=0)
+    plan.set_params(**_cv_params(4, 16))
+    ti = [torch.from_numpy(np.ascontiguousarray(v.T)).cuda() for v in (a, b, c, d)]
+    x = tds.solve_interleaved(plan, *ti)
+    torch.cuda.synchronize()
+    check(a, b, c, d, x.cpu().numpy().T, np.float32)
+
+
 # ------------------------------------- the paper's strided base-kernel variant
 
 SV_CASES = [  # (dtype, n, m, k)

@@ -200,3 +200,27 @@ def test_aborting_cost_leaves_the_plan(tds):
     with pytest.raises(tds.TdsError):
         p.tune_search(lambda q: 1e30)  # the seed refused
     assert p.info == before
+
+
+def test_load_variants_are_a_tuner_dimension(tds):
+    """The paper's two base-kernel load variants, chosen by the
+    tuner per workload: when the coalesced variant with global
+    fallback (strided = 2) is cheapest at the one-pass k <= 4 plans it is
+    kept, and its Thomas switch T is then searched (its form is PCR-Thomas);
+    when the strided gather is cheapest, that one is kept."""
+    def coalesced_fast(q):
+        if q["strided"] == 2:
+            return 0.3 + 0.05 * abs(l2(q["thomas_chains"]) - 4)  # optimum T = 16
+        return 1.0 if q["k"] <= 4 else 2.0
+    p, seen = run(tds, coalesced_fast, n=65536, m=256)
+    i = p.info
+    assert i["strided"] == 2 and i["passes"] == 1 and i["k"] <= 4 and i["onchip_form"] == 0
+    assert i["thomas_chains"] == 16 and i["cr_levels"] == 0 and i["tl_levels"] == 0
+    assert {q["thomas_chains"] for q in seen if q["strided"] == 2} >= {64, 32, 16, 8}
+
+    def strided_fast(q):  # the strided gather is a variant of the warp form (tl_levels = 5): reached through it
+        if q["k"] > 4:
+            return 2.0
+        return 0.5 if q["strided"] == 1 else (0.9 if q["tl_levels"] == 5 and q["strided"] == 0 else 1.0)
+    p1, seen1 = run(tds, strided_fast, n=65536, m=256)
+    assert p1.info["strided"] == 1 and any(q["strided"] == 2 for q in seen1)
