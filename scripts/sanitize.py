@@ -38,7 +38,7 @@ CASES = [  # (label, dtype, n, m, params or None for the static plan)
     ("f64 strided k2", F64, 9001, 2, dict(k_pass=[2], cr_levels=3, thomas_chains=1, tl_levels=5, strided=1)),
     ("coalesced k3 (global fallback)", F32, 65536, 2, dict(k_pass=[3], cr_levels=0, thomas_chains=64, tl_levels=0,
                                                           strided=2)),
-    ("f64 coalesced k2", F64, 9001, 2, dict(k_pass=[2], cr_levels=0, thomas_chains=32, tl_levels=0, strided=2)),
+    ("f64 coalesced k2", F64, 9000, 2, dict(k_pass=[2], cr_levels=0, thomas_chains=32, tl_levels=0, strided=2)),
 ]
 
 bad = 0
