@@ -57,7 +57,9 @@ def _cases():
     return out
 
 
-CV = [(dt, n, m, tgp._cv_params(k, T), tgp.cv_stride(dt, n)) for dt, n, m, k, T in tgp.CV_CASES]
+CV = [(dt, n, m, tgp._cv_params(k, T), tgp.cv_stride(dt, n)) for dt, n, m, k, T in tgp.CV_CASES] + \
+    [(dt, 16384, 7, dict(tgp._cv_params(3, 64), chunk_systems=ch), 16384) for dt, ch in [(np.float32, 2),
+                                                                                       (np.float64, 3)]]
 
 
 @pytest.mark.parametrize("dtype,n,m,params,stride", CV)

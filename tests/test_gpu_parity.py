@@ -919,6 +919,20 @@ def test_coalesced_variant(tds, dtype, n, m, k, T):
     check(a, b, c, d, np.ascontiguousarray(xs[:, :n]), dtype)
 
 
+@pytest.mark.parametrize("dtype,chunk", [(np.float32, 2), (np.float64, 3)])
+def test_coalesced_variant_chunked(tds, dtype, chunk):
+    """Chunked plans (chunk_systems): every chunk reuses the workspace (both
+    buffers of the global fallback); x matches the unchunked plan bit for bit
+    (same arithmetic per system) and the oracle."""
+    n, m = 16384, 7
+    a, b, c, d = inputs.generate(n, m, dtype, seed=181)
+    x0, _ = run(tds, a, b, c, d, params=_cv_params(3, 64))
+    x1, plan = run(tds, a, b, c, d, params=dict(_cv_params(3, 64), chunk_systems=chunk))
+    assert plan.info["chunks"] == -(-m // chunk)
+    assert np.array_equal(x0, x1)
+    check(a, b, c, d, x1, dtype)
+
+
 def test_coalesced_variant_stride_and_alignment(tds):
     """A padded batch stride leaves the padding; unaligned input rows are
     refused (UNSUPPORTED: the variant reads the TMA split's in-place output),
