@@ -118,6 +118,31 @@ def main():
         emit({"study": "fig6_smem", "T": T, "ms_median": med, "eq_per_s": n * m / (med / 1e3),
               "plan": plan_summary(plan.info)})
 
+    del ta, tb, tc, td, x
+    # ---- the paper's load variants (tuned per workload P:L713-721) on Fig. 7's
+    # 2Kx2K and 4Kx4K workloads at one-pass k = 3 / 4: de-interleaved (strided 0, warp form),
+    # strided gather (1), coalesced groups with global fallback (2) over a Fig. 6 T sweep
+    for name, n, m in FIG7[1:3]:
+        a, b, c, d = inputs.generate(n, m, np.float32, seed=4)
+        ta, tb, tc, td = (torch.from_numpy(v).cuda() for v in (a, b, c, d))
+        x = torch.empty_like(td)
+        for k in (3, 4):
+            runs = [(0, dict(cr_levels=4, thomas_chains=1, tl_levels=5)), (1, dict(cr_levels=4, thomas_chains=1,
+                                                                                    tl_levels=5))]
+            runs += [(2, dict(cr_levels=0, thomas_chains=T, tl_levels=0)) for T in (1, 4, 16, 64)]
+            for sv, kw in runs:
+                plan = tds.Plan(n, m, "float32", device=0)
+                try:
+                    plan.set_params(k_pass=[k], cluster=1, strided=sv, **kw)
+                except tds.TdsError as e:
+                    emit({"study": "load_variants", "workload": name, "k": k, "strided": sv, "error": str(e)})
+                    continue
+                med, mn = time_plan(tds, plan, ta, tb, tc, td, x, args.reps)
+                emit({"study": "load_variants", "workload": name, "k": k, "strided": sv, "T": kw["thomas_chains"],
+                      "n_sub": -(-n >> k), "ms_median": med, "eq_per_s": n * m / (med / 1e3),
+                      "plan": plan_summary(plan.info)})
+        del ta, tb, tc, td, x
+
     with open(args.out + ".jsonl", "w") as f:
         for r in lines:
             f.write(json.dumps(r) + "\n")
@@ -138,6 +163,12 @@ def main():
     for r in lines:
         if r.get("study", "").startswith("fig6") and "ms_median" in r:
             md.append(f"| {r['study'][5:]} | {r['T']} | {r['ms_median']:.4f} | {r['eq_per_s']:.3g} |")
+    md += ["", "| load variant (P:L279-295) | workload | k | n_sub | T | ms | eq/s |", "|---|---|---|---|---|---|---|"]
+    names = {0: "de-interleaved (B200 primary, warp form)", 1: "strided gather", 2: "coalesced + global fallback"}
+    for r in lines:
+        if r.get("study") == "load_variants" and "ms_median" in r:
+            md.append(f"| {names[r['strided']]} | {r['workload']} | {r['k']} | {r['n_sub']} | {r['T']} | "
+                      f"{r['ms_median']:.4f} | {r['eq_per_s']:.3g} |")
     with open(args.out + ".md", "w") as f:
         f.write("\n".join(md) + "\n")
 

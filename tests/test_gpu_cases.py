@@ -59,12 +59,14 @@ def _cases():
 
 CV = [(dt, n, m, tgp._cv_params(k, T), tgp.cv_stride(dt, n)) for dt, n, m, k, T in tgp.CV_CASES] + \
     [(dt, 16384, 7, dict(tgp._cv_params(3, 64), chunk_systems=ch), 16384) for dt, ch in [(np.float32, 2),
-                                                                                       (np.float64, 3)]]
+                                                                                       (np.float64, 3)]] + \
+    [(dt, n, m, p, 0) for dt, n, m, k, T in tgp.CV_BITEXACT for p in (tgp._cv_params(k, T),
+                                                                    dict(tgp._cv_params(k, T), strided=0))]
 
 
 @pytest.mark.parametrize("dtype,n,m,params,stride", CV)
 def test_coalesced_case_is_accepted(tds, dtype, n, m, params, stride):
-    assert _accepts(tds, dtype, n, m, params, stride)["strided"] == 2
+    assert _accepts(tds, dtype, n, m, params, stride)["strided"] == params["strided"]
 
 
 CASES = _cases()

@@ -919,6 +919,25 @@ def test_coalesced_variant(tds, dtype, n, m, k, T):
     check(a, b, c, d, np.ascontiguousarray(xs[:, :n]), dtype)
 
 
+CV_BITEXACT = [  # (dtype, n, m, k, T): subsystems of <= 1024 rows, where the de-interleaved plan with the
+    # same switch point (c = 0, c2 = 0, T, one CTA) runs the paper's PCR-Thomas base kernel (onchip.cu)
+    (np.float32, 2048, 64, 3, 16), (np.float32, 16384, 9, 4, 64), (np.float32, 4000, 5, 3, 8),
+    (np.float64, 4096, 6, 2, 32), (np.float64, 3002, 3, 3, 1)]
+
+
+@pytest.mark.parametrize("dtype,n,m,k,T", CV_BITEXACT)
+def test_coalesced_variant_bit_identical_to_deinterleaved(tds, dtype, n, m, k, T):
+    """The coalesced variant changes only where the rows live (sector groups,
+    global fallback), not the arithmetic: x is bit-identical to the
+    de-interleaved path's PCR-Thomas base kernel under the same (k, T)."""
+    a, b, c, d = inputs.generate(n, m, dtype, seed=182 + k)
+    x2, p2 = run(tds, a, b, c, d, params=_cv_params(k, T))
+    x0, p0 = run(tds, a, b, c, d, params=dict(_cv_params(k, T), strided=0))
+    assert p0.info["onchip_form"] == p2.info["onchip_form"] == 0 and p0.info["launches"] == 3
+    assert np.array_equal(x2, x0)
+    check(a, b, c, d, x2, dtype)
+
+
 @pytest.mark.parametrize("dtype,chunk", [(np.float32, 2), (np.float64, 3)])
 def test_coalesced_variant_chunked(tds, dtype, chunk):
     """Chunked plans (chunk_systems): every chunk reuses the workspace (both
