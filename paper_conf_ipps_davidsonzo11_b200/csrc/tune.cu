@@ -403,6 +403,7 @@ static tds_status commit(tds_plan_st *plan, const tds_params &best, int trials, 
 struct TuneCtx {
     tds_plan_st *plan;
     cudaStream_t st;
+    cudaStream_t cap = nullptr;  // private stream for graph-timed trials (created on first use)
     void *a = nullptr, *b = nullptr, *c = nullptr, *d = nullptr, *x = nullptr, *ws = nullptr;
     size_t ws_bytes = 0;
     int reps = 7;
@@ -421,11 +422,62 @@ static bool ensure_ws(TuneCtx &C, size_t need) {
     return true;
 }
 
+// Launch-bound solves (a back-to-back eager solve under kGraphTrialMs) are
+// timed as CUDA-graph replays of `inner` captured solves: eager launches of a
+// few-microsecond solve measure the host's launch rate (~7 us per solve for
+// every candidate of config 1), not the kernels, so the climb could not tell
+// the plans apart (gpurun_out/r02aj: 3.0 vs 4.2 us per solve under graph
+// replay for two plans that both time 7.0 us eagerly).  Returns the median ms
+// per solve, kRejected if the capture is refused, NaN on a device fault.
+constexpr float kGraphTrialMs = 0.03f;
+
+static double graph_trial(TuneCtx &C, tds_plan_st &tmp, int inner) {
+    if (!C.cap && cudaStreamCreateWithFlags(&C.cap, cudaStreamNonBlocking) != cudaSuccess) {
+        cudaGetLastError();
+        C.cap = nullptr;
+        return kRejected;
+    }
+    if (cudaStreamSynchronize(C.st) != cudaSuccess) return NAN;  // trial data and workspace are ready
+    cudaGraph_t g = nullptr;
+    cudaGraphExec_t ge = nullptr;
+    bool ok = cudaStreamBeginCapture(C.cap, cudaStreamCaptureModeThreadLocal) == cudaSuccess;
+    for (int i = 0; i < inner && ok; ++i)
+        ok = tds_solve_batched(&tmp, C.a, C.b, C.c, C.d, C.x, C.ws, C.ws_bytes, C.cap) == TDS_OK;
+    const cudaError_t ec = cudaStreamEndCapture(C.cap, &g);
+    ok = ok && ec == cudaSuccess && g && cudaGraphInstantiate(&ge, g, 0) == cudaSuccess;
+    if (!ok) {
+        if (ge) cudaGraphExecDestroy(ge);
+        if (g) cudaGraphDestroy(g);
+        cudaGetLastError();
+        return kRejected;
+    }
+    cudaEvent_t e0, e1;
+    if (cudaEventCreate(&e0) != cudaSuccess || cudaEventCreate(&e1) != cudaSuccess) return NAN;
+    std::vector<float> ms;
+    bool fault = false;
+    for (int r = 0; r < C.reps + 1 && !fault; ++r) {
+        cudaEventRecord(e0, C.cap);
+        cudaGraphLaunch(ge, C.cap);
+        cudaEventRecord(e1, C.cap);
+        if (cudaEventSynchronize(e1) != cudaSuccess) fault = true;
+        float t = 0;
+        cudaEventElapsedTime(&t, e0, e1);
+        if (r >= 1) ms.push_back(t / float(inner));
+    }
+    cudaEventDestroy(e0);
+    cudaEventDestroy(e1);
+    cudaGraphExecDestroy(ge);
+    cudaGraphDestroy(g);
+    if (fault || cudaStreamSynchronize(C.cap) != cudaSuccess) return NAN;
+    std::sort(ms.begin(), ms.end());
+    return ms[ms.size() / 2];
+}
+
 // Median time (ms) of the full solve with parameters p (already validated),
 // measured as bench.py runs it: `inner` solves back to back between two
-// events (inner chosen so one sample spans >= ~0.4 ms; small problems would
-// otherwise time the host launch gaps, not the kernels); kRejected if the
-// solve refuses to launch; NaN on a device fault (sticky: the search stops).
+// events (inner chosen so one sample spans >= ~0.4 ms); launch-bound solves
+// by graph replay (graph_trial); kRejected if the solve refuses to launch;
+// NaN on a device fault (sticky: the search stops).
 static double trial(TuneCtx &C, const tds_params &p) {
     tds_plan_st tmp = *C.plan;
     if (derive(tmp.info, tmp.props, p) != TDS_OK) return kRejected;
@@ -454,7 +506,13 @@ static double trial(TuneCtx &C, const tds_params &p) {
         return kRejected;
     }
     std::sort(ms.begin(), ms.end());
-    return ms[ms.size() / 2];
+    const double eager = ms[ms.size() / 2];
+    if (eager < kGraphTrialMs) {
+        const double gt = graph_trial(C, tmp, std::max(inner, 16));
+        if (std::isnan(gt)) return gt;
+        if (gt < kRejected) return gt;
+    }
+    return eager;
 }
 
 // max |x - y| and max |y| over the rows of m systems (padding excluded);
@@ -582,6 +640,7 @@ extern "C" tds_status tds_tune(tds_plan_t plan, void *cuda_stream, const char *c
     const int trials = S.trials;
     if (result == TDS_OK) result = commit(plan, best, trials, path, key);
     cudaStreamSynchronize(C.st);
+    if (C.cap) cudaStreamDestroy(C.cap);
     for (auto p : bufs) cudaFree(*p);
     if (C.ws) cudaFree(C.ws);
     if (result == TDS_OK) clear_error();
