@@ -207,7 +207,11 @@ tds_status tds_plan_destroy(tds_plan_t plan);
  * text file of saved results keyed by device, dtype, n and m ("save those
  * results for future runs"); a hit skips the search.  A trial
  * is the median over several samples of back-to-back solves (>= ~0.4 ms per
- * sample); the Thomas switch T is not searched in the warp form (no T).  A
+ * sample; a solve under 30 us is timed as CUDA-graph replays of captured
+ * solves on a private stream, since eager launches would time the host's
+ * launch rate); the Thomas switch T is not searched in the warp form (no T);
+ * the x placement (x_group) and the paper's load variant (strided 0 / 1 / 2)
+ * are searched with the on-chip switch.  A
  * trial that faults the device (sticky CUDA error) aborts the search with
  * TUNE; the chosen parameters must reproduce the seed plan's x on the trial
  * systems (relative 2e-4 fp32 / 1e-9 fp64) before they and the cache line
