@@ -29,21 +29,35 @@ constexpr int kMaxPasses = TDS_MAX_PASSES;
 
 // Reciprocal.  fp32: the SFU approximation (MUFU.RCP, <= 1 ulp) -- the
 // north_star's fp32 tolerance (1e-4 error, 1e-5 residual) leaves room for it
-// (reading R16).  fp64: the SFU seed (MUFU.RCP64H) refined by two
-// Newton steps (relative error ~1 ulp, R16) instead of IEEE
+// (reading R16).  fp64: the SFU seed (MUFU.RCP64H) refined by one
+// cubic step (relative error <= 2 ulp, R16, below) instead of IEEE
 // division, whose special-case slow path costs a call per row update.
 __device__ __forceinline__ float rcp(float x) {
     float r;
     asm("rcp.approx.ftz.f32 %0, %1;" : "=f"(r) : "f"(x));
     return r;
 }
+// fp64 refinement: with e = 1 - x r0, 1/x = r0 / (1 - e) = r0 (1 + e + e^2
+// + ...); r0 (1 + e + e^2) = fma(r0, fma(e, e, e), r0) leaves a relative
+// error ~e^3 (seed <= 9.9e-7 ~ 2^-20 -> 2^-60) plus rounding: <= 2 ulp over
+// 2^26 inputs, in 3 dependent DFMA instead of the two Newton steps' 4 (0 ulp
+// measured; -DTDS_RCP64_CUBIC=0): config 3 fp64 step -3 %
+// (scripts/probes/rcp64_probe.cu, profiles/r02am_rcp64.md).
+#ifndef TDS_RCP64_CUBIC
+#define TDS_RCP64_CUBIC 1
+#endif
 __device__ __forceinline__ double rcp(double x) {
     double r;
     asm("rcp.approx.ftz.f64 %0, %1;" : "=d"(r) : "d"(x));
+#if TDS_RCP64_CUBIC
+    const double e = fma(-x, r, 1.0);
+    return fma(r, fma(e, e, e), r);
+#else
     double e = fma(-x, r, 1.0);
     r = fma(r, e, r);
     e = fma(-x, r, 1.0);
     return fma(r, e, r);
+#endif
 }
 
 // One PCR/CR row update in NORMALISED form (every row scaled so b = 1).
