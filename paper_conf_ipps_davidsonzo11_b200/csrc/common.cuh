@@ -60,25 +60,6 @@ __device__ __forceinline__ double rcp(double x) {
 #endif
 }
 
-// One PCR/CR row update in NORMALISED form (every row scaled so b = 1).
-// With the textbook update (SURVEY.md §8(c); Hockney & Jesshope [11], cited
-// PAPER.md P:L199-200) applied to normalised rows and the result rescaled
-// by 1/b':
-//   r  = 1 / (1 - a_i c_{i-s} - c_i a_{i+s})
-//   a' = -a_i a_{i-s} r,  c' = -c_i c_{i+s} r,  d' = (d_i - a_i d_{i-s} - c_i d_{i+s}) r
-// Identity neighbours (outside the system) are (a, c, d) = (0, 0, 0).
-template <typename T>
-__device__ __forceinline__ void row_update(T &a, T &c, T &d, T al, T cl, T dl, T ar, T cr, T dr) {
-    const T den = fma(-c, ar, fma(-a, cl, T(1)));
-    const T r = rcp(den);
-    const T ma = -a * r;
-    const T mc = -c * r;
-    const T nd = fma(ma, dl, fma(mc, dr, d * r));
-    a = ma * al;
-    c = mc * cr;
-    d = nd;
-}
-
 // The same update with the other operation order: the products a_i a_{i-s},
 // c_i c_{i+s} and the numerator d_i - a_i d_{i-s} - c_i d_{i+s} do not depend
 // on r, so they are formed while the reciprocal is in flight and each output
@@ -96,6 +77,32 @@ __device__ __forceinline__ void row_update_early(T &a, T &c, T &d, T al, T cl, T
     a = -pa * r;
     c = -pc * r;
     d = num * r;
+}
+
+// One PCR/CR row update in NORMALISED form (every row scaled so b = 1).
+// With the textbook update (SURVEY.md §8(c); Hockney & Jesshope [11], cited
+// PAPER.md P:L199-200) applied to normalised rows and the result rescaled
+// by 1/b':
+//   r  = 1 / (1 - a_i c_{i-s} - c_i a_{i+s})
+//   a' = -a_i a_{i-s} r,  c' = -c_i c_{i+s} r,  d' = (d_i - a_i d_{i-s} - c_i d_{i+s}) r
+// Identity neighbours (outside the system) are (a, c, d) = (0, 0, 0).
+#ifndef TDS_FP64_EARLY
+#define TDS_FP64_EARLY 0
+#endif
+template <typename T>
+__device__ __forceinline__ void row_update(T &a, T &c, T &d, T al, T cl, T dl, T ar, T cr, T dr) {
+    if constexpr (TDS_FP64_EARLY && sizeof(T) == 8) {  // experiment: fp64 in the early order (below)
+        row_update_early(a, c, d, al, cl, dl, ar, cr, dr);
+        return;
+    }
+    const T den = fma(-c, ar, fma(-a, cl, T(1)));
+    const T r = rcp(den);
+    const T ma = -a * r;
+    const T mc = -c * r;
+    const T nd = fma(ma, dl, fma(mc, dr, d * r));
+    a = ma * al;
+    c = mc * cr;
+    d = nd;
 }
 
 // The same update on two independent rows at once with the packed fp32x2
