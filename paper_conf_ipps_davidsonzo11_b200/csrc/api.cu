@@ -208,8 +208,9 @@ static tds_status solve_impl(const tds_plan_info &I, const T *a, const T *b, con
             WsBufs<T> w = ws_bufs<T>(I, ws);
             int l2t = 0;
             while ((1 << l2t) < P.thomas_chains) ++l2t;
-            err = launch_onchip_coalesced<T>(w.a, w.c, w.d, x, I.n, I.m, I.batch_stride,
-                                             natural_stride<T>(I.n), P.k, l2t, int64_t(smem_optin_current()) - kSmemReserve, st);
+            const int64_t smem_budget = int64_t(smem_optin_current()) - kSmemReserve;
+            err = launch_onchip_coalesced<T>(w.a, w.c, w.d, x, I.n, I.m, I.batch_stride, natural_stride<T>(I.n), P.k,
+                                             l2t, smem_budget, st);
         } else if (strided_ok) {
             // gather residue classes with stride 2^k from the in-place split output, x scattered in place
             A.x = x;
