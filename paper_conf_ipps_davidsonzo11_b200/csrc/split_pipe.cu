@@ -60,6 +60,11 @@ __constant__ int tds_split_ablation;
 #ifndef TDS_SPLIT_TRC64
 #define TDS_SPLIT_TRC64 1
 #endif
+// fp32 512-thread tiles: the bank-conflict-free sub-row class transpose
+// (split_reg.cuh, tr34_phys); -DTDS_SPLIT_TR34=0 restores the swizzled [rho][m] rows.
+#ifndef TDS_SPLIT_TR34
+#define TDS_SPLIT_TR34 1
+#endif
 
 template <int KP, int NT_>
 struct SplitShape {
@@ -101,14 +106,24 @@ struct SplitShape {
     template <typename T>
     __host__ __device__ static constexpr bool tstore() { return !TDS_SPLIT_STG && (PT * int(sizeof(T))) % 16 == 0; }
     template <typename T>
+    __host__ __device__ static constexpr bool tr34() { return TDS_SPLIT_TR34 && sizeof(T) == 4 && NT == 512 && KP > 4; }
+    template <typename T>
     __host__ __device__ static constexpr int tbuf_elems() {
-        const int tr = KP > 4 ? ((sizeof(T) == 4 || TDS_SPLIT_TRC64) ? 3 : 1) * AV * 16 : 0;
+        const int tr = !(KP > 4)  ? 0
+                       : tr34<T>() ? 3 * 16 * kTr34C + 32
+                                   : ((sizeof(T) == 4 || TDS_SPLIT_TRC64) ? 3 : 1) * AV * 16;
         const int so = tstore<T>() ? 3 * TV : 0;
         return tr > so ? tr : so;
     }
+    // the transpose / staging buffer follows the last array's window (the stages are
+    // 1024-byte aligned for the swizzled TMA boxes; the buffer only needs 128 bytes)
+    template <typename T>
+    __host__ __device__ static constexpr int tbuf_off(int na) {
+        return tr34<T>() ? (na - 1) * stage_elems<T>() + ROWS : na * stage_elems<T>();
+    }
     template <typename T>
     static constexpr size_t smem_bytes(bool raw) {
-        return 1024 + (size_t(raw ? 4 : 3) * stage_elems<T>() + size_t(tbuf_elems<T>())) * sizeof(T);
+        return 1024 + (size_t(tbuf_off<T>(raw ? 4 : 3)) + size_t(tbuf_elems<T>())) * sizeof(T);
     }
 };
 
@@ -125,7 +140,8 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
     constexpr int NTR = KP > 4 ? ((sizeof(T) == 4 || TDS_SPLIT_TRC64) ? 3 : 1) : 0;  // arrays per transpose round
     extern __shared__ __align__(1024) unsigned char smem_raw[];
     T *stage = reinterpret_cast<T *>(smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u));  // 1024-aligned
-    T *tbuf = stage + NA * STG;  // [NTR][AV * 16] transpose buffer / [3][TV] output staging
+    T *tbuf = stage + S::template tbuf_off<T>(NA);  // [NTR][AV * 16] transpose buffer / [3][TV] output staging
+    static_assert((ROWS * sizeof(T)) % 128 == 0, "128-byte aligned transpose / staging buffer");
     constexpr bool TSTORE = S::template tstore<T>();
     constexpr int PT = S::PT, BOXP = S::BOXP, NBOX = S::NBOX, NRES = 1 << KP;
     // staging index of (residue rr, tile position p): [box][residue][BOXP]
@@ -396,7 +412,20 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
             const int rho = t / CH, b = t % CH;
             const int mb = LEFT - 16 + 16 * b;  // member of u = 0
             const bool wr = lane >= 1 && lane <= 30;
-            if constexpr (NTR == 3 && sizeof(T) == 4) {  // fp32, one round: 3 class-major buffers [rho][m]
+            if constexpr (S::template tr34<T>()) {  // fp32 512 threads: conflict-free sub-row transpose
+                constexpr int CW = kTr34C, AW = 16 * CW;  // class row / array strides
+                if (wr) {
+                    const int pm = tr34_phys(ablk - 1);
+                    trc_write<T, R, CW>(ra, tbuf + pm);
+                    trc_write<T, R, CW>(rc, tbuf + AW + pm);
+                    trc_write<T, R, CW>(rd, tbuf + 2 * AW + pm);
+                }
+                __syncthreads();
+                const float *rp = tbuf + rho * CW + b - 1;
+                tr34_read<R, LEFT>(ra, rp);
+                tr34_read<R, LEFT>(rc, rp + AW);
+                tr34_read<R, LEFT>(rd, rp + 2 * AW);
+            } else if constexpr (NTR == 3 && sizeof(T) == 4) {  // fp32, one round: 3 class-major buffers [rho][m]
                 if (wr) {
                     const int pm = trc_phys(ablk - 1);
                     trc_write<T, R, AV>(ra, tbuf + pm);

@@ -226,6 +226,33 @@ __device__ __forceinline__ void trc_read(float (&x)[R], const float *row, const 
     }
 }
 
+// fp32, 512-thread tiles (TDS_SPLIT_TR34): the class transpose without bank
+// conflicts in either direction.  Class row rho holds its members as 16
+// sub-rows (m mod 16) of 34 words, member m at (m & 15) * 34 + (m >> 4).
+// Layout-A stores (30 consecutive m across a warp, one class per store)
+// land on banks (2 (m & 15) + (m >> 4)) mod 32: distinct, because members
+// one sub-row column apart differ in parity and members two columns apart
+// would need (m & 15) to step by one across a whole window.  Layout-B loads
+// (one class per warp, lanes b 16 members apart, member u of every lane in
+// one load) read 32 consecutive words: one wavefront each.  Costs 16 scalar
+// loads per array instead of 4 LDS.128 (the same wavefronts) and 2.3 KB more
+// buffer per array (the [rho][m] swizzle keeps ~1.6 wavefronts per store).
+constexpr int kTr34W = 34;
+// class-row stride: the last stored member of a class is 15 * 34 + 29 (AV = 480);
+// the halo lanes' reads run up to 2 words further (into the next class, or into the
+// 32 spare words after the buffer).  Any stride keeps the banks: one class per access.
+constexpr int kTr34C = 540;
+__device__ __forceinline__ int tr34_phys(int m) { return (m & 15) * kTr34W + (m >> 4); }
+
+// members mb + u, u = 0..R-1, of the class whose row starts at row; mb = LEFT - 16 + 16 b
+// and p = row + b - 1, so member mb + u is p[((LEFT + u) & 15) * 34 + ((LEFT + u) >> 4)]:
+// a compile-time offset from one per-thread base (halo lanes read padding / neighbours)
+template <int R, int LEFT>
+__device__ __forceinline__ void tr34_read(float (&x)[R], const float *p) {
+#pragma unroll
+    for (int u = 0; u < R; ++u) x[u] = p[((LEFT + u) & 15) * kTr34W + ((LEFT + u) >> 4)];
+}
+
 // fp64 class-major buffer [rho][m] (row stride AV doubles): member m at
 // 2 * (c ^ ((c >> 3) & 7)) + (m & 1), c = m >> 1 (16-byte chunks of two
 // members XOR-swizzled by the 128-byte block).  Layout-A writes are 16 scalar
