@@ -173,7 +173,25 @@ __global__ void __launch_bounds__(kPlaceThreads) place_x_tile_kernel(const Place
 // along j per tile; loads run two tiles ahead; stores are TMA tensor stores.
 // Rows past floor(n / 2^K) * 2^K (fewer than 2^K per system) are copied last
 // with plain loads and stores.
-constexpr int kTpBoxes = 4, kTpThreads = 256;
+// Tile shape of the TMA transposer: 2 boxes per tile, 128 threads (~25 KB, 9 CTAs per
+// SM) measured fastest on config 3 (place_x 22.4 -> 20.8 us, gpurun_out/r02b9, r02b10):
+// more, smaller CTAs beat deeper pipelines (3-4 input stages or double-buffered
+// output boxes: 24-29 us) and 4-box / 256- or 512-thread tiles (22.3-22.8 us).
+#ifndef TDS_TP_BOXES
+#define TDS_TP_BOXES 2
+#endif
+#ifndef TDS_TP_THREADS
+#define TDS_TP_THREADS 128
+#endif
+constexpr int kTpBoxes = TDS_TP_BOXES, kTpThreads = TDS_TP_THREADS;
+// pipeline depth of the TMA transposer: input stages in flight, output boxes in flight
+#ifndef TDS_TP_STAGES
+#define TDS_TP_STAGES 2
+#endif
+#ifndef TDS_TP_OUTBUF
+#define TDS_TP_OUTBUF 1
+#endif
+constexpr int kTpStages = TDS_TP_STAGES, kTpOut = TDS_TP_OUTBUF;
 
 template <typename T, bool XS>
 __global__ void __launch_bounds__(kTpThreads) place_x_tma_kernel(const PlaceArgs<T> A, const __grid_constant__ TmapSet tm,
@@ -184,9 +202,10 @@ __global__ void __launch_bounds__(kTpThreads) place_x_tma_kernel(const PlaceArgs
     constexpr int BOX = E * E;  // elements per box
     extern __shared__ __align__(1024) unsigned char smem_raw[];
     T *base = reinterpret_cast<T *>(smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u));
-    T *sin = base;                   // [2][NBX][E slots][E positions]
-    T *sout = base + 2 * NBX * BOX;  // [NBX][E j][E residues]
-    __shared__ __align__(8) uint64_t full[2];
+    constexpr int NS = kTpStages, NO = kTpOut;
+    T *sin = base;                    // [NS][NBX][E slots][E positions]
+    T *sout0 = base + NS * NBX * BOX;  // [NO][NBX][E j][E residues]
+    __shared__ __align__(8) uint64_t full[NS];
     const int t = threadIdx.x;
     const int64_t rtiles = (int64_t(1) << A.K) / E;
     auto coords = [&](int64_t w, int64_t &sys, int64_t &rt, int64_t &jt) {
@@ -211,26 +230,27 @@ __global__ void __launch_bounds__(kTpThreads) place_x_tma_kernel(const PlaceArgs
     };
     pdl_wait();  // the previous kernel on the stream is complete before any global access
     if (t == 0) {
-        mbar_init(&full[0], 1);
-        mbar_init(&full[1], 1);
+#pragma unroll
+        for (int q = 0; q < NS; ++q) mbar_init(&full[q], 1);
         asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
-        issue(blockIdx.x, 0);
-        issue(int64_t(blockIdx.x) + gridDim.x, 1);
+#pragma unroll
+        for (int q = 0; q < NS; ++q) issue(int64_t(blockIdx.x) + q * int64_t(gridDim.x), q);
     }
     __syncthreads();
     for (int64_t it = 0;; ++it) {
         const int64_t w = int64_t(blockIdx.x) + it * gridDim.x;
         if (w >= ntiles) break;
         pdl_trigger_if_last(w + gridDim.x >= ntiles);
-        const int s = int(it & 1);
-        mbar_wait(&full[s], uint32_t((it >> 1) & 1));
+        const int s = int(it % NS);
+        T *sout = sout0 + int(it % NO) * NBX * BOX;
+        mbar_wait(&full[s], uint32_t((it / NS) & 1));
         if (l2_discard && t < NBX * E) {  // the x-slot lines of this tile are dead once in shared memory
             int64_t sys, rt, jt;
             coords(w, sys, rt, jt);
             const int64_t pos = (jt * NBX + t / E) * E;
             if (pos + E <= lfull) l2_discard_line(A.xs + ((sys << A.K) + rt * E + t % E) * A.slot + pos);
         }
-        if (t == 0) bulk_wait_read0();  // the previous tile's stores have read sout
+        if (t == 0) bulk_wait_read<NO - 1>();  // the stores of tile it - NO have read this sout
         __syncthreads();
         // transpose: task = (box, slot r, chunk jq); LDS.128 of slot r's chunk jq,
         // CH scalar stores into rows j = jq*CH + e of the output box
@@ -272,7 +292,7 @@ __global__ void __launch_bounds__(kTpThreads) place_x_tma_kernel(const PlaceArgs
                 }
             }
             bulk_commit();
-            issue(w + 2 * int64_t(gridDim.x), s);  // stage s is free: every thread passed the barrier
+            issue(w + NS * int64_t(gridDim.x), s);  // stage s is free: every thread passed the barrier
         }
     }
     if (t == 0) bulk_wait_all();
@@ -319,7 +339,7 @@ cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batc
         const int64_t rtiles = (int64_t(1) << K) / E;
         const int64_t jtiles = lfull / (kTpBoxes * E);
         const int64_t ntiles = m * rtiles * jtiles;
-        const size_t smem = 1024 + size_t(3 * kTpBoxes * E * E) * sizeof(T);
+        const size_t smem = 1024 + size_t((kTpStages + kTpOut) * kTpBoxes * E * E) * sizeof(T);
         auto kern = place_x_tma_kernel<T, true>;
         int occ = 1;
         cudaError_t e = kernel_setup((const void *)kern, kTpThreads, smem, 1, &occ);
@@ -354,7 +374,7 @@ cudaError_t launch_place_x(const T *xs, T *x, int64_t n, int64_t m, int64_t batc
         if ((m << K) < (int64_t(1) << 31) &&
             encode_box3_tmap(&tm.m[0], xs, int(sizeof(T)), din, sin_, bin) &&
             encode_box3_tmap(&tm.m[1], x, int(sizeof(T)), dout, sout_, bout)) {
-            const size_t smem = 1024 + size_t(3 * kTpBoxes * E * E) * sizeof(T);
+            const size_t smem = 1024 + size_t((kTpStages + kTpOut) * kTpBoxes * E * E) * sizeof(T);
             auto kern = place_x_tma_kernel<T, false>;
             int occ = 1;
             cudaError_t e = kernel_setup((const void *)kern, kTpThreads, smem, 1, &occ);
