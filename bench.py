@@ -773,6 +773,10 @@ def run_huge(args):
 
 def main():
     args = parse()
+    # diagnostics only: a run still going after 10 minutes prints every thread's
+    # Python stack to stderr (and keeps running), so a stall shows where it sits
+    import faulthandler
+    faulthandler.dump_traceback_later(600, repeat=True, exit=False)
     if args.impl == "reference":
         return run_reference(args)
     return run_tds(args)
