@@ -60,8 +60,8 @@ __constant__ int tds_split_ablation;
 #ifndef TDS_SPLIT_TRC64
 #define TDS_SPLIT_TRC64 1
 #endif
-// fp32 512-thread tiles: the bank-conflict-free sub-row class transpose
-// (split_reg.cuh, tr34_phys); -DTDS_SPLIT_TR34=0 restores the swizzled [rho][m] rows.
+// fp32 512-thread and fp64 256-thread tiles: the bank-conflict-free sub-row class
+// transpose (split_reg.cuh, Tr34); -DTDS_SPLIT_TR34=0 restores the swizzled [rho][m] rows.
 #ifndef TDS_SPLIT_TR34
 #define TDS_SPLIT_TR34 1
 #endif
@@ -106,11 +106,13 @@ struct SplitShape {
     template <typename T>
     __host__ __device__ static constexpr bool tstore() { return !TDS_SPLIT_STG && (PT * int(sizeof(T))) % 16 == 0; }
     template <typename T>
-    __host__ __device__ static constexpr bool tr34() { return TDS_SPLIT_TR34 && sizeof(T) == 4 && NT == 512 && KP > 4; }
+    __host__ __device__ static constexpr bool tr34() {
+        return TDS_SPLIT_TR34 && KP > 4 && ((sizeof(T) == 4 && NT == 512) || (sizeof(T) == 8 && NT == 256));
+    }
     template <typename T>
     __host__ __device__ static constexpr int tbuf_elems() {
         const int tr = !(KP > 4)  ? 0
-                       : tr34<T>() ? 3 * 16 * kTr34C + 32
+                       : tr34<T>() ? 3 * 16 * Tr34<T>::C + Tr34<T>::SLACK
                                    : ((sizeof(T) == 4 || TDS_SPLIT_TRC64) ? 3 : 1) * AV * 16;
         const int so = tstore<T>() ? 3 * TV : 0;
         return tr > so ? tr : so;
@@ -412,16 +414,16 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
             const int rho = t / CH, b = t % CH;
             const int mb = LEFT - 16 + 16 * b;  // member of u = 0
             const bool wr = lane >= 1 && lane <= 30;
-            if constexpr (S::template tr34<T>()) {  // fp32 512 threads: conflict-free sub-row transpose
-                constexpr int CW = kTr34C, AW = 16 * CW;  // class row / array strides
+            if constexpr (S::template tr34<T>()) {  // conflict-free sub-row transpose (fp32 512 / fp64 256 threads)
+                constexpr int CW = Tr34<T>::C, AW = 16 * CW;  // class row / array strides
                 if (wr) {
-                    const int pm = tr34_phys(ablk - 1);
+                    const int pm = tr34_phys<T>(ablk - 1);
                     trc_write<T, R, CW>(ra, tbuf + pm);
                     trc_write<T, R, CW>(rc, tbuf + AW + pm);
                     trc_write<T, R, CW>(rd, tbuf + 2 * AW + pm);
                 }
                 __syncthreads();
-                const float *rp = tbuf + rho * CW + b - 1;
+                const T *rp = tbuf + rho * CW + b - 1;
                 tr34_read<R, LEFT>(ra, rp);
                 tr34_read<R, LEFT>(rc, rp + AW);
                 tr34_read<R, LEFT>(rd, rp + 2 * AW);

@@ -226,31 +226,45 @@ __device__ __forceinline__ void trc_read(float (&x)[R], const float *row, const 
     }
 }
 
-// fp32, 512-thread tiles (TDS_SPLIT_TR34): the class transpose without bank
-// conflicts in either direction.  Class row rho holds its members as 16
-// sub-rows (m mod 16) of 34 words, member m at (m & 15) * 34 + (m >> 4).
-// Layout-A stores (30 consecutive m across a warp, one class per store)
-// land on banks (2 (m & 15) + (m >> 4)) mod 32: distinct, because members
-// one sub-row column apart differ in parity and members two columns apart
-// would need (m & 15) to step by one across a whole window.  Layout-B loads
-// (one class per warp, lanes b 16 members apart, member u of every lane in
-// one load) read 32 consecutive words: one wavefront each.  Costs 16 scalar
-// loads per array instead of 4 LDS.128 (the same wavefronts) and 2.3 KB more
-// buffer per array (the [rho][m] swizzle keeps ~1.6 wavefronts per store).
-constexpr int kTr34W = 34;
-// class-row stride: the last stored member of a class is 15 * 34 + 29 (AV = 480);
-// the halo lanes' reads run up to 2 words further (into the next class, or into the
-// 32 spare words after the buffer).  Any stride keeps the banks: one class per access.
-constexpr int kTr34C = 540;
-__device__ __forceinline__ int tr34_phys(int m) { return (m & 15) * kTr34W + (m >> 4); }
+// fp32 512-thread and fp64 256-thread tiles (TDS_SPLIT_TR34): the class
+// transpose without bank conflicts in either direction.  Class row rho holds
+// its members as 16 sub-rows (m mod 16) of W elements, member m at
+// (m & 15) * W + (m >> 4).
+// fp32, W = 34 words: layout-A stores (30 consecutive m across a warp, one
+// class per store) land on banks (2 (m & 15) + (m >> 4)) mod 32: distinct,
+// because members one sub-row column apart differ in parity and members two
+// columns apart would need (m & 15) to step by one across a whole window.
+// Layout-B loads (one class per warp, lanes b 16 members apart, member u of
+// every lane in one load) read 32 consecutive words.
+// fp64, W = 17 doubles: an 8-byte store is served per half-warp (15
+// consecutive members, lanes 1..15 / 16..30), whose 8-byte bank pairs
+// ((m & 15) + (m >> 4)) mod 16 are distinct (a window spans two sub-row
+// columns, and m, m' one column apart collide only if (m & 15) - (m' & 15) = 1,
+// i.e. never inside one window); layout-B loads (one class per half-warp)
+// read 16 consecutive doubles.  Each direction is one wavefront per access:
+// 16 scalar loads per array instead of 4 LDS.128 (fp32) / 8 (fp64), the same
+// wavefronts; the [rho][m] swizzles keep ~1.6 (fp32) / ~1.7 (fp64) wavefronts
+// per store.
+template <typename T>
+struct Tr34 {
+    static constexpr int W = sizeof(T) == 4 ? 34 : 17;
+    // class-row stride: the last stored member is 15 W + AV / 16 - 1 (AV = 480 / 240);
+    // the halo lanes' reads run to sub-row column 15 of the last sub-row (fp64: inside
+    // the class; fp32: 2 words into the next class or the 32 spare words after the
+    // buffer).  Any stride keeps the banks: one class per access (per half-warp).
+    static constexpr int C = sizeof(T) == 4 ? 540 : 271;
+    static constexpr int SLACK = sizeof(T) == 4 ? 32 : 0;
+};
+template <typename T>
+__device__ __forceinline__ int tr34_phys(int m) { return (m & 15) * Tr34<T>::W + (m >> 4); }
 
 // members mb + u, u = 0..R-1, of the class whose row starts at row; mb = LEFT - 16 + 16 b
-// and p = row + b - 1, so member mb + u is p[((LEFT + u) & 15) * 34 + ((LEFT + u) >> 4)]:
+// and p = row + b - 1, so member mb + u is p[((LEFT + u) & 15) * W + ((LEFT + u) >> 4)]:
 // a compile-time offset from one per-thread base (halo lanes read padding / neighbours)
-template <int R, int LEFT>
-__device__ __forceinline__ void tr34_read(float (&x)[R], const float *p) {
+template <int R, int LEFT, typename T>
+__device__ __forceinline__ void tr34_read(T (&x)[R], const T *p) {
 #pragma unroll
-    for (int u = 0; u < R; ++u) x[u] = p[((LEFT + u) & 15) * kTr34W + ((LEFT + u) >> 4)];
+    for (int u = 0; u < R; ++u) x[u] = p[((LEFT + u) & 15) * Tr34<T>::W + ((LEFT + u) >> 4)];
 }
 
 // fp64 class-major buffer [rho][m] (row stride AV doubles): member m at
