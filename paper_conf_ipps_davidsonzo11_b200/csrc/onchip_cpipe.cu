@@ -32,15 +32,23 @@ namespace cg = cooperative_groups;
 
 namespace tds {
 
+// The cluster top solve's 32 lane rows by PCR (5 levels, no lane back
+// substitution) instead of CR (5 + 5 levels): config 2 0.0810 -> 0.0784 ms
+// (gpurun_out/r02b18, profiles/r02b18/).  -DTDS_CPIPE_LANE_PCR=0 restores CR.
+#ifndef TDS_CPIPE_LANE_PCR
+#define TDS_CPIPE_LANE_PCR 1
+#endif
+
 template <int C>
 __device__ __forceinline__ void csync() {
     if constexpr (C > 1) cg::this_cluster().sync(); else __syncthreads();
 }
 
 // One warp solves a system of 32 * RZ normalised rows (lane l holds rows
-// l RZ .. l RZ + RZ - 1) by cyclic reduction: log2(RZ) levels in registers,
-// 5 across the lanes (shuffles), back substitution in reverse order; rows
-// outside the system are identity rows.  No barrier (the cluster's top rows,
+// l RZ .. l RZ + RZ - 1): cyclic reduction over log2(RZ) levels in registers,
+// then the 32 lane rows by PCR across the lanes (shuffles; every row
+// decouples), then back substitution of the register levels; rows outside
+// the system are identity rows.  No barrier (the cluster's top rows,
 // C = 4 / 8, replace 6 / 7 shared-memory PCR levels with 14 barriers).
 template <typename T, int RZ>
 __device__ __forceinline__ void warp_cr_solve(T (&ra)[RZ], T (&rc)[RZ], T (&rd)[RZ], int lane) {
@@ -60,6 +68,21 @@ __device__ __forceinline__ void warp_cr_solve(T (&ra)[RZ], T (&rc)[RZ], T (&rd)[
         }
     }
     T za = ra[RZ - 1], zc = rc[RZ - 1], zd = rd[RZ - 1];
+#if TDS_CPIPE_LANE_PCR
+    // the 32 lane rows by PCR: every lane updates at every level, so after 5
+    // levels each row is decoupled (x = d) and no lane back substitution follows
+#pragma unroll
+    for (int l = 1; l <= 5; ++l) {
+        const int s = 1 << (l - 1);
+        const T la = __shfl_up_sync(FULL, za, s), lc = __shfl_up_sync(FULL, zc, s), ld = __shfl_up_sync(FULL, zd, s);
+        const T xa = __shfl_down_sync(FULL, za, s), xc = __shfl_down_sync(FULL, zc, s),
+                xd = __shfl_down_sync(FULL, zd, s);
+        const bool hl = lane >= s, hr = lane + s < 32 && !TDS_MUT(3, s >= 4);
+        row_update_early(za, zc, zd, hl ? la : T(0), hl ? lc : T(0), hl ? ld : T(0), hr ? xa : T(0),
+                         hr ? xc : T(0), hr ? xd : T(0));
+    }
+    const T xw = zd;
+#else
 #pragma unroll
     for (int l = 1; l <= 5; ++l) {
         const int s = 1 << (l - 1);
@@ -83,6 +106,7 @@ __device__ __forceinline__ void warp_cr_solve(T (&ra)[RZ], T (&rc)[RZ], T (&rd)[
         const T xn = zd - za * (lane >= s ? xl : T(0)) - zc * (lane + s < 32 ? xr : T(0));
         xw = (lane & ((1 << l) - 1)) == s - 1 ? xn : xw;
     }
+#endif
     T xleft = __shfl_up_sync(FULL, xw, 1);
     if (lane == 0) xleft = T(0);
     rd[RZ - 1] = xw;
