@@ -46,6 +46,21 @@ __device__ __forceinline__ void reduced_solve_pipe(T *z, int Z, int NT, int t, i
 // row s-1 per register level, lane s-1's row per lane level; both depend on
 // nothing beyond their own warp).  Every warp then solves the one-row-per-warp
 // system itself (no barrier to distribute its x).
+// Row updates on the warp form's serial path (lane CR, the deferred chains,
+// the top PCR): -DTDS_PIPE_SER_EARLY=1 uses the early operation order there
+// (1 dependent op after the reciprocal); the register levels keep row_update.
+// Measured neutral on config 3 (on-chip 52.8 vs 52.8 us, gpurun_out/r02b21).
+#ifndef TDS_PIPE_SER_EARLY
+#define TDS_PIPE_SER_EARLY 0
+#endif
+template <typename T>
+__device__ __forceinline__ void row_update_ser(T &a, T &c, T &d, T al, T cl, T dl, T ar, T cr, T dr) {
+    if constexpr (TDS_PIPE_SER_EARLY)
+        row_update_early(a, c, d, al, cl, dl, ar, cr, dr);
+    else
+        row_update(a, c, d, al, cl, dl, ar, cr, dr);
+}
+
 template <typename T, int R, typename Hook>
 __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[R], T *scr, int lane, int warp,
                                                 int nwarps, Hook &&after_barrier) {
@@ -102,7 +117,7 @@ __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[
             f[2] = zd;
         }
         T na2 = za, nc2 = zc, nd2 = zd;
-        row_update(na2, nc2, nd2, la, lc, ld, xa, xc, xd);
+        row_update_ser(na2, nc2, nd2, la, lc, ld, xa, xc, xd);
         const bool upd = (lane & ((1 << l) - 1)) == (1 << l) - 1 && lane != 31;
         za = upd ? na2 : za;
         zc = upd ? nc2 : zc;
@@ -116,7 +131,7 @@ __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[
         for (int l = 1; l <= CR; ++l) {
             const int s = 1 << (l - 1);
             const T *e = e_in + ((warp + 1) * CR + l - 1) * 3;
-            row_update(ra[R - 1], rc[R - 1], rd[R - 1], ra[R - 1 - s], rc[R - 1 - s], rd[R - 1 - s],
+            row_update_ser(ra[R - 1], rc[R - 1], rd[R - 1], ra[R - 1 - s], rc[R - 1 - s], rd[R - 1 - s],
                        h ? e[0] : T(0), h ? e[1] : T(0), h ? e[2] : T(0));
         }
         za = ra[R - 1];
@@ -126,7 +141,7 @@ __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[
         for (int l = 1; l <= 5; ++l) {
             const T *f = lft + (warp * 5 + l - 1) * 3;
             const T *w = w_in + ((warp + 1) * 5 + l - 1) * 3;
-            row_update(za, zc, zd, f[0], f[1], f[2], h ? w[0] : T(0), h ? w[1] : T(0), h ? w[2] : T(0));
+            row_update_ser(za, zc, zd, f[0], f[1], f[2], h ? w[0] : T(0), h ? w[1] : T(0), h ? w[2] : T(0));
         }
         top[warp] = za;
         top[32 + warp] = zc;
@@ -146,7 +161,7 @@ __device__ __forceinline__ void solve_item_warp(T (&ra)[R], T (&rc)[R], T (&rd)[
                     xd = __shfl_down_sync(FULL, d, s);
             const bool hl = lane >= s, hr = lane + s < nwarps && !TDS_MUT(1, s >= 2);
             T na = a, nc = c, nd = d;
-            row_update(na, nc, nd, hl ? la : T(0), hl ? lc : T(0), hl ? ld : T(0), hr ? xa : T(0), hr ? xc : T(0),
+            row_update_ser(na, nc, nd, hl ? la : T(0), hl ? lc : T(0), hl ? ld : T(0), hr ? xa : T(0), hr ? xc : T(0),
                        hr ? xd : T(0));
             a = lane < nwarps ? na : a;
             c = lane < nwarps ? nc : c;
