@@ -272,6 +272,12 @@ __device__ __forceinline__ void tma_store_4d(const CUtensorMap *map, const void 
                  "r"(smem_u32(src)), "r"(c0), "r"(c1), "r"(c2), "r"(c3)
                  : "memory");
 }
+__device__ __forceinline__ void tma_store_5d(const CUtensorMap *map, const void *src, int c0, int c1, int c2, int c3,
+                                             int c4) {
+    asm volatile("cp.async.bulk.tensor.5d.global.shared::cta.bulk_group [%0, {%2, %3, %4, %5, %6}], [%1];" ::"l"(map),
+                 "r"(smem_u32(src)), "r"(c0), "r"(c1), "r"(c2), "r"(c3), "r"(c4)
+                 : "memory");
+}
 __device__ __forceinline__ void bulk_commit() { asm volatile("cp.async.bulk.commit_group;" ::: "memory"); }
 // the committed bulk stores have finished READING shared memory
 __device__ __forceinline__ void bulk_wait_read0() { asm volatile("cp.async.bulk.wait_group.read 0;" ::: "memory"); }
@@ -287,6 +293,11 @@ __device__ __forceinline__ void fence_proxy_async_smem() {
 // sys < msys} -- with a box of {box_pos, 1, nrho, 1}.
 bool encode_out_tmap(CUtensorMap *out, const void *base, int dsize, int64_t slot, int64_t nr, int64_t nrho,
                      int64_t msys, int box_pos);
+// the same output view with the residue split as rho = rho_lo + 16 mu (dims {position,
+// r, rho_lo < 16, mu < nrho / 16, system}), box {box_pos, 1, 1, nrho / 16, 1}: one warp's
+// residues rho_lo + 16 mu of a tile in one store
+bool encode_out5_tmap(CUtensorMap *out, const void *base, int dsize, int64_t slot, int64_t nr, int64_t nrho,
+                      int64_t msys, int box_pos);
 
 // R consecutive rows to stage row s0 of a swizzled stage (the inverse of lds_rows_sw).
 template <typename T, int R>

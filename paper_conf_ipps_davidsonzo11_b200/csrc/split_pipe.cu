@@ -65,6 +65,15 @@ __constant__ int tds_split_ablation;
 #ifndef TDS_SPLIT_TR34
 #define TDS_SPLIT_TR34 1
 #endif
+// Experiment switch (-DTDS_SPLIT_WSTORE=1), fp32 512-thread sub-row tiles: every warp
+// (one residue class rho mod 16) stages its outputs in its own class rows of the
+// transpose buffer and stores them by its own 5-D TMA tensor store -- no CTA barrier
+// between the layout-B levels and the stores.  Correct (300 split / coupling / fuzz GPU
+// tests) but slower: config 3 split 101.5 vs 97.0 us (48 stores of 1.8 KB per tile
+// instead of 3 of 28 KB; gpurun_out/r02b22, profiles/r02b22/).  Default off.
+#ifndef TDS_SPLIT_WSTORE
+#define TDS_SPLIT_WSTORE 0
+#endif
 
 template <int KP, int NT_>
 struct SplitShape {
@@ -110,6 +119,10 @@ struct SplitShape {
         return TDS_SPLIT_TR34 && KP > 4 && ((sizeof(T) == 4 && NT == 512) || (sizeof(T) == 8 && NT == 256));
     }
     template <typename T>
+    __host__ __device__ static constexpr bool wstore() {
+        return TDS_SPLIT_WSTORE && tr34<T>() && sizeof(T) == 4 && tstore<T>() && NBOX == 1;
+    }
+    template <typename T>
     __host__ __device__ static constexpr int tbuf_elems() {
         const int tr = !(KP > 4)  ? 0
                        : tr34<T>() ? 3 * 16 * Tr34<T>::C + Tr34<T>::SLACK
@@ -145,6 +158,7 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
     T *tbuf = stage + S::template tbuf_off<T>(NA);  // [NTR][AV * 16] transpose buffer / [3][TV] output staging
     static_assert((ROWS * sizeof(T)) % 128 == 0, "128-byte aligned transpose / staging buffer");
     constexpr bool TSTORE = S::template tstore<T>();
+    constexpr bool WST = S::template wstore<T>() && !SC;  // per-warp staging and stores (fp32 512-thread sub-row tiles)
     constexpr int PT = S::PT, BOXP = S::BOXP, NBOX = S::NBOX, NRES = 1 << KP;
     // staging index of (residue rr, tile position p): [box][residue][BOXP]
     auto sidx = [](int rr, int p) { return (p / BOXP) * (NRES * BOXP) + rr * BOXP + p % BOXP; };
@@ -330,7 +344,7 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
         if constexpr (KP >= 4) reg_level_w<T, R, 8, 32>(ra, rc, rd);
         }
         if constexpr (TSTORE) {  // tbuf is written next: the previous tile's TMA store must have read it
-            if (t == 0) bulk_wait_read0();
+            if (WST ? lane == 0 : t == 0) bulk_wait_read0();  // WST: each warp's own stores
             __syncthreads();
         }
         if constexpr (KP <= 4) {
@@ -475,6 +489,41 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
             if constexpr (KQ >= 4) reg_level_w<T, R, 8, CH>(ra, rc, rd);
             }
             // member LEFT + 16(b-1) + u is row t0 + 16(16(b-1) + u) + rho
+            if constexpr (WST) {
+                // this warp's outputs (residues rho + 16 mu, mu < NQ, positions 0..PT) into its
+                // own class rows ([mu][PT] from the first 128-byte boundary of row rho: only this
+                // warp reads these rows, apart from halo lanes whose values are discarded), then
+                // one 5-D tensor store per array by lane 0 -- no CTA barrier
+                constexpr int CW = Tr34<T>::C, AW = 16 * CW, PT = S::PT;
+                static_assert(NQ * PT + 31 <= CW, "a warp's staging fits its class row");
+                T *wb = tbuf + ((rho * CW + 31) & ~31);
+                if (b >= 1 && b <= NB) {
+#pragma unroll
+                    for (int mu = 0; mu < NQ; ++mu) {  // residue rho + 16 mu, positions G(b-1) + q
+                        T va[G], vc[G], vd[G];
+#pragma unroll
+                        for (int q = 0; q < G; ++q) {
+                            va[q] = ra[mu + NQ * q];
+                            vc[q] = rc[mu + NQ * q];
+                            vd[q] = rd[mu + NQ * q];
+                        }
+                        const int o = mu * PT + G * (b - 1);
+                        store_run<T, G>(wb + o, va);
+                        store_run<T, G>(wb + AW + o, vc);
+                        store_run<T, G>(wb + 2 * AW + o, vd);
+                    }
+                }
+                fence_proxy_async_smem();  // generic-proxy smem writes -> visible to the TMA
+                __syncwarp();
+                if (lane == 0 && !TDS_ABL(4)) {
+                    const int j0 = int(t0 >> KP), r = int(sigma & ((int64_t(1) << kprev) - 1)),
+                              sys = int(sigma >> kprev);
+#pragma unroll
+                    for (int q = 0; q < 3; ++q) tma_store_5d(&tmo.m[q], wb + q * AW, j0, r, rho, 0, sys);
+                    bulk_commit();
+                }
+                continue;
+            }
             if constexpr (TSTORE) {
                 __syncthreads();  // every layout-B read of tbuf is done: reuse it as the staging buffer
                 if (b >= 1 && b <= NB) {
@@ -530,7 +579,7 @@ __global__ void __launch_bounds__(NT, (sizeof(T) == 4 && NT == 256) ? 2 : 1)
         }
     }
     if constexpr (TSTORE) {
-        if (t == 0) bulk_wait_all();
+        if (WST ? lane == 0 : t == 0) bulk_wait_all();
     }
 }
 
@@ -597,10 +646,14 @@ static cudaError_t launch_sp(const SplitArgs<T> &A, int64_t m_in, int64_t max_le
     } else if constexpr (S::template tstore<T>()) {  // output view {position, r, rho, system}
         T *outs[3] = {A.oa, A.oc, A.od};
         const int64_t msys = m_in >> kprev;
-        for (int q = 0; q < 3; ++q)
-            if (!encode_out_tmap(&tmo.m[q], outs[q], int(sizeof(T)), A.out_slot, int64_t(1) << kprev, int64_t(1) << KP,
-                                 msys, S::BOXP))
-                return cudaErrorInvalidValue;
+        for (int q = 0; q < 3; ++q) {
+            const bool ok = S::template wstore<T>()  // {position, r, rho mod 16, rho / 16, system}: one warp's box
+                                ? encode_out5_tmap(&tmo.m[q], outs[q], int(sizeof(T)), A.out_slot, int64_t(1) << kprev,
+                                                   int64_t(1) << KP, msys, S::BOXP)
+                                : encode_out_tmap(&tmo.m[q], outs[q], int(sizeof(T)), A.out_slot, int64_t(1) << kprev,
+                                                  int64_t(1) << KP, msys, S::BOXP);
+            if (!ok) return cudaErrorInvalidValue;
+        }
     }
     const int64_t grid = std::min<int64_t>(nitems, int64_t(std::max(occ, 1)) * sm_count_current());
 #ifdef TDS_SPLIT_ABLATION

@@ -50,6 +50,25 @@ bool encode_out_tmap(CUtensorMap *out, const void *base, int dsize, int64_t slot
     return r == CUDA_SUCCESS;
 }
 
+bool encode_out5_tmap(CUtensorMap *out, const void *base, int dsize, int64_t slot, int64_t nr, int64_t nrho,
+                      int64_t msys, int box_pos) {
+    const PFN_cuTensorMapEncodeTiled_v12000 fn = encode_fn();
+    if (!fn || slot < 1 || nr < 1 || nrho < 16 || nrho % 16 != 0 || nrho > 4096 || msys < 1 || box_pos < 1 ||
+        box_pos > 256)
+        return false;
+    const cuuint64_t ds = cuuint64_t(dsize);
+    const cuuint64_t dims[5] = {cuuint64_t(slot), cuuint64_t(nr), 16, cuuint64_t(nrho / 16), cuuint64_t(msys)};
+    const cuuint64_t strides[4] = {cuuint64_t(slot) * ds, cuuint64_t(slot * nr) * ds, cuuint64_t(slot * nr * 16) * ds,
+                                   cuuint64_t(slot * nr * nrho) * ds};
+    const cuuint32_t box[5] = {cuuint32_t(box_pos), 1, 1, cuuint32_t(nrho / 16), 1};
+    const cuuint32_t estr[5] = {1, 1, 1, 1, 1};
+    const CUresult r = fn(out, dsize == 4 ? CU_TENSOR_MAP_DATA_TYPE_FLOAT32 : CU_TENSOR_MAP_DATA_TYPE_FLOAT64, 5,
+                          const_cast<void *>(base), dims, strides, box, estr, CU_TENSOR_MAP_INTERLEAVE_NONE,
+                          CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_NONE,
+                          CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+    return r == CUDA_SUCCESS;
+}
+
 bool encode_box3_tmap(CUtensorMap *out, const void *base, int dsize, const uint64_t dims[3], const uint64_t strides[2],
                       const uint32_t box[3]) {
     const PFN_cuTensorMapEncodeTiled_v12000 fn = encode_fn();
